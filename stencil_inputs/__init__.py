@@ -1,0 +1,295 @@
+"""Seeded synthetic workloads shared by the oracle side and the CUDA side.
+
+This module holds NO stencil arithmetic.  It only says *what* is computed
+(extents, pad/slide arguments, boundary kinds, weights, op constants) and
+draws the seeded fp32 input grids.  Both ``oracle/`` (test infrastructure) and
+the CUDA path's tests/bench import it; neither imports the other.
+
+Workload recipe:
+  * grids are contiguous fp32, row-major, extents slowest-first (PAPER.md
+    P:336-337, ``[[T]_m]_n`` has n outermost);
+  * values come from ``numpy.random.default_rng(seed).random(shape, float32)``
+    (PCG64, U[0,1)) and are mapped affinely in fp32 per workload;
+  * seeds 1001..1007 follow SURVEY.md §8(d).
+
+Weights/constants are the readings A13, A14, A16, A18, A19, A20 of DESIGN.md
+(the paper prints none: Table 1, gives only dims/points/sizes).
+"""
+from __future__ import annotations
+
+from dataclasses import dataclass, field
+from typing import Dict, List, Optional, Sequence, Tuple
+
+import numpy as np
+
+# Boundary kinds — numeric values are the C-ABI enum ``stencil_pad``.
+CLAMP, MIRROR, WRAP, CONSTANT, REFLECT = 0, 1, 2, 3, 4
+KIND_NAMES = {CLAMP: "clamp", MIRROR: "mirror", WRAP: "wrap",
+              CONSTANT: "constant", REFLECT: "reflect"}
+
+# Ops — numeric values are the C-ABI enum ``stencil_op``.
+WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC = 0, 1, 2, 3, 4
+OP_NAMES = {WEIGHTED: "weighted", HOTSPOT3D: "hotspot3d", SRAD1: "srad1",
+            SRAD2: "srad2", ACOUSTIC: "acoustic"}
+
+# Number of input grids per op (zip arity).
+N_INPUTS = {WEIGHTED: 1, HOTSPOT3D: 2, SRAD1: 1, SRAD2: 2, ACOUSTIC: 2}
+
+
+@dataclass
+class StencilSpec:
+    """Arguments of ``map_n(f, slide_n(size, step, pad_n(l, r, h, input)))``
+     plus the op id/constants of the map function."""
+    extents: Tuple[int, ...]            # n_d, slowest first
+    size: Tuple[int, ...]               # slide size per dim
+    step: Tuple[int, ...]               # slide step per dim
+    pad_lo: Tuple[int, ...]             # pad l per dim
+    pad_hi: Tuple[int, ...]             # pad r per dim
+    kind: Tuple[int, ...]               # boundary function h per dim
+    pad_value: float = 0.0              # value for CONSTANT
+    op: int = WEIGHTED
+    weights: Optional[np.ndarray] = None    # float32, shape == size (WEIGHTED)
+    params: Tuple[float, ...] = ()          # float32 op constants
+
+    @property
+    def ndim(self) -> int:
+        return len(self.extents)
+
+    def out_extents(self) -> Tuple[int, ...]:
+        """o_d = floor((n_d + l_d + r_d - size_d) / step_d) + 1 (A6)."""
+        return tuple((n + l + r - s) // st + 1 for n, l, r, s, st in
+                     zip(self.extents, self.pad_lo, self.pad_hi, self.size, self.step))
+
+
+def f32(x) -> np.ndarray:
+    return np.asarray(x, dtype=np.float32)
+
+
+# --------------------------------------------------------------------------
+# Weights (A13, A14). Row-major over the neighbourhood, slowest dim
+# first, offset -r first.
+# --------------------------------------------------------------------------
+def weights_j2d5() -> np.ndarray:
+    """Jacobi 2D 5-point (A13): N=.10 W=.15 C=.45 E=.10 S=.20, asymmetric."""
+    return f32([[0.0, 0.10, 0.0],
+                [0.15, 0.45, 0.10],
+                [0.0, 0.20, 0.0]])
+
+
+def weights_j2d9() -> np.ndarray:
+    """Jacobi 2D 9-point (box), normalised, asymmetric (NEXT-1 shape)."""
+    w = np.array([[0.05, 0.10, 0.06],
+                  [0.12, 0.30, 0.08],
+                  [0.07, 0.14, 0.08]], dtype=np.float64)
+    return f32(w)
+
+
+def weights_j3d7() -> np.ndarray:
+    """Jacobi 3D 7-point star (A13): C=.40, z-1=.05, z+1=.15, y+-1=.10, x-1=.08, x+1=.12."""
+    w = np.zeros((3, 3, 3), np.float32)
+    w[1, 1, 1] = 0.40
+    w[0, 1, 1] = 0.05
+    w[2, 1, 1] = 0.15
+    w[1, 0, 1] = 0.10
+    w[1, 2, 1] = 0.10
+    w[1, 1, 0] = 0.08
+    w[1, 1, 2] = 0.12
+    return w
+
+
+def weights_j3d13() -> np.ndarray:
+    """Jacobi 3D 13-point star, radius 2 (A13): C=.28, +-1 taps .08, +-2 taps .04."""
+    w = np.zeros((5, 5, 5), np.float32)
+    w[2, 2, 2] = 0.28
+    for d in range(3):
+        for off, val in ((1, 0.08), (2, 0.04)):
+            for sgn in (-1, 1):
+                idx = [2, 2, 2]
+                idx[d] = 2 + sgn * off
+                w[tuple(idx)] = val
+    return w
+
+
+def weights_gauss5() -> np.ndarray:
+    """Gaussian 5x5 binomial [1,4,6,4,1] (x) [1,4,6,4,1] / 256 (A14); exact in fp32."""
+    b = np.array([1, 4, 6, 4, 1], np.float64)
+    return f32(np.outer(b, b) / 256.0)
+
+
+def weights_laplacian(ndim: int) -> np.ndarray:
+    """Discrete Laplacian (A13, tests only): centre -2*ndim, faces +1."""
+    w = np.zeros((3,) * ndim, np.float32)
+    c = (1,) * ndim
+    w[c] = -2.0 * ndim
+    for d in range(ndim):
+        for s in (0, 2):
+            idx = list(c)
+            idx[d] = s
+            w[tuple(idx)] = 1.0
+    return w
+
+
+# --------------------------------------------------------------------------
+# Op constants (A16, A18, A19, A20)
+# --------------------------------------------------------------------------
+def params_hotspot3d() -> Tuple[float, ...]:
+    """Rodinia v3.1 hotspot3D constants for a (8, 512, 512) chip (A16).
+    Order: cc, cn, cs, ce, cw, ct, cb, sdc, amb."""
+    ce = cw = cn = cs = 0.0341333
+    ct = cb = 5.33333e-4
+    cc = 1.0 - (2 * ce + 2 * cn + 3 * ct)
+    sdc = 0.341333
+    amb = 80.0
+    return tuple(float(np.float32(v)) for v in (cc, cn, cs, ce, cw, ct, cb, sdc, amb))
+
+
+def params_srad1(q0sqr: float) -> Tuple[float, ...]:
+    return (float(np.float32(q0sqr)),)
+
+
+def params_srad2(lam: float = 0.5) -> Tuple[float, ...]:
+    return (float(np.float32(lam)),)
+
+
+def params_acoustic(points: int) -> Tuple[float, ...]:
+    """(lambda^2, loss1, loss2) (A19/A20): zeta = 0.1, loss1 = 1/(1+zeta),
+    loss2 = 1 - zeta; lambda^2 = 0.25 (7-point) or 0.15 (13-point)."""
+    zeta = 0.1
+    l2 = 0.25 if points == 7 else 0.15
+    return tuple(float(np.float32(v)) for v in (l2, 1.0 / (1.0 + zeta), 1.0 - zeta))
+
+
+def srad_q0sqr(image: np.ndarray) -> float:
+    """Rodinia's q0sqr = var/mean^2 of the image (A18), computed once on the
+    host in fp64 from the input and passed to both sides as an fp32 param.
+    This is a workload parameter (a statistic of the input), not stencil work."""
+    x = image.astype(np.float64)
+    m = x.mean()
+    return float(np.float32(x.var() / (m * m)))
+
+
+# --------------------------------------------------------------------------
+# Seeded grids
+# --------------------------------------------------------------------------
+def uniform(shape: Sequence[int], seed: int, lo: float = 0.0, hi: float = 1.0) -> np.ndarray:
+    """U[lo, hi) fp32 from PCG64(seed); the affine map is done in fp32."""
+    rng = np.random.default_rng(seed)
+    u = rng.random(tuple(shape), dtype=np.float32)
+    if lo != 0.0 or hi != 1.0:
+        u *= np.float32(hi - lo)
+        u += np.float32(lo)
+    return u
+
+
+@dataclass
+class Workload:
+    """One named configuration: a spec plus how to draw its inputs."""
+    name: str
+    spec: StencilSpec
+    seeds: Tuple[int, ...]
+    ranges: Tuple[Tuple[float, float], ...]
+    steps: int = 1                      # time steps (iterate), 1 = single sweep
+    transform: Tuple[str, ...] = ()     # per-input post-transform ('exp' for SRAD)
+    note: str = ""
+
+    def make_inputs(self) -> List[np.ndarray]:
+        xs = []
+        for i, (seed, (lo, hi)) in enumerate(zip(self.seeds, self.ranges)):
+            x = uniform(self.spec.extents, seed, lo, hi)
+            if i < len(self.transform) and self.transform[i] == "exp":
+                x = np.exp(x).astype(np.float32)
+            xs.append(x)
+        return xs
+
+
+def _spec(extents, size, op=WEIGHTED, weights=None, params=(), kind=CLAMP,
+          pad=None, step=None, pad_value=0.0) -> StencilSpec:
+    nd = len(extents)
+    size = tuple(size) if isinstance(size, (tuple, list)) else (size,) * nd
+    r = tuple(s // 2 for s in size) if pad is None else (
+        tuple(pad) if isinstance(pad, (tuple, list)) else (pad,) * nd)
+    kind = tuple(kind) if isinstance(kind, (tuple, list)) else (kind,) * nd
+    step = (1,) * nd if step is None else tuple(step)
+    return StencilSpec(tuple(extents), size, step, r, r, kind, pad_value, op,
+                       None if weights is None else f32(weights), tuple(params))
+
+
+def workload(name: str, scale: Optional[Tuple[int, ...]] = None) -> Workload:
+    """Named workloads of BASELINE.json ``configs`` (C1..C5) and the
+    paper-shaped extras.  ``scale`` overrides the extents (parity-sized runs)."""
+    W = _WORKLOADS[name]
+    w = W()
+    if scale is not None:
+        w.spec.extents = tuple(scale)
+    return w
+
+
+def _c1():
+    return Workload("j2d5_256_clamp", _spec((256, 256), 3, weights=weights_j2d5()),
+                    (1001,), ((0.5, 1.5),), 1, note="C1: Jacobi 2D 5-point, clamp, single sweep")
+
+
+def _c2():
+    return Workload("gauss5_8192_mirror", _spec((8192, 8192), 5, weights=weights_gauss5(), kind=MIRROR),
+                    (1002,), ((0.5, 1.5),), 1, note="C2: Gaussian 5x5, mirror (symmetric), single sweep")
+
+
+def _c3():
+    return Workload("j3d7_512_clamp", _spec((512, 512, 512), 3, weights=weights_j3d7()),
+                    (1003,), ((0.5, 1.5),), 100, note="C3: Jacobi 3D 7-point, clamp, 100 time steps")
+
+
+def _c4a():
+    return Workload("hotspot3d_8x512x512", _spec((8, 512, 512), 3, op=HOTSPOT3D, params=params_hotspot3d()),
+                    (1004, 1005), ((300.0, 350.0), (0.0, 1e-2)), 1, note="C4a: Rodinia Hotspot3D, clamp")
+
+
+def _c4b1():
+    return Workload("srad1_4096", _spec((4096, 4096), 3, op=SRAD1), (1006,), ((0.0, 1.0),), 1,
+                    transform=("exp",), note="C4b: Rodinia SRAD1 (I -> c), clamp; q0sqr from the input")
+
+
+def _c4b2():
+    return Workload("srad2_4096", _spec((4096, 4096), 3, op=SRAD2, params=params_srad2()),
+                    (1008, 1006), ((0.0, 1.0), (0.0, 1.0)), 1, transform=("", "exp"),
+                    note="C4b: Rodinia SRAD2 ((c, I) -> I'), clamp")
+
+
+def _c5a():
+    return Workload("acoustic7_1024", _spec((1024, 1024, 1024), 3, op=ACOUSTIC, params=params_acoustic(7),
+                                           kind=CONSTANT, pad_value=0.0),
+                    (1007, 1007), ((-1.0, 1.0), (-1.0, 1.0)), 100,
+                    note="C5a: Acoustic 7-point (Listing 3), zero pad, prev = cur")
+
+
+def _c5b():
+    return Workload("acoustic13_1024", _spec((1024, 1024, 1024), 5, op=ACOUSTIC, params=params_acoustic(13),
+                                            kind=CONSTANT, pad_value=0.0),
+                    (1007, 1007), ((-1.0, 1.0), (-1.0, 1.0)), 100,
+                    note="C5b: Acoustic 13-point (A20 extrapolation), zero pad, prev = cur")
+
+
+_WORKLOADS = {
+    "j2d5_256_clamp": _c1,
+    "gauss5_8192_mirror": _c2,
+    "j3d7_512_clamp": _c3,
+    "hotspot3d_8x512x512": _c4a,
+    "srad1_4096": _c4b1,
+    "srad2_4096": _c4b2,
+    "acoustic7_1024": _c5a,
+    "acoustic13_1024": _c5b,
+}
+
+WORKLOAD_NAMES = tuple(_WORKLOADS)
+
+
+def make_workload_inputs(w: Workload) -> Tuple[List[np.ndarray], StencilSpec]:
+    """Draw inputs; fills input-derived params (SRAD1 q0sqr) into the spec."""
+    xs = w.make_inputs()
+    spec = w.spec
+    if spec.op == SRAD1:
+        spec.params = params_srad1(srad_q0sqr(xs[0]))
+    if spec.op == SRAD2:
+        # c must lie in [0, 1]; draw it as U[0,1) (seed 1008), I = exp(U).
+        pass
+    return xs, spec
