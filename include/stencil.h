@@ -1,0 +1,193 @@
+/*
+ * stencil.h — C ABI of the B200 Lift-stencil hot path.
+ *
+ * The operation is the paper's problem statement (§3.4):
+ *
+ *     out = map_n(f, slide_n(size, step, pad_n(l, r, h, input)))
+ *
+ *   pad  grows each dimension d by l_d on the left and r_d on
+ *                       the right; padded index j reads input[h_d(j - l_d, n_d)]
+ *                       (reindexing variant) or the constant pad_value
+ *                       (value variant).  h may differ per dimension.
+ *   slide  (P:467-479,  window o is padded indices o*step + k, k in [0,size);
+ *           P:567-630)  o_d in [0, floor((n_d + l_d + r_d - size_d)/step_d) + 1).
+ *   map  f is applied to every window; extra grids are zipped
+ *                       point-wise (zip; Listing 3).
+ *   iterate     repeats the step, feeding the output back.
+ *
+ * Conventions (all functions):
+ *   - grids are contiguous fp32, row-major, extents slowest-first
+ *     (``[[T]_m]_n`` has n outermost); ndim in {1, 2, 3};
+ *   - every grid pointer passed to apply/iterate is a DEVICE pointer owned by
+ *     the caller; weights/params are HOST pointers copied into the plan;
+ *   - ``stream`` is a cudaStream_t passed as void* (NULL = legacy default
+ *     stream); apply/apply_region/iterate are asynchronous, stream-ordered,
+ *     allocate nothing and are CUDA-graph capturable;
+ *   - every function returns a stencil_status; nothing aborts and no C++
+ *     exception crosses the ABI; stencil_last_error() gives a thread-local
+ *     message for the last failure.  Asynchronous kernel faults surface at the
+ *     caller's next synchronisation, as with any CUDA library.
+ *   - there is no CPU fallback: without a usable CUDA device every call that
+ *     launches work returns STENCIL_E_CUDA.
+ */
+#ifndef LIFT_STENCIL_H
+#define LIFT_STENCIL_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct stencil_plan_s* stencil_plan;   /* opaque, owned by the library */
+
+typedef enum {
+  STENCIL_OK = 0,
+  STENCIL_E_INVALID = 1,      /* argument violates the pad/slide/map types  */
+  STENCIL_E_UNSUPPORTED = 2,  /* valid, but not built (e.g. ndim > 3)        */
+  STENCIL_E_CUDA = 3,         /* a CUDA call or launch failed               */
+  STENCIL_E_NOMEM = 4
+} stencil_status;
+
+/* Boundary index functions h of pad (A1-A5). */
+typedef enum {
+  STENCIL_PAD_CLAMP = 0,      /* (i<0) ? 0 : ((i>=n) ? n-1 : i) */
+  STENCIL_PAD_MIRROR = 1,     /* symmetric, edge repeated (numpy 'symmetric')  A2 */
+  STENCIL_PAD_WRAP = 2,       /* ((i mod n) + n) mod n                         A3 */
+  STENCIL_PAD_CONSTANT = 3,   /* value variant of pad: pad_value              A4 */
+  STENCIL_PAD_REFLECT = 4     /* edge not repeated (numpy 'reflect')          A2 */
+} stencil_pad;
+
+/* Neighbourhood functions f of map (A13-A20). */
+typedef enum {
+  STENCIL_OP_WEIGHTED = 0,   /* sum_k w_k W[k], taps in row-major order; 1 input   */
+  STENCIL_OP_HOTSPOT3D = 1,  /* Rodinia hotspot3D (A16): inputs {T (slid), P};
+                                params {cc,cn,cs,ce,cw,ct,cb,sdc,amb}; 3D, size 3  */
+  STENCIL_OP_SRAD1 = 2,      /* Rodinia SRAD kernel 1 (A18): input {I} -> c;
+                                params {q0sqr}; 2D, size 3                         */
+  STENCIL_OP_SRAD2 = 3,      /* Rodinia SRAD kernel 2 (A18): inputs {c, I} -> I';
+                                params {lambda}; 2D, size 3                        */
+  STENCIL_OP_ACOUSTIC = 4    /* Listing 3 (A19/A20): inputs {prev
+                                (point-wise), cur (slid)} -> next; params
+                                {lambda^2, loss1, loss2}; 3D, size 3 (7-pt) or
+                                5 (13-pt); ``out`` may alias ``prev``              */
+} stencil_op;
+
+/* Which kernel family executes a plan (stencil_plan_variant). */
+typedef enum {
+  STENCIL_VARIANT_AUTO = -1,
+  STENCIL_VARIANT_GENERIC = 0,   /* K0: one thread per output, remapped loads  */
+  STENCIL_VARIANT_TILE2D = 1,    /* K1: TMA halo tile, 2D                       */
+  STENCIL_VARIANT_SWEEP3D = 2    /* K2: TMA plane ring, 2.5D sweep along z      */
+} stencil_variant;
+
+/*
+ * Create a plan for one stencil.
+ *   out        : receives the plan handle (NULL on failure).
+ *   device     : CUDA device ordinal the plan's launches target.
+ *   ndim       : 1, 2 or 3.
+ *   extents    : [ndim] input extents n_d, slowest first, each >= 1.
+ *   size, step : [ndim] slide(size_d, step_d), each >= 1.
+ *   pad_lo/hi  : [ndim] pad(l_d, r_d), each >= 0; n_d + l_d + r_d >= size_d.
+ *   kind       : [ndim] stencil_pad per dimension.
+ *   pad_value  : value for STENCIL_PAD_CONSTANT dimensions.
+ *   op         : stencil_op.
+ *   weights    : host, prod(size) floats, row-major over the window (tap k is
+ *                padded index o*step + k: cross-correlation, reading A7);
+ *                required for WEIGHTED (at most 125 non-zero taps), NULL
+ *                otherwise; copied.
+ *   params     : host, n_params op constants (see stencil_op); copied.
+ * Errors: E_INVALID for any type violation listed above, a wrong op/ndim
+ * combination or a NULL weights pointer for WEIGHTED; E_UNSUPPORTED for
+ * ndim > 3 or more than 125 non-zero taps.
+ */
+stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim,
+                                   const int64_t* extents, const int32_t* size,
+                                   const int32_t* step, const int32_t* pad_lo,
+                                   const int32_t* pad_hi, const int32_t* kind,
+                                   float pad_value, int32_t op,
+                                   const float* weights, const float* params,
+                                   int32_t n_params);
+
+/* Output extents o_d = floor((n_d + l_d + r_d - size_d) / step_d) + 1. */
+stencil_status stencil_plan_output_extents(stencil_plan plan, int64_t* out_extents);
+
+/*
+ * Slab mode (multi-GPU decomposition along dimension 0, 3D plans only).
+ * The plan's extents are the OWNED slab (n0_local, n1, n2) of a global grid
+ * with n0 = global_n0 planes; the slab's first owned plane is global plane
+ * z_offset.  Every grid buffer passed to apply/iterate then holds
+ * n0_local + 2*ghost planes: ghost planes [0, ghost) precede the owned planes
+ * and [ghost + n0_local, n0_local + 2*ghost) follow them; pointers point at
+ * plane 0 of the allocation.  Output planes are written at the same offsets
+ * (owned planes only).  Planes outside the global domain are handled by pad
+ * against the GLOBAL extent; WRAP in dimension 0 reads the ghost planes (the
+ * caller fills them from the ring neighbour).  ghost >= max(pad_lo[0],
+ * pad_hi[0]); requires step[0] == 1 and output extents == input extents.
+ */
+stencil_status stencil_plan_set_slab(stencil_plan plan, int64_t z_offset,
+                                     int64_t global_n0, int32_t ghost);
+
+/* Force a kernel family (tests: tiling independence) or AUTO. E_UNSUPPORTED if
+ * the requested family cannot run this plan. */
+stencil_status stencil_plan_set_variant(stencil_plan plan, int32_t variant);
+/* The family AUTO (or the forced one) selects for the given pointers. */
+int32_t stencil_plan_variant(stencil_plan plan);
+
+/*
+ * out = map(f, slide(pad(inputs))) — one application.
+ *   inputs   : [n_inputs] device pointers (op arity, stencil_op).
+ *   out      : device pointer, output extents (slab: allocation layout).
+ * Errors: E_INVALID for wrong n_inputs, NULL pointers, or ``out`` aliasing a
+ * slid input; E_CUDA on launch failure.
+ */
+stencil_status stencil_apply(stencil_plan plan, const float* const* inputs,
+                             int32_t n_inputs, float* out, void* stream);
+
+/* Same, restricted to output planes [o0_begin, o0_end) of dimension 0
+ * (slab interior / boundary split).  Results are bitwise identical to the
+ * corresponding planes of stencil_apply. */
+stencil_status stencil_apply_region(stencil_plan plan, const float* const* inputs,
+                                    int32_t n_inputs, float* out, int64_t o0_begin,
+                                    int64_t o0_end, void* stream);
+
+/*
+ * iterate(in, f, n_steps) with the state rotation of reading A21:
+ *   WEIGHTED  : state {X0, X1}            X_{t+1} = S(X_t), ping-pong
+ *   HOTSPOT3D : state {T0, T1}, aux {P}   T_{t+1} = S(T_t, P)
+ *   ACOUSTIC  : state {prev, cur}         next overwrites prev; roles swap
+ * *result_index receives the index into ``state`` holding the newest grid.
+ * Requires output extents == input extents.
+ */
+stencil_status stencil_iterate(stencil_plan plan, float* const* state, int32_t n_state,
+                               const float* const* aux, int32_t n_aux, int32_t n_steps,
+                               void* stream, int32_t* result_index);
+
+/*
+ * End-to-end entry with HOST buffers (pinned or pageable): copies the state
+ * and aux grids host->device into plan-owned device buffers, runs
+ * stencil_iterate (n_steps >= 1; n_steps == 1 with a non-iterable op is one
+ * stencil_apply), copies the newest grid back to host_out (output extents),
+ * and synchronises ``stream``.  The device workspace is allocated on first
+ * use, kept by the plan and freed by stencil_plan_destroy.
+ */
+stencil_status stencil_run_host(stencil_plan plan, const float* const* host_state,
+                                int32_t n_state, const float* const* host_aux,
+                                int32_t n_aux, int32_t n_steps, float* host_out,
+                                void* stream);
+
+/* Frees the plan (host memory and any stencil_run_host workspace).  Safe once
+ * the caller has synchronised the plan's in-flight work. */
+void stencil_plan_destroy(stencil_plan plan);
+
+const char* stencil_status_string(stencil_status status);
+const char* stencil_last_error(void);
+
+/* Library build/version string. */
+const char* stencil_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+
+#endif /* LIFT_STENCIL_H */

@@ -1,0 +1,457 @@
+// api.cu — the C ABI of include/stencil.h: plan creation and validation
+// (the pad/slide/map types of PAPER.md P:416-422),
+// kernel-family dispatch, apply / apply_region / iterate / run_host.
+#include <cuda_runtime.h>
+
+#include <cstdio>
+#include <cstring>
+#include <new>
+#include <string>
+#include <vector>
+
+#include "../../include/stencil.h"
+#include "common.cuh"
+#include "launch.hpp"
+
+using namespace lift;
+
+struct stencil_plan_s {
+  int device = 0;
+  int ndim = 0;
+  int num_sms = 148;
+  StencilParams p{};
+  int64_t user_out_ext[3] = {0, 0, 0};
+  int32_t forced_variant = STENCIL_VARIANT_AUTO;
+  int32_t last_variant = STENCIL_VARIANT_GENERIC;
+  // stencil_run_host workspace (device)
+  std::vector<float*> ws;
+  size_t ws_elems = 0;
+};
+
+namespace {
+
+thread_local std::string g_last_error;
+
+stencil_status fail(stencil_status s, const std::string& msg) {
+  g_last_error = msg;
+  return s;
+}
+
+stencil_status cuda_fail(cudaError_t e, const char* what) {
+  g_last_error = std::string(what) + ": " + cudaGetErrorString(e);
+  return STENCIL_E_CUDA;
+}
+
+// Saves/restores the caller's current device around library calls.
+struct DeviceGuard {
+  int prev = -1;
+  cudaError_t err = cudaSuccess;
+  explicit DeviceGuard(int dev) {
+    err = cudaGetDevice(&prev);
+    if (err == cudaSuccess && prev != dev) err = cudaSetDevice(dev);
+  }
+  ~DeviceGuard() {
+    int cur = -1;
+    if (prev >= 0 && cudaGetDevice(&cur) == cudaSuccess && cur != prev) cudaSetDevice(prev);
+  }
+};
+
+int op_arity(int op) {
+  switch (op) {
+    case OP_WEIGHTED: return 1;
+    case OP_HOTSPOT3D: return 2;
+    case OP_SRAD1: return 1;
+    case OP_SRAD2: return 2;
+    case OP_ACOUSTIC: return 2;
+    default: return -1;
+  }
+}
+
+// index of the slid input(s) for aliasing checks: bit i set if input i is slid
+int slid_mask(int op) {
+  switch (op) {
+    case OP_WEIGHTED: return 1;
+    case OP_HOTSPOT3D: return 1;      // T slid, P point-wise
+    case OP_SRAD1: return 1;
+    case OP_SRAD2: return 3;          // c and I both slid
+    case OP_ACOUSTIC: return 2;       // prev point-wise, cur slid
+    default: return 0;
+  }
+}
+
+bool same_extents(const StencilParams& p) {
+  return p.o[0] == p.n[0] && p.o[1] == p.n[1] && p.o[2] == p.n[2];
+}
+
+bool aligned16(const void* ptr) { return (reinterpret_cast<uintptr_t>(ptr) & 15u) == 0; }
+
+int choose_variant(stencil_plan_s* pl, const float* in0, const float* in1, const float* out) {
+  const StencilParams& p = pl->p;
+  const bool ptr_ok = aligned16(in0) && (in1 == nullptr || aligned16(in1)) && aligned16(out);
+  auto want = [&](int v) {
+    if (v == STENCIL_VARIANT_SWEEP3D) return ptr_ok && sweep3d_supported(p);
+    if (v == STENCIL_VARIANT_TILE2D) return ptr_ok && tile2d_supported(p);
+    return v == STENCIL_VARIANT_GENERIC;
+  };
+  if (pl->forced_variant != STENCIL_VARIANT_AUTO)
+    return want(pl->forced_variant) ? pl->forced_variant : -1;
+  if (pl->ndim == 3 && want(STENCIL_VARIANT_SWEEP3D)) return STENCIL_VARIANT_SWEEP3D;
+  if (pl->ndim == 2 && want(STENCIL_VARIANT_TILE2D)) return STENCIL_VARIANT_TILE2D;
+  return STENCIL_VARIANT_GENERIC;
+}
+
+stencil_status launch(stencil_plan_s* pl, const StencilParams& p, const float* in0, const float* in1,
+                      float* out, cudaStream_t stream) {
+  const int v = choose_variant(pl, in0, in1, out);
+  if (v < 0) return fail(STENCIL_E_UNSUPPORTED, "forced kernel variant cannot run this plan/pointers");
+  pl->last_variant = v;
+  std::string err;
+  cudaError_t e;
+  switch (v) {
+    case STENCIL_VARIANT_SWEEP3D:
+      e = launch_sweep3d(p, in0, in1, out, stream, pl->num_sms, &err);
+      break;
+    case STENCIL_VARIANT_TILE2D:
+      e = launch_tile2d(p, in0, in1, out, stream, pl->num_sms, &err);
+      break;
+    default:
+      e = launch_generic(p, in0, in1, out, stream, pl->num_sms);
+  }
+  if (e != cudaSuccess) {
+    g_last_error = std::string("kernel launch failed: ") + cudaGetErrorString(e) + (err.empty() ? "" : " (" + err + ")");
+    return STENCIL_E_CUDA;
+  }
+  if (!err.empty()) return fail(STENCIL_E_CUDA, err);
+  return STENCIL_OK;
+}
+
+stencil_status check_inputs(stencil_plan_s* pl, const float* const* inputs, int32_t n_inputs,
+                            const float* out) {
+  const int ar = op_arity(pl->p.op);
+  if (n_inputs != ar) return fail(STENCIL_E_INVALID, "n_inputs does not match the op's arity");
+  if (!inputs || !out) return fail(STENCIL_E_INVALID, "NULL input/output pointer");
+  for (int i = 0; i < n_inputs; ++i)
+    if (!inputs[i]) return fail(STENCIL_E_INVALID, "NULL input pointer");
+  const int m = slid_mask(pl->p.op);
+  for (int i = 0; i < n_inputs; ++i)
+    if ((m >> i) & 1)
+      if (inputs[i] == out) return fail(STENCIL_E_INVALID, "output aliases a slid input");
+  return STENCIL_OK;
+}
+
+}  // namespace
+
+extern "C" {
+
+const char* stencil_version(void) { return "lift-stencil-b200 0.1 (sm_100a)"; }
+
+const char* stencil_status_string(stencil_status s) {
+  switch (s) {
+    case STENCIL_OK: return "ok";
+    case STENCIL_E_INVALID: return "invalid argument";
+    case STENCIL_E_UNSUPPORTED: return "unsupported";
+    case STENCIL_E_CUDA: return "CUDA error";
+    case STENCIL_E_NOMEM: return "out of memory";
+  }
+  return "unknown status";
+}
+
+const char* stencil_last_error(void) { return g_last_error.c_str(); }
+
+stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, const int64_t* extents,
+                                   const int32_t* size, const int32_t* step, const int32_t* pad_lo,
+                                   const int32_t* pad_hi, const int32_t* kind, float pad_value,
+                                   int32_t op, const float* weights, const float* params,
+                                   int32_t n_params) {
+  if (!out) return fail(STENCIL_E_INVALID, "out is NULL");
+  *out = nullptr;
+  if (ndim > 3) return fail(STENCIL_E_UNSUPPORTED, "ndim > 3 is not built");
+  if (ndim < 1) return fail(STENCIL_E_INVALID, "ndim must be 1, 2 or 3");
+  if (!extents || !size || !step || !pad_lo || !pad_hi || !kind)
+    return fail(STENCIL_E_INVALID, "NULL array argument");
+  if (op < 0 || op > OP_ACOUSTIC) return fail(STENCIL_E_INVALID, "unknown op");
+  if (n_params < 0 || n_params > kMaxParams || (n_params > 0 && !params))
+    return fail(STENCIL_E_INVALID, "bad params");
+
+  StencilParams p{};
+  const int off = 3 - ndim;
+  for (int d = 0; d < 3; ++d) {
+    p.n[d] = 1; p.size[d] = 1; p.step[d] = 1; p.lo[d] = 0; p.hi[d] = 0; p.kind[d] = PAD_CLAMP;
+  }
+  for (int d = 0; d < ndim; ++d) {
+    if (extents[d] < 1 || size[d] < 1 || step[d] < 1 || pad_lo[d] < 0 || pad_hi[d] < 0)
+      return fail(STENCIL_E_INVALID, "extents/size/step must be >= 1 and pads >= 0");
+    if (kind[d] < PAD_CLAMP || kind[d] > PAD_REFLECT) return fail(STENCIL_E_INVALID, "unknown pad kind");
+    if (extents[d] + pad_lo[d] + pad_hi[d] < size[d])
+      return fail(STENCIL_E_INVALID, "n + l + r < size: slide yields no window");
+    if (extents[d] > (int64_t)1 << 40 || size[d] > 4096 || pad_lo[d] > (1 << 20) || pad_hi[d] > (1 << 20))
+      return fail(STENCIL_E_INVALID, "extent/size/pad out of supported range");
+    p.n[off + d] = extents[d];
+    p.size[off + d] = size[d];
+    p.step[off + d] = step[d];
+    p.lo[off + d] = pad_lo[d];
+    p.hi[off + d] = pad_hi[d];
+    p.kind[off + d] = kind[d];
+  }
+  for (int d = 0; d < 3; ++d) p.o[d] = (p.n[d] + p.lo[d] + p.hi[d] - p.size[d]) / p.step[d] + 1;
+  p.row = p.n[2];
+  p.plane = p.n[1] * p.n[2];
+  p.pad_value = pad_value;
+  p.op = op;
+  p.z_off = 0;
+  p.gnz = p.n[0];
+  p.ghost = 0;
+  p.slab = 0;
+  p.reg0 = 0;
+  p.reg1 = p.o[0];
+  for (int i = 0; i < n_params; ++i) p.prm[i] = params[i];
+
+  // op-specific shape rules (stencil.h / DESIGN.md A16-A20)
+  auto centred = [&](int r) {
+    for (int d = off; d < 3; ++d)
+      if (p.size[d] != 2 * r + 1 || p.lo[d] != r || p.hi[d] != r || p.step[d] != 1) return false;
+    return true;
+  };
+  switch (op) {
+    case OP_WEIGHTED: {
+      if (!weights) return fail(STENCIL_E_INVALID, "WEIGHTED needs weights");
+      int64_t ntot = 1;
+      for (int d = 0; d < ndim; ++d) ntot *= size[d];
+      if (ntot > (int64_t)1 << 24) return fail(STENCIL_E_INVALID, "window too large");
+      int nt = 0;
+      const int64_t s1 = p.size[1], s2 = p.size[2];
+      for (int64_t k = 0; k < ntot; ++k) {
+        if (weights[k] == 0.0f) continue;
+        if (nt >= kMaxTaps) return fail(STENCIL_E_UNSUPPORTED, "more than 125 non-zero taps");
+        const int64_t kz = k / (s1 * s2), ky = (k / s2) % s1, kx = k % s2;
+        p.tap[nt][0] = (int16_t)kz;
+        p.tap[nt][1] = (int16_t)ky;
+        p.tap[nt][2] = (int16_t)kx;
+        p.w[nt] = weights[k];
+        ++nt;
+      }
+      p.ntaps = nt;
+      if (ntot <= kMaxTaps)
+        for (int64_t k = 0; k < ntot; ++k) p.wbox[k] = weights[k];
+      // radius for the fast kernels: symmetric centred window
+      int r = p.size[2] / 2;
+      p.radius = centred(r) ? r : -1;
+      break;
+    }
+    case OP_HOTSPOT3D:
+      if (ndim != 3 || !centred(1)) return fail(STENCIL_E_INVALID, "HOTSPOT3D needs ndim 3, size 3, pad 1, step 1");
+      if (n_params < 9) return fail(STENCIL_E_INVALID, "HOTSPOT3D needs 9 params");
+      p.radius = 1;
+      break;
+    case OP_SRAD1:
+    case OP_SRAD2:
+      if (ndim != 2 || !centred(1)) return fail(STENCIL_E_INVALID, "SRAD needs ndim 2, size 3, pad 1, step 1");
+      if (n_params < 1) return fail(STENCIL_E_INVALID, "SRAD needs 1 param");
+      p.radius = 1;
+      break;
+    case OP_ACOUSTIC:
+      if (ndim != 3 || !(centred(1) || centred(2)))
+        return fail(STENCIL_E_INVALID, "ACOUSTIC needs ndim 3, size 3 or 5, pad r, step 1");
+      if (n_params < 3) return fail(STENCIL_E_INVALID, "ACOUSTIC needs 3 params");
+      p.radius = p.size[2] / 2;
+      break;
+  }
+
+  stencil_plan_s* pl = new (std::nothrow) stencil_plan_s();
+  if (!pl) return fail(STENCIL_E_NOMEM, "plan allocation failed");
+  pl->device = device;
+  pl->ndim = ndim;
+  pl->p = p;
+  for (int d = 0; d < ndim; ++d) pl->user_out_ext[d] = p.o[off + d];
+  int sms = 0;
+  if (cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, device) == cudaSuccess && sms > 0)
+    pl->num_sms = sms;
+  else
+    cudaGetLastError();  // no device here: plan creation is host-only
+  *out = pl;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_output_extents(stencil_plan pl, int64_t* out_ext) {
+  if (!pl || !out_ext) return fail(STENCIL_E_INVALID, "NULL argument");
+  for (int d = 0; d < pl->ndim; ++d) out_ext[d] = pl->user_out_ext[d];
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_set_slab(stencil_plan pl, int64_t z_offset, int64_t global_n0, int32_t ghost) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  StencilParams& p = pl->p;
+  if (pl->ndim != 3) return fail(STENCIL_E_UNSUPPORTED, "slab mode is built for 3D plans");
+  if (!same_extents(p) || p.step[0] != 1) return fail(STENCIL_E_INVALID, "slab mode needs output extents == input extents and step 1");
+  if (ghost < p.lo[0] || ghost < p.hi[0]) return fail(STENCIL_E_INVALID, "ghost < pad in dimension 0");
+  if (z_offset < 0 || global_n0 < z_offset + p.n[0]) return fail(STENCIL_E_INVALID, "slab outside the global grid");
+  p.z_off = z_offset;
+  p.gnz = global_n0;
+  p.ghost = ghost;
+  p.slab = 1;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_set_variant(stencil_plan pl, int32_t variant) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  if (variant < STENCIL_VARIANT_AUTO || variant > STENCIL_VARIANT_SWEEP3D)
+    return fail(STENCIL_E_INVALID, "unknown variant");
+  if (variant == STENCIL_VARIANT_SWEEP3D && !sweep3d_supported(pl->p))
+    return fail(STENCIL_E_UNSUPPORTED, "SWEEP3D cannot run this plan");
+  if (variant == STENCIL_VARIANT_TILE2D && !tile2d_supported(pl->p))
+    return fail(STENCIL_E_UNSUPPORTED, "TILE2D cannot run this plan");
+  pl->forced_variant = variant;
+  return STENCIL_OK;
+}
+
+int32_t stencil_plan_variant(stencil_plan pl) {
+  if (!pl) return -1;
+  if (pl->forced_variant != STENCIL_VARIANT_AUTO) return pl->forced_variant;
+  const StencilParams& p = pl->p;
+  if (pl->ndim == 3 && sweep3d_supported(p)) return STENCIL_VARIANT_SWEEP3D;
+  if (pl->ndim == 2 && tile2d_supported(p)) return STENCIL_VARIANT_TILE2D;
+  return STENCIL_VARIANT_GENERIC;
+}
+
+stencil_status stencil_apply_region(stencil_plan pl, const float* const* inputs, int32_t n_inputs,
+                                    float* out, int64_t o0_begin, int64_t o0_end, void* stream) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  stencil_status s = check_inputs(pl, inputs, n_inputs, out);
+  if (s != STENCIL_OK) return s;
+  // region is along the plan's dimension 0 (the slowest user dimension)
+  const int off = 3 - pl->ndim;
+  if (off != 0) {
+    if (!(o0_begin == 0 && o0_end == pl->user_out_ext[0]))
+      return fail(STENCIL_E_UNSUPPORTED, "apply_region is built for 3D plans");
+    o0_begin = 0;            // canonical dimension 0 has extent 1
+    o0_end = pl->p.o[0];
+  }
+  if (o0_begin < 0 || o0_end > pl->p.o[0] || o0_begin > o0_end)
+    return fail(STENCIL_E_INVALID, "region outside the output extents");
+  if (o0_begin == o0_end) return STENCIL_OK;
+  DeviceGuard g(pl->device);
+  if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+  StencilParams p = pl->p;
+  p.reg0 = o0_begin;
+  p.reg1 = o0_end;
+  return launch(pl, p, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out, (cudaStream_t)stream);
+}
+
+stencil_status stencil_apply(stencil_plan pl, const float* const* inputs, int32_t n_inputs, float* out,
+                             void* stream) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  return stencil_apply_region(pl, inputs, n_inputs, out, 0, pl->user_out_ext[0], stream);
+}
+
+stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_state, const float* const* aux,
+                               int32_t n_aux, int32_t n_steps, void* stream, int32_t* result_index) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  const StencilParams& p = pl->p;
+  if (!same_extents(p)) return fail(STENCIL_E_INVALID, "iterate needs output extents == input extents");
+  if (n_steps < 0) return fail(STENCIL_E_INVALID, "n_steps < 0");
+  if (!state || n_state != 2) return fail(STENCIL_E_INVALID, "iterate needs 2 state buffers");
+  if (!state[0] || !state[1] || state[0] == state[1]) return fail(STENCIL_E_INVALID, "bad state buffers");
+  int ri = (p.op == OP_ACOUSTIC) ? 1 : 0;
+  if (p.op == OP_WEIGHTED) {
+    if (n_aux != 0) return fail(STENCIL_E_INVALID, "WEIGHTED iterate takes no aux grids");
+    for (int t = 0; t < n_steps; ++t) {
+      const float* in[1] = {state[ri]};
+      stencil_status s = stencil_apply(pl, in, 1, state[1 - ri], stream);
+      if (s != STENCIL_OK) return s;
+      ri = 1 - ri;
+    }
+  } else if (p.op == OP_HOTSPOT3D) {
+    if (n_aux != 1 || !aux || !aux[0]) return fail(STENCIL_E_INVALID, "HOTSPOT3D iterate needs aux {P}");
+    for (int t = 0; t < n_steps; ++t) {
+      const float* in[2] = {state[ri], aux[0]};
+      stencil_status s = stencil_apply(pl, in, 2, state[1 - ri], stream);
+      if (s != STENCIL_OK) return s;
+      ri = 1 - ri;
+    }
+  } else if (p.op == OP_ACOUSTIC) {
+    if (n_aux != 0) return fail(STENCIL_E_INVALID, "ACOUSTIC iterate takes no aux grids");
+    // state {prev, cur}: next overwrites prev, then roles swap (A21)
+    for (int t = 0; t < n_steps; ++t) {
+      const int prev = 1 - ri;
+      const float* in[2] = {state[prev], state[ri]};
+      stencil_status s = stencil_apply(pl, in, 2, state[prev], stream);
+      if (s != STENCIL_OK) return s;
+      ri = prev;
+    }
+  } else {
+    return fail(STENCIL_E_UNSUPPORTED, "iterate is built for WEIGHTED, HOTSPOT3D and ACOUSTIC");
+  }
+  if (result_index) *result_index = ri;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_run_host(stencil_plan pl, const float* const* host_state, int32_t n_state,
+                                const float* const* host_aux, int32_t n_aux, int32_t n_steps,
+                                float* host_out, void* stream) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  if (!host_state || !host_out || n_state < 1 || n_state > 2 || n_aux < 0 || n_aux > 1)
+    return fail(STENCIL_E_INVALID, "bad host buffers");
+  const StencilParams& p = pl->p;
+  DeviceGuard g(pl->device);
+  if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+  cudaStream_t st = (cudaStream_t)stream;
+  const size_t in_elems = (size_t)(p.n[0] + 2 * p.ghost) * p.plane;
+  const size_t out_elems = (size_t)(p.o[0] + 2 * p.ghost) * p.o[1] * p.o[2];
+  const size_t elems = in_elems > out_elems ? in_elems : out_elems;
+  const int nbuf = 4;  // state0, state1, aux0, out
+  if (pl->ws_elems < elems) {
+    for (float* b : pl->ws) cudaFree(b);
+    pl->ws.clear();
+    pl->ws_elems = 0;
+    for (int i = 0; i < nbuf; ++i) {
+      float* b = nullptr;
+      cudaError_t e = cudaMalloc(&b, elems * sizeof(float));
+      if (e != cudaSuccess) return cuda_fail(e, "cudaMalloc (run_host workspace)");
+      pl->ws.push_back(b);
+    }
+    pl->ws_elems = elems;
+  }
+  cudaError_t e;
+  for (int i = 0; i < n_state; ++i) {
+    e = cudaMemcpyAsync(pl->ws[i], host_state[i], in_elems * sizeof(float), cudaMemcpyHostToDevice, st);
+    if (e != cudaSuccess) return cuda_fail(e, "H2D copy");
+  }
+  for (int i = 0; i < n_aux; ++i) {
+    e = cudaMemcpyAsync(pl->ws[2], host_aux[i], in_elems * sizeof(float), cudaMemcpyHostToDevice, st);
+    if (e != cudaSuccess) return cuda_fail(e, "H2D copy");
+  }
+  const float* result = nullptr;
+  const bool iterable = (p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D || p.op == OP_ACOUSTIC) && same_extents(p);
+  if (iterable && (p.op != OP_ACOUSTIC || n_state == 2)) {
+    // WEIGHTED/HOTSPOT3D: state {X, scratch}; ACOUSTIC: state {prev, cur}
+    float* state[2] = {pl->ws[0], pl->ws[1]};
+    const float* aux[1] = {pl->ws[2]};
+    int32_t ri = 0;
+    stencil_status s = stencil_iterate(pl, state, 2, aux, n_aux, n_steps, stream, &ri);
+    if (s != STENCIL_OK) return s;
+    result = state[ri];
+  } else {
+    if (n_steps != 1) return fail(STENCIL_E_UNSUPPORTED, "run_host: op is not iterable; use n_steps = 1");
+    const float* in[2] = {pl->ws[0], n_state > 1 ? pl->ws[1] : (n_aux ? pl->ws[2] : nullptr)};
+    int nin = op_arity(p.op);
+    stencil_status s = stencil_apply(pl, in, nin, pl->ws[3], stream);
+    if (s != STENCIL_OK) return s;
+    result = pl->ws[3];
+  }
+  e = cudaMemcpyAsync(host_out, result, out_elems * sizeof(float), cudaMemcpyDeviceToHost, st);
+  if (e != cudaSuccess) return cuda_fail(e, "D2H copy");
+  e = cudaStreamSynchronize(st);
+  if (e != cudaSuccess) return cuda_fail(e, "stream synchronize");
+  return STENCIL_OK;
+}
+
+void stencil_plan_destroy(stencil_plan pl) {
+  if (!pl) return;
+  if (!pl->ws.empty()) {
+    DeviceGuard g(pl->device);
+    for (float* b : pl->ws) cudaFree(b);
+  }
+  delete pl;
+}
+
+}  // extern "C"

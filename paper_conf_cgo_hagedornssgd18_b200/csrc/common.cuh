@@ -1,0 +1,86 @@
+// common.cuh — launch parameters and index arithmetic shared by all kernels.
+//
+// The plan canonicalises every stencil to 3 dimensions (a 1D/2D grid gets
+// leading dimensions of extent 1, size 1, step 1, pad 0), so every kernel
+// indexes (z, y, x) with x contiguous.  Parameters travel by value as a
+// __grid_constant__ struct: the plan owns no device memory and plans never
+// share __constant__ symbols.
+#pragma once
+#include <cstdint>
+
+namespace lift {
+
+enum PadKind : int { PAD_CLAMP = 0, PAD_MIRROR = 1, PAD_WRAP = 2, PAD_CONSTANT = 3, PAD_REFLECT = 4 };
+enum OpKind : int { OP_WEIGHTED = 0, OP_HOTSPOT3D = 1, OP_SRAD1 = 2, OP_SRAD2 = 3, OP_ACOUSTIC = 4 };
+
+constexpr int kMaxTaps = 125;     // 5x5x5
+constexpr int kMaxParams = 16;
+constexpr int kMaxInputs = 2;
+
+struct StencilParams {
+  // canonical 3D geometry (index 0 = z, slowest)
+  int64_t n[3];          // owned input extents
+  int64_t o[3];          // output extents
+  int64_t row;           // elements per row (= n[2])
+  int64_t plane;         // elements per plane (= n[1]*n[2])
+  int32_t size[3], step[3], lo[3], hi[3];
+  int32_t kind[3];
+  float pad_value;
+  int32_t op;
+  int32_t radius;        // star/box radius for non-WEIGHTED ops and fast kernels
+  // slab mode along z (ghost == 0 and z_off == 0 and gnz == n[0] otherwise)
+  int64_t z_off;         // global index of owned plane 0
+  int64_t gnz;           // global extent of dimension 0
+  int32_t ghost;         // ghost planes before/after the owned ones in every buffer
+  int32_t slab;          // 1 when the plan is a slab of a larger grid
+  // output region along dimension 0: [reg0, reg1)
+  int64_t reg0, reg1;
+  // WEIGHTED: non-zero taps in row-major window order
+  int32_t ntaps;
+  int16_t tap[kMaxTaps][3];   // window index k per dimension
+  float w[kMaxTaps];
+  float wbox[kMaxTaps];        // dense row-major window weights (fast kernels)
+  float prm[kMaxParams];
+};
+
+// h(i, n) of the reindexing pad (A1-A5).
+// i is the unpadded index (padded index minus l).  Only called when i is out
+// of [0, n).
+__host__ __device__ __forceinline__ int64_t pad_remap(int64_t i, int64_t n, int kind) {
+  switch (kind) {
+    case PAD_CLAMP:
+      return i < 0 ? 0 : (i >= n ? n - 1 : i);
+    case PAD_MIRROR: {
+      if (i < 0) i = -1 - i;               // now i >= 0
+      const int64_t p = 2 * n;
+      i %= p;
+      return i >= n ? p - 1 - i : i;
+    }
+    case PAD_WRAP: {
+      i %= n;
+      return i < 0 ? i + n : i;
+    }
+    case PAD_REFLECT: {
+      if (n == 1) return 0;
+      const int64_t p = 2 * n - 2;
+      i %= p;
+      if (i < 0) i += p;
+      return i >= n ? p - i : i;
+    }
+    default:
+      return i;
+  }
+}
+
+// Local plane index (within a buffer of n0 + 2*ghost planes) of the input
+// plane with GLOBAL index gz, or -1 when the padded value is the constant.
+__host__ __device__ __forceinline__ int64_t plane_of(const StencilParams& p, int64_t gz) {
+  if (gz < 0 || gz >= p.gnz) {
+    if (p.kind[0] == PAD_CONSTANT) return -1;
+    if (!(p.slab && p.kind[0] == PAD_WRAP)) gz = pad_remap(gz, p.gnz, p.kind[0]);
+    // slab + wrap: ring neighbour's planes are in the ghosts
+  }
+  return gz - p.z_off + p.ghost;
+}
+
+}  // namespace lift

@@ -1,0 +1,32 @@
+// launch.hpp — host-side entry points of the kernel families (internal).
+#pragma once
+#include <cuda.h>
+#include <cuda_runtime.h>
+
+#include <cstdint>
+#include <string>
+
+#include "common.cuh"
+
+namespace lift {
+
+// K0 — generic remap kernel (any plan).
+cudaError_t launch_generic(const StencilParams& p, const float* in0, const float* in1, float* out,
+                           cudaStream_t stream, int num_sms);
+
+// TMA tensor-map encoder (cuTensorMapEncodeTiled through the runtime's
+// driver entry point; no -lcuda).  Returns false and sets ``err`` on failure.
+bool encode_tensor_map_3d(CUtensorMap* map, const float* base, int64_t nx, int64_t ny, int64_t nz,
+                          uint32_t box_x, uint32_t box_y, uint32_t box_z, std::string* err);
+
+// K2 — 3D TMA plane-ring z-sweep (weighted star/box r<=2, hotspot3d, acoustic).
+bool sweep3d_supported(const StencilParams& p);
+cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float* in1, float* out,
+                           cudaStream_t stream, int num_sms, std::string* err);
+
+// K1 — 2D TMA halo-tile kernel (weighted box r<=4, srad1, srad2).
+bool tile2d_supported(const StencilParams& p);
+cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,
+                          cudaStream_t stream, int num_sms, std::string* err);
+
+}  // namespace lift

@@ -1,0 +1,138 @@
+// ops.cuh — the neighbourhood functions f of map.
+//
+// Every kernel family (K0 generic, K1 2D tile, K2 3D sweep) evaluates f
+// through these functions, so each output point sees exactly the same fp32
+// operation sequence whatever kernel, tile shape or GPU count produced it
+// (tiling independence; A12).  The library is compiled
+// with -fmad=false: the only fused multiply-adds are the explicit __fmaf_rn
+// below, so the compiler cannot contract differently in different kernels.
+//
+// An accessor ``W`` exposes the window: ``W.template at<DZ, DY, DX>()`` is
+// the padded input at offset (DZ, DY, DX) from the window centre (for the
+// centred ops below); point-wise zipped inputs are passed as values.
+#pragma once
+#include "common.cuh"
+
+namespace lift {
+
+// ---- Hotspot3D (Rodinia v3.1 hotspot3D; A16) ---------------------
+// T' = cc*C + cn*N + cs*S + ce*E + cw*W + ct*T + cb*B + sdc*P + ct*amb
+// N = y-1, S = y+1, W = x-1, E = x+1, B = z-1, T = z+1.
+template <class Acc>
+__device__ __forceinline__ float op_hotspot3d(const Acc& T, float Pc, const float* prm) {
+  const float cc = prm[0], cn = prm[1], cs = prm[2], ce = prm[3], cw = prm[4];
+  const float ct = prm[5], cb = prm[6], sdc = prm[7], amb = prm[8];
+  float acc = __fmul_rn(cc, T.template at<0, 0, 0>());
+  acc = __fmaf_rn(cn, T.template at<0, -1, 0>(), acc);
+  acc = __fmaf_rn(cs, T.template at<0, 1, 0>(), acc);
+  acc = __fmaf_rn(ce, T.template at<0, 0, 1>(), acc);
+  acc = __fmaf_rn(cw, T.template at<0, 0, -1>(), acc);
+  acc = __fmaf_rn(ct, T.template at<1, 0, 0>(), acc);
+  acc = __fmaf_rn(cb, T.template at<-1, 0, 0>(), acc);
+  acc = __fmaf_rn(sdc, Pc, acc);
+  acc = __fmaf_rn(ct, amb, acc);
+  return acc;
+}
+
+// ---- SRAD kernel 1: I -> c (Rodinia v3.1 srad; A18) --------------
+template <class Acc>
+__device__ __forceinline__ float op_srad1(const Acc& I, const float* prm) {
+  const float q0 = prm[0];
+  const float Ic = I.template at<0, 0, 0>();
+  const float dN = __fsub_rn(I.template at<0, -1, 0>(), Ic);
+  const float dS = __fsub_rn(I.template at<0, 1, 0>(), Ic);
+  const float dW = __fsub_rn(I.template at<0, 0, -1>(), Ic);
+  const float dE = __fsub_rn(I.template at<0, 0, 1>(), Ic);
+  float g = __fmul_rn(dN, dN);
+  g = __fadd_rn(g, __fmul_rn(dS, dS));
+  g = __fadd_rn(g, __fmul_rn(dW, dW));
+  g = __fadd_rn(g, __fmul_rn(dE, dE));
+  const float G2 = __fdiv_rn(g, __fmul_rn(Ic, Ic));
+  const float L = __fdiv_rn(__fadd_rn(__fadd_rn(__fadd_rn(dN, dS), dW), dE), Ic);
+  const float num = __fsub_rn(__fmul_rn(0.5f, G2), __fmul_rn(0.0625f, __fmul_rn(L, L)));
+  const float den = __fadd_rn(1.0f, __fmul_rn(0.25f, L));
+  const float q = __fdiv_rn(num, __fmul_rn(den, den));
+  const float d = __fdiv_rn(__fsub_rn(q, q0), __fmul_rn(q0, __fadd_rn(1.0f, q0)));
+  float c = __fdiv_rn(1.0f, __fadd_rn(1.0f, d));
+  c = c < 0.0f ? 0.0f : (c > 1.0f ? 1.0f : c);
+  return c;
+}
+
+// ---- SRAD kernel 2: (c, I) -> I' (Rodinia v3.1 srad; A18) --------
+template <class AccC, class AccI>
+__device__ __forceinline__ float op_srad2(const AccC& C, const AccI& I, const float* prm) {
+  const float lam = prm[0];
+  const float Ic = I.template at<0, 0, 0>();
+  const float dN = __fsub_rn(I.template at<0, -1, 0>(), Ic);
+  const float dS = __fsub_rn(I.template at<0, 1, 0>(), Ic);
+  const float dW = __fsub_rn(I.template at<0, 0, -1>(), Ic);
+  const float dE = __fsub_rn(I.template at<0, 0, 1>(), Ic);
+  const float cC = C.template at<0, 0, 0>();
+  const float cS = C.template at<0, 1, 0>();
+  const float cE = C.template at<0, 0, 1>();
+  float D = __fmul_rn(cC, dN);
+  D = __fmaf_rn(cS, dS, D);
+  D = __fmaf_rn(cC, dW, D);
+  D = __fmaf_rn(cE, dE, D);
+  return __fmaf_rn(__fmul_rn(0.25f, lam), D, Ic);
+}
+
+// ---- Acoustic (Listing 3; A19/A20) --------------------
+// next = cf(K,l1) * ((2 - l2*K)*u_c + l2*sum_nbr u - cf(K,l2loss)*prev)
+// Neighbours are summed in row-major tap order (Listing 3 lines 5-6).
+template <int R, class Acc>
+__device__ __forceinline__ float acoustic_sum(const Acc& U) {
+  float s;
+  if constexpr (R == 1) {
+    s = U.template at<-1, 0, 0>();
+    s = __fadd_rn(s, U.template at<0, -1, 0>());
+    s = __fadd_rn(s, U.template at<0, 0, -1>());
+    s = __fadd_rn(s, U.template at<0, 0, 1>());
+    s = __fadd_rn(s, U.template at<0, 1, 0>());
+    s = __fadd_rn(s, U.template at<1, 0, 0>());
+  } else {
+    s = U.template at<-2, 0, 0>();
+    s = __fadd_rn(s, U.template at<-1, 0, 0>());
+    s = __fadd_rn(s, U.template at<0, -2, 0>());
+    s = __fadd_rn(s, U.template at<0, -1, 0>());
+    s = __fadd_rn(s, U.template at<0, 0, -2>());
+    s = __fadd_rn(s, U.template at<0, 0, -1>());
+    s = __fadd_rn(s, U.template at<0, 0, 1>());
+    s = __fadd_rn(s, U.template at<0, 0, 2>());
+    s = __fadd_rn(s, U.template at<0, 1, 0>());
+    s = __fadd_rn(s, U.template at<0, 2, 0>());
+    s = __fadd_rn(s, U.template at<1, 0, 0>());
+    s = __fadd_rn(s, U.template at<2, 0, 0>());
+  }
+  return s;
+}
+
+// Number of star neighbours (+-1..+-R per axis) inside the global domain
+// (computeNumNeighbors): generated on the fly, 0 bytes.
+template <int R>
+__device__ __forceinline__ int acoustic_K(int64_t gz, int64_t gy, int64_t gx, int64_t nz,
+                                          int64_t ny, int64_t nx) {
+  int K = 0;
+#pragma unroll
+  for (int off = 1; off <= R; ++off) {
+    K += (gz - off >= 0) + (gz + off < nz);
+    K += (gy - off >= 0) + (gy + off < ny);
+    K += (gx - off >= 0) + (gx + off < nx);
+  }
+  return K;
+}
+
+template <int R, class Acc>
+__device__ __forceinline__ float op_acoustic(const Acc& U, float prev, int K, const float* prm) {
+  const float l2 = prm[0], loss1 = prm[1], loss2 = prm[2];
+  constexpr int kmax = 6 * R;
+  const float cf1 = K < kmax ? loss1 : 1.0f;
+  const float cf2 = K < kmax ? loss2 : 1.0f;
+  const float s = acoustic_sum<R>(U);
+  float t = __fmul_rn(__fsub_rn(2.0f, __fmul_rn(l2, (float)K)), U.template at<0, 0, 0>());
+  t = __fmaf_rn(l2, s, t);
+  t = __fmaf_rn(-cf2, prev, t);
+  return __fmul_rn(cf1, t);
+}
+
+}  // namespace lift

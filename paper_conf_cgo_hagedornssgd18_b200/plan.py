@@ -1,0 +1,145 @@
+"""Torch-facing convenience layer over the C ABI (device memory and streams
+only — PyTorch is plumbing here; all stencil work runs in libstencil.so).
+
+    plan = Plan(extents=(512, 512, 512), size=3, pad=1, kind="clamp",
+                op="weighted", weights=w)
+    y = plan.apply(x)                      # x: contiguous fp32 CUDA tensor
+    idx = plan.iterate([x, scratch], n_steps=100)
+"""
+from __future__ import annotations
+
+from typing import Optional, Sequence, Union
+
+import numpy as np
+import torch
+
+from . import _lib as L
+
+KINDS = {"clamp": L.PAD_CLAMP, "mirror": L.PAD_MIRROR, "symmetric": L.PAD_MIRROR, "wrap": L.PAD_WRAP,
+         "constant": L.PAD_CONSTANT, "zero": L.PAD_CONSTANT, "reflect": L.PAD_REFLECT}
+OPS = {"weighted": L.OP_WEIGHTED, "hotspot3d": L.OP_HOTSPOT3D, "srad1": L.OP_SRAD1, "srad2": L.OP_SRAD2,
+       "acoustic": L.OP_ACOUSTIC}
+VARIANTS = {"auto": L.VARIANT_AUTO, "generic": L.VARIANT_GENERIC, "tile2d": L.VARIANT_TILE2D,
+            "sweep3d": L.VARIANT_SWEEP3D}
+
+
+def _tuple(v, nd):
+    if isinstance(v, (list, tuple)):
+        assert len(v) == nd
+        return tuple(int(x) for x in v)
+    return (int(v),) * nd
+
+
+def _kind(k):
+    return KINDS[k] if isinstance(k, str) else int(k)
+
+
+def _stream_handle(stream: Optional[torch.cuda.Stream]) -> int:
+    s = stream if stream is not None else torch.cuda.current_stream()
+    return int(s.cuda_stream)
+
+
+class Plan:
+    """map_n(f, slide_n(size, step, pad_n(l, r, h, input)))."""
+
+    def __init__(self, extents: Sequence[int], size: Union[int, Sequence[int]] = 3,
+                 step: Union[int, Sequence[int]] = 1, pad: Union[None, int, Sequence[int]] = None,
+                 pad_hi: Union[None, int, Sequence[int]] = None, kind="clamp", pad_value: float = 0.0,
+                 op="weighted", weights=None, params: Sequence[float] = (), device: Optional[int] = None):
+        nd = len(extents)
+        self.ndim = nd
+        self.extents = tuple(int(e) for e in extents)
+        self.size = _tuple(size, nd)
+        self.step = _tuple(step, nd)
+        self.pad_lo = tuple(s // 2 for s in self.size) if pad is None else _tuple(pad, nd)
+        self.pad_hi = self.pad_lo if pad_hi is None and pad is not None else (
+            tuple(s - 1 - l for s, l in zip(self.size, self.pad_lo)) if pad_hi is None else _tuple(pad_hi, nd))
+        kinds = kind if isinstance(kind, (list, tuple)) else [kind] * nd
+        self.kind = tuple(_kind(k) for k in kinds)
+        self.pad_value = float(pad_value)
+        self.op = OPS[op] if isinstance(op, str) else int(op)
+        self.weights = None if weights is None else np.asarray(weights, np.float32)
+        self.params = tuple(float(p) for p in params)
+        self.device = torch.cuda.current_device() if device is None else int(device)
+        self.handle = L.stencil_plan_create(self.device, self.extents, self.size, self.step, self.pad_lo,
+                                            self.pad_hi, self.kind, self.pad_value, self.op, self.weights,
+                                            self.params)
+        self.out_extents = L.stencil_plan_output_extents(self.handle, nd)
+        self.ghost = 0
+        self.alloc_extents = self.extents
+        self.out_alloc_extents = self.out_extents
+
+    @classmethod
+    def from_spec(cls, spec, device: Optional[int] = None) -> "Plan":
+        """Build from a stencil_inputs.StencilSpec-like object (duck-typed)."""
+        return cls(spec.extents, spec.size, spec.step, spec.pad_lo, spec.pad_hi, list(spec.kind),
+                   spec.pad_value, spec.op, spec.weights, spec.params, device)
+
+    def set_slab(self, z_offset: int, global_n0: int, ghost: int):
+        L.stencil_plan_set_slab(self.handle, z_offset, global_n0, ghost)
+        self.ghost = int(ghost)
+        self.alloc_extents = (self.extents[0] + 2 * ghost,) + self.extents[1:]
+        self.out_alloc_extents = self.alloc_extents
+
+    def set_variant(self, variant):
+        L.stencil_plan_set_variant(self.handle, VARIANTS[variant] if isinstance(variant, str) else int(variant))
+
+    @property
+    def variant(self) -> int:
+        return L.stencil_plan_variant(self.handle)
+
+    def _check(self, t: torch.Tensor, shape, name):
+        if not isinstance(t, torch.Tensor) or not t.is_cuda:
+            raise TypeError(f"{name} must be a CUDA tensor (no CPU fallback)")
+        if t.dtype != torch.float32 or not t.is_contiguous():
+            raise TypeError(f"{name} must be contiguous float32")
+        if tuple(t.shape) != tuple(shape):
+            raise ValueError(f"{name} has shape {tuple(t.shape)}, expected {tuple(shape)}")
+
+    def empty_output(self) -> torch.Tensor:
+        return torch.empty(self.out_alloc_extents, dtype=torch.float32, device=f"cuda:{self.device}")
+
+    def apply(self, *inputs: torch.Tensor, out: Optional[torch.Tensor] = None,
+              stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+        for i, x in enumerate(inputs):
+            self._check(x, self.alloc_extents, f"input {i}")
+        if out is None:
+            out = self.empty_output()
+        self._check(out, self.out_alloc_extents, "out")
+        L.stencil_apply(self.handle, [x.data_ptr() for x in inputs], out.data_ptr(), _stream_handle(stream))
+        return out
+
+    def apply_region(self, *inputs: torch.Tensor, out: torch.Tensor, begin: int, end: int,
+                     stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+        for i, x in enumerate(inputs):
+            self._check(x, self.alloc_extents, f"input {i}")
+        self._check(out, self.out_alloc_extents, "out")
+        L.stencil_apply_region(self.handle, [x.data_ptr() for x in inputs], out.data_ptr(), begin, end,
+                               _stream_handle(stream))
+        return out
+
+    def iterate(self, state: Sequence[torch.Tensor], n_steps: int, aux: Sequence[torch.Tensor] = (),
+                stream: Optional[torch.cuda.Stream] = None) -> int:
+        for i, x in enumerate(list(state) + list(aux)):
+            self._check(x, self.alloc_extents, f"state/aux {i}")
+        return L.stencil_iterate(self.handle, [x.data_ptr() for x in state], [x.data_ptr() for x in aux],
+                                 n_steps, _stream_handle(stream))
+
+    def run_host(self, host_state: Sequence[np.ndarray], n_steps: int = 1,
+                 host_aux: Sequence[np.ndarray] = (), out: Optional[np.ndarray] = None,
+                 stream: Optional[torch.cuda.Stream] = None) -> np.ndarray:
+        if out is None:
+            out = np.empty(self.out_alloc_extents, np.float32)
+        L.stencil_run_host(self.handle, list(host_state), list(host_aux), n_steps, out, _stream_handle(stream))
+        return out
+
+    def close(self):
+        if getattr(self, "handle", None):
+            L.stencil_plan_destroy(self.handle)
+            self.handle = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass

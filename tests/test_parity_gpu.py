@@ -1,0 +1,300 @@
+"""GPU parity: the CUDA path (through the C ABI) against the fp64 oracle,
+element by element on seeded inputs, plus bitwise cross-kernel invariants.
+
+Tolerance (north_star; A22): max_p |g_p - o_p| / max(|o_p|, A_p)
+<= 1e-5 for one application, <= 1e-4 after 10 iterated steps (Acoustic,
+whose field changes sign: |g - o| <= 1e-4 * max|o|).
+"""
+import itertools
+
+import numpy as np
+import pytest
+import torch
+
+import stencil_inputs as si
+from oracle import stencil_oracle as orc
+from stencil_inputs import CLAMP, CONSTANT, MIRROR, REFLECT, WRAP
+
+pytestmark = pytest.mark.gpu
+
+TOL1 = 1e-5
+TOL10 = 1e-4
+KINDS = [CLAMP, MIRROR, WRAP, CONSTANT, REFLECT]
+
+
+@pytest.fixture(scope="module")
+def lift():
+    import __graft_entry__
+    __graft_entry__.build()
+    import paper_conf_cgo_hagedornssgd18_b200 as m
+    torch.cuda.set_device(0)
+    return m
+
+
+def spec(extents, size, weights=None, kind=CLAMP, lo=None, hi=None, step=None, value=0.0,
+         op=si.WEIGHTED, params=()):
+    nd = len(extents)
+    size = tuple(size) if isinstance(size, (tuple, list)) else (size,) * nd
+    lo = tuple(s // 2 for s in size) if lo is None else tuple(lo)
+    hi = tuple(s - 1 - l for s, l in zip(size, lo)) if hi is None else tuple(hi)
+    kind = (kind,) * nd if isinstance(kind, int) else tuple(kind)
+    step = (1,) * nd if step is None else tuple(step)
+    return si.StencilSpec(tuple(extents), size, step, lo, hi, kind, value, op,
+                          None if weights is None else si.f32(weights), tuple(params))
+
+
+def run_gpu(lift, sp, xs, variant=None):
+    plan = lift.Plan.from_spec(sp)
+    if variant is not None:
+        plan.set_variant(variant)
+    dev = [torch.from_numpy(np.ascontiguousarray(x)).cuda() for x in xs]
+    y = plan.apply(*dev)
+    torch.cuda.synchronize()
+    return y.cpu().numpy(), plan
+
+
+def check(lift, sp, xs, tol=TOL1, variant=None):
+    y, plan = run_gpu(lift, sp, xs, variant)
+    Y, A = orc.apply(sp, xs)
+    assert y.shape == Y.shape
+    err = orc.max_rel_err(y, Y, A)
+    assert err <= tol, f"max rel err {err:.3e} > {tol} (variant {plan.variant})"
+    return y, plan
+
+
+def rnd(shape, seed, lo=0.5, hi=1.5):
+    return si.uniform(shape, seed, lo, hi)
+
+
+# ------------------------------------------------------------- 1D ---------
+@pytest.mark.parametrize("kind", KINDS)
+def test_1d(lift, kind):
+    x = rnd((1001,), 1)
+    check(lift, spec((1001,), 3, [1, 1, 1], kind, value=0.25), [x])
+    check(lift, spec((1001,), 5, [0.1, -0.2, 0.5, 0.3, 0.7], kind, lo=(3,), hi=(1,), step=(2,), value=-1.5), [x])
+    check(lift, spec((7,), 4, [1, 2, 3, 4], kind, lo=(9,), hi=(6,), value=2.0), [rnd((7,), 2)])  # pad > n
+
+
+# ------------------------------------------------------------- 2D ---------
+@pytest.mark.parametrize("kind", KINDS)
+def test_2d_weighted(lift, kind):
+    x = rnd((67, 300), 3)
+    check(lift, spec(x.shape, 3, si.weights_j2d5(), kind, value=0.75), [x])
+    x = rnd((130, 516), 4)
+    check(lift, spec(x.shape, 5, si.weights_gauss5(), kind, value=0.75), [x])
+    check(lift, spec(x.shape, 3, si.weights_j2d9(), kind, value=0.75), [x])
+    w = np.random.default_rng(5).standard_normal((7, 9)).astype(np.float32)
+    check(lift, spec(x.shape, (7, 9), w, kind, value=0.75), [x])
+
+
+def test_2d_valid_asymmetric_strided(lift):
+    x = rnd((61, 203), 6)
+    w = np.random.default_rng(7).standard_normal((3, 4)).astype(np.float32)
+    check(lift, spec(x.shape, (3, 4), w, CLAMP, lo=(0, 0), hi=(0, 0)), [x])          # valid mode
+    check(lift, spec(x.shape, (3, 4), w, MIRROR, lo=(2, 0), hi=(1, 3)), [x])         # asymmetric
+    check(lift, spec(x.shape, (3, 4), w, (WRAP, CONSTANT), lo=(1, 2), hi=(1, 1), step=(2, 3), value=0.1), [x])
+
+
+def test_2d_mixed_kinds(lift):
+    x = rnd((70, 132), 8)
+    for k0, k1 in itertools.product(KINDS, KINDS):
+        check(lift, spec(x.shape, 5, si.weights_gauss5(), (k0, k1), value=-0.5), [x])
+
+
+def test_srad(lift):
+    I = np.exp(rnd((130, 260), 9, 0.0, 1.0)).astype(np.float32)
+    sp1 = spec(I.shape, 3, op=si.SRAD1, params=si.params_srad1(si.srad_q0sqr(I)))
+    c, _ = check(lift, sp1, [I])
+    assert c.min() >= 0 and c.max() <= 1
+    sp2 = spec(I.shape, 3, op=si.SRAD2, params=si.params_srad2())
+    check(lift, sp2, [c.astype(np.float32), I])
+    check(lift, sp2, [rnd(I.shape, 10, 0.0, 1.0), I])
+
+
+# ------------------------------------------------------------- 3D ---------
+@pytest.mark.parametrize("kind", KINDS)
+def test_3d_weighted(lift, kind):
+    x = rnd((37, 70, 260), 11)
+    check(lift, spec(x.shape, 3, si.weights_j3d7(), kind, value=0.3), [x])
+    x = rnd((21, 40, 132), 12)
+    check(lift, spec(x.shape, 5, si.weights_j3d13(), kind, value=0.3), [x])
+    w = np.random.default_rng(13).standard_normal((3, 3, 3)).astype(np.float32)
+    check(lift, spec(x.shape, 3, w, kind, value=0.3), [x])
+
+
+def test_3d_mixed_kinds(lift):
+    x = rnd((18, 22, 68), 14)
+    for ks in [(CLAMP, WRAP, MIRROR), (CONSTANT, CLAMP, WRAP), (WRAP, CONSTANT, REFLECT), (MIRROR, MIRROR, CONSTANT)]:
+        check(lift, spec(x.shape, 3, si.weights_j3d7(), ks, value=0.9), [x])
+        check(lift, spec(x.shape, 5, si.weights_j3d13(), ks, value=0.9), [x])
+
+
+def test_hotspot3d(lift):
+    T = rnd((8, 64, 132), 15, 300.0, 350.0)
+    P = rnd(T.shape, 16, 0.0, 1e-2)
+    check(lift, spec(T.shape, 3, op=si.HOTSPOT3D, params=si.params_hotspot3d()), [T, P])
+
+
+@pytest.mark.parametrize("pts,sz", [(7, 3), (13, 5)])
+def test_acoustic(lift, pts, sz):
+    u0 = rnd((20, 36, 132), 17, -1.0, 1.0)
+    u1 = rnd(u0.shape, 18, -1.0, 1.0)
+    check(lift, spec(u0.shape, sz, op=si.ACOUSTIC, params=si.params_acoustic(pts), kind=CONSTANT), [u0, u1])
+
+
+# ------------------------------------------------------ edge cases --------
+def test_degenerate_extents(lift):
+    for shape in [(1, 1, 4), (2, 3, 4), (1, 5, 8), (3, 1, 1)]:
+        x = rnd(shape, 19)
+        for kind in KINDS:
+            check(lift, spec(shape, 3, si.weights_j3d7(), kind, value=0.5), [x])
+    check(lift, spec((1, 4), 3, si.weights_j2d5(), MIRROR), [rnd((1, 4), 20)])
+
+
+def test_unaligned_and_odd_width_fall_back(lift):
+    x = rnd((20, 30, 66), 21)          # nx % 4 != 0
+    check(lift, spec(x.shape, 3, si.weights_j3d7(), CLAMP), [x])
+    big = torch.from_numpy(rnd((20 * 30 * 68 + 1,), 22)).cuda()
+    xin = big[1:].view(20, 30, 68)     # 4-byte aligned, not 16-byte aligned
+    sp = spec((20, 30, 68), 3, si.weights_j3d7(), CLAMP)
+    plan = lift.Plan.from_spec(sp)
+    y = plan.apply(xin).cpu().numpy()
+    Y, A = orc.apply(sp, [xin.cpu().numpy()])
+    assert orc.max_rel_err(y, Y, A) <= TOL1
+
+
+def test_alias_rejected(lift):
+    x = torch.from_numpy(rnd((8, 8, 8), 23)).cuda()
+    plan = lift.Plan.from_spec(spec((8, 8, 8), 3, si.weights_j3d7()))
+    with pytest.raises(lift.StencilError):
+        plan.apply(x, out=x)
+
+
+# ------------------------------------------ bitwise cross-kernel pins ------
+def _variants(plan_nd):
+    return ["generic", "tile2d"] if plan_nd == 2 else ["generic", "sweep3d"]
+
+
+@pytest.mark.parametrize("case", ["j2d5", "gauss", "j3d7", "j3d13", "hotspot", "acoustic13", "srad1", "srad2"])
+def test_kernel_families_bitwise_equal(lift, case):
+    """Tiling independence: every kernel family gives the same bits."""
+    rng = np.random.default_rng(24)
+    if case == "j2d5":
+        sp, xs = spec((130, 388), 3, si.weights_j2d5(), MIRROR), [rnd((130, 388), 25)]
+    elif case == "gauss":
+        sp, xs = spec((130, 388), 5, si.weights_gauss5(), WRAP), [rnd((130, 388), 26)]
+    elif case == "j3d7":
+        sp, xs = spec((19, 37, 264), 3, si.weights_j3d7(), CLAMP), [rnd((19, 37, 264), 27)]
+    elif case == "j3d13":
+        sp, xs = spec((19, 37, 136), 5, si.weights_j3d13(), REFLECT), [rnd((19, 37, 136), 28)]
+    elif case == "hotspot":
+        sp = spec((8, 40, 136), 3, op=si.HOTSPOT3D, params=si.params_hotspot3d())
+        xs = [rnd((8, 40, 136), 29, 300, 350), rnd((8, 40, 136), 30, 0, 1e-2)]
+    elif case == "acoustic13":
+        sp = spec((19, 37, 136), 5, op=si.ACOUSTIC, params=si.params_acoustic(13), kind=CONSTANT)
+        xs = [rnd((19, 37, 136), 31, -1, 1), rnd((19, 37, 136), 32, -1, 1)]
+    elif case == "srad1":
+        I = np.exp(rnd((130, 264), 33, 0, 1)).astype(np.float32)
+        sp, xs = spec(I.shape, 3, op=si.SRAD1, params=si.params_srad1(si.srad_q0sqr(I))), [I]
+    else:
+        I = np.exp(rnd((130, 264), 34, 0, 1)).astype(np.float32)
+        sp, xs = spec(I.shape, 3, op=si.SRAD2, params=si.params_srad2()), [rnd(I.shape, 35, 0, 1), I]
+    outs = []
+    for v in _variants(sp.ndim):
+        try:
+            y, _ = run_gpu(lift, sp, xs, v)
+        except lift.StencilError as e:
+            if e.status == 2:
+                continue           # family not built for this plan
+            raise
+        outs.append(y)
+    for y in outs[1:]:
+        np.testing.assert_array_equal(y, outs[0])
+
+
+def test_apply_region_pieces_bitwise(lift):
+    x = rnd((33, 40, 136), 36)
+    sp = spec(x.shape, 3, si.weights_j3d7(), CLAMP)
+    full, plan = run_gpu(lift, sp, [x])
+    xd = torch.from_numpy(x).cuda()
+    out = torch.full(x.shape, float("nan"), device="cuda")
+    for a, b in [(0, 1), (1, 7), (7, 32), (32, 33)]:
+        plan.apply_region(xd, out=out, begin=a, end=b)
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(out.cpu().numpy(), full)
+
+
+def test_constant_field_bitwise(lift):
+    for sp_ in [spec((9, 40, 132), 3, [[[0, 0, 0], [0, .125, 0], [0, 0, 0]],
+                                       [[0, .125, 0], [.125, .25, .125], [0, .125, 0]],
+                                       [[0, 0, 0], [0, .125, 0], [0, 0, 0]]], WRAP),
+                spec((70, 132), 5, si.weights_gauss5(), MIRROR)]:
+        x = np.full(sp_.extents, 0.8125, np.float32)
+        y, _ = run_gpu(lift, sp_, [x])
+        assert np.all(y == np.float32(0.8125))
+
+
+def test_wrap_translation_bitwise(lift):
+    x = rnd((16, 36, 132), 37)
+    sp = spec(x.shape, 3, si.weights_j3d7(), WRAP)
+    y, _ = run_gpu(lift, sp, [x])
+    ys, _ = run_gpu(lift, sp, [np.ascontiguousarray(np.roll(x, (3, -5, 8), axis=(0, 1, 2)))])
+    np.testing.assert_array_equal(ys, np.roll(y, (3, -5, 8), axis=(0, 1, 2)))
+
+
+# ------------------------------------------------------------ iterate -----
+def test_iterate_weighted_10_steps(lift):
+    x = rnd((24, 40, 136), 38)
+    sp = spec(x.shape, 3, si.weights_j3d7(), CLAMP)
+    plan = lift.Plan.from_spec(sp)
+    a = torch.from_numpy(x).cuda()
+    b = torch.empty_like(a)
+    ri = plan.iterate([a, b], 10)
+    g = (a, b)[ri].cpu().numpy()
+    ref = orc.iterate(sp, [x], [], 10)[0]
+    assert np.max(np.abs(g - ref) / np.abs(ref)) <= TOL10
+    # iterate == 10 x apply with the same rotation, bitwise
+    c = torch.from_numpy(x).cuda()
+    d = torch.empty_like(c)
+    for _ in range(10):
+        plan.apply(c, out=d)
+        c, d = d, c
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(c.cpu().numpy(), g)
+
+
+def test_iterate_hotspot_10_steps(lift):
+    T = rnd((8, 40, 136), 39, 300, 350)
+    P = rnd(T.shape, 40, 0, 1e-2)
+    sp = spec(T.shape, 3, op=si.HOTSPOT3D, params=si.params_hotspot3d())
+    plan = lift.Plan.from_spec(sp)
+    a, b, p = (torch.from_numpy(v).cuda() for v in (T, np.empty_like(T), P))
+    ri = plan.iterate([a, b], 10, aux=[p])
+    g = (a, b)[ri].cpu().numpy()
+    ref = orc.iterate(sp, [T], [P], 10)[0]
+    assert np.max(np.abs(g - ref) / np.abs(ref)) <= TOL10
+
+
+@pytest.mark.parametrize("pts,sz", [(7, 3), (13, 5)])
+def test_iterate_acoustic_10_steps(lift, pts, sz):
+    u = rnd((20, 36, 132), 41, -1, 1)
+    sp = spec(u.shape, sz, op=si.ACOUSTIC, params=si.params_acoustic(pts), kind=CONSTANT)
+    plan = lift.Plan.from_spec(sp)
+    a = torch.from_numpy(u).cuda()
+    b = torch.from_numpy(u.copy()).cuda()
+    ri = plan.iterate([a, b], 10)
+    g = (a, b)[ri].cpu().numpy()
+    ref = orc.iterate(sp, [u, u], [], 10)[1]
+    assert np.max(np.abs(g - ref)) <= TOL10 * np.max(np.abs(ref))
+
+
+def test_run_host_matches_device(lift):
+    x = rnd((24, 40, 136), 42)
+    sp = spec(x.shape, 3, si.weights_j3d7(), MIRROR)
+    plan = lift.Plan.from_spec(sp)
+    a = torch.from_numpy(x).cuda()
+    b = torch.empty_like(a)
+    ri = plan.iterate([a, b], 3)
+    dev = (a, b)[ri].cpu().numpy()
+    host = plan.run_host([x], n_steps=3)
+    np.testing.assert_array_equal(host, dev)
