@@ -11,9 +11,38 @@
 // the padded input at offset (DZ, DY, DX) from the window centre (for the
 // centred ops below); point-wise zipped inputs are passed as values.
 #pragma once
+#include <utility>
+
 #include "common.cuh"
 
 namespace lift {
+
+// compile-time loop: f(std::integral_constant<int, 0..N-1>) in order
+template <class F, int... Is>
+__device__ __forceinline__ void static_for_impl(F&& f, std::integer_sequence<int, Is...>) {
+  (f(std::integral_constant<int, Is>{}), ...);
+}
+template <int N, class F>
+__device__ __forceinline__ void static_for(F&& f) {
+  static_for_impl(f, std::make_integer_sequence<int, N>{});
+}
+
+// ---- WEIGHTED: sum_k w_k * W[k] over a centred (2RZ+1)x(2RY+1)x(2RX+1) window,
+// taps in row-major window order (the order K0 uses for its non-zero taps;
+// a zero-weight tap is an exact no-op: fma(0, x, acc) == acc for finite x).
+// STAR restricts the taps to the axes (7/13-point Jacobi); otherwise the box.
+template <int RZ, int RY, int RX, bool STAR, class Acc>
+__device__ __forceinline__ float op_weighted(const Acc& W, const float* wbox) {
+  constexpr int SZ = 2 * RZ + 1, SY = 2 * RY + 1, SX = 2 * RX + 1;
+  float acc = 0.0f;
+  static_for<SZ * SY * SX>([&](auto K) {
+    constexpr int k = decltype(K)::value;
+    constexpr int kz = k / (SY * SX), ky = (k / SX) % SY, kx = k % SX;
+    constexpr int nax = (kz != RZ) + (ky != RY) + (kx != RX);
+    if constexpr (!STAR || nax <= 1) acc = __fmaf_rn(wbox[k], W.template at<kz - RZ, ky - RY, kx - RX>(), acc);
+  });
+  return acc;
+}
 
 // ---- Hotspot3D (Rodinia v3.1 hotspot3D; A16) ---------------------
 // T' = cc*C + cn*N + cs*S + ce*E + cw*W + ct*T + cb*B + sdc*P + ct*amb

@@ -201,15 +201,30 @@ def test_kernel_families_bitwise_equal(lift, case):
         sp, xs = spec(I.shape, 3, op=si.SRAD2, params=si.params_srad2()), [rnd(I.shape, 35, 0, 1), I]
     outs = []
     for v in _variants(sp.ndim):
-        try:
-            y, _ = run_gpu(lift, sp, xs, v)
-        except lift.StencilError as e:
-            if e.status == 2:
-                continue           # family not built for this plan
-            raise
+        y, plan = run_gpu(lift, sp, xs, v)
+        assert plan.variant == lift.plan.VARIANTS[v]
         outs.append(y)
-    for y in outs[1:]:
-        np.testing.assert_array_equal(y, outs[0])
+    assert len(outs) == 2
+    np.testing.assert_array_equal(outs[1], outs[0])
+    Y, A = orc.apply(sp, xs)
+    assert orc.max_rel_err(outs[1], Y, A) <= TOL1
+
+
+def test_variant_selection(lift):
+    """AUTO must pick the TMA kernels for the configs' shapes (no silent K0)."""
+    cases = [(spec((64, 64, 128), 3, si.weights_j3d7()), "sweep3d"),
+             (spec((64, 64, 128), 5, si.weights_j3d13(), MIRROR), "sweep3d"),
+             (spec((8, 64, 128), 3, op=si.HOTSPOT3D, params=si.params_hotspot3d()), "sweep3d"),
+             (spec((16, 64, 128), 5, op=si.ACOUSTIC, params=si.params_acoustic(13), kind=CONSTANT), "sweep3d"),
+             (spec((64, 128), 3, si.weights_j2d5()), "tile2d"),
+             (spec((64, 128), 5, si.weights_gauss5(), MIRROR), "tile2d"),
+             (spec((64, 128), 3, op=si.SRAD1, params=(0.1,)), "tile2d"),
+             (spec((64, 128), 3, op=si.SRAD2, params=(0.5,)), "tile2d"),
+             (spec((64, 64, 130), 3, si.weights_j3d7()), "generic"),
+             (spec((64, 64, 128), 3, np.ones((3, 3, 3), np.float32)), "generic")]
+    for sp, v in cases:
+        plan = lift.Plan.from_spec(sp)
+        assert plan.variant == lift.plan.VARIANTS[v], (sp, v)
 
 
 def test_apply_region_pieces_bitwise(lift):
