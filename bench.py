@@ -1,0 +1,416 @@
+#!/usr/bin/env python
+"""Benchmark of the Lift-stencil hot path on B200 (driver contract).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--workload NAME] [--impl reference]
+
+Default workload: BASELINE.json config "Jacobi 3D 7-point, 512^3 fp32, clamp
+boundary, 100 time steps" — the config the metric's 1/2/4/8-GPU numbers are
+quoted on (north_star: iterated sweeps at 2/4/8 GPUs, weak scaling for the
+iterated 3D Jacobi).  One bench step = one full stencil_iterate of 100 time
+steps (pad -> slide -> map -> store, iterated) over 512^3 points per GPU.
+At N GPUs the global grid is (512*N, 512, 512), slab-decomposed along z with a
+per-time-step halo exchange (NCCL send/recv) overlapped with interior compute
+(weak scaling).  Inputs (512 MiB per grid) are larger than L2 (126 MB), so no
+L2 flush is needed between timed iterations.
+
+Other single-GPU workloads (--workload): the remaining BASELINE.json configs
+(gauss5_8192_mirror, j2d5_256_clamp, hotspot3d_8x512x512, srad1_4096,
+srad2_4096, acoustic7_1024, acoustic13_1024).
+
+Metric: stencil Gpoints/s = output points x time steps / time (PAPER.md
+P:958-959 "elements updated per second"); roofline: algorithmic HBM bytes per
+launch / average launch time vs MEASURED_PEAKS.json hbm_gbs.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "stencil Gpoints/s & achieved HBM GB/s vs 8 TB/s at 1/2/4/8 B200"
+
+# algorithmic (compulsory) HBM bytes per output point per launch
+BYTES_PER_POINT = {0: 8, 1: 12, 2: 8, 3: 12, 4: 12}
+KERNEL_NAME = {"j3d7_512_clamp": "k2_sweep", "acoustic7_1024": "k2_sweep", "acoustic13_1024": "k2_sweep",
+               "hotspot3d_8x512x512": "k2_sweep", "gauss5_8192_mirror": "k1_tile", "j2d5_256_clamp": "k1_tile",
+               "srad1_4096": "k1_tile", "srad2_4096": "k1_tile"}
+
+
+def env_int(k, d):
+    try:
+        return int(os.environ.get(k, d))
+    except ValueError:
+        return d
+
+
+def peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        with open(p) as f:
+            d = json.load(f)
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    return 6650.0, "fallback (B200_PROFILING.md)"
+
+
+def ncu_traffic(workload):
+    """dram bytes per launch of the dominant kernel from the committed ncu capture."""
+    p = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    if not os.path.exists(p):
+        return None
+    with open(p) as f:
+        d = json.load(f)
+    v = d.get(workload)
+    return None if v is None else v.get("dram_bytes_per_launch")
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons sampled during the timed region."""
+
+    Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+         "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, gpu_index):
+        self.idx = gpu_index
+        self.samples = []
+        self.stop = threading.Event()
+        self.t = threading.Thread(target=self.run, daemon=True)
+
+    def run(self):
+        while not self.stop.is_set():
+            try:
+                r = subprocess.run(["nvidia-smi", "-i", str(self.idx), f"--query-gpu={self.Q}",
+                                    "--format=csv,noheader,nounits"], capture_output=True, text=True, timeout=5)
+                vals = [v.strip() for v in r.stdout.strip().split(",")]
+                if len(vals) == 6:
+                    self.samples.append(vals)
+            except Exception:
+                pass
+            self.stop.wait(0.2)
+
+    def __enter__(self):
+        self.t.start()
+        return self
+
+    def __exit__(self, *a):
+        self.stop.set()
+        self.t.join(timeout=10)
+
+    def summary(self):
+        if not self.samples:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unsampled"], "samples": 0}
+        sm = [float(s[0]) for s in self.samples if s[0].replace(".", "").isdigit()]
+        mx = [float(s[1]) for s in self.samples if s[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for s in self.samples for i in range(4) if s[2 + i].lower() == "active"})
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": reasons, "samples": len(self.samples)}
+
+
+# ----------------------------------------------------------------------------
+# reference arm / cpu baseline: the fp64 oracle on a bounded sample
+# ----------------------------------------------------------------------------
+def oracle_sample_spec(workload):
+    """A bounded sub-grid of the workload (same op/kind/weights), ~seconds of CPU."""
+    import stencil_inputs as si
+    w = si.workload(workload)
+    ext = w.spec.extents
+    if len(ext) == 3:
+        sub = (min(ext[0], 16), min(ext[1], 512), min(ext[2], 512))
+    else:
+        sub = (min(ext[0], 1024), min(ext[1], 1024))
+    ws = si.workload(workload, scale=sub)
+    xs, spec = si.make_workload_inputs(ws)
+    return xs, spec, sub
+
+
+def time_oracle(workload, min_seconds=10.0, max_reps=50):
+    from oracle import stencil_oracle as orc
+    xs, spec, sub = oracle_sample_spec(workload)
+    pts = int(np.prod(spec.out_extents()))
+    reps = 0
+    t0 = time.perf_counter()
+    while True:
+        orc.apply(spec, xs)
+        reps += 1
+        el = time.perf_counter() - t0
+        if el >= min_seconds or reps >= max_reps:
+            break
+    gpts = pts * reps / el / 1e9
+    sample = f"{reps} x one sweep of a {'x'.join(map(str, sub))} sub-grid of {workload} (numpy fp64 oracle)"
+    return gpts, sample, el
+
+
+def reference_arm(args, workload):
+    rank = env_int("RANK", 0)
+    if rank != 0:
+        return
+    per_step = []
+    gp_all = []
+    for _ in range(args.warmup):
+        time_oracle(workload, min_seconds=0.0, max_reps=1)
+    sample = ""
+    for _ in range(args.steps):
+        gp, sample, el = time_oracle(workload, min_seconds=2.0, max_reps=20)
+        gp_all.append(gp)
+        per_step.append(el)
+    gpts = statistics.median(gp_all)
+    line = {"impl": "reference", "metric": METRIC, "value": gpts, "unit": "Gpoints/s", "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * statistics.median(per_step),
+            "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+            "config": {"workload": workload},
+            "cpu_baseline": {"value": gpts, "unit": "Gpoints/s", "cores": 1, "kind": "oracle", "sample": sample},
+            "e2e": {"value": gpts, "unit": "Gpoints/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+# ----------------------------------------------------------------------------
+# CUDA arm
+# ----------------------------------------------------------------------------
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--workload", default="j3d7_512_clamp")
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu", action="store_true")
+    args = ap.parse_args()
+    args.warmup = max(args.warmup, 3)
+
+    if args.impl == "reference":
+        reference_arm(args, args.workload)
+        return
+
+    import torch
+    import torch.distributed as dist
+
+    import stencil_inputs as si
+    import paper_conf_cgo_hagedornssgd18_b200 as lift
+    from paper_conf_cgo_hagedornssgd18_b200.slab import SlabPlan
+
+    world = env_int("WORLD_SIZE", 1)
+    rank = env_int("RANK", 0)
+    local = env_int("LOCAL_RANK", 0)
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device(f"cuda:{local}"))
+    dev = torch.device(f"cuda:{local}")
+
+    w = si.workload(args.workload)
+    steps_per_iter = w.steps
+    spec = w.spec
+    ext1 = spec.extents
+    iterable = spec.op in (si.WEIGHTED, si.HOTSPOT3D, si.ACOUSTIC) and steps_per_iter > 1
+    slabbed = world > 1 and iterable and len(ext1) == 3
+
+    # ---- inputs: seeded synthetic grids resident in HBM (host copies kept for e2e)
+    local_ext = ext1
+    if slabbed:
+        # weak scaling: the per-rank slab is the single-GPU workload
+        gext = (ext1[0] * world,) + tuple(ext1[1:])
+        ws = si.workload(args.workload)
+        ws.spec.extents = ext1
+        seeds = tuple(s + 7919 * rank for s in ws.seeds)
+        ws.seeds = seeds
+        xs, spec = si.make_workload_inputs(ws)
+    else:
+        ws = si.workload(args.workload)
+        ws.seeds = tuple(s + 7919 * rank for s in ws.seeds)
+        xs, spec = si.make_workload_inputs(ws)
+    npts_local = int(np.prod(spec.out_extents()))
+
+    if slabbed:
+        sp = SlabPlan(gext, rank, world, spec.size, spec.pad_lo, list(spec.kind), spec.pad_value, spec.op,
+                      spec.weights, spec.params, device=local)
+        plan = sp.plan
+        host = [torch.from_numpy(x).pin_memory() for x in xs]
+        bufs = []
+        for x in host:
+            b = sp.empty()
+            sp.owned(b).copy_(x, non_blocking=True)
+            bufs.append(b)
+    else:
+        plan = lift.Plan.from_spec(spec, device=local)
+        host = [torch.from_numpy(x).pin_memory() for x in xs]
+        bufs = [x.to(dev, non_blocking=True) for x in host]
+    torch.cuda.synchronize()
+
+    # state/aux layout per op
+    op = spec.op
+    if iterable:
+        if op == si.ACOUSTIC:
+            state = [bufs[0], bufs[1]]          # prev, cur
+            aux = []
+        elif op == si.HOTSPOT3D:
+            state = [bufs[0], torch.empty_like(bufs[0])]
+            aux = [bufs[1]]
+        else:
+            state = [bufs[0], torch.empty_like(bufs[0])]
+            aux = []
+        launches_per_step = steps_per_iter * (3 if slabbed else 1)
+    else:
+        out = plan.empty_output()
+        launches_per_step = 1
+
+    stream = torch.cuda.current_stream()
+
+    def step():
+        if iterable:
+            if slabbed:
+                return sp.iterate(state, steps_per_iter, aux)
+            return plan.iterate(state, steps_per_iter, aux)
+        plan.apply(*bufs, out=out)
+        return 0
+
+    def barrier():
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+
+    # warm-up
+    for _ in range(args.warmup):
+        step()
+    barrier()
+
+    # timed region: exactly K steps, barrier + sync on both sides, events on the launching stream
+    ev0 = torch.cuda.Event(enable_timing=True)
+    ev1 = torch.cuda.Event(enable_timing=True)
+    with ClockSampler(local) as clk:
+        barrier()
+        ev0.record(stream)
+        for _ in range(args.steps):
+            step()
+        ev1.record(stream)
+        barrier()
+    t_ms = ev0.elapsed_time(ev1)
+    t_max = t_ms
+    if world > 1:
+        tt = torch.tensor([t_ms], device=dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        t_max = float(tt.item())
+    ms_per_step = t_max / args.steps
+    points = npts_local * world * steps_per_iter * args.steps
+    value = points / (t_max * 1e-3) / 1e9
+
+    # per-launch kernel duration of the dominant kernel: a step is back-to-back
+    # launches of it on one stream (single GPU), so avg launch = step time / launches
+    bpp = BYTES_PER_POINT[op]
+    if not slabbed:
+        avg_launch_s = (t_ms * 1e-3) / (args.steps * launches_per_step)
+        alg_bytes = npts_local * bpp
+    else:
+        # time the owned-slab sweep alone (all planes in one launch) on this rank
+        e0 = torch.cuda.Event(enable_timing=True)
+        e1 = torch.cuda.Event(enable_timing=True)
+        nrep = 20
+        ins = (state[0],) + tuple(aux) if op != si.ACOUSTIC else (state[0], state[1])
+        dst = state[1] if op != si.ACOUSTIC else state[0]
+        e0.record(stream)
+        for _ in range(nrep):
+            plan.apply(*ins, out=dst)
+        e1.record(stream)
+        torch.cuda.synchronize()
+        avg_launch_s = e0.elapsed_time(e1) * 1e-3 / nrep
+        alg_bytes = npts_local * bpp
+    peak, peak_src = peaks()
+    achieved = alg_bytes / avg_launch_s / 1e9
+
+    # ---- e2e: the C-ABI call with HOST buffers (H2D + compute + D2H timed), single GPU path
+    e2e = None
+    if not args.no_e2e and not slabbed:
+        h_state = [x.numpy() for x in host]
+        h_aux = []
+        if op == si.HOTSPOT3D:                   # T is the state, P the fixed aux grid
+            h_state, h_aux = [host[0].numpy()], [host[1].numpy()]
+        out_h = torch.empty(plan.out_alloc_extents, dtype=torch.float32).pin_memory().numpy()
+        n_e2e = max(1, min(args.steps, 3))
+        nsteps = steps_per_iter if iterable else 1
+        plan.run_host(h_state, nsteps, h_aux, out=out_h)      # warm (workspace allocation)
+        torch.cuda.synchronize()
+        t0 = time.perf_counter()
+        for _ in range(n_e2e):
+            plan.run_host(h_state, nsteps, h_aux, out=out_h)
+        el = (time.perf_counter() - t0) / n_e2e
+        h2d = sum(a.nbytes for a in h_state) + sum(a.nbytes for a in h_aux)
+        e2e = {"value": npts_local * nsteps / el / 1e9, "unit": "Gpoints/s", "h2d_bytes_per_step": int(h2d),
+               "d2h_bytes_per_step": int(out_h.nbytes), "ms_per_step": el * 1e3,
+               "timing": "host wall clock around stencil_run_host (synchronising)"}
+    elif not args.no_e2e and slabbed:
+        # per rank: H2D of the owned slab(s) from pinned host memory, the slab
+        # iterate (with its halo exchange), D2H of the newest owned grid
+        n_e2e = max(1, min(args.steps, 3))
+        res_h = torch.empty(sp.owned(state[0]).shape, dtype=torch.float32).pin_memory()
+        def e2e_step():
+            for b, x in zip(bufs, host):
+                sp.owned(b).copy_(x, non_blocking=True)
+            ri = sp.iterate(state, steps_per_iter, aux)
+            res_h.copy_(sp.owned(state[ri]), non_blocking=True)
+        e2e_step()
+        barrier()
+        q0 = torch.cuda.Event(enable_timing=True)
+        q1 = torch.cuda.Event(enable_timing=True)
+        q0.record(stream)
+        for _ in range(n_e2e):
+            e2e_step()
+        q1.record(stream)
+        barrier()
+        te = q0.elapsed_time(q1)
+        tt = torch.tensor([te], device=dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        te = float(tt.item()) / n_e2e
+        h2d = sum(int(x.numel()) * 4 for x in host)
+        e2e = {"value": npts_local * world * steps_per_iter / (te * 1e-3) / 1e9, "unit": "Gpoints/s",
+               "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": int(res_h.numel()) * 4, "ms_per_step": te,
+               "timing": "CUDA events, max over ranks, pinned host buffers"}
+
+    # ---- cpu baseline: the oracle on a bounded sample (rank 0, N=1 only)
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu:
+        gp, sample, _ = time_oracle(args.workload, min_seconds=10.0, max_reps=20)
+        cpu = {"value": gp, "unit": "Gpoints/s", "cores": 1, "kind": "oracle", "sample": sample}
+
+    clocks = clk.summary()
+    if rank == 0:
+        line = {
+            "metric": METRIC, "value": value, "unit": "Gpoints/s", "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "weak",
+            "vs_baseline": None, "dtype": "f32", "data": "synthetic",
+            "config": {"workload": args.workload, "extents_per_gpu": list(ext1),
+                       "global_extents": list(gext) if slabbed else list(ext1),
+                       "time_steps_per_bench_step": steps_per_iter if iterable else 1,
+                       "op": si.OP_NAMES[op], "boundary": [si.KIND_NAMES[k] for k in spec.kind],
+                       "window": list(spec.size), "parallelism": f"slab-z x{world}" if slabbed else
+                       (f"replicas x{world}" if world > 1 else "single"),
+                       "l2": "inputs larger than L2 (no flush needed)" if npts_local * 4 > 126e6
+                       else "L2-resident working set (no flush; reported as such)",
+                       "variant": {0: "K0 generic", 1: "K1 tile2d (TMA)", 2: "K2 sweep3d (TMA)"}[plan.variant]},
+            "hbm_gbs_per_gpu_whole_step": value * bpp / world,
+            "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                         "frac": achieved / peak, "traffic": ncu_traffic(args.workload),
+                         "kernel": KERNEL_NAME.get(args.workload), "peak_source": peak_src,
+                         "alg_bytes_per_launch": alg_bytes, "avg_launch_us": avg_launch_s * 1e6,
+                         "frac_of_8TBs": achieved / 8000.0},
+            "cpu_baseline": cpu,
+            "e2e": e2e,
+            "gpu_launches": int(args.steps * launches_per_step),
+            "clocks": clocks,
+        }
+        print(json.dumps(line), flush=True)
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -97,10 +97,10 @@ __global__ void __launch_bounds__(256) k0_generic(const __grid_constant__ Stenci
         const float prev = __ldg(in0 + (g.oz + p.ghost) * p.plane + g.oy * p.row + g.ox);
         const int64_t gz = p.z_off + g.oz;
         if (p.radius == 1) {
-          const int K = acoustic_K<1>(gz, g.oy, g.ox, p.gnz, p.n[1], p.n[2]);
+          const int K = acoustic_K<1, int64_t>(gz, g.oy, g.ox, p.gnz, p.n[1], p.n[2]);
           v = op_acoustic<1>(CentredAcc{p, in1, g}, prev, K, p.prm);
         } else {
-          const int K = acoustic_K<2>(gz, g.oy, g.ox, p.gnz, p.n[1], p.n[2]);
+          const int K = acoustic_K<2, int64_t>(gz, g.oy, g.ox, p.gnz, p.n[1], p.n[2]);
           v = op_acoustic<2>(CentredAcc{p, in1, g}, prev, K, p.prm);
         }
         break;

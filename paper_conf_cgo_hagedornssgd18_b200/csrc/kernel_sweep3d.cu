@@ -1,36 +1,45 @@
 // kernel_sweep3d.cu — K2: the 3D stencil as a 2.5D sweep along z.
 //
-// slide_3 over a 3D grid: each CTA owns a 128 x TY tile of the
-// (y, x) plane and a chunk of consecutive output planes.  It streams the
-// input planes z-R .. z_end+R-1 through a ring of S shared-memory stages: one
-// elected producer thread issues one TMA tensor load per plane (a halo'd box
-// of (128+8) x (TY+2R) floats: x from x0-4 so the centre columns stay 16-B
-// aligned; y from y0-R), completing on the stage's mbarrier; 8 consumer warps
-// compute output plane z from stages z-R..z+R as soon as stage z+R lands,
-// then release stage z-R.  This is overlapped tiling with the
-// overlap size-step = 2R, staged in local (shared) memory, with
-// the z-overlap reused through the ring instead of re-read.
+// slide_3 over a 3D grid.  Work items are (z-chunk, 128 x TY tile
+// of the (y, x) plane) in chunk-major order; persistent CTAs (grid = SMs x
+// resident CTAs) draw items from a dynamic ticket counter, so the CTAs in
+// flight always work on neighbouring tiles of the same z range (their halo'd
+// boxes overlap in L2) and there is no tail wave.
 //
-// Inside a plane, lane l of warp w owns 4 consecutive x outputs of TY/8 rows:
-// the in-row neighbourhood comes from the neighbouring lanes' float4 through
-// warp shuffles (lanes 0/31 read the halo columns), the y and z neighbours
-// are 128-bit shared loads, and the 4 results leave as one st.global.v4.
+// Per CTA an elected producer thread streams the input planes of its items
+// (z-R .. z_end+R-1 per item) through an S-stage shared-memory ring: one TMA
+// tensor load per plane of a halo'd box of (128+8) x (TY+2R) floats (x from
+// x0-4 so the centre columns stay 16-B aligned; y from y0-R), completing on
+// the stage's mbarrier.  This is overlapped tiling with overlap
+// size-step = 2R, staged in local (shared) memory.
 //
-// pad is folded into the loads: the producer remaps the plane
-// index (h on z, or "constant plane" without a load); TMA zero-fills the
-// (y, x) cells outside the grid, and only edge tiles rewrite those halo cells
-// in shared memory with h-remapped values (or pad_value) before use.  The
-// neighbourhood function goes through ops.cuh, so every output has the bits
-// K0 computes.
+// 8 consumer warps: lane l of warp w owns 4 consecutive x outputs of TY/8
+// rows.  The centre float4 of every plane is read from shared memory once,
+// when the plane lands, into a per-thread register ring of 2R+1 planes (the
+// z-neighbours); when plane z is the centre, its y-neighbours are 128-bit
+// shared loads and its in-row neighbours come from the adjacent lanes by warp
+// shuffles (lanes 0/31 read the halo columns).  A plane's stage is released as
+// soon as it has served as the centre, so the ring needs only R+1 live stages
+// plus prefetch.  Results leave as one st.global.v4 per lane and row.
+//
+// pad is folded into index computation: the producer remaps the
+// plane index (or marks a constant plane, which is never loaded); inside a
+// plane, clamp / mirror / reflect / constant rows are redirected to the
+// remapped box row, and out-of-grid x taps are selected from the lane's own
+// registers; only WRAP in x or y rewrites the halo cells in shared memory from
+// global memory (halo.cuh).  f goes through ops.cuh: every output has exactly
+// the bits K0 computes.
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#include <atomic>
+#include <climits>
 #include <mutex>
 #include <string>
 
 #include "common.cuh"
-#include "launch.hpp"
 #include "halo.cuh"
+#include "launch.hpp"
 #include "ops.cuh"
 #include "tma.cuh"
 
@@ -43,6 +52,11 @@ constexpr int BX = TX + 2 * XH;
 constexpr int NW = 8;          // consumer warps
 constexpr int NCONS = NW * 32;
 constexpr unsigned FULL = 0xffffffffu;
+constexpr int kTickets = 4096;
+
+// dynamic work counters (one per in-flight launch slot; reset by the last CTA)
+__device__ unsigned int g_ticket[kTickets];
+__device__ unsigned int g_done[kTickets];
 
 enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2 };
 
@@ -50,18 +64,17 @@ template <int R, int RPW, int S>
 struct Cfg {
   static constexpr int TY = NW * RPW;
   static constexpr int BY = TY + 2 * R;
-  static constexpr int TX_BYTES = BX * BY * 4;                         // bytes one TMA box delivers
+  static constexpr int TX_BYTES = BX * BY * 4;
   static constexpr int STAGE_FLOATS = ((TX_BYTES + 127) / 128) * 128 / 4;
-  static constexpr int SMEM = S * STAGE_FLOATS * 4 + 2 * S * 8 + 128;  // + barriers + align slack
+  static constexpr int SMEM = S * STAGE_FLOATS * 4 + 2 * S * 8 + 2 * S * 4 + 128 + 128;
 };
 
-// Registers holding one output row's neighbourhood for the 4 x-outputs of a lane.
 template <int R>
 struct Win {
   float x[4 + 2 * R];   // centre row, x offsets -R .. 3+R
-  float ym[R][4];       // ym[k-1][i]: y - k
+  float ym[R][4];
   float yp[R][4];
-  float zm[R][4];       // zm[k-1][i]: z - k
+  float zm[R][4];
   float zp[R][4];
 };
 
@@ -84,39 +97,46 @@ __device__ __forceinline__ void set4(float (&d)[4], float4 v) {
 }
 
 template <int OP, int R, int I>
-__device__ __forceinline__ float eval(const StencilParams& p, const Win<R>& w, const float (&pw)[4], int64_t gz,
-                                      int64_t gy, int64_t gx0) {
+__device__ __forceinline__ float eval(const StencilParams& p, const Win<R>& w, const float4& pw, int gz, int gy,
+                                      int gx0) {
   WinAcc<R, I> a{w};
   if constexpr (OP == K2_WSTAR) {
     return op_weighted<R, R, R, true>(a, p.wbox);
   } else if constexpr (OP == K2_HOTSPOT) {
-    return op_hotspot3d(a, pw[I], p.prm);
+    return op_hotspot3d(a, f4get(pw, I), p.prm);
   } else {
-    const int K = acoustic_K<R>(gz, gy, gx0 + I, p.gnz, p.n[1], p.n[2]);
-    return op_acoustic<R>(a, pw[I], K, p.prm);
+    const int K = acoustic_K<R, int>(gz, gy, gx0 + I, (int)p.gnz, (int)p.n[1], (int)p.n[2]);
+    return op_acoustic<R>(a, f4get(pw, I), K, p.prm);
   }
 }
 
+// Out-of-grid x taps of a lane's window (x = xo - R + m outside [0, nx)) for
+// CLAMP / MIRROR / REFLECT / CONSTANT: the remapped tap lies in the lane's own
+// float4 (R <= 2 < 4 <= nx), selected without dynamic register indexing.
+__device__ __forceinline__ float pick4(int s, const float4& c, float pv) {
+  return s < 0 ? pv : (s == 0 ? c.x : (s == 1 ? c.y : (s == 2 ? c.z : c.w)));
+}
+
 template <int OP, int R, int RPW, int S>
-__global__ void __launch_bounds__(NCONS + 32)
+__global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
-             const float* __restrict__ src, const float* pw_in, float* out, int ntx, int nty, int zc) {
+             const float* __restrict__ src, const float* pw_in, float* out, int ntx, int nty, int zc,
+             int nchunk, int slot) {
   using C = Cfg<R, RPW, S>;
   constexpr int TY = C::TY;
-  extern __shared__ __align__(128) unsigned char smem_raw[];
-  float* stages = reinterpret_cast<float*>((reinterpret_cast<uintptr_t>(smem_raw) + 127) & ~uintptr_t(127));
-  uint64_t* full = reinterpret_cast<uint64_t*>(stages + S * C::STAGE_FLOATS);
+  constexpr int NR = 2 * R + 1;                 // planes in the z register ring
+  constexpr int SF4 = C::STAGE_FLOATS / 4;      // stage size in float4
+  constexpr int BX4 = BX / 4;
+  // dynamic smem (no static smem in this kernel, so it starts the CTA's window):
+  // [S stages][full S][empty S][stage_item S][stage_const S]
+  extern __shared__ __align__(128) float4 dsm4[];
+  uint64_t* full = reinterpret_cast<uint64_t*>(dsm4 + S * SF4);
   uint64_t* empty = full + S;
+  int* stage_item = reinterpret_cast<int*>(empty + S);
+  int* stage_const = stage_item + S;
 
   const int ntile = ntx * nty;
-  const int tile = blockIdx.x % ntile;
-  const int chunk = blockIdx.x / ntile;
-  const int x0 = (tile % ntx) * TX;
-  const int y0 = (tile / ntx) * TY;
-  const int64_t zs = p.reg0 + (int64_t)chunk * zc;
-  const int64_t ze = min(zs + (int64_t)zc, p.reg1);
-  if (zs >= ze) return;
-  const int nzc = (int)(ze - zs);
+  const int nitems = ntile * nchunk;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
 
   if (threadIdx.x == 0) {
@@ -129,102 +149,190 @@ __global__ void __launch_bounds__(NCONS + 32)
   __syncthreads();
 
   if (warp == NW) {
-    // ---------------- producer: one TMA box per input plane ----------------
+    // ---------------- producer: items from the ticket counter, one TMA box per plane ----------------
     if (lane == 0) {
       prefetch_tmap(&tmap);
-      const int nload = nzc + 2 * R;
-      for (int i = 0; i < nload; ++i) {
-        const int s = i % S, k = i / S;
-        if (k > 0) mbar_wait(&empty[s], (k - 1) & 1);
-        const int64_t lz = plane_of(p, p.z_off + zs - R + i);
-        if (lz >= 0) {
-          mbar_arrive_expect_tx(&full[s], C::TX_BYTES);
-          tma_load_3d(stages + s * C::STAGE_FLOATS, &tmap, &full[s], x0 - XH, y0 - R, (int)lz);
-        } else {
-          mbar_arrive(&full[s]);   // constant plane (value pad): nothing to load
+      int s = 0;
+      uint32_t pass = 0;
+      while (true) {
+        const int item = (int)atomicAdd(&g_ticket[slot], 1u);
+        const bool done = item >= nitems;
+        int nload = 1, x0 = 0, y0 = 0;
+        int64_t zs = 0;
+        if (!done) {
+          const int chunk = item / ntile, tile = item % ntile;
+          x0 = (tile % ntx) * TX;
+          y0 = (tile / ntx) * TY;
+          zs = p.reg0 + (int64_t)chunk * zc;
+          const int64_t ze = min(zs + (int64_t)zc, p.reg1);
+          nload = (int)(ze - zs) + 2 * R;
         }
+        // a "done" marker occupies one stage so the consumers see it in order
+        for (int i = 0; i < nload; ++i) {
+          if (pass > 0) mbar_wait(&empty[s], (pass - 1) & 1);
+          const int64_t lz = done ? -1 : plane_of(p, p.z_off + zs - R + i);
+          if (i == 0) stage_item[s] = done ? -1 : item;
+          stage_const[s] = lz < 0;
+          if (lz >= 0) {
+            mbar_arrive_expect_tx(&full[s], C::TX_BYTES);
+            tma_load_3d(dsm4 + s * SF4, &tmap, &full[s], x0 - XH, y0 - R, (int)lz);
+          } else {
+            mbar_arrive(&full[s]);   // constant plane (value pad) or end marker: nothing to load
+          }
+          if (++s == S) { s = 0; ++pass; }
+        }
+        if (done) break;
       }
     }
-    return;
-  }
-
-  // ---------------- consumers ----------------
-  const int64_t nx = p.n[2], ny = p.n[1];
-  const bool edge = (x0 == 0) || (x0 + TX + R > nx) || (y0 < R) || (y0 + TY + R > ny);
-  const bool zero_fill_ok = p.pad_value == 0.0f && p.kind[1] == PAD_CONSTANT && p.kind[2] == PAD_CONSTANT;
-  const bool need_fix = edge && !zero_fill_ok;
-  const int64_t out_plane = p.plane;
-  const int xo = x0 + 4 * lane;
-  const bool x_ok = xo < nx;
-
-  for (int i = 0; i < 2 * R; ++i) mbar_wait(&full[i % S], (i / S) & 1);
-
-  for (int j = 0; j < nzc; ++j) {
-    const int inew = j + 2 * R;
-    mbar_wait(&full[inew % S], (inew / S) & 1);
-    const int64_t z = zs + j;
-    const int64_t gz = p.z_off + z;
-    const int sc = (j + R) % S;
-    float* cst = stages + sc * C::STAGE_FLOATS;
-    if (need_fix) {
-      fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, cst, src, plane_of(p, gz), x0, y0, threadIdx.x);
-      fence_proxy_async_smem();
-      named_bar_sync(1, NCONS);
-    }
-    // which z-neighbour planes are constant (value pad) planes
-    bool zconst_m[R], zconst_p[R];
+  } else {
+    // ---------------- consumers ----------------
+    const int nx = (int)p.n[2], ny = (int)p.n[1];
+    const int kx = p.kind[2], ky = p.kind[1];
+    const float pv = p.pad_value;
+    const float4 pv4 = make_float4(pv, pv, pv, pv);
+    const bool wrap_fix = (kx == PAD_WRAP || ky == PAD_WRAP);
+    // float4 offsets (within a stage) of this thread's first row: centre column, halo column
+    const int roff4 = (warp * RPW + R) * BX4 + XH / 4 + lane;
+    const int eoff4 = (warp * RPW + R) * BX4 + (lane == 0 ? 0 : (TX + XH) / 4);
+    // out-of-grid x taps for CLAMP/MIRROR/REFLECT/CONSTANT come from the lane's
+    // own float4 (R <= 2 < 4 <= nx): source element per halo slot, -1 = pad_value
+    int sl[R], sr[R];
 #pragma unroll
     for (int k = 1; k <= R; ++k) {
-      zconst_m[k - 1] = plane_of(p, gz - k) < 0;
-      zconst_p[k - 1] = plane_of(p, gz + k) < 0;
+      sl[k - 1] = kx == PAD_CONSTANT ? -1 : (int)pad_remap(-k, nx, kx);
+      sr[k - 1] = kx == PAD_CONSTANT ? -1 : (int)(pad_remap(nx - 1 + k, nx, kx) - (nx - 4));
     }
+    int sn = 0;            // stage of the next load to wait for
+    uint32_t pn = 0;       // its pass (barrier phase parity)
+    while (true) {
+      mbar_wait(&full[sn], pn & 1);
+      const int item = stage_item[sn];
+      if (item < 0) {
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&empty[sn]);
+        break;
+      }
+      const int chunk = item / ntile, tile = item % ntile;
+      const int x0 = (tile % ntx) * TX;
+      const int y0 = (tile / ntx) * TY;
+      const int64_t zs = p.reg0 + (int64_t)chunk * zc;
+      const int nzc = (int)(min(zs + (int64_t)zc, p.reg1) - zs);
+      const int xo = x0 + 4 * lane;
+      const bool x_ok = xo < nx;
+      const bool y_edge = (y0 < R) || (y0 + TY + R > ny);
+      const bool fix = wrap_fix && ((x0 == 0) || (x0 + TX + R > nx) || y_edge);
+      const bool pl = !wrap_fix && x0 == 0 && lane == 0;      // left x-halo out of grid
+      const bool pr = !wrap_fix && xo + 4 == nx;              // right x-halo out of grid
+      const bool yr = !wrap_fix && y_edge;
+      // Stages of the 2R+1 planes around the current output plane z: zst[k]
+      // holds plane z - R + k (stage index, or -1 for a constant value plane).
+      int zst[2 * R + 1];
 #pragma unroll
-    for (int jj = 0; jj < RPW; ++jj) {
-      const int rr = warp * RPW + jj;           // tile row
-      const int64_t gy = y0 + rr;
-      const int off = (rr + R) * BX + XH + 4 * lane;
-      Win<R> w;
-      const float4 c = lds128(cst + off);
-      const float4 e = lds128(cst + (rr + R) * BX + (lane == 0 ? 0 : TX + XH));
-      float l1 = __shfl_up_sync(FULL, c.w, 1);
-      float r1 = __shfl_down_sync(FULL, c.x, 1);
-      if (lane == 0) l1 = e.w;
-      if (lane == 31) r1 = e.x;
-      if constexpr (R == 1) {
-        w.x[0] = l1; w.x[1] = c.x; w.x[2] = c.y; w.x[3] = c.z; w.x[4] = c.w; w.x[5] = r1;
-      } else {
-        float l2 = __shfl_up_sync(FULL, c.z, 1);
-        float r2 = __shfl_down_sync(FULL, c.y, 1);
-        if (lane == 0) l2 = e.z;
-        if (lane == 31) r2 = e.y;
-        w.x[0] = l2; w.x[1] = l1; w.x[2] = c.x; w.x[3] = c.y; w.x[4] = c.z; w.x[5] = c.w; w.x[6] = r1; w.x[7] = r2;
+      for (int k = 0; k < 2 * R; ++k) {
+        if (k > 0) mbar_wait(&full[sn], pn & 1);
+        zst[k] = stage_const[sn] ? -1 - sn : sn;
+        if (++sn == S) { sn = 0; ++pn; }
       }
+      float* orow = out + ((zs + p.ghost) * p.plane + (int64_t)(y0 + warp * RPW) * nx + xo);
+      const float* prow = pw_in + ((zs + p.ghost) * p.plane + (int64_t)(y0 + warp * RPW) * nx + xo);
+      for (int j = 0; j < nzc; ++j) {
+        mbar_wait(&full[sn], pn & 1);
+        zst[2 * R] = stage_const[sn] ? -1 - sn : sn;
+        if (++sn == S) { sn = 0; ++pn; }
+        const int gz = (int)(p.z_off + zs + j);
+        const int cbase = zst[R] * SF4;             // the centre plane is inside the grid
+        if (fix) {
+          fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + cbase), src,
+                                                 plane_of(p, (int64_t)gz), x0, y0, threadIdx.x);
+          fence_proxy_async_smem();
+          named_bar_sync(1, NCONS);
+        }
 #pragma unroll
-      for (int k = 1; k <= R; ++k) {
-        set4(w.ym[k - 1], lds128(cst + off - k * BX));
-        set4(w.yp[k - 1], lds128(cst + off + k * BX));
-        const float4 zm = zconst_m[k - 1] ? make_float4(p.pad_value, p.pad_value, p.pad_value, p.pad_value)
-                                          : lds128(stages + ((j + R - k) % S) * C::STAGE_FLOATS + off);
-        const float4 zp = zconst_p[k - 1] ? make_float4(p.pad_value, p.pad_value, p.pad_value, p.pad_value)
-                                          : lds128(stages + ((j + R + k) % S) * C::STAGE_FLOATS + off);
-        set4(w.zm[k - 1], zm);
-        set4(w.zp[k - 1], zp);
+        for (int jj = 0; jj < RPW; ++jj) {
+          const int rr = warp * RPW + jj;
+          const int gy = y0 + rr;
+          const bool ok = x_ok && gy < ny;
+          float4 pw = make_float4(0.f, 0.f, 0.f, 0.f);
+          if constexpr (OP != K2_WSTAR) {
+            if (ok) pw = ldg128(prow + jj * nx);
+          }
+          const int rb = roff4 + jj * BX4;          // row offset within a stage
+          Win<R> w;
+          const float4 c = dsm4[cbase + rb];
+          const float4 e = dsm4[cbase + eoff4 + jj * BX4];
+          {
+            const float cv[4] = {c.x, c.y, c.z, c.w};
+            const float ev[4] = {e.x, e.y, e.z, e.w};
+#pragma unroll
+            for (int k = 1; k <= R; ++k) {
+              float l = __shfl_up_sync(FULL, cv[4 - k], 1);
+              float r = __shfl_down_sync(FULL, cv[k - 1], 1);
+              if (lane == 0) l = ev[4 - k];
+              if (lane == 31) r = ev[k - 1];
+              if (pl) l = pick4(sl[k - 1], c, pv);
+              if (pr) r = pick4(sr[k - 1], c, pv);
+              w.x[R - k] = l;
+              w.x[R + 3 + k] = r;
+            }
+#pragma unroll
+            for (int i = 0; i < 4; ++i) w.x[R + i] = cv[i];
+          }
+#pragma unroll
+          for (int k = 1; k <= R; ++k) {
+            int m = -k * BX4, q = k * BX4;      // float4 offsets of rows y-k, y+k
+            bool cm = false, cq = false;
+            if (yr) {                              // pad redirect (edge items only)
+              if (gy - k < 0) {
+                if (ky == PAD_CONSTANT) cm = true;
+                else m = (min(max((int)pad_remap(gy - k, ny, ky) - y0 + R, 0), C::BY - 1) - (rr + R)) * BX4;
+              }
+              if (gy + k >= ny) {
+                if (ky == PAD_CONSTANT) cq = true;
+                else q = (min(max((int)pad_remap(gy + k, ny, ky) - y0 + R, 0), C::BY - 1) - (rr + R)) * BX4;
+              }
+            }
+            set4(w.ym[k - 1], cm ? pv4 : dsm4[cbase + rb + m]);
+            set4(w.yp[k - 1], cq ? pv4 : dsm4[cbase + rb + q]);
+            const int am = zst[R - k], ap = zst[R + k];
+            set4(w.zm[k - 1], am < 0 ? pv4 : dsm4[am * SF4 + rb]);
+            set4(w.zp[k - 1], ap < 0 ? pv4 : dsm4[ap * SF4 + rb]);
+          }
+          float4 res;
+          res.x = eval<OP, R, 0>(p, w, pw, gz, gy, xo);
+          res.y = eval<OP, R, 1>(p, w, pw, gz, gy, xo);
+          res.z = eval<OP, R, 2>(p, w, pw, gz, gy, xo);
+          res.w = eval<OP, R, 3>(p, w, pw, gz, gy, xo);
+          if (ok) stg128(orow + jj * nx, res);
+        }
+        orow += p.plane;
+        prow += p.plane;
+        // plane z - R is no longer needed (pre-chunk planes included)
+        __syncwarp();
+        if (lane == 0) {
+          const int t = zst[0] < 0 ? -1 - zst[0] : zst[0];
+          mbar_arrive(&empty[t]);
+        }
+#pragma unroll
+        for (int k = 0; k < 2 * R; ++k) zst[k] = zst[k + 1];
       }
-      const bool ok = x_ok && gy < ny;
-      const int64_t go = (z + p.ghost) * out_plane + gy * nx + xo;
-      float pw[4] = {0.f, 0.f, 0.f, 0.f};
-      if constexpr (OP != K2_WSTAR) {
-        if (ok) set4(pw, ldg128(pw_in + go));
+      // the chunk's last 2R planes (z_end - R .. z_end + R - 1) are still held
+      __syncwarp();
+      if (lane == 0) {
+#pragma unroll
+        for (int k = 0; k < 2 * R; ++k) mbar_arrive(&empty[zst[k] < 0 ? -1 - zst[k] : zst[k]]);
       }
-      float4 res;
-      res.x = eval<OP, R, 0>(p, w, pw, gz, gy, xo);
-      res.y = eval<OP, R, 1>(p, w, pw, gz, gy, xo);
-      res.z = eval<OP, R, 2>(p, w, pw, gz, gy, xo);
-      res.w = eval<OP, R, 3>(p, w, pw, gz, gy, xo);
-      if (ok) stg128(out + go, res);
     }
-    __syncwarp();
-    if (lane == 0) mbar_arrive(&empty[j % S]);   // plane z-R is no longer needed
+  }
+  // last CTA out resets the launch slot's counters (graph-replay safe)
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    __threadfence();
+    const unsigned prev = atomicAdd(&g_done[slot], 1u);
+    if (prev == gridDim.x - 1) {
+      g_ticket[slot] = 0;
+      g_done[slot] = 0;
+      __threadfence();
+    }
   }
 }
 
@@ -267,12 +375,11 @@ Launcher get_launcher() {
 
 Launcher pick(const StencilParams& p) {
   const int R = p.radius;
-  if (p.op == OP_WEIGHTED) return R == 1 ? get_launcher<K2_WSTAR, 1, 2, 5>() : get_launcher<K2_WSTAR, 2, 2, 7>();
-  if (p.op == OP_HOTSPOT3D) return get_launcher<K2_HOTSPOT, 1, 2, 5>();
-  return R == 1 ? get_launcher<K2_ACOUSTIC, 1, 2, 5>() : get_launcher<K2_ACOUSTIC, 2, 2, 7>();
+  if (p.op == OP_WEIGHTED) return R == 1 ? get_launcher<K2_WSTAR, 1, 2, 7>() : get_launcher<K2_WSTAR, 2, 2, 8>();
+  if (p.op == OP_HOTSPOT3D) return get_launcher<K2_HOTSPOT, 1, 2, 7>();
+  return R == 1 ? get_launcher<K2_ACOUSTIC, 1, 2, 7>() : get_launcher<K2_ACOUSTIC, 2, 2, 8>();
 }
 
-// small cache of encoded tensor maps (pointer + geometry)
 struct MapEntry {
   const float* base;
   int64_t nx, ny, nz;
@@ -296,6 +403,8 @@ bool get_map(const float* base, int64_t nx, int64_t ny, int64_t nz, int by, CUte
   return true;
 }
 
+std::atomic<unsigned> g_slot{0};
+
 }  // namespace
 
 bool sweep3d_supported(const StencilParams& p) {
@@ -311,7 +420,7 @@ bool sweep3d_supported(const StencilParams& p) {
     return false;
   }
   if (p.n[2] % 4 != 0) return false;
-  if (p.n[2] >= (1ll << 31) || p.n[1] >= (1ll << 31) || p.n[0] + 2 * p.ghost >= (1ll << 31)) return false;
+  if (p.n[2] * p.n[1] >= (1ll << 31) || p.gnz >= (1ll << 31) || p.n[0] + 2 * p.ghost >= (1ll << 31)) return false;
   return true;
 }
 
@@ -321,7 +430,6 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   if (nz_reg <= 0) return cudaSuccess;
   const Launcher L = pick(p);
   const int R = p.radius;
-  // slid input and point-wise input per op (stencil.h input order)
   const float* slid = (p.op == OP_ACOUSTIC) ? in1 : in0;
   const float* pw = (p.op == OP_ACOUSTIC) ? in0 : (p.op == OP_HOTSPOT3D ? in1 : nullptr);
   CUtensorMap map;
@@ -330,15 +438,18 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);
   const int64_t tiles = (int64_t)ntx * nty;
   const int64_t slots = (int64_t)num_sms * L.ctas_per_sm;
-  int64_t nchunk = (4 * slots + tiles - 1) / tiles;
-  if (nchunk < 1) nchunk = 1;
-  int64_t zc = (nz_reg + nchunk - 1) / nchunk;
-  if (zc < 4 && nz_reg >= 4) zc = 4;
-  nchunk = (nz_reg + zc - 1) / zc;
-  const int64_t grid = tiles * nchunk;
-  if (grid > 0x7fffffff) return cudaErrorInvalidConfiguration;
-  int ntx_i = ntx, nty_i = nty, zc_i = (int)zc;
-  void* args[] = {(void*)&p, (void*)&map, (void*)&slid, (void*)&pw, (void*)&out, &ntx_i, &nty_i, &zc_i};
+  // z-chunk: ~8 items per CTA for dynamic balance, at least 16 planes (halo re-load <= 2R/16)
+  int64_t zc = (nz_reg * tiles + 8 * slots - 1) / (8 * slots);
+  if (zc < 16) zc = 16;
+  if (zc > nz_reg) zc = nz_reg;
+  const int64_t nchunk = (nz_reg + zc - 1) / zc;
+  const int64_t items = tiles * nchunk;
+  if (items > 0x7fffffff) return cudaErrorInvalidConfiguration;
+  int64_t grid = slots < items ? slots : items;
+  int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk;
+  int slot = (int)(g_slot.fetch_add(1) % kTickets);
+  void* args[] = {(void*)&p, (void*)&map, (void*)&slid, (void*)&pw, (void*)&out,
+                  &ntx_i, &nty_i, &zc_i, &nch_i, &slot};
   return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
 }
 

@@ -138,9 +138,8 @@ __device__ __forceinline__ float acoustic_sum(const Acc& U) {
 
 // Number of star neighbours (+-1..+-R per axis) inside the global domain
 // (computeNumNeighbors): generated on the fly, 0 bytes.
-template <int R>
-__device__ __forceinline__ int acoustic_K(int64_t gz, int64_t gy, int64_t gx, int64_t nz,
-                                          int64_t ny, int64_t nx) {
+template <int R, class Int>
+__device__ __forceinline__ int acoustic_K(Int gz, Int gy, Int gx, Int nz, Int ny, Int nx) {
   int K = 0;
 #pragma unroll
   for (int off = 1; off <= R; ++off) {
