@@ -117,7 +117,7 @@ __device__ __forceinline__ float pick4(int s, const float4& c, float pv) {
   return s < 0 ? pv : (s == 0 ? c.x : (s == 1 ? c.y : (s == 2 ? c.z : c.w)));
 }
 
-template <int OP, int R, int RPW, int S>
+template <int OP, int R, int RPW, int S, bool ZC>
 __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
              const float* __restrict__ src, const float* pw_in, float* out, int ntx, int nty, int zc,
@@ -190,7 +190,11 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
     const int kx = p.kind[2], ky = p.kind[1];
     const float pv = p.pad_value;
     const float4 pv4 = make_float4(pv, pv, pv, pv);
-    const bool wrap_fix = (kx == PAD_WRAP || ky == PAD_WRAP);
+    // WRAP and non-zero CONSTANT in x/y rewrite the halo cells in shared memory;
+    // zero CONSTANT is TMA's out-of-bounds fill; CLAMP/MIRROR/REFLECT are folded
+    // into row offsets (y) and register selects (x)
+    const bool wrap_fix = (kx == PAD_WRAP || ky == PAD_WRAP) ||
+                          ((kx == PAD_CONSTANT || ky == PAD_CONSTANT) && pv != 0.0f);
     // float4 offsets (within a stage) of this thread's first row: centre column, halo column
     const int roff4 = (warp * RPW + R) * BX4 + XH / 4 + lane;
     const int eoff4 = (warp * RPW + R) * BX4 + (lane == 0 ? 0 : (TX + XH) / 4);
@@ -199,7 +203,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
     int sl[R], sr[R];
 #pragma unroll
     for (int k = 1; k <= R; ++k) {
-      sl[k - 1] = kx == PAD_CONSTANT ? -1 : (int)pad_remap(-k, nx, kx);
+      sl[k - 1] = kx == PAD_CONSTANT ? -1 : (int)pad_remap(-k, nx, kx);          // -1: zero (TMA fill)
       sr[k - 1] = kx == PAD_CONSTANT ? -1 : (int)(pad_remap(nx - 1 + k, nx, kx) - (nx - 4));
     }
     int sn = 0;            // stage of the next load to wait for
@@ -221,23 +225,40 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
       const bool x_ok = xo < nx;
       const bool y_edge = (y0 < R) || (y0 + TY + R > ny);
       const bool fix = wrap_fix && ((x0 == 0) || (x0 + TX + R > nx) || y_edge);
-      const bool pl = !wrap_fix && x0 == 0 && lane == 0;      // left x-halo out of grid
-      const bool pr = !wrap_fix && xo + 4 == nx;              // right x-halo out of grid
-      const bool yr = !wrap_fix && y_edge;
+      const bool pl = !wrap_fix && kx != PAD_CONSTANT && x0 == 0 && lane == 0;   // left x-halo out of grid
+      const bool pr = !wrap_fix && kx != PAD_CONSTANT && xo + 4 == nx;           // right x-halo out of grid
+      const bool yr = !wrap_fix && ky != PAD_CONSTANT && y_edge;
+      // float4 offsets of rows y-k / y+k relative to row y (pad redirect folded in)
+      int om[RPW][R], oq[RPW][R];
+#pragma unroll
+      for (int jj = 0; jj < RPW; ++jj) {
+        const int rr = warp * RPW + jj, gy = y0 + rr;
+#pragma unroll
+        for (int k = 1; k <= R; ++k) {
+          om[jj][k - 1] = -k * BX4;
+          oq[jj][k - 1] = k * BX4;
+          if (yr) {
+            if (gy - k < 0)
+              om[jj][k - 1] = (min(max((int)pad_remap(gy - k, ny, ky) - y0 + R, 0), C::BY - 1) - (rr + R)) * BX4;
+            if (gy + k >= ny)
+              oq[jj][k - 1] = (min(max((int)pad_remap(gy + k, ny, ky) - y0 + R, 0), C::BY - 1) - (rr + R)) * BX4;
+          }
+        }
+      }
       // Stages of the 2R+1 planes around the current output plane z: zst[k]
       // holds plane z - R + k (stage index, or -1 for a constant value plane).
       int zst[2 * R + 1];
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k) {
         if (k > 0) mbar_wait(&full[sn], pn & 1);
-        zst[k] = stage_const[sn] ? -1 - sn : sn;
+        zst[k] = (ZC && stage_const[sn]) ? -1 - sn : sn;
         if (++sn == S) { sn = 0; ++pn; }
       }
       float* orow = out + ((zs + p.ghost) * p.plane + (int64_t)(y0 + warp * RPW) * nx + xo);
       const float* prow = pw_in + ((zs + p.ghost) * p.plane + (int64_t)(y0 + warp * RPW) * nx + xo);
       for (int j = 0; j < nzc; ++j) {
         mbar_wait(&full[sn], pn & 1);
-        zst[2 * R] = stage_const[sn] ? -1 - sn : sn;
+        zst[2 * R] = (ZC && stage_const[sn]) ? -1 - sn : sn;
         if (++sn == S) { sn = 0; ++pn; }
         const int gz = (int)(p.z_off + zs + j);
         const int cbase = zst[R] * SF4;             // the centre plane is inside the grid
@@ -269,8 +290,8 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
               float r = __shfl_down_sync(FULL, cv[k - 1], 1);
               if (lane == 0) l = ev[4 - k];
               if (lane == 31) r = ev[k - 1];
-              if (pl) l = pick4(sl[k - 1], c, pv);
-              if (pr) r = pick4(sr[k - 1], c, pv);
+              if (pl) l = pick4(sl[k - 1], c, 0.0f);
+              if (pr) r = pick4(sr[k - 1], c, 0.0f);
               w.x[R - k] = l;
               w.x[R + 3 + k] = r;
             }
@@ -279,23 +300,16 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
           }
 #pragma unroll
           for (int k = 1; k <= R; ++k) {
-            int m = -k * BX4, q = k * BX4;      // float4 offsets of rows y-k, y+k
-            bool cm = false, cq = false;
-            if (yr) {                              // pad redirect (edge items only)
-              if (gy - k < 0) {
-                if (ky == PAD_CONSTANT) cm = true;
-                else m = (min(max((int)pad_remap(gy - k, ny, ky) - y0 + R, 0), C::BY - 1) - (rr + R)) * BX4;
-              }
-              if (gy + k >= ny) {
-                if (ky == PAD_CONSTANT) cq = true;
-                else q = (min(max((int)pad_remap(gy + k, ny, ky) - y0 + R, 0), C::BY - 1) - (rr + R)) * BX4;
-              }
-            }
-            set4(w.ym[k - 1], cm ? pv4 : dsm4[cbase + rb + m]);
-            set4(w.yp[k - 1], cq ? pv4 : dsm4[cbase + rb + q]);
+            set4(w.ym[k - 1], dsm4[cbase + rb + om[jj][k - 1]]);
+            set4(w.yp[k - 1], dsm4[cbase + rb + oq[jj][k - 1]]);
             const int am = zst[R - k], ap = zst[R + k];
-            set4(w.zm[k - 1], am < 0 ? pv4 : dsm4[am * SF4 + rb]);
-            set4(w.zp[k - 1], ap < 0 ? pv4 : dsm4[ap * SF4 + rb]);
+            if constexpr (ZC) {
+              set4(w.zm[k - 1], am < 0 ? pv4 : dsm4[am * SF4 + rb]);
+              set4(w.zp[k - 1], ap < 0 ? pv4 : dsm4[ap * SF4 + rb]);
+            } else {
+              set4(w.zm[k - 1], dsm4[am * SF4 + rb]);
+              set4(w.zp[k - 1], dsm4[ap * SF4 + rb]);
+            }
           }
           float4 res;
           res.x = eval<OP, R, 0>(p, w, pw, gz, gy, xo);
@@ -357,13 +371,13 @@ struct Launcher {
   int ctas_per_sm;
 };
 
-template <int OP, int R, int RPW, int S>
+template <int OP, int R, int RPW, int S, bool ZC>
 Launcher get_launcher() {
   static Launcher L{};
   static std::once_flag once;
   std::call_once(once, [] {
     using C = Cfg<R, RPW, S>;
-    auto fn = k2_sweep<OP, R, RPW, S>;
+    auto fn = k2_sweep<OP, R, RPW, S, ZC>;
     cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
     int occ = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, NCONS + 32, C::SMEM) != cudaSuccess) occ = 1;
@@ -375,9 +389,15 @@ Launcher get_launcher() {
 
 Launcher pick(const StencilParams& p) {
   const int R = p.radius;
-  if (p.op == OP_WEIGHTED) return R == 1 ? get_launcher<K2_WSTAR, 1, 2, 7>() : get_launcher<K2_WSTAR, 2, 2, 8>();
-  if (p.op == OP_HOTSPOT3D) return get_launcher<K2_HOTSPOT, 1, 2, 7>();
-  return R == 1 ? get_launcher<K2_ACOUSTIC, 1, 2, 7>() : get_launcher<K2_ACOUSTIC, 2, 2, 8>();
+  const bool zc = p.kind[0] == PAD_CONSTANT;   // value-pad planes in z are possible
+  if (p.op == OP_WEIGHTED) {
+    if (R == 1) return zc ? get_launcher<K2_WSTAR, 1, 2, 7, true>() : get_launcher<K2_WSTAR, 1, 2, 7, false>();
+    return zc ? get_launcher<K2_WSTAR, 2, 2, 8, true>() : get_launcher<K2_WSTAR, 2, 2, 8, false>();
+  }
+  if (p.op == OP_HOTSPOT3D)
+    return zc ? get_launcher<K2_HOTSPOT, 1, 2, 7, true>() : get_launcher<K2_HOTSPOT, 1, 2, 7, false>();
+  if (R == 1) return zc ? get_launcher<K2_ACOUSTIC, 1, 2, 7, true>() : get_launcher<K2_ACOUSTIC, 1, 2, 7, false>();
+  return zc ? get_launcher<K2_ACOUSTIC, 2, 2, 8, true>() : get_launcher<K2_ACOUSTIC, 2, 2, 8, false>();
 }
 
 struct MapEntry {
