@@ -1,0 +1,101 @@
+"""Slab decomposition on the GPU (single device): the decomposed iterate must be
+bitwise equal to the single-plan iterate (same per-point kernel code), and the
+single-plan iterate matches the oracle (test_parity_gpu).
+
+  * virtual slabs: G slab plans on one device, ghosts filled by D2D copies
+    (slab.virtual_slab_iterate) — checks partition, ghost layout, global pad
+    handling in z (stencil_plan_set_slab) and the Acoustic global neighbour
+    count;
+  * SlabPlan with world = 1: the boundary / interior apply_region split, the
+    comm side stream and the exchange hook of the multi-GPU path.
+"""
+import numpy as np
+import pytest
+import torch
+
+import stencil_inputs as si
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def lift():
+    import __graft_entry__
+    __graft_entry__.build()
+    import paper_conf_cgo_hagedornssgd18_b200 as m
+    torch.cuda.set_device(0)
+    return m
+
+
+def single_iterate(lift, spec, state, aux, n):
+    plan = lift.Plan.from_spec(spec)
+    st = [torch.from_numpy(x).cuda() for x in state]
+    if len(st) == 1:
+        st.append(torch.empty_like(st[0]))
+    ax = [torch.from_numpy(x).cuda() for x in aux]
+    ri = plan.iterate(st, n, ax)
+    torch.cuda.synchronize()
+    if spec.op == si.ACOUSTIC:
+        return [st[1 - ri].cpu().numpy(), st[ri].cpu().numpy()]
+    return [st[ri].cpu().numpy()]
+
+
+def kw(spec):
+    return dict(size=spec.size, pad=spec.pad_lo, kind=list(spec.kind), pad_value=spec.pad_value, op=spec.op,
+                weights=spec.weights, params=spec.params)
+
+
+@pytest.mark.parametrize("kind", [si.CLAMP, si.WRAP, si.CONSTANT, si.MIRROR, si.REFLECT])
+@pytest.mark.parametrize("world", [2, 3])
+def test_virtual_slab_weighted_bitwise(lift, kind, world):
+    from paper_conf_cgo_hagedornssgd18_b200.slab import virtual_slab_iterate
+    ext = (30, 40, 136)
+    sp = si.StencilSpec(ext, (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (kind,) * 3, 0.5, si.WEIGHTED,
+                        si.weights_j3d7(), ())
+    x = si.uniform(ext, 77, 0.5, 1.5)
+    ref = single_iterate(lift, sp, [x], [], 5)[0]
+    got = virtual_slab_iterate(ext, world, [torch.from_numpy(x).cuda()], 5, **kw(sp))[0]
+    np.testing.assert_array_equal(got.cpu().numpy(), ref)
+
+
+@pytest.mark.parametrize("pts,sz", [(7, 3), (13, 5)])
+def test_virtual_slab_acoustic_bitwise(lift, pts, sz):
+    from paper_conf_cgo_hagedornssgd18_b200.slab import virtual_slab_iterate
+    ext = (24, 36, 132)
+    r = sz // 2
+    sp = si.StencilSpec(ext, (sz,) * 3, (1,) * 3, (r,) * 3, (r,) * 3, (si.CONSTANT,) * 3, 0.0, si.ACOUSTIC, None,
+                        si.params_acoustic(pts))
+    u0 = si.uniform(ext, 78, -1, 1)
+    u1 = si.uniform(ext, 79, -1, 1)
+    ref = single_iterate(lift, sp, [u0, u1], [], 4)
+    got = virtual_slab_iterate(ext, 3, [torch.from_numpy(u0).cuda(), torch.from_numpy(u1).cuda()], 4, **kw(sp))
+    np.testing.assert_array_equal(got[1].cpu().numpy(), ref[1])
+    np.testing.assert_array_equal(got[0].cpu().numpy(), ref[0])
+
+
+def test_virtual_slab_hotspot_bitwise(lift):
+    from paper_conf_cgo_hagedornssgd18_b200.slab import virtual_slab_iterate
+    ext = (8, 64, 128)
+    sp = si.StencilSpec(ext, (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.CLAMP,) * 3, 0.0, si.HOTSPOT3D, None,
+                        si.params_hotspot3d())
+    T = si.uniform(ext, 80, 300, 350)
+    P = si.uniform(ext, 81, 0, 1e-2)
+    ref = single_iterate(lift, sp, [T], [P], 6)[0]
+    got = virtual_slab_iterate(ext, 2, [torch.from_numpy(T).cuda()], 6, [torch.from_numpy(P).cuda()], **kw(sp))[0]
+    np.testing.assert_array_equal(got.cpu().numpy(), ref)
+
+
+@pytest.mark.parametrize("kind", [si.CLAMP, si.WRAP])
+def test_slabplan_world1_split_bitwise(lift, kind):
+    from paper_conf_cgo_hagedornssgd18_b200.slab import SlabPlan
+    ext = (20, 40, 136)
+    sp = si.StencilSpec(ext, (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (kind,) * 3, 0.0, si.WEIGHTED,
+                        si.weights_j3d7(), ())
+    x = si.uniform(ext, 82, 0.5, 1.5)
+    ref = single_iterate(lift, sp, [x], [], 7)[0]
+    slab = SlabPlan(ext, 0, 1, **kw(sp))
+    a = slab.scatter(torch.from_numpy(x).cuda())
+    b = slab.empty()
+    ri = slab.iterate([a, b], 7)
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(slab.owned((a, b)[ri]).cpu().numpy(), ref)
