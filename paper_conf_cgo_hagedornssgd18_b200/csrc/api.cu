@@ -3,6 +3,7 @@
 // kernel-family dispatch, apply / apply_region / iterate / run_host.
 #include <cuda_runtime.h>
 
+#include <cmath>
 #include <cstdio>
 #include <cstring>
 #include <new>
@@ -233,6 +234,34 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
       p.ntaps = nt;
       if (ntot <= kMaxTaps)
         for (int64_t k = 0; k < ntot; ++k) p.wbox[k] = weights[k];
+      // separable (rank-1) 2D weights: w[i][j] == su[i] * sv[j] exactly (checked
+      // in double, where fp32 x fp32 products are exact); the factors are scaled
+      // by sqrt of the largest tap so that e.g. the binomial Gaussian factors
+      // into its exact 1D binomials
+      p.sep = 0;
+      if (ndim == 2 && p.size[1] <= kMaxSep && p.size[2] <= kMaxSep) {
+        const int SY = p.size[1], SX = p.size[2];
+        int bi = 0, bj = 0;
+        for (int i = 0; i < SY; ++i)
+          for (int j = 0; j < SX; ++j)
+            if (std::fabs(weights[i * SX + j]) > std::fabs(weights[bi * SX + bj])) { bi = i; bj = j; }
+        const float wc = weights[bi * SX + bj];
+        if (wc != 0.0f) {
+          const float sc = std::sqrt(std::fabs(wc));
+          float u[kMaxSep], v[kMaxSep];
+          for (int j = 0; j < SX; ++j) v[j] = weights[bi * SX + j] / sc;
+          for (int i = 0; i < SY; ++i) u[i] = weights[i * SX + bj] / (wc / sc);
+          bool ok = true;
+          for (int i = 0; i < SY && ok; ++i)
+            for (int j = 0; j < SX && ok; ++j)
+              ok = (double)u[i] * (double)v[j] == (double)weights[i * SX + j];
+          if (ok) {
+            p.sep = 1;
+            for (int i = 0; i < SY; ++i) p.su[i] = u[i];
+            for (int j = 0; j < SX; ++j) p.sv[j] = v[j];
+          }
+        }
+      }
       // radius for the fast kernels: symmetric centred window
       int r = p.size[2] / 2;
       p.radius = centred(r) ? r : -1;

@@ -16,6 +16,7 @@ enum OpKind : int { OP_WEIGHTED = 0, OP_HOTSPOT3D = 1, OP_SRAD1 = 2, OP_SRAD2 = 
 constexpr int kMaxTaps = 125;     // 5x5x5
 constexpr int kMaxParams = 16;
 constexpr int kMaxInputs = 2;
+constexpr int kMaxSep = 16;
 
 struct StencilParams {
   // canonical 3D geometry (index 0 = z, slowest)
@@ -40,6 +41,10 @@ struct StencilParams {
   int16_t tap[kMaxTaps][3];   // window index k per dimension
   float w[kMaxTaps];
   float wbox[kMaxTaps];        // dense row-major window weights (fast kernels)
+  // 2D WEIGHTED with exactly rank-1 weights w[ky][kx] = su[ky] * sv[kx]:
+  // every kernel family evaluates sum_ky su[ky] * (sum_kx sv[kx] * x) in this order
+  int32_t sep;
+  float su[kMaxSep], sv[kMaxSep];
   float prm[kMaxParams];
 };
 

@@ -74,9 +74,18 @@ __global__ void __launch_bounds__(256) k0_generic(const __grid_constant__ Stenci
         const int64_t bz = p.z_off + g.oz * p.step[0] - p.lo[0];
         const int64_t by = g.oy * p.step[1] - p.lo[1];
         const int64_t bx = g.ox * p.step[2] - p.lo[2];
-        for (int t = 0; t < p.ntaps; ++t) {
-          const float x = fetch(p, in0, bz + p.tap[t][0], by + p.tap[t][1], bx + p.tap[t][2]);
-          acc = __fmaf_rn(p.w[t], x, acc);
+        if (p.sep) {
+          // separable 2D weights: rows first (x taps in order), then the column
+          for (int ky = 0; ky < p.size[1]; ++ky) {
+            float h = 0.0f;
+            for (int kx = 0; kx < p.size[2]; ++kx) h = __fmaf_rn(p.sv[kx], fetch(p, in0, bz, by + ky, bx + kx), h);
+            acc = __fmaf_rn(p.su[ky], h, acc);
+          }
+        } else {
+          for (int t = 0; t < p.ntaps; ++t) {
+            const float x = fetch(p, in0, bz + p.tap[t][0], by + p.tap[t][1], bx + p.tap[t][2]);
+            acc = __fmaf_rn(p.w[t], x, acc);
+          }
         }
         v = acc;
         break;

@@ -1,22 +1,26 @@
 // kernel_tile2d.cu — K1: the 2D stencil on TMA-staged halo'd tiles.
 //
 // map_2(f, slide_2(size, step, pad_2(...))) over a 2D
-// grid.  The output is cut into 128 x TY tiles (overlapped tiling, P:693-822:
+// grid.  The output is cut into 128 x 48 tiles (overlapped tiling, P:693-822:
 // each tile's input box carries the 2R-wide overlap).  Persistent CTAs (one
-// wave: grid = SMs x resident CTAs) take contiguous runs of tiles in
-// row-major tile order, so neighbouring tiles — whose boxes overlap — are in
-// flight at the same time and the overlap is served by L2.  Per CTA an
-// elected producer thread streams the tiles' boxes ((128+8) x (TY+2RY)
-// floats per input grid) through an S-stage shared-memory ring with TMA and
-// mbarriers; 8 consumer warps each sweep TY/8 output rows down the box,
-// keeping the 2RY+1 rows of x-windows in registers (each box row is read from
-// shared memory once per warp) and taking the in-row neighbours from the
-// adjacent lanes with warp shuffles; 4 outputs per lane leave as one
-// st.global.v4.  Edge tiles rewrite their out-of-grid halo cells (halo.cuh)
-// before use.  f goes through ops.cuh (bitwise equal to K0).
+// wave: grid = SMs x resident CTAs) take tiles with a grid stride, so in every
+// round the CTAs cover a band of consecutive tiles in row-major order and the
+// overlap rows/columns of neighbouring tiles come from L2.  Per CTA an elected
+// producer thread streams each tile's box ((128+8) x (48+2RY) floats per input
+// grid) into a 2-stage shared-memory ring with TMA and mbarriers; 8 consumer
+// warps each sweep 6 output rows down the box.  Every box row is read from
+// shared memory once per warp (one LDS.128 per lane; the in-row neighbours
+// come from the adjacent lanes by warp shuffles) and immediately added to the
+// 2RY+1 output rows in flight, so each output's FMA chain runs in row-major
+// tap order — the order K0 uses.  Separable weights (the binomial Gaussian)
+// take the row sum once per box row and then one FMA per output row
+// (10 instead of 25 FMA per point), star weights skip the off-axis taps.
+// 4 outputs per lane leave as one st.global.v4.  Edge tiles rewrite their
+// out-of-grid halo cells (halo.cuh) before use.
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#include <cstdlib>
 #include <mutex>
 #include <string>
 
@@ -36,7 +40,7 @@ constexpr int NW = 8;
 constexpr int NCONS = NW * 32;
 constexpr unsigned FULL = 0xffffffffu;
 
-enum K1Op { K1_WBOX = 0, K1_SRAD1 = 1, K1_SRAD2 = 2 };
+enum K1Op { K1_WBOX = 0, K1_SRAD1 = 1, K1_SRAD2 = 2, K1_WSTAR = 3, K1_WSEP = 4 };
 
 template <int RY, int RPW, int S, int NIN>
 struct Cfg {
@@ -49,10 +53,11 @@ struct Cfg {
 };
 
 // x-window of one box row for the 4 outputs of a lane: offsets -RX .. 3+RX
+// (centre float4 from shared memory, neighbours from the adjacent lanes)
 template <int RX>
-__device__ __forceinline__ void load_row(const float* row, int lane, float (&xw)[4 + 2 * RX]) {
-  const float4 c = lds128(row + XH + 4 * lane);
-  const float4 e = lds128(row + (lane == 0 ? 0 : TX + XH));
+__device__ __forceinline__ void load_row(const float4* row4, int lane, float (&xw)[4 + 2 * RX]) {
+  const float4 c = row4[XH / 4 + lane];
+  const float4 e = row4[lane == 0 ? 0 : (TX + XH) / 4];
   const float cv[4] = {c.x, c.y, c.z, c.w};
   const float ev[4] = {e.x, e.y, e.z, e.w};
 #pragma unroll
@@ -68,10 +73,10 @@ __device__ __forceinline__ void load_row(const float* row, int lane, float (&xw)
   for (int i = 0; i < 4; ++i) xw[RX + i] = cv[i];
 }
 
-// Accessor over the register ring: rows[(DY + RY) slot][I + RX + DX].
+// Accessor over a ring of x-windows (SRAD): rows[DY + RY][I + RX + DX].
 template <int RY, int RX, int I>
 struct RingAcc {
-  const float (*rows)[4 + 2 * RX];   // rows[0..2RY] ordered y-RY .. y+RY
+  const float (*rows)[4 + 2 * RX];
   template <int DZ, int DY, int DX>
   __device__ __forceinline__ float at() const {
     static_assert(DZ == 0, "2D");
@@ -79,35 +84,28 @@ struct RingAcc {
   }
 };
 
-template <int OP, int RY, int RX, int I>
-__device__ __forceinline__ float eval(const StencilParams& p, const float (*a)[4 + 2 * RX],
-                                      const float (*b)[4 + 2 * RX]) {
-  if constexpr (OP == K1_WBOX) {
-    return op_weighted<0, RY, RX, false>(RingAcc<RY, RX, I>{a}, p.wbox);
-  } else if constexpr (OP == K1_SRAD1) {
-    return op_srad1(RingAcc<RY, RX, I>{a}, p.prm);
-  } else {
-    return op_srad2(RingAcc<RY, RX, I>{a}, RingAcc<RY, RX, I>{b}, p.prm);   // (c, I)
-  }
-}
-
-template <int OP, int RY, int RX, int RPW, int S, int NIN>
-__global__ void __launch_bounds__(NCONS + 32)
+template <int OP, int RY, int RX, int RPW, int S, int NIN, int MINB>
+__global__ void __launch_bounds__(NCONS + 32, MINB)
     k1_tile(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap map0,
             const __grid_constant__ CUtensorMap map1, const float* __restrict__ src0,
             const float* __restrict__ src1, float* __restrict__ out, int ntx, int nty) {
   using C = Cfg<RY, RPW, S, NIN>;
   constexpr int TY = C::TY;
   constexpr int W = 4 + 2 * RX;
-  extern __shared__ __align__(128) unsigned char smem_raw[];
-  float* stages = reinterpret_cast<float*>((reinterpret_cast<uintptr_t>(smem_raw) + 127) & ~uintptr_t(127));
-  uint64_t* full = reinterpret_cast<uint64_t*>(stages + S * C::STAGE_FLOATS);
+  constexpr int SY = 2 * RY + 1, SX = 2 * RX + 1;
+  constexpr int BX4 = BX / 4;
+  constexpr int SF4 = C::STAGE_FLOATS / 4;
+  constexpr int BF4 = C::BOX_FLOATS / 4;
+  extern __shared__ __align__(128) float4 dsm4[];
+  uint64_t* full = reinterpret_cast<uint64_t*>(dsm4 + S * SF4);
   uint64_t* empty = full + S;
 
+  // strided tile assignment: in round k all CTAs work on tiles
+  // [k*grid, (k+1)*grid) of the row-major tile order, so the tiles above and
+  // below (whose rows are this tile's halo) are in flight in the same or the
+  // neighbouring round and the overlap comes from L2
   const int64_t ntiles = (int64_t)ntx * nty;
-  const int64_t t0 = ntiles * blockIdx.x / gridDim.x;
-  const int64_t t1 = ntiles * (blockIdx.x + 1) / gridDim.x;
-  const int nt = (int)(t1 - t0);
+  const int nt = (int)((ntiles - blockIdx.x + gridDim.x - 1) / gridDim.x);
   if (nt <= 0) return;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
 
@@ -124,70 +122,129 @@ __global__ void __launch_bounds__(NCONS + 32)
     if (lane == 0) {
       prefetch_tmap(&map0);
       if (NIN > 1) prefetch_tmap(&map1);
+      int s = 0;
+      uint32_t pass = 0;
       for (int i = 0; i < nt; ++i) {
-        const int s = i % S, k = i / S;
-        if (k > 0) mbar_wait(&empty[s], (k - 1) & 1);
-        const int64_t t = t0 + i;
+        if (pass > 0) mbar_wait(&empty[s], (pass - 1) & 1);
+        const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
         const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
-        float* st = stages + s * C::STAGE_FLOATS;
         mbar_arrive_expect_tx(&full[s], NIN * C::BOX_BYTES);
-        tma_load_3d(st, &map0, &full[s], x0 - XH, y0 - RY, 0);
-        if constexpr (NIN > 1) tma_load_3d(st + C::BOX_FLOATS, &map1, &full[s], x0 - XH, y0 - RY, 0);
+        tma_load_3d(dsm4 + s * SF4, &map0, &full[s], x0 - XH, y0 - RY, 0);
+        if constexpr (NIN > 1) tma_load_3d(dsm4 + s * SF4 + BF4, &map1, &full[s], x0 - XH, y0 - RY, 0);
+        if (++s == S) { s = 0; ++pass; }
       }
     }
     return;
   }
 
-  const int64_t nx = p.n[2], ny = p.n[1];
+  const int nx = (int)p.n[2], ny = (int)p.n[1];
   const bool zero_fill_ok = p.pad_value == 0.0f && p.kind[1] == PAD_CONSTANT && p.kind[2] == PAD_CONSTANT;
+  const int r0 = warp * RPW;   // first output row of this warp (tile-relative)
+  int s = 0;
+  uint32_t pass = 0;
   for (int i = 0; i < nt; ++i) {
-    const int s = i % S;
-    mbar_wait(&full[s], (i / S) & 1);
-    const int64_t t = t0 + i;
+    mbar_wait(&full[s], pass & 1);
+    const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
     const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
-    float* st = stages + s * C::STAGE_FLOATS;
     const bool edge = (x0 == 0) || (x0 + TX + RX > nx) || (y0 < RY) || (y0 + TY + RY > ny);
     if (edge && !zero_fill_ok) {
-      fixup_tile<RY, RX, XH, BX, C::BY, NCONS>(p, st, src0, 0, x0, y0, threadIdx.x);
-      if constexpr (NIN > 1) fixup_tile<RY, RX, XH, BX, C::BY, NCONS>(p, st + C::BOX_FLOATS, src1, 0, x0, y0, threadIdx.x);
+      fixup_tile<RY, RX, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + s * SF4), src0, 0, x0, y0,
+                                               threadIdx.x);
+      if constexpr (NIN > 1)
+        fixup_tile<RY, RX, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + s * SF4 + BF4), src1, 0, x0,
+                                                 y0, threadIdx.x);
       fence_proxy_async_smem();
       named_bar_sync(1, NCONS);
     }
     const int xo = x0 + 4 * lane;
     const bool x_ok = xo < nx;
-    const int r0 = warp * RPW;   // first output row of this warp (tile-relative)
-    // register ring of 2RY+1 box rows, filled as the warp sweeps down
-    float ra[2 * RY + 1][W];
-    float rb[(NIN > 1) ? 2 * RY + 1 : 1][W];
+    const float4* box0 = dsm4 + s * SF4 + r0 * BX4;     // box row r0 = output row r0 - RY
+    float* orow = out + ((int64_t)(y0 + r0) * nx + xo);
+    auto store = [&](int o, const float (&v)[4]) {
+      if (x_ok && y0 + r0 + o < ny) stg128(orow + (int64_t)o * nx, make_float4(v[0], v[1], v[2], v[3]));
+    };
+
+    if constexpr (OP == K1_WBOX || OP == K1_WSTAR || OP == K1_WSEP) {
+      // Box rows stream in top to bottom; each row adds its taps to the 2RY+1
+      // outputs in flight, so every output's chain runs in row-major tap order.
+      float acc[SY][4];
+      static_for<RPW + 2 * RY>([&](auto KR) {
+        constexpr int kr = decltype(KR)::value;
+        float xw[W];
+        load_row<RX>(box0 + kr * BX4, lane, xw);
+        float h[4];
+        if constexpr (OP == K1_WSEP) {
 #pragma unroll
-    for (int k = 0; k < 2 * RY; ++k) {
-      load_row<RX>(st + (r0 + k) * BX, lane, ra[k]);
-      if constexpr (NIN > 1) load_row<RX>(st + C::BOX_FLOATS + (r0 + k) * BX, lane, rb[k]);
-    }
+          for (int q = 0; q < 4; ++q) {
+            float a = 0.0f;
 #pragma unroll
-    for (int jj = 0; jj < RPW; ++jj) {
-      // box row of (output row r0+jj) + RY enters the ring
-      load_row<RX>(st + (r0 + jj + 2 * RY) * BX, lane, ra[2 * RY]);
-      if constexpr (NIN > 1) load_row<RX>(st + C::BOX_FLOATS + (r0 + jj + 2 * RY) * BX, lane, rb[2 * RY]);
-      const int64_t gy = y0 + r0 + jj;
-      float4 res;
-      res.x = eval<OP, RY, RX, 0>(p, ra, rb);
-      res.y = eval<OP, RY, RX, 1>(p, ra, rb);
-      res.z = eval<OP, RY, RX, 2>(p, ra, rb);
-      res.w = eval<OP, RY, RX, 3>(p, ra, rb);
-      if (x_ok && gy < ny) stg128(out + gy * nx + xo, res);
-      // rotate
-#pragma unroll
-      for (int k = 0; k < 2 * RY; ++k) {
-#pragma unroll
-        for (int q = 0; q < W; ++q) {
-          ra[k][q] = ra[k + 1][q];
-          if constexpr (NIN > 1) rb[k][q] = rb[k + 1][q];
+            for (int kx = 0; kx < SX; ++kx) a = __fmaf_rn(p.sv[kx], xw[q + kx], a);
+            h[q] = a;
+          }
         }
-      }
+        static_for<SY>([&](auto KY) {
+          constexpr int ky = decltype(KY)::value;
+          constexpr int o = kr - ky;                  // output row (warp-relative) this box row feeds
+          if constexpr (o >= 0 && o < RPW) {
+            constexpr int slot = o % SY;
+#pragma unroll
+            for (int q = 0; q < 4; ++q) {
+              float a = ky == 0 ? 0.0f : acc[slot][q];
+              if constexpr (OP == K1_WSEP) {
+                a = __fmaf_rn(p.su[ky], h[q], a);
+              } else if constexpr (OP == K1_WSTAR) {
+                if constexpr (ky == RY) {
+#pragma unroll
+                  for (int kx = 0; kx < SX; ++kx) a = __fmaf_rn(p.wbox[ky * SX + kx], xw[q + kx], a);
+                } else {
+                  a = __fmaf_rn(p.wbox[ky * SX + RX], xw[q + RX], a);
+                }
+              } else {
+#pragma unroll
+                for (int kx = 0; kx < SX; ++kx) a = __fmaf_rn(p.wbox[ky * SX + kx], xw[q + kx], a);
+              }
+              acc[slot][q] = a;
+            }
+            if constexpr (ky == 2 * RY) store(o, acc[slot]);
+          }
+        });
+      });
+    } else {
+      // SRAD: all taps of an output at once from a ring of 2RY+1 x-windows
+      float ra[SY][W];
+      float rb[(NIN > 1) ? SY : 1][W];
+      static_for<RPW + 2 * RY>([&](auto KR) {
+        constexpr int kr = decltype(KR)::value;
+        constexpr int slot = kr % SY;
+        load_row<RX>(box0 + kr * BX4, lane, ra[slot]);
+        if constexpr (NIN > 1) load_row<RX>(box0 + BF4 + kr * BX4, lane, rb[slot]);
+        constexpr int o = kr - 2 * RY;
+        if constexpr (o >= 0) {
+          // rows o .. o+2RY of the box sit in slots (o + k) % SY
+          float wa[SY][W], wb[(NIN > 1) ? SY : 1][W];
+#pragma unroll
+          for (int k = 0; k < SY; ++k)
+#pragma unroll
+            for (int q = 0; q < W; ++q) {
+              wa[k][q] = ra[(o + k) % SY][q];
+              if constexpr (NIN > 1) wb[k][q] = rb[(o + k) % SY][q];
+            }
+          float v[4];
+          static_for<4>([&](auto I) {
+            constexpr int ii = decltype(I)::value;
+            if constexpr (OP == K1_SRAD1) {
+              v[ii] = op_srad1(RingAcc<RY, RX, ii>{wa}, p.prm);
+            } else {
+              v[ii] = op_srad2(RingAcc<RY, RX, ii>{wa}, RingAcc<RY, RX, ii>{wb}, p.prm);   // (c, I)
+            }
+          });
+          store(o, v);
+        }
+      });
     }
     __syncwarp();
     if (lane == 0) mbar_arrive(&empty[s]);
+    if (++s == S) { s = 0; ++pass; }
   }
 }
 
@@ -200,13 +257,13 @@ struct Launcher {
   int ctas_per_sm;
 };
 
-template <int OP, int RY, int RX, int RPW, int S, int NIN>
+template <int OP, int RY, int RX, int RPW, int S, int NIN, int MINB = 3>
 Launcher get_launcher() {
   static Launcher L{};
   static std::once_flag once;
   std::call_once(once, [] {
     using C = Cfg<RY, RPW, S, NIN>;
-    auto fn = k1_tile<OP, RY, RX, RPW, S, NIN>;
+    auto fn = k1_tile<OP, RY, RX, RPW, S, NIN, MINB>;
     cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
     int occ = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, NCONS + 32, C::SMEM) != cudaSuccess) occ = 1;
@@ -216,17 +273,50 @@ Launcher get_launcher() {
   return L;
 }
 
+bool star2d(const StencilParams& p, int RY, int RX) {
+  const int SX = 2 * RX + 1;
+  for (int ky = 0; ky < 2 * RY + 1; ++ky)
+    for (int kx = 0; kx < SX; ++kx)
+      if (ky != RY && kx != RX && p.wbox[ky * SX + kx] != 0.0f) return false;
+  return true;
+}
+
+#define K1_PICK(OPV, RYV, RXV, NINV) get_launcher<OPV, RYV, RXV, 6, 2, NINV>()
+
 bool pick(const StencilParams& p, Launcher* L) {
   const int ry = p.lo[1], rx = p.lo[2];
   if (p.op == OP_WEIGHTED) {
-    if (ry == 1 && rx == 1) { *L = get_launcher<K1_WBOX, 1, 1, 4, 3, 1>(); return true; }
-    if (ry == 2 && rx == 2) { *L = get_launcher<K1_WBOX, 2, 2, 4, 3, 1>(); return true; }
-    if (ry == 1 && rx == 2) { *L = get_launcher<K1_WBOX, 1, 2, 4, 3, 1>(); return true; }
-    if (ry == 2 && rx == 1) { *L = get_launcher<K1_WBOX, 2, 1, 4, 3, 1>(); return true; }
+    const int mode = p.sep ? K1_WSEP : (star2d(p, ry, rx) ? K1_WSTAR : K1_WBOX);
+    // tile-shape sweep hook (NEXT-4 / ATF role): LIFT_K1_VARIANT
+    // selects alternative (rows per warp, stages, CTAs per SM) for the
+    // separable radius-2 case; the default is the tuned one
+    static const int tv = [] { const char* e = getenv("LIFT_K1_VARIANT"); return e ? atoi(e) : 0; }();
+    if (mode == K1_WSEP && ry == 2 && rx == 2 && tv != 0) {
+      switch (tv) {
+        case 1: *L = get_launcher<K1_WSEP, 2, 2, 8, 2, 1, 3>(); return true;
+        case 2: *L = get_launcher<K1_WSEP, 2, 2, 4, 2, 1, 4>(); return true;
+        case 3: *L = get_launcher<K1_WSEP, 2, 2, 2, 4, 1, 4>(); return true;
+        case 4: *L = get_launcher<K1_WSEP, 2, 2, 8, 3, 1, 2>(); return true;
+        case 5: *L = get_launcher<K1_WSEP, 2, 2, 4, 3, 1, 3>(); return true;
+        default: break;
+      }
+    }
+#define K1_CASE(RYV, RXV)                                                     \
+  if (ry == RYV && rx == RXV) {                                              \
+    if (mode == K1_WSEP) *L = K1_PICK(K1_WSEP, RYV, RXV, 1);                 \
+    else if (mode == K1_WSTAR) *L = K1_PICK(K1_WSTAR, RYV, RXV, 1);          \
+    else *L = K1_PICK(K1_WBOX, RYV, RXV, 1);                                 \
+    return true;                                                             \
+  }
+    K1_CASE(1, 1)
+    K1_CASE(2, 2)
+    K1_CASE(1, 2)
+    K1_CASE(2, 1)
+#undef K1_CASE
     return false;
   }
-  if (p.op == OP_SRAD1) { *L = get_launcher<K1_SRAD1, 1, 1, 4, 3, 1>(); return true; }
-  if (p.op == OP_SRAD2) { *L = get_launcher<K1_SRAD2, 1, 1, 4, 3, 2>(); return true; }
+  if (p.op == OP_SRAD1) { *L = K1_PICK(K1_SRAD1, 1, 1, 1); return true; }
+  if (p.op == OP_SRAD2) { *L = K1_PICK(K1_SRAD2, 1, 1, 2); return true; }
   return false;
 }
 
