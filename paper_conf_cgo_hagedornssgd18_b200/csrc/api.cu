@@ -276,6 +276,10 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
     case OP_SRAD2:
       if (ndim != 2 || !centred(1)) return fail(STENCIL_E_INVALID, "SRAD needs ndim 2, size 3, pad 1, step 1");
       if (n_params < 1) return fail(STENCIL_E_INVALID, "SRAD needs 1 param");
+      if (op == OP_SRAD1) {
+        if (!(params[0] > 0.0f)) return fail(STENCIL_E_INVALID, "SRAD1 needs q0sqr > 0");
+        p.prm[1] = 1.0f / (params[0] * (1.0f + params[0]));   // derived plan constant
+      }
       p.radius = 1;
       break;
     case OP_ACOUSTIC:

@@ -32,6 +32,7 @@
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#include <algorithm>
 #include <atomic>
 #include <climits>
 #include <mutex>
@@ -458,9 +459,13 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);
   const int64_t tiles = (int64_t)ntx * nty;
   const int64_t slots = (int64_t)num_sms * L.ctas_per_sm;
-  // z-chunk: ~8 items per CTA for dynamic balance, at least 16 planes (halo re-load <= 2R/16)
-  int64_t zc = (nz_reg * tiles + 8 * slots - 1) / (8 * slots);
-  if (zc < 16) zc = 16;
+  // z-chunk: ~8 items per CTA for dynamic balance, at least 16 planes (halo
+  // re-load <= 2R/16) — unless the grid is too small to give every CTA two
+  // items (e.g. Hotspot3D's 8 planes), then parallelism wins over halo reuse
+  const int64_t work = nz_reg * tiles;
+  int64_t zc = (work + 8 * slots - 1) / (8 * slots);
+  const int64_t zmin = std::min<int64_t>(16, std::max<int64_t>(2, (work + 2 * slots - 1) / (2 * slots)));
+  if (zc < zmin) zc = zmin;
   if (zc > nz_reg) zc = nz_reg;
   const int64_t nchunk = (nz_reg + zc - 1) / zc;
   const int64_t items = tiles * nchunk;

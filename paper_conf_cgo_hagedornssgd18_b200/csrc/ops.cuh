@@ -64,25 +64,30 @@ __device__ __forceinline__ float op_hotspot3d(const Acc& T, float Pc, const floa
 }
 
 // ---- SRAD kernel 1: I -> c (Rodinia v3.1 srad; A18) --------------
+// The divisions of the definition are evaluated as correctly rounded
+// reciprocals (__frcp_rn) times the numerator; 1/(q0*(1+q0)) is a plan
+// constant (prm[1], computed once on the host).  q >= 0 keeps 1 + d >= 1/(1+q0)
+// away from 0, so the reciprocals are well conditioned (A18).
 template <class Acc>
 __device__ __forceinline__ float op_srad1(const Acc& I, const float* prm) {
-  const float q0 = prm[0];
+  const float q0 = prm[0], qinv = prm[1];
   const float Ic = I.template at<0, 0, 0>();
   const float dN = __fsub_rn(I.template at<0, -1, 0>(), Ic);
   const float dS = __fsub_rn(I.template at<0, 1, 0>(), Ic);
   const float dW = __fsub_rn(I.template at<0, 0, -1>(), Ic);
   const float dE = __fsub_rn(I.template at<0, 0, 1>(), Ic);
+  const float rI = __frcp_rn(Ic);
   float g = __fmul_rn(dN, dN);
   g = __fadd_rn(g, __fmul_rn(dS, dS));
   g = __fadd_rn(g, __fmul_rn(dW, dW));
   g = __fadd_rn(g, __fmul_rn(dE, dE));
-  const float G2 = __fdiv_rn(g, __fmul_rn(Ic, Ic));
-  const float L = __fdiv_rn(__fadd_rn(__fadd_rn(__fadd_rn(dN, dS), dW), dE), Ic);
+  const float G2 = __fmul_rn(g, __fmul_rn(rI, rI));
+  const float L = __fmul_rn(__fadd_rn(__fadd_rn(__fadd_rn(dN, dS), dW), dE), rI);
   const float num = __fsub_rn(__fmul_rn(0.5f, G2), __fmul_rn(0.0625f, __fmul_rn(L, L)));
   const float den = __fadd_rn(1.0f, __fmul_rn(0.25f, L));
-  const float q = __fdiv_rn(num, __fmul_rn(den, den));
-  const float d = __fdiv_rn(__fsub_rn(q, q0), __fmul_rn(q0, __fadd_rn(1.0f, q0)));
-  float c = __fdiv_rn(1.0f, __fadd_rn(1.0f, d));
+  const float q = __fmul_rn(num, __frcp_rn(__fmul_rn(den, den)));
+  const float d = __fmul_rn(__fsub_rn(q, q0), qinv);
+  float c = __frcp_rn(__fadd_rn(1.0f, d));
   c = c < 0.0f ? 0.0f : (c > 1.0f ? 1.0f : c);
   return c;
 }
