@@ -278,7 +278,9 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
       if (n_params < 1) return fail(STENCIL_E_INVALID, "SRAD needs 1 param");
       if (op == OP_SRAD1) {
         if (!(params[0] > 0.0f)) return fail(STENCIL_E_INVALID, "SRAD1 needs q0sqr > 0");
-        p.prm[1] = 1.0f / (params[0] * (1.0f + params[0]));   // derived plan constant
+        const double q0 = params[0];                       // derived plan constants (A18b)
+        p.prm[1] = (float)(q0 / (1.0 + q0));
+        p.prm[2] = (float)(1.0 / (q0 * (1.0 + q0)));
       }
       p.radius = 1;
       break;

@@ -61,13 +61,16 @@ __device__ unsigned int g_done[kTickets];
 
 enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2 };
 
-template <int R, int RPW, int S>
+template <int R, int RPW, int S, bool PW>
 struct Cfg {
   static constexpr int TY = NW * RPW;
   static constexpr int BY = TY + 2 * R;
   static constexpr int TX_BYTES = BX * BY * 4;
   static constexpr int STAGE_FLOATS = ((TX_BYTES + 127) / 128) * 128 / 4;
-  static constexpr int SMEM = S * STAGE_FLOATS * 4 + 2 * S * 8 + 2 * S * 4 + 128 + 128;
+  static constexpr int PS = PW ? 3 : 0;                 // point-wise ring slots
+  static constexpr int PW_BYTES = TX * TY * 4;
+  static constexpr int PW_FLOATS = TX * TY;
+  static constexpr int SMEM = S * STAGE_FLOATS * 4 + PS * PW_BYTES + 2 * (S + PS) * 8 + 2 * S * 4 + 128 + 128;
 };
 
 template <int R>
@@ -121,19 +124,23 @@ __device__ __forceinline__ float pick4(int s, const float4& c, float pv) {
 template <int OP, int R, int RPW, int S, bool ZC>
 __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
-             const float* __restrict__ src, const float* pw_in, float* out, int ntx, int nty, int zc,
-             int nchunk, int slot) {
-  using C = Cfg<R, RPW, S>;
+             const __grid_constant__ CUtensorMap pwmap, const float* __restrict__ src, float* out, int ntx,
+             int nty, int zc, int nchunk, int slot) {
+  using C = Cfg<R, RPW, S, OP != K2_WSTAR>;
+  constexpr bool PW = OP != K2_WSTAR;           // a point-wise zipped grid (Hotspot P, Acoustic prev)
+  constexpr int PS = C::PS;                     // point-wise ring slots
+  constexpr int PWF4 = C::PW_FLOATS / 4;
   constexpr int TY = C::TY;
-  constexpr int NR = 2 * R + 1;                 // planes in the z register ring
   constexpr int SF4 = C::STAGE_FLOATS / 4;      // stage size in float4
   constexpr int BX4 = BX / 4;
   // dynamic smem (no static smem in this kernel, so it starts the CTA's window):
-  // [S stages][full S][empty S][stage_item S][stage_const S]
+  // [S plane stages][PS point-wise slots][full S][empty S][pwfull PS][pwempty PS][stage_item S][stage_const S]
   extern __shared__ __align__(128) float4 dsm4[];
-  uint64_t* full = reinterpret_cast<uint64_t*>(dsm4 + S * SF4);
+  uint64_t* full = reinterpret_cast<uint64_t*>(dsm4 + S * SF4 + PS * PWF4);
   uint64_t* empty = full + S;
-  int* stage_item = reinterpret_cast<int*>(empty + S);
+  uint64_t* pwfull = empty + S;
+  uint64_t* pwempty = pwfull + PS;
+  int* stage_item = reinterpret_cast<int*>(pwempty + PS);
   int* stage_const = stage_item + S;
 
   const int ntile = ntx * nty;
@@ -145,6 +152,10 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
       mbar_init(&full[s], 1);
       mbar_init(&empty[s], NW);
     }
+    for (int s = 0; s < PS; ++s) {
+      mbar_init(&pwfull[s], 1);
+      mbar_init(&pwempty[s], NW);
+    }
     fence_mbar_init();
   }
   __syncthreads();
@@ -153,8 +164,11 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
     // ---------------- producer: items from the ticket counter, one TMA box per plane ----------------
     if (lane == 0) {
       prefetch_tmap(&tmap);
+      if constexpr (PW) prefetch_tmap(&pwmap);
       int s = 0;
       uint32_t pass = 0;
+      int ps = 0;
+      uint32_t ppass = 0;
       while (true) {
         const int item = (int)atomicAdd(&g_ticket[slot], 1u);
         const bool done = item >= nitems;
@@ -181,6 +195,16 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
             mbar_arrive(&full[s]);   // constant plane (value pad) or end marker: nothing to load
           }
           if (++s == S) { s = 0; ++pass; }
+          if constexpr (PW) {
+            // the point-wise box of output plane zs + i - R rides with that plane's load
+            if (!done && i >= R && i < nload - R) {
+              if (ppass > 0) mbar_wait(&pwempty[ps], (ppass - 1) & 1);
+              mbar_arrive_expect_tx(&pwfull[ps], C::PW_BYTES);
+              tma_load_3d(dsm4 + S * SF4 + ps * PWF4, &pwmap, &pwfull[ps], x0, y0,
+                          (int)(zs - R + i + p.ghost));
+              if (++ps == PS) { ps = 0; ++ppass; }
+            }
+          }
         }
         if (done) break;
       }
@@ -209,6 +233,8 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
     }
     int sn = 0;            // stage of the next load to wait for
     uint32_t pn = 0;       // its pass (barrier phase parity)
+    int psc = 0;           // point-wise ring slot of the current output plane
+    uint32_t ppc = 0;
     while (true) {
       mbar_wait(&full[sn], pn & 1);
       const int item = stage_item[sn];
@@ -256,7 +282,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
         if (++sn == S) { sn = 0; ++pn; }
       }
       float* orow = out + ((zs + p.ghost) * p.plane + (int64_t)(y0 + warp * RPW) * nx + xo);
-      const float* prow = pw_in + ((zs + p.ghost) * p.plane + (int64_t)(y0 + warp * RPW) * nx + xo);
+
       for (int j = 0; j < nzc; ++j) {
         mbar_wait(&full[sn], pn & 1);
         zst[2 * R] = (ZC && stage_const[sn]) ? -1 - sn : sn;
@@ -269,19 +295,19 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
           fence_proxy_async_smem();
           named_bar_sync(1, NCONS);
         }
+        // point-wise input of this output plane: its own TMA ring (no halo)
+        if constexpr (PW) mbar_wait(&pwfull[psc], ppc & 1);
 #pragma unroll
         for (int jj = 0; jj < RPW; ++jj) {
           const int rr = warp * RPW + jj;
           const int gy = y0 + rr;
           const bool ok = x_ok && gy < ny;
           float4 pw = make_float4(0.f, 0.f, 0.f, 0.f);
-          if constexpr (OP != K2_WSTAR) {
-            if (ok) pw = ldg128(prow + jj * nx);
-          }
+          if constexpr (PW) pw = dsm4[S * SF4 + psc * PWF4 + (warp * RPW + jj) * (TX / 4) + lane];
           const int rb = roff4 + jj * BX4;          // row offset within a stage
-          Win<R> w;
           const float4 c = dsm4[cbase + rb];
           const float4 e = dsm4[cbase + eoff4 + jj * BX4];
+          float xw[4 + 2 * R];                      // centre row, x offsets -R .. 3+R
           {
             const float cv[4] = {c.x, c.y, c.z, c.w};
             const float ev[4] = {e.x, e.y, e.z, e.w};
@@ -293,39 +319,87 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
               if (lane == 31) r = ev[k - 1];
               if (pl) l = pick4(sl[k - 1], c, 0.0f);
               if (pr) r = pick4(sr[k - 1], c, 0.0f);
-              w.x[R - k] = l;
-              w.x[R + 3 + k] = r;
+              xw[R - k] = l;
+              xw[R + 3 + k] = r;
             }
 #pragma unroll
-            for (int i = 0; i < 4; ++i) w.x[R + i] = cv[i];
+            for (int i = 0; i < 4; ++i) xw[R + i] = cv[i];
           }
-#pragma unroll
-          for (int k = 1; k <= R; ++k) {
-            set4(w.ym[k - 1], dsm4[cbase + rb + om[jj][k - 1]]);
-            set4(w.yp[k - 1], dsm4[cbase + rb + oq[jj][k - 1]]);
-            const int am = zst[R - k], ap = zst[R + k];
-            if constexpr (ZC) {
-              set4(w.zm[k - 1], am < 0 ? pv4 : dsm4[am * SF4 + rb]);
-              set4(w.zp[k - 1], ap < 0 ? pv4 : dsm4[ap * SF4 + rb]);
-            } else {
-              set4(w.zm[k - 1], dsm4[am * SF4 + rb]);
-              set4(w.zp[k - 1], dsm4[ap * SF4 + rb]);
-            }
-          }
+          auto zrow = [&](int k) -> float4 {       // centre float4 of plane z + k
+            const int a = zst[R + k];
+            if constexpr (ZC) return a < 0 ? pv4 : dsm4[a * SF4 + rb];
+            return dsm4[a * SF4 + rb];
+          };
           float4 res;
-          res.x = eval<OP, R, 0>(p, w, pw, gz, gy, xo);
-          res.y = eval<OP, R, 1>(p, w, pw, gz, gy, xo);
-          res.z = eval<OP, R, 2>(p, w, pw, gz, gy, xo);
-          res.w = eval<OP, R, 3>(p, w, pw, gz, gy, xo);
+          if constexpr (OP == K2_ACOUSTIC) {
+            // ordered neighbour sum (acoustic_sum's row-major order), accumulated
+            // as the taps are loaded: z-R..z-1, y-R..y-1, x-R..x-1, x+1..x+R,
+            // y+1..y+R, z+1..z+R
+            float sm[4];
+            bool first = true;
+            auto add4 = [&](const float4& v) {
+              const float vv[4] = {v.x, v.y, v.z, v.w};
+#pragma unroll
+              for (int i = 0; i < 4; ++i) sm[i] = first ? vv[i] : __fadd_rn(sm[i], vv[i]);
+              first = false;
+            };
+#pragma unroll
+            for (int k = R; k >= 1; --k) add4(zrow(-k));
+#pragma unroll
+            for (int k = R; k >= 1; --k) add4(dsm4[cbase + rb + om[jj][k - 1]]);
+#pragma unroll
+            for (int k = R; k >= 1; --k) add4(make_float4(xw[0 + R - k], xw[1 + R - k], xw[2 + R - k], xw[3 + R - k]));
+#pragma unroll
+            for (int k = 1; k <= R; ++k) add4(make_float4(xw[0 + R + k], xw[1 + R + k], xw[2 + R + k], xw[3 + R + k]));
+#pragma unroll
+            for (int k = 1; k <= R; ++k) add4(dsm4[cbase + rb + oq[jj][k - 1]]);
+#pragma unroll
+            for (int k = 1; k <= R; ++k) add4(zrow(k));
+            const int Kzy = [&] {
+              int K = 0;
+#pragma unroll
+              for (int o = 1; o <= R; ++o)
+                K += (gz - o >= 0) + (gz + o < (int)p.gnz) + (gy - o >= 0) + (gy + o < ny);
+              return K;
+            }();
+            const float pwv[4] = {pw.x, pw.y, pw.z, pw.w};
+            float rv[4];
+#pragma unroll
+            for (int i = 0; i < 4; ++i) {
+              int K = Kzy;
+#pragma unroll
+              for (int o = 1; o <= R; ++o) K += (xo + i - o >= 0) + (xo + i + o < nx);
+              rv[i] = acoustic_combine<R>(sm[i], xw[R + i], pwv[i], K, p.prm);
+            }
+            res = make_float4(rv[0], rv[1], rv[2], rv[3]);
+          } else {
+            Win<R> w;
+#pragma unroll
+            for (int i = 0; i < 4 + 2 * R; ++i) w.x[i] = xw[i];
+#pragma unroll
+            for (int k = 1; k <= R; ++k) {
+              set4(w.ym[k - 1], dsm4[cbase + rb + om[jj][k - 1]]);
+              set4(w.yp[k - 1], dsm4[cbase + rb + oq[jj][k - 1]]);
+              set4(w.zm[k - 1], zrow(-k));
+              set4(w.zp[k - 1], zrow(k));
+            }
+            res.x = eval<OP, R, 0>(p, w, pw, gz, gy, xo);
+            res.y = eval<OP, R, 1>(p, w, pw, gz, gy, xo);
+            res.z = eval<OP, R, 2>(p, w, pw, gz, gy, xo);
+            res.w = eval<OP, R, 3>(p, w, pw, gz, gy, xo);
+          }
           if (ok) stg128(orow + jj * nx, res);
         }
         orow += p.plane;
-        prow += p.plane;
         // plane z - R is no longer needed (pre-chunk planes included)
         __syncwarp();
         if (lane == 0) {
           const int t = zst[0] < 0 ? -1 - zst[0] : zst[0];
           mbar_arrive(&empty[t]);
+          if constexpr (PW) mbar_arrive(&pwempty[psc]);
+        }
+        if constexpr (PW) {
+          if (++psc == PS) { psc = 0; ++ppc; }
         }
 #pragma unroll
         for (int k = 0; k < 2 * R; ++k) zst[k] = zst[k + 1];
@@ -377,7 +451,7 @@ Launcher get_launcher() {
   static Launcher L{};
   static std::once_flag once;
   std::call_once(once, [] {
-    using C = Cfg<R, RPW, S>;
+    using C = Cfg<R, RPW, S, OP != K2_WSTAR>;
     auto fn = k2_sweep<OP, R, RPW, S, ZC>;
     cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
     int occ = 0;
@@ -396,28 +470,29 @@ Launcher pick(const StencilParams& p) {
     return zc ? get_launcher<K2_WSTAR, 2, 2, 8, true>() : get_launcher<K2_WSTAR, 2, 2, 8, false>();
   }
   if (p.op == OP_HOTSPOT3D)
-    return zc ? get_launcher<K2_HOTSPOT, 1, 2, 7, true>() : get_launcher<K2_HOTSPOT, 1, 2, 7, false>();
-  if (R == 1) return zc ? get_launcher<K2_ACOUSTIC, 1, 2, 7, true>() : get_launcher<K2_ACOUSTIC, 1, 2, 7, false>();
+    return zc ? get_launcher<K2_HOTSPOT, 1, 2, 5, true>() : get_launcher<K2_HOTSPOT, 1, 2, 5, false>();
+  if (R == 1) return zc ? get_launcher<K2_ACOUSTIC, 1, 2, 5, true>() : get_launcher<K2_ACOUSTIC, 1, 2, 5, false>();
   return zc ? get_launcher<K2_ACOUSTIC, 2, 2, 8, true>() : get_launcher<K2_ACOUSTIC, 2, 2, 8, false>();
 }
 
 struct MapEntry {
   const float* base;
   int64_t nx, ny, nz;
-  int by;
+  int bx, by;
   CUtensorMap map;
 };
 
-bool get_map(const float* base, int64_t nx, int64_t ny, int64_t nz, int by, CUtensorMap* out, std::string* err) {
+bool get_map(const float* base, int64_t nx, int64_t ny, int64_t nz, int bx, int by, CUtensorMap* out,
+             std::string* err) {
   thread_local MapEntry cache[8];
   thread_local int next = 0;
   for (auto& e : cache)
-    if (e.base == base && e.nx == nx && e.ny == ny && e.nz == nz && e.by == by) {
+    if (e.base == base && e.nx == nx && e.ny == ny && e.nz == nz && e.bx == bx && e.by == by) {
       *out = e.map;
       return true;
     }
-  MapEntry e{base, nx, ny, nz, by, {}};
-  if (!encode_tensor_map_3d(&e.map, base, nx, ny, nz, BX, (uint32_t)by, 1, err)) return false;
+  MapEntry e{base, nx, ny, nz, bx, by, {}};
+  if (!encode_tensor_map_3d(&e.map, base, nx, ny, nz, (uint32_t)bx, (uint32_t)by, 1, err)) return false;
   cache[next] = e;
   next = (next + 1) % 8;
   *out = e.map;
@@ -453,8 +528,13 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   const int R = p.radius;
   const float* slid = (p.op == OP_ACOUSTIC) ? in1 : in0;
   const float* pw = (p.op == OP_ACOUSTIC) ? in0 : (p.op == OP_HOTSPOT3D ? in1 : nullptr);
-  CUtensorMap map;
-  if (!get_map(slid, p.n[2], p.n[1], p.n[0] + 2 * p.ghost, L.ty + 2 * R, &map, err)) return cudaErrorInvalidValue;
+  CUtensorMap map, pwmap;
+  if (!get_map(slid, p.n[2], p.n[1], p.n[0] + 2 * p.ghost, BX, L.ty + 2 * R, &map, err)) return cudaErrorInvalidValue;
+  if (pw) {
+    if (!get_map(pw, p.n[2], p.n[1], p.n[0] + 2 * p.ghost, TX, L.ty, &pwmap, err)) return cudaErrorInvalidValue;
+  } else {
+    pwmap = map;
+  }
   const int ntx = (int)((p.n[2] + TX - 1) / TX);
   const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);
   const int64_t tiles = (int64_t)ntx * nty;
@@ -473,7 +553,7 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   int64_t grid = slots < items ? slots : items;
   int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk;
   int slot = (int)(g_slot.fetch_add(1) % kTickets);
-  void* args[] = {(void*)&p, (void*)&map, (void*)&slid, (void*)&pw, (void*)&out,
+  void* args[] = {(void*)&p, (void*)&map, (void*)&pwmap, (void*)&slid, (void*)&out,
                   &ntx_i, &nty_i, &zc_i, &nch_i, &slot};
   return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
 }

@@ -64,30 +64,30 @@ __device__ __forceinline__ float op_hotspot3d(const Acc& T, float Pc, const floa
 }
 
 // ---- SRAD kernel 1: I -> c (Rodinia v3.1 srad; A18) --------------
-// The divisions of the definition are evaluated as correctly rounded
-// reciprocals (__frcp_rn) times the numerator; 1/(q0*(1+q0)) is a plan
-// constant (prm[1], computed once on the host).  q >= 0 keeps 1 + d >= 1/(1+q0)
-// away from 0, so the reciprocals are well conditioned (A18).
+// Definition: G2 = g/Ic^2, L = sd/Ic (g = sum dX^2, sd = sum dX),
+// q = (G2/2 - L^2/16) / (1 + L/4)^2, d = (q - q0)/(q0(1+q0)), c = 1/(1+d).
+// Multiplying through by Ic^2 gives the same function with one reciprocal and
+// only non-negative terms (reading A18b):
+//   D = Ic + sd/4,  n0 = g/2 - sd^2/16 (>= g/4 by Cauchy-Schwarz),
+//   c = D^2 / (a*D^2 + b*n0),  a = q0/(1+q0),  b = 1/(q0(1+q0))
+// with a, b plan constants (prm[1], prm[2]); then c is clamped to [0, 1].
 template <class Acc>
 __device__ __forceinline__ float op_srad1(const Acc& I, const float* prm) {
-  const float q0 = prm[0], qinv = prm[1];
+  const float a = prm[1], b = prm[2];
   const float Ic = I.template at<0, 0, 0>();
   const float dN = __fsub_rn(I.template at<0, -1, 0>(), Ic);
   const float dS = __fsub_rn(I.template at<0, 1, 0>(), Ic);
   const float dW = __fsub_rn(I.template at<0, 0, -1>(), Ic);
   const float dE = __fsub_rn(I.template at<0, 0, 1>(), Ic);
-  const float rI = __frcp_rn(Ic);
   float g = __fmul_rn(dN, dN);
-  g = __fadd_rn(g, __fmul_rn(dS, dS));
-  g = __fadd_rn(g, __fmul_rn(dW, dW));
-  g = __fadd_rn(g, __fmul_rn(dE, dE));
-  const float G2 = __fmul_rn(g, __fmul_rn(rI, rI));
-  const float L = __fmul_rn(__fadd_rn(__fadd_rn(__fadd_rn(dN, dS), dW), dE), rI);
-  const float num = __fsub_rn(__fmul_rn(0.5f, G2), __fmul_rn(0.0625f, __fmul_rn(L, L)));
-  const float den = __fadd_rn(1.0f, __fmul_rn(0.25f, L));
-  const float q = __fmul_rn(num, __frcp_rn(__fmul_rn(den, den)));
-  const float d = __fmul_rn(__fsub_rn(q, q0), qinv);
-  float c = __frcp_rn(__fadd_rn(1.0f, d));
+  g = __fmaf_rn(dS, dS, g);
+  g = __fmaf_rn(dW, dW, g);
+  g = __fmaf_rn(dE, dE, g);
+  const float sd = __fadd_rn(__fadd_rn(__fadd_rn(dN, dS), dW), dE);
+  const float n0 = __fmaf_rn(-0.0625f, __fmul_rn(sd, sd), __fmul_rn(0.5f, g));
+  const float D = __fmaf_rn(0.25f, sd, Ic);
+  const float D2 = __fmul_rn(D, D);
+  float c = __fmul_rn(D2, __frcp_rn(__fmaf_rn(a, D2, __fmul_rn(b, n0))));
   c = c < 0.0f ? 0.0f : (c > 1.0f ? 1.0f : c);
   return c;
 }
@@ -155,17 +155,22 @@ __device__ __forceinline__ int acoustic_K(Int gz, Int gy, Int gx, Int nz, Int ny
   return K;
 }
 
-template <int R, class Acc>
-__device__ __forceinline__ float op_acoustic(const Acc& U, float prev, int K, const float* prm) {
+// the point update given the ordered neighbour sum s and the centre uc
+template <int R>
+__device__ __forceinline__ float acoustic_combine(float s, float uc, float prev, int K, const float* prm) {
   const float l2 = prm[0], loss1 = prm[1], loss2 = prm[2];
   constexpr int kmax = 6 * R;
   const float cf1 = K < kmax ? loss1 : 1.0f;
   const float cf2 = K < kmax ? loss2 : 1.0f;
-  const float s = acoustic_sum<R>(U);
-  float t = __fmul_rn(__fsub_rn(2.0f, __fmul_rn(l2, (float)K)), U.template at<0, 0, 0>());
+  float t = __fmul_rn(__fsub_rn(2.0f, __fmul_rn(l2, (float)K)), uc);
   t = __fmaf_rn(l2, s, t);
   t = __fmaf_rn(-cf2, prev, t);
   return __fmul_rn(cf1, t);
+}
+
+template <int R, class Acc>
+__device__ __forceinline__ float op_acoustic(const Acc& U, float prev, int K, const float* prm) {
+  return acoustic_combine<R>(acoustic_sum<R>(U), U.template at<0, 0, 0>(), prev, K, prm);
 }
 
 }  // namespace lift
