@@ -290,6 +290,9 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
         const int gz = (int)(p.z_off + zs + j);
         const int cbase = zst[R] * SF4;             // the centre plane is inside the grid
         if (fix) {
+          // all warps are past the previous plane (which read this stage as its
+          // z+1 neighbour, including the padding lanes/rows of ragged tiles)
+          named_bar_sync(1, NCONS);
           fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + cbase), src,
                                                  plane_of(p, (int64_t)gz), x0, y0, threadIdx.x);
           fence_proxy_async_smem();
