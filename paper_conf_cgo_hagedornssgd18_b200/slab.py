@@ -114,7 +114,7 @@ class SlabPlan:
 
     def __init__(self, global_extents: Sequence[int], rank: int, world: int, size=3, pad=None, kind="clamp",
                  pad_value: float = 0.0, op="weighted", weights=None, params=(), group=None,
-                 device: Optional[int] = None, exchange=None):
+                 device: Optional[int] = None, exchange=None, exchange_factory=None):
         from .plan import Plan, KINDS, _kind
         self.global_extents = tuple(int(e) for e in global_extents)
         self.rank, self.world = rank, world
@@ -127,8 +127,8 @@ class SlabPlan:
             raise ValueError("slab thinner than the ghost width")
         self.plan.set_slab(self.z0, self.global_extents[0], self.g)
         self.wrap = self.plan.kind[0] == WRAP
-        self.exchange = exchange if exchange is not None else DistExchange(rank, world, self.n, self.g, self.wrap,
-                                                                            group)
+        factory = exchange_factory if exchange_factory is not None else DistExchange
+        self.exchange = exchange if exchange is not None else factory(rank, world, self.n, self.g, self.wrap, group)
         self.comm = torch.cuda.Stream(device=self.plan.device)
         self.alloc_shape = self.plan.alloc_extents
 
