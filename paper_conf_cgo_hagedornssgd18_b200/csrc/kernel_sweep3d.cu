@@ -35,6 +35,7 @@
 #include <algorithm>
 #include <atomic>
 #include <climits>
+#include <cstdlib>
 #include <mutex>
 #include <string>
 
@@ -70,7 +71,7 @@ struct Cfg {
   static constexpr int PS = PW ? 3 : 0;                 // point-wise ring slots
   static constexpr int PW_BYTES = TX * TY * 4;
   static constexpr int PW_FLOATS = TX * TY;
-  static constexpr int SMEM = S * STAGE_FLOATS * 4 + PS * PW_BYTES + 2 * (S + PS) * 8 + 2 * S * 4 + 128 + 128;
+  static constexpr int SMEM = S * STAGE_FLOATS * 4 + PS * PW_BYTES + 2 * (S + PS + 4) * 8 + (2 * S + 4) * 4 + 256;
 };
 
 template <int R>
@@ -122,13 +123,14 @@ __device__ __forceinline__ float pick4(int s, const float4& c, float pv) {
 }
 
 template <int OP, int R, int RPW, int S, bool ZC>
-__global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
+__global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
              const __grid_constant__ CUtensorMap pwmap, const float* __restrict__ src, float* out, int ntx,
              int nty, int zc, int nchunk, int slot) {
   using C = Cfg<R, RPW, S, OP != K2_WSTAR>;
   constexpr bool PW = OP != K2_WSTAR;           // a point-wise zipped grid (Hotspot P, Acoustic prev)
   constexpr int PS = C::PS;                     // point-wise ring slots
+  constexpr int QN = 4;                         // item queue between the two producer lanes
   constexpr int PWF4 = C::PW_FLOATS / 4;
   constexpr int TY = C::TY;
   constexpr int SF4 = C::STAGE_FLOATS / 4;      // stage size in float4
@@ -140,8 +142,11 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
   uint64_t* empty = full + S;
   uint64_t* pwfull = empty + S;
   uint64_t* pwempty = pwfull + PS;
-  int* stage_item = reinterpret_cast<int*>(pwempty + PS);
+  uint64_t* itemfull = pwempty + PS;
+  uint64_t* itemempty = itemfull + QN;
+  int* stage_item = reinterpret_cast<int*>(itemempty + QN);
   int* stage_const = stage_item + S;
+  int* item_q = stage_const + S;
 
   const int ntile = ntx * nty;
   const int nitems = ntile * nchunk;
@@ -156,22 +161,35 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
       mbar_init(&pwfull[s], 1);
       mbar_init(&pwempty[s], NW);
     }
+    for (int s = 0; s < QN; ++s) {
+      mbar_init(&itemfull[s], 1);
+      mbar_init(&itemempty[s], 1);
+    }
     fence_mbar_init();
   }
   __syncthreads();
 
   if (warp == NW) {
-    // ---------------- producer: items from the ticket counter, one TMA box per plane ----------------
+    // ---------------- producers ----------------
+    // lane 0: items from the ticket counter, one TMA box per input plane;
+    // lane 1 (point-wise ops): the point-wise box of every output plane, fed
+    // the item sequence through a small queue so that a full point-wise ring
+    // never holds back the plane prefetch
     if (lane == 0) {
       prefetch_tmap(&tmap);
-      if constexpr (PW) prefetch_tmap(&pwmap);
       int s = 0;
       uint32_t pass = 0;
-      int ps = 0;
-      uint32_t ppass = 0;
+      int q = 0;
+      uint32_t qpass = 0;
       while (true) {
         const int item = (int)atomicAdd(&g_ticket[slot], 1u);
         const bool done = item >= nitems;
+        if constexpr (PW) {
+          if (qpass > 0) mbar_wait(&itemempty[q], (qpass - 1) & 1);
+          item_q[q] = done ? -1 : item;
+          mbar_arrive(&itemfull[q]);
+          if (++q == QN) { q = 0; ++qpass; }
+        }
         int nload = 1, x0 = 0, y0 = 0;
         int64_t zs = 0;
         if (!done) {
@@ -195,18 +213,29 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
             mbar_arrive(&full[s]);   // constant plane (value pad) or end marker: nothing to load
           }
           if (++s == S) { s = 0; ++pass; }
-          if constexpr (PW) {
-            // the point-wise box of output plane zs + i - R rides with that plane's load
-            if (!done && i >= R && i < nload - R) {
-              if (ppass > 0) mbar_wait(&pwempty[ps], (ppass - 1) & 1);
-              mbar_arrive_expect_tx(&pwfull[ps], C::PW_BYTES);
-              tma_load_3d(dsm4 + S * SF4 + ps * PWF4, &pwmap, &pwfull[ps], x0, y0,
-                          (int)(zs - R + i + p.ghost));
-              if (++ps == PS) { ps = 0; ++ppass; }
-            }
-          }
         }
         if (done) break;
+      }
+    } else if (PW && lane == 1) {
+      prefetch_tmap(&pwmap);
+      int ps = 0, q = 0;
+      uint32_t ppass = 0, qpass = 0;
+      while (true) {
+        mbar_wait(&itemfull[q], qpass & 1);
+        const int item = item_q[q];
+        mbar_arrive(&itemempty[q]);
+        if (++q == QN) { q = 0; ++qpass; }
+        if (item < 0) break;
+        const int chunk = item / ntile, tile = item % ntile;
+        const int x0 = (tile % ntx) * TX, y0 = (tile / ntx) * TY;
+        const int64_t zs = p.reg0 + (int64_t)chunk * zc;
+        const int nzc = (int)(min(zs + (int64_t)zc, p.reg1) - zs);
+        for (int j = 0; j < nzc; ++j) {
+          if (ppass > 0) mbar_wait(&pwempty[ps], (ppass - 1) & 1);
+          mbar_arrive_expect_tx(&pwfull[ps], C::PW_BYTES);
+          tma_load_3d(dsm4 + S * SF4 + ps * PWF4, &pwmap, &pwfull[ps], x0, y0, (int)(zs + j + p.ghost));
+          if (++ps == PS) { ps = 0; ++ppass; }
+        }
       }
     }
   } else {
@@ -255,6 +284,18 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
       const bool pl = !wrap_fix && kx != PAD_CONSTANT && x0 == 0 && lane == 0;   // left x-halo out of grid
       const bool pr = !wrap_fix && kx != PAD_CONSTANT && xo + 4 == nx;           // right x-halo out of grid
       const bool yr = !wrap_fix && ky != PAD_CONSTANT && y_edge;
+      // Acoustic: x part of the in-domain neighbour count of the lane's 4
+      // outputs, packed 4 bits each (computed once per item)
+      int kxp = 0;
+      if constexpr (OP == K2_ACOUSTIC) {
+#pragma unroll
+        for (int i = 0; i < 4; ++i) {
+          int kxi = 0;
+#pragma unroll
+          for (int o = 1; o <= R; ++o) kxi += (xo + i - o >= 0) + (xo + i + o < nx);
+          kxp |= kxi << (4 * i);
+        }
+      }
       // float4 offsets of rows y-k / y+k relative to row y (pad redirect folded in)
       int om[RPW][R], oq[RPW][R];
 #pragma unroll
@@ -368,12 +409,8 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 ? 3 : 2))
             const float pwv[4] = {pw.x, pw.y, pw.z, pw.w};
             float rv[4];
 #pragma unroll
-            for (int i = 0; i < 4; ++i) {
-              int K = Kzy;
-#pragma unroll
-              for (int o = 1; o <= R; ++o) K += (xo + i - o >= 0) + (xo + i + o < nx);
-              rv[i] = acoustic_combine<R>(sm[i], xw[R + i], pwv[i], K, p.prm);
-            }
+            for (int i = 0; i < 4; ++i)
+              rv[i] = acoustic_combine<R>(sm[i], xw[R + i], pwv[i], Kzy + ((kxp >> (4 * i)) & 15), p.prm);
             res = make_float4(rv[0], rv[1], rv[2], rv[3]);
           } else {
             Win<R> w;
@@ -475,6 +512,16 @@ Launcher pick(const StencilParams& p) {
   if (p.op == OP_HOTSPOT3D)
     return zc ? get_launcher<K2_HOTSPOT, 1, 2, 5, true>() : get_launcher<K2_HOTSPOT, 1, 2, 5, false>();
   if (R == 1) return zc ? get_launcher<K2_ACOUSTIC, 1, 2, 5, true>() : get_launcher<K2_ACOUSTIC, 1, 2, 5, false>();
+  // tile-shape sweep hook (NEXT-4 / ATF role): LIFT_K2_VARIANT
+  static const int tv = [] { const char* e = getenv("LIFT_K2_VARIANT"); return e ? atoi(e) : 0; }();
+  if (zc) {
+    switch (tv) {
+      case 1: return get_launcher<K2_ACOUSTIC, 2, 1, 8, true>();
+      case 2: return get_launcher<K2_ACOUSTIC, 2, 2, 6, true>();
+      case 3: return get_launcher<K2_ACOUSTIC, 2, 1, 10, true>();
+      default: break;
+    }
+  }
   return zc ? get_launcher<K2_ACOUSTIC, 2, 2, 8, true>() : get_launcher<K2_ACOUSTIC, 2, 2, 8, false>();
 }
 
