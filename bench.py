@@ -186,6 +186,11 @@ def main():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--no-graph", action="store_true", help="launch single sweeps eagerly instead of a CUDA graph")
+    ap.add_argument("--force-slab", action="store_true",
+                    help="run the slab (multi-GPU) path even at world size 1 (launch under torchrun)")
+    ap.add_argument("--halo", default="nccl", choices=["nccl", "fused"],
+                    help="multi-GPU ghost exchange: NCCL send/recv overlapped with the interior (default), or the "
+                         "fused boundary kernel storing into the neighbours' ghosts over NVLink peer memory")
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
 
@@ -198,13 +203,15 @@ def main():
 
     import stencil_inputs as si
     import paper_conf_cgo_hagedornssgd18_b200 as lift
-    from paper_conf_cgo_hagedornssgd18_b200.slab import SlabPlan
+    from paper_conf_cgo_hagedornssgd18_b200.slab import SlabPlan, symmetric_fused_halo
 
     world = env_int("WORLD_SIZE", 1)
+    sym, fused = None, None
     rank = env_int("RANK", 0)
     local = env_int("LOCAL_RANK", 0)
     torch.cuda.set_device(local)
-    if world > 1:
+    use_pg = world > 1 or (args.force_slab and "MASTER_ADDR" in os.environ)
+    if use_pg:
         dist.init_process_group("nccl", device_id=torch.device(f"cuda:{local}"))
     dev = torch.device(f"cuda:{local}")
 
@@ -213,7 +220,7 @@ def main():
     spec = w.spec
     ext1 = spec.extents
     iterable = spec.op in (si.WEIGHTED, si.HOTSPOT3D, si.ACOUSTIC) and steps_per_iter > 1
-    slabbed = world > 1 and iterable and len(ext1) == 3
+    slabbed = (world > 1 or (args.force_slab and use_pg)) and iterable and len(ext1) == 3
 
     # ---- inputs: seeded synthetic grids resident in HBM (host copies kept for e2e)
     local_ext = ext1
@@ -237,8 +244,13 @@ def main():
         plan = sp.plan
         host = [torch.from_numpy(x).pin_memory() for x in xs]
         bufs = []
-        for x in host:
-            b = sp.empty()
+        fused = None
+        if args.halo == "fused":
+            sym, fused = symmetric_fused_halo(sp)
+        for i, x in enumerate(host):
+            # the rotating state lives in symmetric (peer-mapped) memory for the fused path
+            is_state = i == 0 or spec.op == si.ACOUSTIC
+            b = sym[i] if (fused is not None and is_state) else sp.empty()
             sp.owned(b).copy_(x, non_blocking=True)
             bufs.append(b)
     else:
@@ -254,12 +266,14 @@ def main():
             state = [bufs[0], bufs[1]]          # prev, cur
             aux = []
         elif op == si.HOTSPOT3D:
-            state = [bufs[0], torch.empty_like(bufs[0])]
+            state = [bufs[0], sym[1] if (slabbed and fused is not None) else torch.empty_like(bufs[0])]
             aux = [bufs[1]]
         else:
-            state = [bufs[0], torch.empty_like(bufs[0])]
+            state = [bufs[0], sym[1] if (slabbed and fused is not None) else torch.empty_like(bufs[0])]
             aux = []
-        launches_per_step = steps_per_iter * (3 if slabbed else 1)
+        # slab + NCCL: boundary low, boundary high, interior per time step;
+        # slab + fused: one launch per time step
+        launches_per_step = steps_per_iter * (3 if (slabbed and args.halo == "nccl") else 1)
     else:
         out = plan.empty_output()
         launches_per_step = 1
@@ -269,7 +283,7 @@ def main():
     def step():
         if iterable:
             if slabbed:
-                return sp.iterate(state, steps_per_iter, aux)
+                return sp.iterate(state, steps_per_iter, aux, fused=fused)
             return plan.iterate(state, steps_per_iter, aux)
         plan.apply(*bufs, out=out)
         return 0
@@ -293,7 +307,7 @@ def main():
             return 0
 
     def barrier():
-        if world > 1:
+        if use_pg:
             dist.barrier()
         torch.cuda.synchronize()
 
@@ -314,7 +328,7 @@ def main():
         barrier()
     t_ms = ev0.elapsed_time(ev1)
     t_max = t_ms
-    if world > 1:
+    if use_pg:
         tt = torch.tensor([t_ms], device=dev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
         t_max = float(tt.item())
@@ -373,7 +387,7 @@ def main():
         def e2e_step():
             for b, x in zip(bufs, host):
                 sp.owned(b).copy_(x, non_blocking=True)
-            ri = sp.iterate(state, steps_per_iter, aux)
+            ri = sp.iterate(state, steps_per_iter, aux, fused=fused)
             res_h.copy_(sp.owned(state[ri]), non_blocking=True)
         e2e_step()
         barrier()
@@ -409,7 +423,9 @@ def main():
                        "global_extents": list(gext) if slabbed else list(ext1),
                        "time_steps_per_bench_step": steps_per_iter if iterable else 1,
                        "op": si.OP_NAMES[op], "boundary": [si.KIND_NAMES[k] for k in spec.kind],
-                       "window": list(spec.size), "parallelism": f"slab-z x{world}" if slabbed else
+                       "window": list(spec.size),
+                       "halo": (args.halo if slabbed else None),
+                       "parallelism": f"slab-z x{world}" if slabbed else
                        (f"replicas x{world}" if world > 1 else "single"),
                        "l2": "inputs larger than L2 (no flush needed)" if npts_local * 4 > 126e6
                        else "L2-resident working set (no flush; reported as such)",
@@ -427,7 +443,7 @@ def main():
             "clocks": clocks,
         }
         print(json.dumps(line), flush=True)
-    if world > 1:
+    if use_pg:
         dist.barrier()
         dist.destroy_process_group()
 

@@ -152,6 +152,45 @@ stencil_status stencil_apply_region(stencil_plan plan, const float* const* input
                                     int64_t o0_end, void* stream);
 
 /*
+ * Fused halo put (slab mode, 3D plans on the TMA sweep kernel): like
+ * stencil_apply_region, and every output plane z < ghost is ALSO stored to
+ * put_lo + z*plane, every plane z >= n0_local - ghost to
+ * put_hi + (z - (n0_local - ghost))*plane — the neighbour ranks' ghost planes
+ * through NVLink peer pointers (NULL = no neighbour on that side).  When all
+ * stores are done, the kernel's last CTA makes them visible system-wide and
+ * release-stores sig_value to *sig_lo / *sig_hi (the neighbours' flags for
+ * this rank; NULL = none).  The region must cover the planes to be put.
+ * Errors: E_UNSUPPORTED if the plan does not run on the sweep kernel (the
+ * caller then exchanges ghosts with stencil_apply_region + NCCL).
+ */
+stencil_status stencil_apply_region_put(stencil_plan plan, const float* const* inputs, int32_t n_inputs,
+                                        float* out, int64_t o0_begin, int64_t o0_end, float* put_lo,
+                                        float* put_hi, uint32_t* sig_lo, uint32_t* sig_hi,
+                                        uint32_t sig_value, void* stream);
+
+/*
+ * One time step of a slab as ONE launch with the halo exchange fused in:
+ * computes all owned output planes; the boundary z-chunks are scheduled first;
+ * before loading the ghost planes of the first / last chunk the kernel waits
+ * (acquire, system scope) until *wait_lo / *wait_hi >= wait_value (this rank's
+ * flags, raised by the neighbours' previous step; NULL = no wait); output planes
+ * z < ghost / z >= n0_local - ghost are also stored to put_lo / put_hi as in
+ * stencil_apply_region_put, and when the first / last chunk is complete the
+ * neighbours' flags *sig_lo / *sig_hi are release-stored with sig_value.
+ * Needs a slab plan on the TMA sweep kernel (E_UNSUPPORTED otherwise).
+ */
+stencil_status stencil_slab_step_fused(stencil_plan plan, const float* const* inputs, int32_t n_inputs,
+                                       float* out, float* put_lo, float* put_hi, uint32_t* sig_lo,
+                                       uint32_t* sig_hi, uint32_t sig_value, const uint32_t* wait_lo,
+                                       const uint32_t* wait_hi, uint32_t wait_value, void* stream);
+
+/* Stream-ordered wait: a one-thread kernel on ``stream`` spins (acquire,
+ * system scope) until *sig_a >= value and *sig_b >= value (wrap-around
+ * compare; NULL pointers are skipped).  Pairs with stencil_apply_region_put. */
+stencil_status stencil_wait_signals(const uint32_t* sig_a, const uint32_t* sig_b, uint32_t value,
+                                    void* stream);
+
+/*
  * iterate(in, f, n_steps) with the state rotation of reading A21:
  *   WEIGHTED  : state {X0, X1}            X_{t+1} = S(X_t), ping-pong
  *   HOTSPOT3D : state {T0, T1}, aux {P}   T_{t+1} = S(T_t, P)

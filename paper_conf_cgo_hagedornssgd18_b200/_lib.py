@@ -17,8 +17,8 @@ _PKG = os.path.dirname(os.path.abspath(__file__))
 LIB_PATH = os.path.join(_PKG, "libstencil.so")
 
 if not os.path.exists(LIB_PATH):
-    raise ImportError(f"{LIB_PATH} is missing: build it with "
-                      "`python -m paper_conf_cgo_hagedornssgd18_b200.build` (no CPU fallback exists)")
+    raise ImportError(f"{LIB_PATH} is missing: build it with `python __graft_entry__.py` or "
+                      "`python paper_conf_cgo_hagedornssgd18_b200/build.py` (no CPU fallback exists)")
 _lib = C.CDLL(LIB_PATH)
 
 # status / enums (include/stencil.h)
@@ -50,6 +50,11 @@ _set_variant = _sig("stencil_plan_set_variant", C.c_int, [_P, C.c_int32])
 _variant = _sig("stencil_plan_variant", C.c_int32, [_P])
 _apply = _sig("stencil_apply", C.c_int, [_P, _FPP, C.c_int32, _P, _P])
 _apply_region = _sig("stencil_apply_region", C.c_int, [_P, _FPP, C.c_int32, _P, C.c_int64, C.c_int64, _P])
+_apply_region_put = _sig("stencil_apply_region_put", C.c_int, [_P, _FPP, C.c_int32, _P, C.c_int64, C.c_int64, _P, _P,
+                                                              _P, _P, C.c_uint32, _P])
+_slab_step_fused = _sig("stencil_slab_step_fused", C.c_int, [_P, _FPP, C.c_int32, _P, _P, _P, _P, _P, C.c_uint32,
+                                                            _P, _P, C.c_uint32, _P])
+_wait_signals = _sig("stencil_wait_signals", C.c_int, [_P, _P, C.c_uint32, _P])
 _iterate = _sig("stencil_iterate", C.c_int, [_P, _FPP, C.c_int32, _FPP, C.c_int32, C.c_int32, _P, _I32P])
 _run_host = _sig("stencil_run_host", C.c_int, [_P, _FPP, C.c_int32, _FPP, C.c_int32, C.c_int32, _P, _P])
 _destroy = _sig("stencil_plan_destroy", None, [_P])
@@ -59,6 +64,7 @@ _version = _sig("stencil_version", C.c_char_p, [])
 
 EXPORTED = ("stencil_plan_create", "stencil_plan_output_extents", "stencil_plan_set_slab",
             "stencil_plan_set_variant", "stencil_plan_variant", "stencil_apply", "stencil_apply_region",
+            "stencil_apply_region_put", "stencil_slab_step_fused", "stencil_wait_signals",
             "stencil_iterate", "stencil_run_host", "stencil_plan_destroy", "stencil_status_string",
             "stencil_last_error", "stencil_version")
 
@@ -141,6 +147,30 @@ def stencil_apply_region(plan: int, inputs: Sequence[int], out: int, o0_begin: i
                          stream: int = 0):
     _check(_apply_region(plan, _ptrs(inputs), len(inputs), C.c_void_p(int(out)), int(o0_begin), int(o0_end),
                          C.c_void_p(int(stream))), "stencil_apply_region")
+
+
+def stencil_apply_region_put(plan: int, inputs: Sequence[int], out: int, o0_begin: int, o0_end: int,
+                             put_lo: int = 0, put_hi: int = 0, sig_lo: int = 0, sig_hi: int = 0, sig_value: int = 0,
+                             stream: int = 0):
+    v = lambda x: C.c_void_p(int(x)) if x else None
+    _check(_apply_region_put(plan, _ptrs(inputs), len(inputs), C.c_void_p(int(out)), int(o0_begin), int(o0_end),
+                             v(put_lo), v(put_hi), v(sig_lo), v(sig_hi), int(sig_value) & 0xffffffff,
+                             C.c_void_p(int(stream))), "stencil_apply_region_put")
+
+
+def stencil_slab_step_fused(plan: int, inputs: Sequence[int], out: int, put_lo: int = 0, put_hi: int = 0,
+                            sig_lo: int = 0, sig_hi: int = 0, sig_value: int = 0, wait_lo: int = 0, wait_hi: int = 0,
+                            wait_value: int = 0, stream: int = 0):
+    v = lambda x: C.c_void_p(int(x)) if x else None
+    _check(_slab_step_fused(plan, _ptrs(inputs), len(inputs), C.c_void_p(int(out)), v(put_lo), v(put_hi), v(sig_lo),
+                            v(sig_hi), int(sig_value) & 0xffffffff, v(wait_lo), v(wait_hi),
+                            int(wait_value) & 0xffffffff, C.c_void_p(int(stream))), "stencil_slab_step_fused")
+
+
+def stencil_wait_signals(sig_a: int, sig_b: int, value: int, stream: int = 0):
+    v = lambda x: C.c_void_p(int(x)) if x else None
+    _check(_wait_signals(v(sig_a), v(sig_b), int(value) & 0xffffffff, C.c_void_p(int(stream))),
+           "stencil_wait_signals")
 
 
 def stencil_iterate(plan: int, state: Sequence[int], aux: Sequence[int], n_steps: int, stream: int = 0) -> int:

@@ -1,6 +1,9 @@
 """Build libstencil.so in-tree with nvcc for sm_100a (no JIT, no torch extension).
 
-    python -m paper_conf_cgo_hagedornssgd18_b200.build [-v]
+    python paper_conf_cgo_hagedornssgd18_b200/build.py [-v] [-f]
+
+(run it as a script, or through __graft_entry__.build(): importing it via the
+package would load libstencil.so before it exists)
 
 Every .cu under csrc/ is compiled separately (in parallel) and linked into
 ``paper_conf_cgo_hagedornssgd18_b200/libstencil.so`` with a static CUDA

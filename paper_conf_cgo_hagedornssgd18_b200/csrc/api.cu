@@ -372,6 +372,63 @@ stencil_status stencil_apply_region(stencil_plan pl, const float* const* inputs,
   return launch(pl, p, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out, (cudaStream_t)stream);
 }
 
+stencil_status stencil_apply_region_put(stencil_plan pl, const float* const* inputs, int32_t n_inputs, float* out,
+                                        int64_t o0_begin, int64_t o0_end, float* put_lo, float* put_hi,
+                                        uint32_t* sig_lo, uint32_t* sig_hi, uint32_t sig_value, void* stream) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  stencil_status s = check_inputs(pl, inputs, n_inputs, out);
+  if (s != STENCIL_OK) return s;
+  if (!pl->p.slab) return fail(STENCIL_E_INVALID, "fused halo put needs a slab plan (stencil_plan_set_slab)");
+  if (o0_begin < 0 || o0_end > pl->p.o[0] || o0_begin >= o0_end)
+    return fail(STENCIL_E_INVALID, "region outside the output extents");
+  if (choose_variant(pl, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out) != STENCIL_VARIANT_SWEEP3D)
+    return fail(STENCIL_E_UNSUPPORTED, "fused halo put is built on the TMA sweep kernel only");
+  DeviceGuard g(pl->device);
+  if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+  StencilParams p = pl->p;
+  p.reg0 = o0_begin;
+  p.reg1 = o0_end;
+  p.put_lo = put_lo;
+  p.put_hi = put_hi;
+  p.sig_lo = sig_lo;
+  p.sig_hi = sig_hi;
+  p.sig_value = sig_value;
+  return launch(pl, p, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out, (cudaStream_t)stream);
+}
+
+stencil_status stencil_slab_step_fused(stencil_plan pl, const float* const* inputs, int32_t n_inputs, float* out,
+                                       float* put_lo, float* put_hi, uint32_t* sig_lo, uint32_t* sig_hi,
+                                       uint32_t sig_value, const uint32_t* wait_lo, const uint32_t* wait_hi,
+                                       uint32_t wait_value, void* stream) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  stencil_status s = check_inputs(pl, inputs, n_inputs, out);
+  if (s != STENCIL_OK) return s;
+  if (!pl->p.slab) return fail(STENCIL_E_INVALID, "fused step needs a slab plan (stencil_plan_set_slab)");
+  if (choose_variant(pl, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out) != STENCIL_VARIANT_SWEEP3D)
+    return fail(STENCIL_E_UNSUPPORTED, "fused step is built on the TMA sweep kernel only");
+  DeviceGuard g(pl->device);
+  if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+  StencilParams p = pl->p;
+  p.reg0 = 0;
+  p.reg1 = p.o[0];
+  p.put_lo = put_lo;
+  p.put_hi = put_hi;
+  p.sig_lo = sig_lo;
+  p.sig_hi = sig_hi;
+  p.sig_value = sig_value;
+  p.wait_lo = wait_lo;
+  p.wait_hi = wait_hi;
+  p.wait_value = wait_value;
+  p.fused_step = 1;
+  return launch(pl, p, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out, (cudaStream_t)stream);
+}
+
+stencil_status stencil_wait_signals(const uint32_t* sig_a, const uint32_t* sig_b, uint32_t value, void* stream) {
+  cudaError_t e = launch_wait_signals(sig_a, sig_b, value, (cudaStream_t)stream);
+  if (e != cudaSuccess) return cuda_fail(e, "wait kernel launch");
+  return STENCIL_OK;
+}
+
 stencil_status stencil_apply(stencil_plan pl, const float* const* inputs, int32_t n_inputs, float* out,
                              void* stream) {
   if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");

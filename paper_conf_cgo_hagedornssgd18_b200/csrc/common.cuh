@@ -46,6 +46,23 @@ struct StencilParams {
   int32_t sep;
   float su[kMaxSep], sv[kMaxSep];
   float prm[kMaxParams];
+  // fused halo put (slab mode, per launch): output plane z < ghost is also
+  // stored at put_lo + z*plane, plane z >= n0 - ghost at put_hi + (z - (n0 -
+  // ghost))*plane (the neighbours' ghost planes, NVLink peer pointers); the
+  // last CTA then release-stores sig_value to sig_lo / sig_hi (system scope)
+  float* put_lo;
+  float* put_hi;
+  unsigned int* sig_lo;
+  unsigned int* sig_hi;
+  unsigned int sig_value;
+  // single-launch fused step: before loading ghost planes (first / last
+  // z-chunk) the producer waits until *wait_lo / *wait_hi >= wait_value
+  // (acquire, system scope); the boundary chunks are scheduled first and the
+  // neighbours' flags are raised as soon as their chunk is complete
+  const unsigned int* wait_lo;
+  const unsigned int* wait_hi;
+  unsigned int wait_value;
+  int32_t fused_step;
 };
 
 // h(i, n) of the reindexing pad (A1-A5).

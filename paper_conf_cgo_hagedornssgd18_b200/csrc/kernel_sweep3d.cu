@@ -59,6 +59,17 @@ constexpr int kTickets = 4096;
 // dynamic work counters (one per in-flight launch slot; reset by the last CTA)
 __device__ unsigned int g_ticket[kTickets];
 __device__ unsigned int g_done[kTickets];
+__device__ unsigned int g_bdone[kTickets][2];   // finished boundary-chunk items (fused step)
+
+// fused step: boundary chunks first (item order: chunk 0, chunk last, then the rest)
+__device__ __forceinline__ int chunk_of(int c, int nchunk, bool fused) {
+  if (!fused || nchunk <= 2) return c;
+  return c == 0 ? 0 : (c == 1 ? nchunk - 1 : c - 1);
+}
+
+__device__ __forceinline__ void spin_until(const unsigned int* f, unsigned int v) {
+  while ((int)(ld_acquire_sys(f) - v) < 0) __nanosleep(32);
+}
 
 enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2 };
 
@@ -193,12 +204,18 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
         int nload = 1, x0 = 0, y0 = 0;
         int64_t zs = 0;
         if (!done) {
-          const int chunk = item / ntile, tile = item % ntile;
+          const int chunk = chunk_of(item / ntile, nchunk, p.fused_step), tile = item % ntile;
           x0 = (tile % ntx) * TX;
           y0 = (tile / ntx) * TY;
           zs = p.reg0 + (int64_t)chunk * zc;
           const int64_t ze = min(zs + (int64_t)zc, p.reg1);
           nload = (int)(ze - zs) + 2 * R;
+          // fused step: the ghost planes of this chunk must hold the neighbours'
+          // previous step before the TMA reads them
+          bool waited = false;
+          if (chunk == 0 && p.wait_lo) { spin_until(p.wait_lo, p.wait_value); waited = true; }
+          if (chunk == nchunk - 1 && p.wait_hi) { spin_until(p.wait_hi, p.wait_value); waited = true; }
+          if (waited) asm volatile("fence.proxy.async.global;" ::: "memory");
         }
         // a "done" marker occupies one stage so the consumers see it in order
         for (int i = 0; i < nload; ++i) {
@@ -226,7 +243,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
         mbar_arrive(&itemempty[q]);
         if (++q == QN) { q = 0; ++qpass; }
         if (item < 0) break;
-        const int chunk = item / ntile, tile = item % ntile;
+        const int chunk = chunk_of(item / ntile, nchunk, p.fused_step), tile = item % ntile;
         const int x0 = (tile % ntx) * TX, y0 = (tile / ntx) * TY;
         const int64_t zs = p.reg0 + (int64_t)chunk * zc;
         const int nzc = (int)(min(zs + (int64_t)zc, p.reg1) - zs);
@@ -272,7 +289,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
         if (lane == 0) mbar_arrive(&empty[sn]);
         break;
       }
-      const int chunk = item / ntile, tile = item % ntile;
+      const int chunk = chunk_of(item / ntile, nchunk, p.fused_step), tile = item % ntile;
       const int x0 = (tile % ntx) * TX;
       const int y0 = (tile / ntx) * TY;
       const int64_t zs = p.reg0 + (int64_t)chunk * zc;
@@ -328,7 +345,8 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
         mbar_wait(&full[sn], pn & 1);
         zst[2 * R] = (ZC && stage_const[sn]) ? -1 - sn : sn;
         if (++sn == S) { sn = 0; ++pn; }
-        const int gz = (int)(p.z_off + zs + j);
+        const int64_t z = zs + j;                  // local output plane
+        const int gz = (int)(p.z_off + z);
         const int cbase = zst[R] * SF4;             // the centre plane is inside the grid
         if (fix) {
           // all warps are past the previous plane (which read this stage as its
@@ -428,7 +446,13 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
             res.z = eval<OP, R, 2>(p, w, pw, gz, gy, xo);
             res.w = eval<OP, R, 3>(p, w, pw, gz, gy, xo);
           }
-          if (ok) stg128(orow + jj * nx, res);
+          if (ok) {
+            stg128(orow + jj * nx, res);
+            // fused halo put: boundary planes also go to the neighbour's ghosts
+            if (z < p.ghost && p.put_lo) stg128(p.put_lo + z * p.plane + (int64_t)gy * nx + xo, res);
+            if (z >= p.n[0] - p.ghost && p.put_hi)
+              stg128(p.put_hi + (z - (p.n[0] - p.ghost)) * p.plane + (int64_t)gy * nx + xo, res);
+          }
         }
         orow += p.plane;
         // plane z - R is no longer needed (pre-chunk planes included)
@@ -449,10 +473,32 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
       if (lane == 0) {
 #pragma unroll
         for (int k = 0; k < 2 * R; ++k) mbar_arrive(&empty[zst[k] < 0 ? -1 - zst[k] : zst[k]]);
+        // fused step: when every warp of every tile of a boundary chunk is done,
+        // publish its peer stores and raise that neighbour's flag
+        if (p.fused_step) {
+          const unsigned need = (unsigned)ntile * NW;
+          if (chunk == 0 && p.sig_lo) {
+            __threadfence_system();
+            if (atomicAdd(&g_bdone[slot][0], 1u) == need - 1) {
+              __threadfence_system();
+              st_release_sys(p.sig_lo, p.sig_value);
+            }
+          }
+          if (chunk == nchunk - 1 && p.sig_hi) {
+            __threadfence_system();
+            if (atomicAdd(&g_bdone[slot][1], 1u) == need - 1) {
+              __threadfence_system();
+              st_release_sys(p.sig_hi, p.sig_value);
+            }
+          }
+        }
       }
     }
   }
-  // last CTA out resets the launch slot's counters (graph-replay safe)
+  // last CTA out resets the launch slot's counters (graph-replay safe) and,
+  // for a fused halo put, publishes the ghost planes to the neighbours
+  const bool puts = p.put_lo || p.put_hi;
+  if (puts) __threadfence_system();     // this thread's peer stores before the CTA's arrival
   __syncthreads();
   if (threadIdx.x == 0) {
     __threadfence();
@@ -460,6 +506,13 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
     if (prev == gridDim.x - 1) {
       g_ticket[slot] = 0;
       g_done[slot] = 0;
+      g_bdone[slot][0] = 0;
+      g_bdone[slot][1] = 0;
+      if (puts && !p.fused_step) {
+        __threadfence_system();
+        if (p.sig_lo) st_release_sys(p.sig_lo, p.sig_value);
+        if (p.sig_hi) st_release_sys(p.sig_hi, p.sig_value);
+      }
       __threadfence();
     }
   }
@@ -596,6 +649,7 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   int64_t zc = (work + 8 * slots - 1) / (8 * slots);
   const int64_t zmin = std::min<int64_t>(16, std::max<int64_t>(2, (work + 2 * slots - 1) / (2 * slots)));
   if (zc < zmin) zc = zmin;
+  if (p.fused_step && zc < p.ghost) zc = p.ghost;     // boundary planes stay in the first / last chunk
   if (zc > nz_reg) zc = nz_reg;
   const int64_t nchunk = (nz_reg + zc - 1) / zc;
   const int64_t items = tiles * nchunk;

@@ -29,4 +29,8 @@ bool tile2d_supported(const StencilParams& p);
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,
                           cudaStream_t stream, int num_sms, std::string* err);
 
+// wait (one thread, acquire.sys) until *a >= value and *b >= value (NULL = skip)
+cudaError_t launch_wait_signals(const unsigned int* a, const unsigned int* b, unsigned int value,
+                                cudaStream_t stream);
+
 }  // namespace lift

@@ -131,6 +131,12 @@ class SlabPlan:
         self.exchange = exchange if exchange is not None else factory(rank, world, self.n, self.g, self.wrap, group)
         self.comm = torch.cuda.Stream(device=self.plan.device)
         self.alloc_shape = self.plan.alloc_extents
+        self.epoch = 0          # fused-halo step counter (flag values only grow)
+
+    def _iterate_fused(self, state, n_steps, aux, fused, ri, acoustic):
+        # the initial ghosts came through ``exchange``; the flags already hold
+        # self.epoch on every rank (all ranks run the same number of steps)
+        return _iterate_fused_impl(self, state, n_steps, aux, fused, ri, acoustic)
 
     def empty(self) -> torch.Tensor:
         return torch.empty(self.alloc_shape, dtype=torch.float32, device=f"cuda:{self.plan.device}")
@@ -156,13 +162,18 @@ class SlabPlan:
             w.wait()                       # on the comm stream
         torch.cuda.current_stream().wait_stream(self.comm)
 
-    def iterate(self, state: Sequence[torch.Tensor], n_steps: int, aux: Sequence[torch.Tensor] = ()) -> int:
+    def iterate(self, state: Sequence[torch.Tensor], n_steps: int, aux: Sequence[torch.Tensor] = (),
+                fused: Optional[FusedHalo] = None) -> int:
         """n time steps with the rotation of stencil_iterate (DESIGN.md A21);
-        returns the index of the state buffer holding the newest grid."""
+        returns the index of the state buffer holding the newest grid.  With
+        ``fused`` the ghosts travel by peer stores from the boundary kernel
+        (stencil_apply_region_put) instead of NCCL."""
         op = self.plan.op
         acoustic = op == 4
         ri = 1 if acoustic else 0
         self._join(self._on_comm(lambda: self.exchange.post(state[ri])))
+        if fused is not None:
+            return self._iterate_fused(state, n_steps, aux, fused, ri, acoustic)
         for _ in range(n_steps):
             if acoustic:
                 dst = 1 - ri
@@ -176,6 +187,87 @@ class SlabPlan:
             self._join(works)
             ri = dst
         return ri
+
+
+def _iterate_fused_impl(slab, state, n_steps, aux, fused, ri, acoustic):
+    stream = torch.cuda.current_stream()
+    for _ in range(n_steps):
+        dst = 1 - ri
+        ins = (state[dst], state[ri]) if acoustic else (state[ri],) + tuple(aux)
+        slab.epoch += 1
+        fused_step(slab, fused, ins, state[dst], dst, slab.epoch, stream)
+        ri = dst
+    return ri
+
+
+class FusedHalo:
+    """Peer view for the fused halo put: the boundary-plane kernel
+    stores its planes into the neighbours' ghost planes through NVLink peer
+    pointers and raises their flags; no NCCL call on the data path.
+
+    ``peer_state[k][r]`` is rank r's state buffer k (a tensor this rank can
+    address: a symmetric-memory peer view on real GPUs, the tensor itself in
+    virtual mode); ``peer_flags[r]`` is rank r's int32[2] flag array
+    ([written by the lower neighbour, written by the upper neighbour]).
+    ``parts`` is the z partition."""
+
+    def __init__(self, rank: int, world: int, parts, wrap: bool, peer_state, peer_flags):
+        self.rank, self.world, self.parts = rank, world, parts
+        self.lo, self.hi = neighbours(rank, world, wrap)
+        self.peer_state, self.peer_flags = peer_state, peer_flags
+
+    def targets(self, k: int, g: int):
+        """(put_lo, put_hi, sig_lo, sig_hi) device addresses for writing state k."""
+        put_lo = put_hi = sig_lo = sig_hi = 0
+        if self.lo is not None:
+            t = self.peer_state[k][self.lo]
+            n_lo = self.parts[self.lo][1] - self.parts[self.lo][0]
+            put_lo = t.data_ptr() + (g + n_lo) * t.stride(0) * 4      # its upper ghost planes
+            sig_lo = self.peer_flags[self.lo].data_ptr() + 4          # its "from upper" flag
+        if self.hi is not None:
+            put_hi = self.peer_state[k][self.hi].data_ptr()           # its lower ghost planes
+            sig_hi = self.peer_flags[self.hi].data_ptr()               # its "from lower" flag
+        return put_lo, put_hi, sig_lo, sig_hi
+
+    def my_flags(self):
+        f = self.peer_flags[self.rank].data_ptr()
+        return (f if self.lo is not None else 0), (f + 4 if self.hi is not None else 0)
+
+
+def fused_step(slab: "SlabPlan", fh: FusedHalo, ins, out: torch.Tensor, out_k: int, value: int, stream) -> None:
+    """One time step as ONE kernel launch on ``stream`` (stencil_slab_step_fused):
+    the boundary z-chunks run first; before loading ghost planes the kernel
+    waits until this rank's flags hold ``value - 1`` (the neighbours' previous
+    step); the boundary planes are also stored into the neighbours' ghost
+    planes, and each neighbour's flag is raised to ``value`` as soon as the
+    chunk it needs is complete."""
+    from . import _lib as L
+    g = slab.g
+    fa, fb = fh.my_flags()
+    put_lo, put_hi, sig_lo, sig_hi = fh.targets(out_k, g)
+    L.stencil_slab_step_fused(slab.plan.handle, [x.data_ptr() for x in ins], out.data_ptr(), put_lo, put_hi, sig_lo,
+                              sig_hi, value, fa, fb, value - 1, int(stream.cuda_stream))
+
+
+def symmetric_fused_halo(slab: "SlabPlan", group=None):
+    """Real multi-GPU setup: two state buffers and the flag array in torch
+    symmetric memory (NVLink peer-mapped), rendezvoused over ``group``.
+    Returns (state buffers, FusedHalo)."""
+    import torch.distributed._symmetric_memory as symm_mem
+    grp = group if group is not None else dist.group.WORLD
+    dev = torch.device(f"cuda:{slab.plan.device}")
+    bufs = [symm_mem.empty(*slab.alloc_shape, dtype=torch.float32, device=dev) for _ in range(2)]
+    hdls = [symm_mem.rendezvous(b, grp) for b in bufs]
+    flags = symm_mem.empty(2, dtype=torch.int32, device=dev)
+    flags.zero_()
+    hf = symm_mem.rendezvous(flags, grp)
+    torch.cuda.synchronize(dev)
+    dist.barrier(group=grp)
+    parts = partition(slab.global_extents[0], slab.world)
+    peer_state = [[hdls[k].get_buffer(r, slab.alloc_shape, torch.float32) for r in range(slab.world)]
+                  for k in range(2)]
+    peer_flags = [hf.get_buffer(r, (2,), torch.int32) for r in range(slab.world)]
+    return bufs, FusedHalo(slab.rank, slab.world, parts, slab.wrap, peer_state, peer_flags)
 
 
 class LocalExchange:
@@ -229,3 +321,38 @@ def virtual_slab_iterate(global_extents, world: int, state_global: Sequence[torc
 class _NoExchange:
     def post(self, buf):
         return []
+
+
+def virtual_slab_iterate_fused(global_extents, world: int, state_global: Sequence[torch.Tensor], n_steps: int,
+                               aux_global: Sequence[torch.Tensor] = (), **plan_kw) -> List[torch.Tensor]:
+    """Fused-halo protocol with G slabs in one process: each slab runs on its
+    own CUDA stream, the boundary kernels store into the neighbour slabs'
+    ghost planes and raise their flags, and the streams synchronise only
+    through those flags (stencil_wait_signals) — the multi-GPU protocol with
+    device-local "peer" pointers."""
+    slabs = [SlabPlan(global_extents, r, world, exchange=_NoExchange(), **plan_kw) for r in range(world)]
+    ex = LocalExchange(slabs)
+    nst = len(state_global)
+    bufs = [[s.scatter(state_global[k]) if k < nst else s.empty() for k in range(2)] for s in slabs]
+    auxs = [[s.scatter(a) for a in aux_global] for s in slabs]
+    acoustic = slabs[0].plan.op == 4
+    ri = 1 if acoustic else 0
+    ex.fill([b[ri] for b in bufs])
+    dev = bufs[0][0].device
+    flags = [torch.zeros(2, dtype=torch.int32, device=dev) for _ in range(world)]
+    parts = partition(global_extents[0], world)
+    peer_state = [[bufs[r][k] for r in range(world)] for k in range(2)]
+    fhs = [FusedHalo(r, world, parts, slabs[r].wrap, peer_state, flags) for r in range(world)]
+    streams = [torch.cuda.Stream(device=dev) for _ in range(world)]
+    torch.cuda.synchronize(dev)
+    # issue step by step across slabs so no stream waits on work not yet enqueued
+    for _ in range(n_steps):
+        dst = 1 - ri
+        for r, (s, b, a) in enumerate(zip(slabs, bufs, auxs)):
+            ins = (b[dst], b[ri]) if acoustic else (b[ri],) + tuple(a)
+            s.epoch += 1
+            fused_step(s, fhs[r], ins, b[dst], dst, s.epoch, streams[r])
+        ri = dst
+    torch.cuda.synchronize(dev)
+    order = [1 - ri, ri] if acoustic else [ri]
+    return [torch.cat([s.owned(b[k]) for s, b in zip(slabs, bufs)], 0) for k in order]

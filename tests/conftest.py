@@ -31,7 +31,7 @@ def pytest_sessionstart(session):
     # libstencil.so is built in-tree (incremental; a no-op when up to date) so the
     # binding can be imported on CPU-only hosts for host-logic tests
     try:
-        from paper_conf_cgo_hagedornssgd18_b200 import build as _b
-        _b.build()
+        import __graft_entry__
+        __graft_entry__._build_module().build()
     except Exception as e:  # pragma: no cover
         print(f"libstencil build failed: {e}")

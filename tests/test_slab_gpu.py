@@ -99,3 +99,44 @@ def test_slabplan_world1_split_bitwise(lift, kind):
     ri = slab.iterate([a, b], 7)
     torch.cuda.synchronize()
     np.testing.assert_array_equal(slab.owned((a, b)[ri]).cpu().numpy(), ref)
+
+
+@pytest.mark.parametrize("kind,world", [(si.CLAMP, 2), (si.CLAMP, 3), (si.WRAP, 2), (si.WRAP, 3), (si.WRAP, 1),
+                                        (si.MIRROR, 4)])
+def test_fused_halo_virtual_bitwise(lift, kind, world):
+    """Fused halo put: boundary kernels store into the neighbour slabs' ghosts
+    and raise their flags; each slab on its own stream, synchronised only by
+    the flags — bitwise equal to the single plan."""
+    from paper_conf_cgo_hagedornssgd18_b200.slab import virtual_slab_iterate_fused
+    ext = (32, 40, 136)
+    sp = si.StencilSpec(ext, (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (kind,) * 3, 0.0, si.WEIGHTED,
+                        si.weights_j3d7(), ())
+    x = si.uniform(ext, 83, 0.5, 1.5)
+    ref = single_iterate(lift, sp, [x], [], 9)[0]
+    got = virtual_slab_iterate_fused(ext, world, [torch.from_numpy(x).cuda()], 9, **kw(sp))[0]
+    np.testing.assert_array_equal(got.cpu().numpy(), ref)
+
+
+def test_fused_halo_virtual_acoustic13(lift):
+    from paper_conf_cgo_hagedornssgd18_b200.slab import virtual_slab_iterate_fused
+    ext = (30, 36, 132)
+    sp = si.StencilSpec(ext, (5,) * 3, (1,) * 3, (2,) * 3, (2,) * 3, (si.CONSTANT,) * 3, 0.0, si.ACOUSTIC, None,
+                        si.params_acoustic(13))
+    u0 = si.uniform(ext, 84, -1, 1)
+    u1 = si.uniform(ext, 85, -1, 1)
+    ref = single_iterate(lift, sp, [u0, u1], [], 6)
+    got = virtual_slab_iterate_fused(ext, 3, [torch.from_numpy(u0).cuda(), torch.from_numpy(u1).cuda()], 6,
+                                     **kw(sp))
+    np.testing.assert_array_equal(got[1].cpu().numpy(), ref[1])
+    np.testing.assert_array_equal(got[0].cpu().numpy(), ref[0])
+
+
+def test_apply_region_put_needs_slab(lift):
+    sp = si.StencilSpec((16, 40, 136), (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.CLAMP,) * 3, 0.0, si.WEIGHTED,
+                        si.weights_j3d7(), ())
+    plan = lift.Plan.from_spec(sp)
+    x = torch.zeros(sp.extents, device="cuda")
+    y = torch.empty_like(x)
+    with pytest.raises(lift.StencilError) as e:
+        lift.stencil_apply_region_put(plan.handle, [x.data_ptr()], y.data_ptr(), 0, 1)
+    assert e.value.status == 1
