@@ -40,7 +40,7 @@ sys.path.insert(0, ROOT)
 METRIC = "stencil Gpoints/s & achieved HBM GB/s vs 8 TB/s at 1/2/4/8 B200"
 
 # algorithmic (compulsory) HBM bytes per output point per launch
-BYTES_PER_POINT = {0: 8, 1: 12, 2: 8, 3: 12, 4: 12}
+BYTES_PER_POINT = {0: 8, 1: 12, 2: 8, 3: 12, 4: 12, 5: 12, 6: 8}
 KERNEL_NAME = {"j3d7_512_clamp": "k2_sweep", "acoustic7_1024": "k2_sweep", "acoustic13_1024": "k2_sweep",
                "hotspot3d_8x512x512": "k2_sweep", "gauss5_8192_mirror": "k1_tile", "j2d5_256_clamp": "k1_tile",
                "srad1_4096": "k1_tile", "srad2_4096": "k1_tile"}
@@ -434,7 +434,8 @@ def main():
             "hbm_gbs_per_gpu_whole_step": value * bpp / world,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": ncu_traffic(args.workload),
-                         "kernel": KERNEL_NAME.get(args.workload), "peak_source": peak_src,
+                         "kernel": {0: "k0_generic", 1: "k1_tile", 2: "k2_sweep"}[plan.variant],
+                         "peak_source": peak_src,
                          "alg_bytes_per_launch": alg_bytes, "avg_launch_us": avg_launch_s * 1e6,
                          "frac_of_8TBs": achieved / 8000.0},
             "cpu_baseline": cpu,

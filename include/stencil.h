@@ -67,10 +67,16 @@ typedef enum {
                                 params {q0sqr}; 2D, size 3                         */
   STENCIL_OP_SRAD2 = 3,      /* Rodinia SRAD kernel 2 (A18): inputs {c, I} -> I';
                                 params {lambda}; 2D, size 3                        */
-  STENCIL_OP_ACOUSTIC = 4    /* Listing 3 (A19/A20): inputs {prev
+  STENCIL_OP_ACOUSTIC = 4,   /* Listing 3 (A19/A20): inputs {prev
                                 (point-wise), cur (slid)} -> next; params
                                 {lambda^2, loss1, loss2}; 3D, size 3 (7-pt) or
                                 5 (13-pt); ``out`` may alias ``prev``              */
+  STENCIL_OP_HOTSPOT2D = 5,  /* Rodinia hotspot (A26, Table 1): inputs {T
+                                (slid), P (point-wise)}; params {step/Cap, 1/Rx,
+                                1/Ry, 1/Rz, amb}; 2D, size 3                       */
+  STENCIL_OP_GRADIENT = 6    /* Rawat et al. 2D gradient (A25, Table 1):
+                                I + 1/sqrt(eps + sum of squared differences to
+                                the 4 neighbours); params {eps}; 2D, size 3        */
 } stencil_op;
 
 /* Which kernel family executes a plan (stencil_plan_variant). */
@@ -193,7 +199,8 @@ stencil_status stencil_wait_signals(const uint32_t* sig_a, const uint32_t* sig_b
 /*
  * iterate(in, f, n_steps) with the state rotation of reading A21:
  *   WEIGHTED  : state {X0, X1}            X_{t+1} = S(X_t), ping-pong
- *   HOTSPOT3D : state {T0, T1}, aux {P}   T_{t+1} = S(T_t, P)
+ *   HOTSPOT3D, HOTSPOT2D : state {T0, T1}, aux {P}   T_{t+1} = S(T_t, P)
+ *   GRADIENT  : state {X0, X1}            ping-pong like WEIGHTED
  *   ACOUSTIC  : state {prev, cur}         next overwrites prev; roles swap
  * *result_index receives the index into ``state`` holding the newest grid.
  * Requires output extents == input extents.

@@ -30,8 +30,9 @@ linear field under the Laplacian, Gaussian separability, wrap translation
 equivariance, mirror symmetry, linearity).
 
 PARITY UNPINNED (the paper prints no formula or values, the definitions are
-external readings, A16/A18/A19): the Hotspot3D point function, the
-SRAD1/SRAD2 point functions and the Acoustic constants.  For these only
+external readings, A16/A18/A19/A25/A26): the Hotspot3D and
+Hotspot2D point functions, the SRAD1/SRAD2 point functions, the Gradient point
+function and the Acoustic constants.  For these only
 structural properties are pinned (fixed points, ranges, brute-force K count).
 """
 from __future__ import annotations
@@ -41,7 +42,7 @@ from typing import Callable, List, Sequence, Tuple
 import numpy as np
 
 CLAMP, MIRROR, WRAP, CONSTANT, REFLECT = 0, 1, 2, 3, 4
-WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC = 0, 1, 2, 3, 4
+WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC, HOTSPOT2D, GRADIENT = 0, 1, 2, 3, 4, 5, 6
 
 
 # ---------------------------------------------------------------------------
@@ -233,6 +234,33 @@ def f_srad2(Wc: Callable, WI: Callable, prm: Sequence[float]) -> Tuple:
     return Y, A
 
 
+def f_hotspot2d(WT: Callable, WP: Callable, prm: Sequence[float]) -> Tuple:
+    """Rodinia v3.1 hotspot (2D) update (reading A26; PARITY UNPINNED formula):
+    T' = T + sdc*(P + (S + N - 2T)/Ry + (E + W - 2T)/Rx + (amb - T)/Rz),
+    with params (sdc, 1/Rx, 1/Ry, 1/Rz, amb); N=y-1, S=y+1, W=x-1, E=x+1."""
+    sdc, rx1, ry1, rz1, amb = (np.float64(v) for v in prm)
+    T = WT((1, 1))
+    terms = (WP((1, 1)), (WT((2, 1)) + WT((0, 1)) - 2.0 * T) * ry1,
+             (WT((1, 2)) + WT((1, 0)) - 2.0 * T) * rx1, (amb - T) * rz1)
+    acc = terms[0] + terms[1] + terms[2] + terms[3]
+    Y = T + sdc * acc
+    aT = np.abs(T)
+    A = aT + np.abs(sdc) * (np.abs(terms[0]) + (np.abs(WT((2, 1))) + np.abs(WT((0, 1))) + 2.0 * aT) * abs(ry1) +
+                            (np.abs(WT((1, 2))) + np.abs(WT((1, 0))) + 2.0 * aT) * abs(rx1) +
+                            (abs(amb) + aT) * abs(rz1))
+    return Y, A
+
+
+def f_gradient(W: Callable, prm: Sequence[float]) -> Tuple:
+    """Rawat et al. [36] 2D gradient (reading A25; PARITY UNPINNED formula):
+    out = I + 1/sqrt(eps + (I-N)^2 + (I-S)^2 + (I-W)^2 + (I-E)^2)."""
+    eps = np.float64(prm[0])
+    Ic = W((1, 1))
+    s = eps + (Ic - W((0, 1))) ** 2 + (Ic - W((2, 1))) ** 2 + (Ic - W((1, 0))) ** 2 + (Ic - W((1, 2))) ** 2
+    Y = Ic + 1.0 / np.sqrt(s)
+    return Y, np.abs(Ic) + np.abs(1.0 / np.sqrt(s))
+
+
 def acoustic_neighbours(o: Sequence, extents: Sequence[int], r: int):
     """computeNumNeighbors (Listing 3 line 14; reading A19):
     K = number of the star neighbour offsets (+-1..+-r on each axis) whose
@@ -281,7 +309,7 @@ def f_acoustic(W: Callable, prev_c, K, r: int, prm: Sequence[float]) -> Tuple:
 def _check_op_shape(spec):
     if spec.op in (HOTSPOT3D, ACOUSTIC):
         assert spec.ndim == 3
-    if spec.op in (SRAD1, SRAD2):
+    if spec.op in (SRAD1, SRAD2, HOTSPOT2D, GRADIENT):
         assert spec.ndim == 2
     if spec.op != WEIGHTED:
         assert all(s == 1 for s in spec.step)
@@ -305,6 +333,10 @@ def apply(spec, inputs: Sequence[np.ndarray]):
         Y, A = f_srad1(tapper(pad(inputs[0])), spec.params)
     elif spec.op == SRAD2:
         Y, A = f_srad2(tapper(pad(inputs[0])), tapper(pad(inputs[1])), spec.params)
+    elif spec.op == HOTSPOT2D:
+        Y, A = f_hotspot2d(tapper(pad(inputs[0])), tapper(pad(inputs[1])), spec.params)
+    elif spec.op == GRADIENT:
+        Y, A = f_gradient(tapper(pad(inputs[0])), spec.params)
     elif spec.op == ACOUSTIC:
         r = spec.size[0] // 2
         o = np.meshgrid(*[np.arange(n) for n in outs], indexing="ij", sparse=True)
@@ -346,6 +378,10 @@ def apply_point(spec, inputs: Sequence[np.ndarray], o: Sequence[int]):
         return f_srad1(tap(inputs[0]), spec.params)
     if spec.op == SRAD2:
         return f_srad2(tap(inputs[0]), tap(inputs[1]), spec.params)
+    if spec.op == HOTSPOT2D:
+        return f_hotspot2d(tap(inputs[0]), tap(inputs[1]), spec.params)
+    if spec.op == GRADIENT:
+        return f_gradient(tap(inputs[0]), spec.params)
     if spec.op == ACOUSTIC:
         r = spec.size[0] // 2
         K = acoustic_neighbours(o, spec.extents, r)
@@ -362,7 +398,7 @@ def iterate(spec, state: Sequence[np.ndarray], aux: Sequence[np.ndarray], n_step
     before feeding it back (not used by the parity tests: the oracle keeps
     fp64 state)."""
     cvt = (lambda a: a.astype(np.float32).astype(np.float64)) if round_fp32 else (lambda a: a)
-    if spec.op in (WEIGHTED, HOTSPOT3D):
+    if spec.op in (WEIGHTED, HOTSPOT3D, HOTSPOT2D, GRADIENT):
         X = np.asarray(state[0], np.float64)
         for _ in range(n_steps):
             X, _A = apply(spec, [X] + list(aux))

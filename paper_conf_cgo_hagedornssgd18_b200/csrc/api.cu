@@ -64,6 +64,8 @@ int op_arity(int op) {
     case OP_SRAD1: return 1;
     case OP_SRAD2: return 2;
     case OP_ACOUSTIC: return 2;
+    case OP_HOTSPOT2D: return 2;
+    case OP_GRADIENT: return 1;
     default: return -1;
   }
 }
@@ -76,6 +78,8 @@ int slid_mask(int op) {
     case OP_SRAD1: return 1;
     case OP_SRAD2: return 3;          // c and I both slid
     case OP_ACOUSTIC: return 2;       // prev point-wise, cur slid
+    case OP_HOTSPOT2D: return 1;      // T slid, P point-wise
+    case OP_GRADIENT: return 1;
     default: return 0;
   }
 }
@@ -170,7 +174,7 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
   if (ndim < 1) return fail(STENCIL_E_INVALID, "ndim must be 1, 2 or 3");
   if (!extents || !size || !step || !pad_lo || !pad_hi || !kind)
     return fail(STENCIL_E_INVALID, "NULL array argument");
-  if (op < 0 || op > OP_ACOUSTIC) return fail(STENCIL_E_INVALID, "unknown op");
+  if (op < 0 || op > OP_GRADIENT) return fail(STENCIL_E_INVALID, "unknown op");
   if (n_params < 0 || n_params > kMaxParams || (n_params > 0 && !params))
     return fail(STENCIL_E_INVALID, "bad params");
 
@@ -232,6 +236,15 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
         ++nt;
       }
       p.ntaps = nt;
+      {
+        // linear tap offsets for K0's interior fast path (needs 32-bit offsets)
+        const int64_t span = (int64_t)(p.size[0] - 1) * p.plane + (int64_t)(p.size[1] - 1) * p.row + p.size[2];
+        if (span < ((int64_t)1 << 31))
+          for (int t = 0; t < nt; ++t)
+            p.tap_off[t] = (int32_t)(p.tap[t][0] * p.plane + p.tap[t][1] * p.row + p.tap[t][2]);
+        else if (nt > 0)
+          p.tap_off[0] = -1;
+      }
       if (ntot <= kMaxTaps)
         for (int64_t k = 0; k < ntot; ++k) p.wbox[k] = weights[k];
       // separable (rank-1) 2D weights: w[i][j] == su[i] * sv[j] exactly (checked
@@ -282,6 +295,16 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
         p.prm[1] = (float)(q0 / (1.0 + q0));
         p.prm[2] = (float)(1.0 / (q0 * (1.0 + q0)));
       }
+      p.radius = 1;
+      break;
+    case OP_HOTSPOT2D:
+      if (ndim != 2 || !centred(1)) return fail(STENCIL_E_INVALID, "HOTSPOT2D needs ndim 2, size 3, pad 1, step 1");
+      if (n_params < 5) return fail(STENCIL_E_INVALID, "HOTSPOT2D needs 5 params");
+      p.radius = 1;
+      break;
+    case OP_GRADIENT:
+      if (ndim != 2 || !centred(1)) return fail(STENCIL_E_INVALID, "GRADIENT needs ndim 2, size 3, pad 1, step 1");
+      if (n_params < 1) return fail(STENCIL_E_INVALID, "GRADIENT needs 1 param (eps)");
       p.radius = 1;
       break;
     case OP_ACOUSTIC:
@@ -444,16 +467,16 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
   if (!state || n_state != 2) return fail(STENCIL_E_INVALID, "iterate needs 2 state buffers");
   if (!state[0] || !state[1] || state[0] == state[1]) return fail(STENCIL_E_INVALID, "bad state buffers");
   int ri = (p.op == OP_ACOUSTIC) ? 1 : 0;
-  if (p.op == OP_WEIGHTED) {
-    if (n_aux != 0) return fail(STENCIL_E_INVALID, "WEIGHTED iterate takes no aux grids");
+  if (p.op == OP_WEIGHTED || p.op == OP_GRADIENT) {
+    if (n_aux != 0) return fail(STENCIL_E_INVALID, "WEIGHTED/GRADIENT iterate takes no aux grids");
     for (int t = 0; t < n_steps; ++t) {
       const float* in[1] = {state[ri]};
       stencil_status s = stencil_apply(pl, in, 1, state[1 - ri], stream);
       if (s != STENCIL_OK) return s;
       ri = 1 - ri;
     }
-  } else if (p.op == OP_HOTSPOT3D) {
-    if (n_aux != 1 || !aux || !aux[0]) return fail(STENCIL_E_INVALID, "HOTSPOT3D iterate needs aux {P}");
+  } else if (p.op == OP_HOTSPOT3D || p.op == OP_HOTSPOT2D) {
+    if (n_aux != 1 || !aux || !aux[0]) return fail(STENCIL_E_INVALID, "HOTSPOT iterate needs aux {P}");
     for (int t = 0; t < n_steps; ++t) {
       const float* in[2] = {state[ri], aux[0]};
       stencil_status s = stencil_apply(pl, in, 2, state[1 - ri], stream);
@@ -471,7 +494,7 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
       ri = prev;
     }
   } else {
-    return fail(STENCIL_E_UNSUPPORTED, "iterate is built for WEIGHTED, HOTSPOT3D and ACOUSTIC");
+    return fail(STENCIL_E_UNSUPPORTED, "iterate is built for WEIGHTED, HOTSPOT3D/2D, GRADIENT and ACOUSTIC");
   }
   if (result_index) *result_index = ri;
   return STENCIL_OK;
@@ -513,7 +536,8 @@ stencil_status stencil_run_host(stencil_plan pl, const float* const* host_state,
     if (e != cudaSuccess) return cuda_fail(e, "H2D copy");
   }
   const float* result = nullptr;
-  const bool iterable = (p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D || p.op == OP_ACOUSTIC) && same_extents(p);
+  const bool iterable = (p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D || p.op == OP_ACOUSTIC ||
+                         p.op == OP_HOTSPOT2D || p.op == OP_GRADIENT) && same_extents(p);
   if (iterable && (p.op != OP_ACOUSTIC || n_state == 2)) {
     // WEIGHTED/HOTSPOT3D: state {X, scratch}; ACOUSTIC: state {prev, cur}
     float* state[2] = {pl->ws[0], pl->ws[1]};

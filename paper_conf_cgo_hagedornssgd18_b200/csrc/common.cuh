@@ -11,7 +11,9 @@
 namespace lift {
 
 enum PadKind : int { PAD_CLAMP = 0, PAD_MIRROR = 1, PAD_WRAP = 2, PAD_CONSTANT = 3, PAD_REFLECT = 4 };
-enum OpKind : int { OP_WEIGHTED = 0, OP_HOTSPOT3D = 1, OP_SRAD1 = 2, OP_SRAD2 = 3, OP_ACOUSTIC = 4 };
+enum OpKind : int {
+  OP_WEIGHTED = 0, OP_HOTSPOT3D = 1, OP_SRAD1 = 2, OP_SRAD2 = 3, OP_ACOUSTIC = 4, OP_HOTSPOT2D = 5, OP_GRADIENT = 6
+};
 
 constexpr int kMaxTaps = 125;     // 5x5x5
 constexpr int kMaxParams = 16;
@@ -39,6 +41,7 @@ struct StencilParams {
   // WEIGHTED: non-zero taps in row-major window order
   int32_t ntaps;
   int16_t tap[kMaxTaps][3];   // window index k per dimension
+  int32_t tap_off[kMaxTaps];   // kz*plane + ky*row + kx (K0 interior fast path; -1 in [0] = disabled)
   float w[kMaxTaps];
   float wbox[kMaxTaps];        // dense row-major window weights (fast kernels)
   // 2D WEIGHTED with exactly rank-1 weights w[ky][kx] = su[ky] * sv[kx]:

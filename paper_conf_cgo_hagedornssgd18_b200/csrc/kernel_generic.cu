@@ -82,9 +82,18 @@ __global__ void __launch_bounds__(256) k0_generic(const __grid_constant__ Stenci
             acc = __fmaf_rn(p.su[ky], h, acc);
           }
         } else {
-          for (int t = 0; t < p.ntaps; ++t) {
-            const float x = fetch(p, in0, bz + p.tap[t][0], by + p.tap[t][1], bx + p.tap[t][2]);
-            acc = __fmaf_rn(p.w[t], x, acc);
+          // interior fast path: the whole window lies inside the grid (and, in
+          // slab mode, inside the global domain), so no tap needs a remap
+          const bool inside = p.tap_off[0] >= 0 && bz >= 0 && bz + p.size[0] <= p.gnz && by >= 0 &&
+                              by + p.size[1] <= p.n[1] && bx >= 0 && bx + p.size[2] <= p.n[2];
+          if (inside) {
+            const float* __restrict__ base = in0 + (bz - p.z_off + p.ghost) * p.plane + by * p.row + bx;
+            for (int t = 0; t < p.ntaps; ++t) acc = __fmaf_rn(p.w[t], __ldg(base + p.tap_off[t]), acc);
+          } else {
+            for (int t = 0; t < p.ntaps; ++t) {
+              const float x = fetch(p, in0, bz + p.tap[t][0], by + p.tap[t][1], bx + p.tap[t][2]);
+              acc = __fmaf_rn(p.w[t], x, acc);
+            }
           }
         }
         v = acc;
@@ -100,6 +109,12 @@ __global__ void __launch_bounds__(256) k0_generic(const __grid_constant__ Stenci
         break;
       case OP_SRAD2:
         v = op_srad2(CentredAcc{p, in0, g}, CentredAcc{p, in1, g}, p.prm);
+        break;
+      case OP_HOTSPOT2D:
+        v = op_hotspot2d(CentredAcc{p, in0, g}, CentredAcc{p, in1, g}, p.prm);
+        break;
+      case OP_GRADIENT:
+        v = op_gradient(CentredAcc{p, in0, g}, p.prm);
         break;
       case OP_ACOUSTIC: {
         // inputs: in0 = prev (point-wise), in1 = cur (slid)

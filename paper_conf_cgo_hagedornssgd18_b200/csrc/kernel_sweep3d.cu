@@ -71,7 +71,7 @@ __device__ __forceinline__ void spin_until(const unsigned int* f, unsigned int v
   while ((int)(ld_acquire_sys(f) - v) < 0) __nanosleep(32);
 }
 
-enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2 };
+enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2, K2_WBOX = 3 };
 
 template <int R, int RPW, int S, bool PW>
 struct Cfg {
@@ -133,13 +133,13 @@ __device__ __forceinline__ float pick4(int s, const float4& c, float pv) {
   return s < 0 ? pv : (s == 0 ? c.x : (s == 1 ? c.y : (s == 2 ? c.z : c.w)));
 }
 
-template <int OP, int R, int RPW, int S, bool ZC>
+template <int OP, int R, int RPW, int S, bool ZC, bool FZ>
 __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
              const __grid_constant__ CUtensorMap pwmap, const float* __restrict__ src, float* out, int ntx,
              int nty, int zc, int nchunk, int slot) {
-  using C = Cfg<R, RPW, S, OP != K2_WSTAR>;
-  constexpr bool PW = OP != K2_WSTAR;           // a point-wise zipped grid (Hotspot P, Acoustic prev)
+  using C = Cfg<R, RPW, S, (OP == K2_HOTSPOT || OP == K2_ACOUSTIC)>;
+  constexpr bool PW = OP == K2_HOTSPOT || OP == K2_ACOUSTIC;           // a point-wise zipped grid (Hotspot P, Acoustic prev)
   constexpr int PS = C::PS;                     // point-wise ring slots
   constexpr int QN = 4;                         // item queue between the two producer lanes
   constexpr int PWF4 = C::PW_FLOATS / 4;
@@ -204,7 +204,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
         int nload = 1, x0 = 0, y0 = 0;
         int64_t zs = 0;
         if (!done) {
-          const int chunk = chunk_of(item / ntile, nchunk, p.fused_step), tile = item % ntile;
+          const int chunk = chunk_of(item / ntile, nchunk, FZ && p.fused_step), tile = item % ntile;
           x0 = (tile % ntx) * TX;
           y0 = (tile / ntx) * TY;
           zs = p.reg0 + (int64_t)chunk * zc;
@@ -212,10 +212,12 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
           nload = (int)(ze - zs) + 2 * R;
           // fused step: the ghost planes of this chunk must hold the neighbours'
           // previous step before the TMA reads them
-          bool waited = false;
-          if (chunk == 0 && p.wait_lo) { spin_until(p.wait_lo, p.wait_value); waited = true; }
-          if (chunk == nchunk - 1 && p.wait_hi) { spin_until(p.wait_hi, p.wait_value); waited = true; }
-          if (waited) asm volatile("fence.proxy.async.global;" ::: "memory");
+          if constexpr (FZ) {
+            bool waited = false;
+            if (chunk == 0 && p.wait_lo) { spin_until(p.wait_lo, p.wait_value); waited = true; }
+            if (chunk == nchunk - 1 && p.wait_hi) { spin_until(p.wait_hi, p.wait_value); waited = true; }
+            if (waited) asm volatile("fence.proxy.async.global;" ::: "memory");
+          }
         }
         // a "done" marker occupies one stage so the consumers see it in order
         for (int i = 0; i < nload; ++i) {
@@ -243,7 +245,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
         mbar_arrive(&itemempty[q]);
         if (++q == QN) { q = 0; ++qpass; }
         if (item < 0) break;
-        const int chunk = chunk_of(item / ntile, nchunk, p.fused_step), tile = item % ntile;
+        const int chunk = chunk_of(item / ntile, nchunk, FZ && p.fused_step), tile = item % ntile;
         const int x0 = (tile % ntx) * TX, y0 = (tile / ntx) * TY;
         const int64_t zs = p.reg0 + (int64_t)chunk * zc;
         const int nzc = (int)(min(zs + (int64_t)zc, p.reg1) - zs);
@@ -289,7 +291,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
         if (lane == 0) mbar_arrive(&empty[sn]);
         break;
       }
-      const int chunk = chunk_of(item / ntile, nchunk, p.fused_step), tile = item % ntile;
+      const int chunk = chunk_of(item / ntile, nchunk, FZ && p.fused_step), tile = item % ntile;
       const int x0 = (tile % ntx) * TX;
       const int y0 = (tile / ntx) * TY;
       const int64_t zs = p.reg0 + (int64_t)chunk * zc;
@@ -333,29 +335,55 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
       // Stages of the 2R+1 planes around the current output plane z: zst[k]
       // holds plane z - R + k (stage index, or -1 for a constant value plane).
       int zst[2 * R + 1];
+      // WRAP / non-zero constant: rewrite a plane's out-of-grid halo cells as
+      // soon as it arrives (no warp has read that stage since its TMA landed),
+      // so every plane of a window — not only the centre — is complete
+      // (box windows read the halo of every plane: fix each plane on arrival;
+      // star windows read only the centre plane's halo: fix the centre)
+      constexpr bool FIX_ON_ARRIVAL = OP == K2_WBOX;
+      auto fix_plane = [&](int stage, int64_t gzp) {
+        if (stage_const[stage]) return;
+        fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + stage * SF4), src,
+                                               plane_of(p, gzp), x0, y0, threadIdx.x);
+        fence_proxy_async_smem();
+      };
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k) {
         if (k > 0) mbar_wait(&full[sn], pn & 1);
         zst[k] = (ZC && stage_const[sn]) ? -1 - sn : sn;
+        if constexpr (FIX_ON_ARRIVAL) {
+          if (fix) fix_plane(sn, p.z_off + zs - R + k);
+        }
         if (++sn == S) { sn = 0; ++pn; }
+      }
+      if constexpr (FIX_ON_ARRIVAL) {
+        if (fix) named_bar_sync(1, NCONS);
       }
       float* orow = out + ((zs + p.ghost) * p.plane + (int64_t)(y0 + warp * RPW) * nx + xo);
 
       for (int j = 0; j < nzc; ++j) {
         mbar_wait(&full[sn], pn & 1);
         zst[2 * R] = (ZC && stage_const[sn]) ? -1 - sn : sn;
-        if (++sn == S) { sn = 0; ++pn; }
         const int64_t z = zs + j;                  // local output plane
         const int gz = (int)(p.z_off + z);
+        if constexpr (FIX_ON_ARRIVAL) {
+          if (fix) {
+            fix_plane(sn, p.z_off + z + R);
+            named_bar_sync(1, NCONS);
+          }
+        }
+        if (++sn == S) { sn = 0; ++pn; }
         const int cbase = zst[R] * SF4;             // the centre plane is inside the grid
-        if (fix) {
-          // all warps are past the previous plane (which read this stage as its
-          // z+1 neighbour, including the padding lanes/rows of ragged tiles)
-          named_bar_sync(1, NCONS);
-          fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + cbase), src,
-                                                 plane_of(p, (int64_t)gz), x0, y0, threadIdx.x);
-          fence_proxy_async_smem();
-          named_bar_sync(1, NCONS);
+        if constexpr (!FIX_ON_ARRIVAL) {
+          if (fix) {
+            // all warps are past the previous plane (which read this stage as its
+            // z+1 neighbour, including the padding lanes/rows of ragged tiles)
+            named_bar_sync(1, NCONS);
+            fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + cbase), src,
+                                                   plane_of(p, (int64_t)gz), x0, y0, threadIdx.x);
+            fence_proxy_async_smem();
+            named_bar_sync(1, NCONS);
+          }
         }
         // point-wise input of this output plane: its own TMA ring (no halo)
         if constexpr (PW) mbar_wait(&pwfull[psc], ppc & 1);
@@ -393,7 +421,37 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
             return dsm4[a * SF4 + rb];
           };
           float4 res;
-          if constexpr (OP == K2_ACOUSTIC) {
+          if constexpr (OP == K2_WBOX) {
+            // 3x3x3 box: every (plane, row) of the window is an x-window; taps
+            // are added in row-major (kz, ky, kx) order — K0's order
+            float acc[4] = {0.f, 0.f, 0.f, 0.f};
+#pragma unroll
+            for (int kz = 0; kz < 3; ++kz) {
+              const int a = zst[kz];
+              const bool cz = ZC && a < 0;
+              const int sb = (cz ? 0 : a) * SF4;
+#pragma unroll
+              for (int kyy = 0; kyy < 3; ++kyy) {
+                const int ro = rb + (kyy == 0 ? om[jj][0] : (kyy == 2 ? oq[jj][0] : 0));
+                const float4 c2 = cz ? pv4 : dsm4[sb + ro];
+                const float4 e2 = cz ? pv4 : dsm4[sb + ro - rb + eoff4 + jj * BX4];
+                float l = __shfl_up_sync(FULL, c2.w, 1);
+                float r = __shfl_down_sync(FULL, c2.x, 1);
+                if (lane == 0) l = e2.w;
+                if (lane == 31) r = e2.x;
+                if (pl && !cz) l = pick4(sl[0], c2, 0.0f);
+                if (pr && !cz) r = pick4(sr[0], c2, 0.0f);
+                const float w6[6] = {l, c2.x, c2.y, c2.z, c2.w, r};
+#pragma unroll
+                for (int kxx = 0; kxx < 3; ++kxx) {
+                  const float wt = p.wbox[(kz * 3 + kyy) * 3 + kxx];
+#pragma unroll
+                  for (int i = 0; i < 4; ++i) acc[i] = __fmaf_rn(wt, w6[i + kxx], acc[i]);
+                }
+              }
+            }
+            res = make_float4(acc[0], acc[1], acc[2], acc[3]);
+          } else if constexpr (OP == K2_ACOUSTIC) {
             // ordered neighbour sum (acoustic_sum's row-major order), accumulated
             // as the taps are loaded: z-R..z-1, y-R..y-1, x-R..x-1, x+1..x+R,
             // y+1..y+R, z+1..z+R
@@ -448,10 +506,12 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
           }
           if (ok) {
             stg128(orow + jj * nx, res);
-            // fused halo put: boundary planes also go to the neighbour's ghosts
-            if (z < p.ghost && p.put_lo) stg128(p.put_lo + z * p.plane + (int64_t)gy * nx + xo, res);
-            if (z >= p.n[0] - p.ghost && p.put_hi)
-              stg128(p.put_hi + (z - (p.n[0] - p.ghost)) * p.plane + (int64_t)gy * nx + xo, res);
+            if constexpr (FZ) {
+              // fused halo put: boundary planes also go to the neighbour's ghosts
+              if (z < p.ghost && p.put_lo) stg128(p.put_lo + z * p.plane + (int64_t)gy * nx + xo, res);
+              if (z >= p.n[0] - p.ghost && p.put_hi)
+                stg128(p.put_hi + (z - (p.n[0] - p.ghost)) * p.plane + (int64_t)gy * nx + xo, res);
+            }
           }
         }
         orow += p.plane;
@@ -475,7 +535,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
         for (int k = 0; k < 2 * R; ++k) mbar_arrive(&empty[zst[k] < 0 ? -1 - zst[k] : zst[k]]);
         // fused step: when every warp of every tile of a boundary chunk is done,
         // publish its peer stores and raise that neighbour's flag
-        if (p.fused_step) {
+        if (FZ && p.fused_step) {
           const unsigned need = (unsigned)ntile * NW;
           if (chunk == 0 && p.sig_lo) {
             __threadfence_system();
@@ -497,7 +557,7 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
   }
   // last CTA out resets the launch slot's counters (graph-replay safe) and,
   // for a fused halo put, publishes the ghost planes to the neighbours
-  const bool puts = p.put_lo || p.put_hi;
+  const bool puts = FZ && (p.put_lo || p.put_hi);
   if (puts) __threadfence_system();     // this thread's peer stores before the CTA's arrival
   __syncthreads();
   if (threadIdx.x == 0) {
@@ -539,13 +599,13 @@ struct Launcher {
   int ctas_per_sm;
 };
 
-template <int OP, int R, int RPW, int S, bool ZC>
+template <int OP, int R, int RPW, int S, bool ZC, bool FZ>
 Launcher get_launcher() {
   static Launcher L{};
   static std::once_flag once;
   std::call_once(once, [] {
-    using C = Cfg<R, RPW, S, OP != K2_WSTAR>;
-    auto fn = k2_sweep<OP, R, RPW, S, ZC>;
+    using C = Cfg<R, RPW, S, (OP == K2_HOTSPOT || OP == K2_ACOUSTIC)>;
+    auto fn = k2_sweep<OP, R, RPW, S, ZC, FZ>;
     cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
     int occ = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, NCONS + 32, C::SMEM) != cudaSuccess) occ = 1;
@@ -555,27 +615,24 @@ Launcher get_launcher() {
   return L;
 }
 
+template <int OP, int R, int RPW, int S>
+Launcher get_launcher_zf(bool zc, bool fz) {
+  if (fz) return zc ? get_launcher<OP, R, RPW, S, true, true>() : get_launcher<OP, R, RPW, S, false, true>();
+  return zc ? get_launcher<OP, R, RPW, S, true, false>() : get_launcher<OP, R, RPW, S, false, false>();
+}
+
 Launcher pick(const StencilParams& p) {
   const int R = p.radius;
   const bool zc = p.kind[0] == PAD_CONSTANT;   // value-pad planes in z are possible
+  const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;   // fused halo launch
   if (p.op == OP_WEIGHTED) {
-    if (R == 1) return zc ? get_launcher<K2_WSTAR, 1, 2, 7, true>() : get_launcher<K2_WSTAR, 1, 2, 7, false>();
-    return zc ? get_launcher<K2_WSTAR, 2, 2, 8, true>() : get_launcher<K2_WSTAR, 2, 2, 8, false>();
+    if (R == 1 && !star_weights(p, 1)) return get_launcher_zf<K2_WBOX, 1, 2, 7>(zc, fz);
+    if (R == 1) return get_launcher_zf<K2_WSTAR, 1, 2, 7>(zc, fz);
+    return get_launcher_zf<K2_WSTAR, 2, 2, 8>(zc, fz);
   }
-  if (p.op == OP_HOTSPOT3D)
-    return zc ? get_launcher<K2_HOTSPOT, 1, 2, 5, true>() : get_launcher<K2_HOTSPOT, 1, 2, 5, false>();
-  if (R == 1) return zc ? get_launcher<K2_ACOUSTIC, 1, 2, 5, true>() : get_launcher<K2_ACOUSTIC, 1, 2, 5, false>();
-  // tile-shape sweep hook (NEXT-4 / ATF role): LIFT_K2_VARIANT
-  static const int tv = [] { const char* e = getenv("LIFT_K2_VARIANT"); return e ? atoi(e) : 0; }();
-  if (zc) {
-    switch (tv) {
-      case 1: return get_launcher<K2_ACOUSTIC, 2, 1, 8, true>();
-      case 2: return get_launcher<K2_ACOUSTIC, 2, 2, 6, true>();
-      case 3: return get_launcher<K2_ACOUSTIC, 2, 1, 10, true>();
-      default: break;
-    }
-  }
-  return zc ? get_launcher<K2_ACOUSTIC, 2, 2, 8, true>() : get_launcher<K2_ACOUSTIC, 2, 2, 8, false>();
+  if (p.op == OP_HOTSPOT3D) return get_launcher_zf<K2_HOTSPOT, 1, 2, 5>(zc, fz);
+  if (R == 1) return get_launcher_zf<K2_ACOUSTIC, 1, 2, 5>(zc, fz);
+  return get_launcher_zf<K2_ACOUSTIC, 2, 2, 8>(zc, fz);
 }
 
 struct MapEntry {
@@ -612,7 +669,7 @@ bool sweep3d_supported(const StencilParams& p) {
   for (int d = 0; d < 3; ++d)
     if (p.size[d] != 2 * R + 1 || p.lo[d] != R || p.hi[d] != R || p.step[d] != 1) return false;
   if (p.op == OP_WEIGHTED) {
-    if (!star_weights(p, R)) return false;
+    if (!star_weights(p, R) && R != 1) return false;      // 3x3x3 boxes run on K2_WBOX
   } else if (p.op == OP_HOTSPOT3D) {
     if (R != 1) return false;
   } else if (p.op != OP_ACOUSTIC) {

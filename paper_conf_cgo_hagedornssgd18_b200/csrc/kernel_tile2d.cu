@@ -40,7 +40,7 @@ constexpr int NW = 8;
 constexpr int NCONS = NW * 32;
 constexpr unsigned FULL = 0xffffffffu;
 
-enum K1Op { K1_WBOX = 0, K1_SRAD1 = 1, K1_SRAD2 = 2, K1_WSTAR = 3, K1_WSEP = 4 };
+enum K1Op { K1_WBOX = 0, K1_SRAD1 = 1, K1_SRAD2 = 2, K1_WSTAR = 3, K1_WSEP = 4, K1_HOT2D = 5, K1_GRAD = 6 };
 
 template <int RY, int RPW, int S, int NIN>
 struct Cfg {
@@ -234,6 +234,10 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
             constexpr int ii = decltype(I)::value;
             if constexpr (OP == K1_SRAD1) {
               v[ii] = op_srad1(RingAcc<RY, RX, ii>{wa}, p.prm);
+            } else if constexpr (OP == K1_GRAD) {
+              v[ii] = op_gradient(RingAcc<RY, RX, ii>{wa}, p.prm);
+            } else if constexpr (OP == K1_HOT2D) {
+              v[ii] = op_hotspot2d(RingAcc<RY, RX, ii>{wa}, RingAcc<RY, RX, ii>{wb}, p.prm);   // (T, P)
             } else {
               v[ii] = op_srad2(RingAcc<RY, RX, ii>{wa}, RingAcc<RY, RX, ii>{wb}, p.prm);   // (c, I)
             }
@@ -317,6 +321,8 @@ bool pick(const StencilParams& p, Launcher* L) {
   }
   if (p.op == OP_SRAD1) { *L = K1_PICK(K1_SRAD1, 1, 1, 1); return true; }
   if (p.op == OP_SRAD2) { *L = K1_PICK(K1_SRAD2, 1, 1, 2); return true; }
+  if (p.op == OP_HOTSPOT2D) { *L = K1_PICK(K1_HOT2D, 1, 1, 2); return true; }
+  if (p.op == OP_GRADIENT) { *L = K1_PICK(K1_GRAD, 1, 1, 1); return true; }
   return false;
 }
 
@@ -352,7 +358,7 @@ bool tile2d_supported(const StencilParams& p) {
   for (int d = 1; d < 3; ++d)
     if (p.step[d] != 1 || p.hi[d] != p.lo[d] || p.size[d] != 2 * p.lo[d] + 1) return false;
   if (ry < 1 || ry > 2 || rx < 1 || rx > 2) return false;
-  if (p.op == OP_SRAD1 || p.op == OP_SRAD2) {
+  if (p.op == OP_SRAD1 || p.op == OP_SRAD2 || p.op == OP_HOTSPOT2D || p.op == OP_GRADIENT) {
     if (ry != 1 || rx != 1) return false;
   } else if (p.op != OP_WEIGHTED) {
     return false;

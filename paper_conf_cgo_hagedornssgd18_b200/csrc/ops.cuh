@@ -111,6 +111,38 @@ __device__ __forceinline__ float op_srad2(const AccC& C, const AccI& I, const fl
   return __fmaf_rn(__fmul_rn(0.25f, lam), D, Ic);
 }
 
+// ---- Hotspot2D (Rodinia v3.1 hotspot; A26) -----------------------
+// T' = T + sdc * (P + (S + N - 2T)*Ry_1 + (E + W - 2T)*Rx_1 + (amb - T)*Rz_1)
+template <class AccT, class AccP>
+__device__ __forceinline__ float op_hotspot2d(const AccT& T, const AccP& P, const float* prm) {
+  const float sdc = prm[0], rx1 = prm[1], ry1 = prm[2], rz1 = prm[3], amb = prm[4];
+  const float Tc = T.template at<0, 0, 0>();
+  const float a = __fmaf_rn(-2.0f, Tc, __fadd_rn(T.template at<0, 1, 0>(), T.template at<0, -1, 0>()));
+  const float b = __fmaf_rn(-2.0f, Tc, __fadd_rn(T.template at<0, 0, 1>(), T.template at<0, 0, -1>()));
+  float acc = P.template at<0, 0, 0>();
+  acc = __fmaf_rn(a, ry1, acc);
+  acc = __fmaf_rn(b, rx1, acc);
+  acc = __fmaf_rn(__fsub_rn(amb, Tc), rz1, acc);
+  return __fmaf_rn(sdc, acc, Tc);
+}
+
+// ---- Gradient (Rawat et al. [36] 2D gradient; A25) ---------------
+// out = I + 1/sqrt(eps + (I-N)^2 + (I-S)^2 + (I-W)^2 + (I-E)^2)
+template <class Acc>
+__device__ __forceinline__ float op_gradient(const Acc& I, const float* prm) {
+  const float eps = prm[0];
+  const float Ic = I.template at<0, 0, 0>();
+  const float d1 = __fsub_rn(Ic, I.template at<0, -1, 0>());
+  const float d2 = __fsub_rn(Ic, I.template at<0, 1, 0>());
+  const float d3 = __fsub_rn(Ic, I.template at<0, 0, -1>());
+  const float d4 = __fsub_rn(Ic, I.template at<0, 0, 1>());
+  float s = __fmaf_rn(d1, d1, eps);
+  s = __fmaf_rn(d2, d2, s);
+  s = __fmaf_rn(d3, d3, s);
+  s = __fmaf_rn(d4, d4, s);
+  return __fadd_rn(Ic, __frsqrt_rn(s));
+}
+
 // ---- Acoustic (Listing 3; A19/A20) --------------------
 // next = cf(K,l1) * ((2 - l2*K)*u_c + l2*sum_nbr u - cf(K,l2loss)*prev)
 // Neighbours are summed in row-major tap order (Listing 3 lines 5-6).

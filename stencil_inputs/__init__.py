@@ -28,12 +28,12 @@ KIND_NAMES = {CLAMP: "clamp", MIRROR: "mirror", WRAP: "wrap",
               CONSTANT: "constant", REFLECT: "reflect"}
 
 # Ops — numeric values are the C-ABI enum ``stencil_op``.
-WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC = 0, 1, 2, 3, 4
+WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC, HOTSPOT2D, GRADIENT = 0, 1, 2, 3, 4, 5, 6
 OP_NAMES = {WEIGHTED: "weighted", HOTSPOT3D: "hotspot3d", SRAD1: "srad1",
-            SRAD2: "srad2", ACOUSTIC: "acoustic"}
+            SRAD2: "srad2", ACOUSTIC: "acoustic", HOTSPOT2D: "hotspot2d", GRADIENT: "gradient"}
 
 # Number of input grids per op (zip arity).
-N_INPUTS = {WEIGHTED: 1, HOTSPOT3D: 2, SRAD1: 1, SRAD2: 2, ACOUSTIC: 2}
+N_INPUTS = {WEIGHTED: 1, HOTSPOT3D: 2, SRAD1: 1, SRAD2: 2, ACOUSTIC: 2, HOTSPOT2D: 2, GRADIENT: 1}
 
 
 @dataclass
@@ -141,6 +141,47 @@ def params_hotspot3d() -> Tuple[float, ...]:
     sdc = 0.341333
     amb = 80.0
     return tuple(float(np.float32(v)) for v in (cc, cn, cs, ce, cw, ct, cb, sdc, amb))
+
+
+def params_hotspot2d(rows: int, cols: int) -> Tuple[float, ...]:
+    """Rodinia v3.1 hotspot constants for a rows x cols chip (A26).
+    Order: step/Cap, 1/Rx, 1/Ry, 1/Rz, amb."""
+    t_chip, chip_h, chip_w = 0.0005, 0.016, 0.016
+    k_si, spec_heat_si, factor_chip, max_pd, precision, amb = 100.0, 1.75e6, 0.5, 3.0e6, 0.001, 80.0
+    gh, gw = chip_h / rows, chip_w / cols
+    cap = factor_chip * spec_heat_si * t_chip * gw * gh
+    rx = gw / (2.0 * k_si * t_chip * gh)
+    ry = gh / (2.0 * k_si * t_chip * gw)
+    rz = t_chip / (k_si * gh * gw)
+    max_slope = max_pd / (factor_chip * t_chip * spec_heat_si)
+    step = precision / max_slope
+    return tuple(float(np.float32(v)) for v in (step / cap, 1.0 / rx, 1.0 / ry, 1.0 / rz, amb))
+
+
+def params_gradient() -> Tuple[float, ...]:
+    """eps of the 2D gradient (A25)."""
+    return (float(np.float32(1e-4)),)
+
+
+def weights_heat7() -> np.ndarray:
+    """Heat 3D 7-point ([35], A13): u + 0.125 * (discrete Laplacian)."""
+    w = np.zeros((3, 3, 3), np.float32)
+    w[1, 1, 1] = 1.0 - 6 * 0.125
+    for d in range(3):
+        for sgn in (0, 2):
+            idx = [1, 1, 1]
+            idx[d] = sgn
+            w[tuple(idx)] = 0.125
+    return w
+
+
+def weights_poisson19() -> np.ndarray:
+    """Poisson 3D 19-point ([35], A13): centre 1/4, 6 faces 1/16, 12 edges 1/32 (normalised, dyadic)."""
+    w = np.zeros((3, 3, 3), np.float32)
+    for k in np.ndindex(3, 3, 3):
+        nax = sum(1 for v in k if v != 1)
+        w[k] = {0: 0.25, 1: 1.0 / 16, 2: 1.0 / 32}.get(nax, 0.0)
+    return w
 
 
 def params_srad1(q0sqr: float) -> Tuple[float, ...]:
@@ -269,6 +310,37 @@ def _c5b():
                     note="C5b: Acoustic 13-point (A20 extrapolation), zero pad, prev = cur")
 
 
+# Table 1 shapes through the same ABI ("paper-shaped sweep", NEXT-1)
+def _t1(name, extents, size, op=WEIGHTED, weights=None, params=(), kind=CLAMP, seeds=(2001,),
+        ranges=((0.5, 1.5),), transform=(), note=""):
+    return lambda: Workload(name, _spec(extents, size, op=op, weights=weights, params=params, kind=kind),
+                            seeds, ranges, 1, transform, note)
+
+
+_TABLE1 = {
+    "t1_stencil2d_4098": _t1("t1_stencil2d_4098", (4098, 4098), 3, weights=weights_j2d9(),
+                             note="SHOC Stencil2D 9-point (weights: A13 J2D9 reading)"),
+    "t1_srad1_504x458": _t1("t1_srad1_504x458", (504, 458), 3, op=SRAD1, transform=("exp",), ranges=((0.0, 1.0),),
+                            note="Rodinia SRAD1 at the paper's size"),
+    "t1_hotspot2d_8192": _t1("t1_hotspot2d_8192", (8192, 8192), 3, op=HOTSPOT2D,
+                             params=params_hotspot2d(8192, 8192), seeds=(2002, 2003),
+                             ranges=((300.0, 350.0), (0.0, 1e-2)), note="Rodinia Hotspot2D (A26)"),
+    "t1_acoustic_404x512x512": _t1("t1_acoustic_404x512x512", (404, 512, 512), 3, op=ACOUSTIC,
+                                   params=params_acoustic(7), kind=CONSTANT, seeds=(2004, 2004),
+                                   ranges=((-1.0, 1.0), (-1.0, 1.0)), note="Acoustic at the paper's size"),
+    "t1_gaussian_4096": _t1("t1_gaussian_4096", (4096, 4096), 5, weights=weights_gauss5(), kind=MIRROR),
+    "t1_gradient_4096": _t1("t1_gradient_4096", (4096, 4096), 3, op=GRADIENT, params=params_gradient(),
+                            note="Rawat 2D gradient (A25)"),
+    "t1_gradient_8192": _t1("t1_gradient_8192", (8192, 8192), 3, op=GRADIENT, params=params_gradient()),
+    "t1_jacobi2d5_8192": _t1("t1_jacobi2d5_8192", (8192, 8192), 3, weights=weights_j2d5()),
+    "t1_jacobi2d9_8192": _t1("t1_jacobi2d9_8192", (8192, 8192), 3, weights=weights_j2d9()),
+    "t1_jacobi3d7_256": _t1("t1_jacobi3d7_256", (256, 256, 256), 3, weights=weights_j3d7()),
+    "t1_jacobi3d13_512": _t1("t1_jacobi3d13_512", (512, 512, 512), 5, weights=weights_j3d13()),
+    "t1_poisson19_512": _t1("t1_poisson19_512", (512, 512, 512), 3, weights=weights_poisson19(),
+                            note="Poisson 19-point (A13 reading)"),
+    "t1_heat7_512": _t1("t1_heat7_512", (512, 512, 512), 3, weights=weights_heat7()),
+}
+
 _WORKLOADS = {
     "j2d5_256_clamp": _c1,
     "gauss5_8192_mirror": _c2,
@@ -280,7 +352,9 @@ _WORKLOADS = {
     "acoustic13_1024": _c5b,
 }
 
+_WORKLOADS.update(_TABLE1)
 WORKLOAD_NAMES = tuple(_WORKLOADS)
+TABLE1_NAMES = tuple(_TABLE1)
 
 
 def make_workload_inputs(w: Workload) -> Tuple[List[np.ndarray], StencilSpec]:
@@ -289,7 +363,4 @@ def make_workload_inputs(w: Workload) -> Tuple[List[np.ndarray], StencilSpec]:
     spec = w.spec
     if spec.op == SRAD1:
         spec.params = params_srad1(srad_q0sqr(xs[0]))
-    if spec.op == SRAD2:
-        # c must lie in [0, 1]; draw it as U[0,1) (seed 1008), I = exp(U).
-        pass
     return xs, spec

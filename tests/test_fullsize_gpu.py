@@ -151,3 +151,14 @@ def test_acoustic_1024(lift, name, pts_):
     idx = samples(spec.extents, 6, 15)[:20]
     gv = {p: v for p, v in zip(idx, g[tuple(torch.tensor(idx).T.cuda())].cpu().numpy())}
     light_cone_check(spec, xs, [], gv, idx, 10, r, 1e-4, acoustic=True)
+
+
+@pytest.mark.parametrize("name", ["t1_stencil2d_4098", "t1_srad1_504x458", "t1_hotspot2d_8192", "t1_gradient_4096",
+                                  "t1_jacobi2d9_8192", "t1_poisson19_512", "t1_heat7_512", "t1_jacobi3d13_512",
+                                  "t1_acoustic_404x512x512"])
+def test_table1_paper_sizes(lift, name):
+    """Table 1 workloads at the paper's sizes, sampled parity."""
+    w = si.workload(name)
+    xs, spec = si.make_workload_inputs(w)
+    y, plan = gpu_apply(lift, spec, xs)
+    check_points(spec, xs, y, samples(spec.extents, 200, 16))

@@ -175,7 +175,8 @@ def _variants(plan_nd):
     return ["generic", "tile2d"] if plan_nd == 2 else ["generic", "sweep3d"]
 
 
-@pytest.mark.parametrize("case", ["j2d5", "gauss", "j3d7", "j3d13", "hotspot", "acoustic13", "srad1", "srad2"])
+@pytest.mark.parametrize("case", ["j2d5", "gauss", "j3d7", "j3d13", "hotspot", "acoustic13", "srad1", "srad2",
+                                  "box27_wrap", "box27_const", "box27_mirror"])
 def test_kernel_families_bitwise_equal(lift, case):
     """Tiling independence: every kernel family gives the same bits."""
     rng = np.random.default_rng(24)
@@ -193,6 +194,10 @@ def test_kernel_families_bitwise_equal(lift, case):
     elif case == "acoustic13":
         sp = spec((19, 37, 136), 5, op=si.ACOUSTIC, params=si.params_acoustic(13), kind=CONSTANT)
         xs = [rnd((19, 37, 136), 31, -1, 1), rnd((19, 37, 136), 32, -1, 1)]
+    elif case.startswith("box27"):
+        k = {"wrap": WRAP, "const": CONSTANT, "mirror": MIRROR}[case.split("_")[1]]
+        w = np.random.default_rng(54).standard_normal((3, 3, 3)).astype(np.float32)
+        sp, xs = spec((19, 37, 264), 3, w, (k, k, k), value=0.7), [rnd((19, 37, 264), 55)]
     elif case == "srad1":
         I = np.exp(rnd((130, 264), 33, 0, 1)).astype(np.float32)
         sp, xs = spec(I.shape, 3, op=si.SRAD1, params=si.params_srad1(si.srad_q0sqr(I))), [I]
@@ -221,7 +226,8 @@ def test_variant_selection(lift):
              (spec((64, 128), 3, op=si.SRAD1, params=(0.1,)), "tile2d"),
              (spec((64, 128), 3, op=si.SRAD2, params=(0.5,)), "tile2d"),
              (spec((64, 64, 130), 3, si.weights_j3d7()), "generic"),
-             (spec((64, 64, 128), 3, np.ones((3, 3, 3), np.float32)), "generic")]
+             (spec((64, 64, 128), 3, np.ones((3, 3, 3), np.float32)), "sweep3d"),
+             (spec((64, 64, 128), 5, np.ones((5, 5, 5), np.float32)), "generic")]
     for sp, v in cases:
         plan = lift.Plan.from_spec(sp)
         assert plan.variant == lift.plan.VARIANTS[v], (sp, v)
@@ -313,3 +319,28 @@ def test_run_host_matches_device(lift):
     dev = (a, b)[ri].cpu().numpy()
     host = plan.run_host([x], n_steps=3)
     np.testing.assert_array_equal(host, dev)
+
+
+# ------------------------------------------------ Table 1 extras (NEXT-1) --
+@pytest.mark.parametrize("kind", [CLAMP, MIRROR, WRAP])
+def test_hotspot2d_and_gradient(lift, kind):
+    T = rnd((100, 260), 50, 300.0, 350.0)
+    P = rnd(T.shape, 51, 0.0, 1e-2)
+    sp = spec(T.shape, 3, op=si.HOTSPOT2D, params=si.params_hotspot2d(512, 512), kind=kind)
+    y, plan = check(lift, sp, [T, P])
+    assert plan.variant == 1
+    y0, _ = run_gpu(lift, sp, [T, P], "generic")
+    np.testing.assert_array_equal(y, y0)
+    I = rnd((100, 260), 52, 0.0, 1.0)
+    sp = spec(I.shape, 3, op=si.GRADIENT, params=si.params_gradient(), kind=kind)
+    y, plan = check(lift, sp, [I])
+    assert plan.variant == 1
+    y0, _ = run_gpu(lift, sp, [I], "generic")
+    np.testing.assert_array_equal(y, y0)
+
+
+def test_poisson19_and_heat7(lift):
+    x = rnd((20, 40, 132), 53)
+    check(lift, spec(x.shape, 3, si.weights_poisson19(), MIRROR), [x])
+    _, plan = check(lift, spec(x.shape, 3, si.weights_heat7(), CLAMP), [x])
+    assert plan.variant == 2
