@@ -134,6 +134,16 @@ stencil_status stencil_plan_output_extents(stencil_plan plan, int64_t* out_exten
 stencil_status stencil_plan_set_slab(stencil_plan plan, int64_t z_offset,
                                      int64_t global_n0, int32_t ghost);
 
+/* Temporal blocking for stencil_iterate: 2 lets iterate
+ * advance two time steps per pass over HBM where the TMA sweep's two-step
+ * kernel applies (WEIGHTED 7-point star, CLAMP/MIRROR/REFLECT); the result is
+ * bitwise identical to single steps.  1 (default) takes one step per pass:
+ * on B200 the single-step sweep already reaches ~0.9 of the HBM roofline and
+ * the two-step kernel is instruction-bound.
+ * stencil_plan_time_block returns the steps per pass iterate will use. */
+stencil_status stencil_plan_set_time_block(stencil_plan plan, int32_t steps);
+int32_t stencil_plan_time_block(stencil_plan plan);
+
 /* Force a kernel family (tests: tiling independence) or AUTO. E_UNSUPPORTED if
  * the requested family cannot run this plan. */
 stencil_status stencil_plan_set_variant(stencil_plan plan, int32_t variant);

@@ -48,6 +48,8 @@ _out_ext = _sig("stencil_plan_output_extents", C.c_int, [_P, _I64P])
 _set_slab = _sig("stencil_plan_set_slab", C.c_int, [_P, C.c_int64, C.c_int64, C.c_int32])
 _set_variant = _sig("stencil_plan_set_variant", C.c_int, [_P, C.c_int32])
 _variant = _sig("stencil_plan_variant", C.c_int32, [_P])
+_set_tb = _sig("stencil_plan_set_time_block", C.c_int, [_P, C.c_int32])
+_tb = _sig("stencil_plan_time_block", C.c_int32, [_P])
 _apply = _sig("stencil_apply", C.c_int, [_P, _FPP, C.c_int32, _P, _P])
 _apply_region = _sig("stencil_apply_region", C.c_int, [_P, _FPP, C.c_int32, _P, C.c_int64, C.c_int64, _P])
 _apply_region_put = _sig("stencil_apply_region_put", C.c_int, [_P, _FPP, C.c_int32, _P, C.c_int64, C.c_int64, _P, _P,
@@ -63,7 +65,8 @@ _last_error = _sig("stencil_last_error", C.c_char_p, [])
 _version = _sig("stencil_version", C.c_char_p, [])
 
 EXPORTED = ("stencil_plan_create", "stencil_plan_output_extents", "stencil_plan_set_slab",
-            "stencil_plan_set_variant", "stencil_plan_variant", "stencil_apply", "stencil_apply_region",
+            "stencil_plan_set_variant", "stencil_plan_variant", "stencil_plan_set_time_block",
+            "stencil_plan_time_block", "stencil_apply", "stencil_apply_region",
             "stencil_apply_region_put", "stencil_slab_step_fused", "stencil_wait_signals",
             "stencil_iterate", "stencil_run_host", "stencil_plan_destroy", "stencil_status_string",
             "stencil_last_error", "stencil_version")
@@ -136,6 +139,14 @@ def stencil_plan_set_variant(plan: int, variant: int):
 
 def stencil_plan_variant(plan: int) -> int:
     return int(_variant(plan))
+
+
+def stencil_plan_set_time_block(plan: int, steps: int):
+    _check(_set_tb(plan, int(steps)), "stencil_plan_set_time_block")
+
+
+def stencil_plan_time_block(plan: int) -> int:
+    return int(_tb(plan))
 
 
 def stencil_apply(plan: int, inputs: Sequence[int], out: int, stream: int = 0):

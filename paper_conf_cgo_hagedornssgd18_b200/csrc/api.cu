@@ -23,6 +23,7 @@ struct stencil_plan_s {
   StencilParams p{};
   int64_t user_out_ext[3] = {0, 0, 0};
   int32_t forced_variant = STENCIL_VARIANT_AUTO;
+  int32_t time_block = 1;          // stencil_iterate: time steps per pass where K2T applies (opt-in, see DESIGN)
   int32_t last_variant = STENCIL_VARIANT_GENERIC;
   // stencil_run_host workspace (device)
   std::vector<float*> ws;
@@ -362,6 +363,18 @@ stencil_status stencil_plan_set_variant(stencil_plan pl, int32_t variant) {
   return STENCIL_OK;
 }
 
+stencil_status stencil_plan_set_time_block(stencil_plan pl, int32_t steps) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  if (steps != 1 && steps != 2) return fail(STENCIL_E_INVALID, "time block must be 1 or 2");
+  pl->time_block = steps;
+  return STENCIL_OK;
+}
+
+int32_t stencil_plan_time_block(stencil_plan pl) {
+  if (!pl) return -1;
+  return (pl->time_block >= 2 && sweep3d_t2_supported(pl->p)) ? 2 : 1;
+}
+
 int32_t stencil_plan_variant(stencil_plan pl) {
   if (!pl) return -1;
   if (pl->forced_variant != STENCIL_VARIANT_AUTO) return pl->forced_variant;
@@ -469,7 +482,22 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
   int ri = (p.op == OP_ACOUSTIC) ? 1 : 0;
   if (p.op == OP_WEIGHTED || p.op == OP_GRADIENT) {
     if (n_aux != 0) return fail(STENCIL_E_INVALID, "WEIGHTED/GRADIENT iterate takes no aux grids");
-    for (int t = 0; t < n_steps; ++t) {
+    int t = 0;
+    // temporal blocking: two steps per pass (K2T) while at least two remain
+    if (pl->time_block >= 2 && n_steps >= 2 && sweep3d_t2_supported(p) &&
+        (pl->forced_variant == STENCIL_VARIANT_AUTO || pl->forced_variant == STENCIL_VARIANT_SWEEP3D) &&
+        aligned16(state[0]) && aligned16(state[1])) {
+      DeviceGuard g(pl->device);
+      if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+      for (; t + 2 <= n_steps; t += 2) {
+        std::string err;
+        cudaError_t e = launch_sweep3d_t2(p, state[ri], state[1 - ri], (cudaStream_t)stream, pl->num_sms, &err);
+        if (e != cudaSuccess)
+          return fail(STENCIL_E_CUDA, std::string("K2T launch failed: ") + cudaGetErrorString(e) + " " + err);
+        ri = 1 - ri;
+      }
+    }
+    for (; t < n_steps; ++t) {
       const float* in[1] = {state[ri]};
       stencil_status s = stencil_apply(pl, in, 1, state[1 - ri], stream);
       if (s != STENCIL_OK) return s;

@@ -579,6 +579,245 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
 }
 
 // ---------------------------------------------------------------------------
+// K2T: two time steps per pass (temporal blocking) for the
+// weighted 7-point star with CLAMP / MIRROR / REFLECT boundaries.
+//
+// X_t planes stream through the same TMA ring as K2 (box (128+8) x (16+2) at
+// (x0-8, y0-2)); for each plane yz the 8 warps compute X_{t+1} on the
+// extended 128 x 16 tile (columns x0-4 .. x0+123, rows y0-1 .. y0+14) into a
+// 4-slot shared-memory ring, then — one barrier later — X_{t+2} on the inner
+// 120 x 14 tile of plane yz-1 from the three ring planes.  Every value goes
+// through op_weighted, so the result is bitwise equal to two single steps.
+// pad applies to X_{t+1} as to any grid: its out-of-grid rows/columns are
+// redirected to the remapped in-grid ones, and a plane outside the grid
+// (global z = -1 or nz) aliases the remapped plane's ring slot.
+// ---------------------------------------------------------------------------
+constexpr int T2_TXO = 120;     // output columns per tile (lanes 1..30)
+constexpr int T2_TYO = 14;      // output rows per tile (Y rows 1..14)
+constexpr int T2_TY = 16;       // X_{t+1} rows per tile (2 per warp)
+constexpr int T2_BY = T2_TY + 2;
+constexpr int T2_YF4 = T2_TY * (TX / 4);   // float4 per X_{t+1} plane slot
+
+template <int S>
+struct CfgT2 {
+  static constexpr int TX_BYTES = BX * T2_BY * 4;
+  static constexpr int STAGE_FLOATS = ((TX_BYTES + 127) / 128) * 128 / 4;
+  static constexpr int SMEM = S * STAGE_FLOATS * 4 + 4 * T2_YF4 * 16 + 2 * S * 8 + 2 * S * 4 + 256;
+};
+
+template <int S>
+__global__ void __launch_bounds__(NCONS + 32, 2)
+    k2t_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap, float* out, int ntx,
+              int nty, int zc, int nchunk, int slot) {
+  using C = CfgT2<S>;
+  constexpr int SF4 = C::STAGE_FLOATS / 4;
+  constexpr int BX4 = BX / 4;
+  constexpr int TX4 = TX / 4;
+  extern __shared__ __align__(128) float4 dsm4[];
+  float4* ysm = dsm4 + S * SF4;                                   // 4 X_{t+1} slots
+  uint64_t* full = reinterpret_cast<uint64_t*>(ysm + 4 * T2_YF4);
+  uint64_t* empty = full + S;
+  int* stage_item = reinterpret_cast<int*>(empty + S);
+
+  const int ntile = ntx * nty;
+  const int nitems = ntile * nchunk;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  if (threadIdx.x == 0) {
+    for (int s = 0; s < S; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NW);
+    }
+    fence_mbar_init();
+  }
+  __syncthreads();
+
+  if (warp == NW) {
+    if (lane == 0) {
+      prefetch_tmap(&tmap);
+      int s = 0;
+      uint32_t pass = 0;
+      while (true) {
+        const int item = (int)atomicAdd(&g_ticket[slot], 1u);
+        const bool done = item >= nitems;
+        int nload = 1, x0 = 0, y0 = 0;
+        int64_t zs = 0;
+        if (!done) {
+          const int chunk = item / ntile, tile = item % ntile;
+          x0 = (tile % ntx) * T2_TXO;
+          y0 = (tile / ntx) * T2_TYO;
+          zs = p.reg0 + (int64_t)chunk * zc;
+          nload = (int)(min(zs + (int64_t)zc, p.reg1) - zs) + 4;   // X planes zs-2 .. ze+1
+        }
+        for (int i = 0; i < nload; ++i) {
+          if (pass > 0) mbar_wait(&empty[s], (pass - 1) & 1);
+          if (i == 0) stage_item[s] = done ? -1 : item;
+          if (!done) {
+            const int64_t lz = plane_of(p, p.z_off + zs - 2 + i);   // never constant (no CONSTANT kind here)
+            mbar_arrive_expect_tx(&full[s], C::TX_BYTES);
+            tma_load_3d(dsm4 + s * SF4, &tmap, &full[s], x0 - 8, y0 - 2, (int)lz);
+          } else {
+            mbar_arrive(&full[s]);
+          }
+          if (++s == S) { s = 0; ++pass; }
+        }
+        if (done) break;
+      }
+    }
+  } else {
+    const int nx = (int)p.n[2], ny = (int)p.n[1];
+    const int kx = p.kind[2], ky = p.kind[1], kz = p.kind[0];
+    const int gnz = (int)p.gnz;
+    const int rsx = (int)pad_remap(-1, nx, kx);                        // source column of x = -1
+    const int rex = (int)(pad_remap(nx, nx, kx) - (nx - 4));           // element of x = nx in the last float4
+    int sn = 0;
+    uint32_t pn = 0;
+    while (true) {
+      mbar_wait(&full[sn], pn & 1);
+      const int item = stage_item[sn];
+      if (item < 0) {
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&empty[sn]);
+        break;
+      }
+      named_bar_sync(1, NCONS);     // previous item's readers are done with the X_{t+1} ring
+      const int chunk = item / ntile, tile = item % ntile;
+      const int x0 = (tile % ntx) * T2_TXO, y0 = (tile / ntx) * T2_TYO;
+      const int64_t zs = p.reg0 + (int64_t)chunk * zc;
+      const int nzc = (int)(min(zs + (int64_t)zc, p.reg1) - zs);
+      const int xo = x0 - 4 + 4 * lane;                 // this lane's X_{t+1} / output columns
+      const bool pl = xo == 0, pr = xo + 4 == nx;       // x-halo out of grid for this lane
+      // X rows (box origin y0-2) and X_{t+1} rows (tile origin y0-1) of this
+      // warp's two rows, with the pad redirect folded into the row offsets
+      int xm[2], xq[2], ym_[2], yq[2];
+#pragma unroll
+      for (int jj = 0; jj < 2; ++jj) {
+        const int rr = warp * 2 + jj, gy = y0 - 1 + rr;
+        xm[jj] = -BX4;
+        xq[jj] = BX4;
+        if (gy - 1 < 0) xm[jj] = (min(max((int)pad_remap(gy - 1, ny, ky) - (y0 - 2), 0), T2_BY - 1) - (rr + 1)) * BX4;
+        if (gy + 1 >= ny) xq[jj] = (min(max((int)pad_remap(gy + 1, ny, ky) - (y0 - 2), 0), T2_BY - 1) - (rr + 1)) * BX4;
+        ym_[jj] = -TX4;
+        yq[jj] = TX4;
+        if (gy - 1 < 0) ym_[jj] = (min(max((int)pad_remap(gy - 1, ny, ky) - (y0 - 1), 0), T2_TY - 1) - rr) * TX4;
+        if (gy + 1 >= ny) yq[jj] = (min(max((int)pad_remap(gy + 1, ny, ky) - (y0 - 1), 0), T2_TY - 1) - rr) * TX4;
+        if (rr == 0) ym_[jj] = 0;                  // rows 0 and 15 produce no output: stay in the slot
+        if (rr == T2_TY - 1) yq[jj] = 0;
+      }
+      int xst[3];                // stages of X planes yz-1, yz, yz+1
+      int yslot[3];              // X_{t+1} ring slots of planes oz-1, oz, oz+1
+      // warm-up: X planes zs-2, zs-1
+      for (int k = 0; k < 2; ++k) {
+        if (k > 0) mbar_wait(&full[sn], pn & 1);
+        xst[k] = sn;
+        if (++sn == S) { sn = 0; ++pn; }
+      }
+      // Y plane i (global zs-1+i) lives in slot i & 3; remember which are real
+      int yreal[3] = {-1, -1, -1};
+      for (int i = 0; i < nzc + 2; ++i) {
+        const int yz = (int)(p.z_off + zs) - 1 + i;     // global plane of X_{t+1}
+        mbar_wait(&full[sn], pn & 1);
+        xst[2] = sn;
+        if (++sn == S) { sn = 0; ++pn; }
+        const int ys = i & 3;
+        const bool inside = yz >= 0 && yz < gnz;
+        if (inside) {
+          // ---- step 1: X_{t+1} plane yz on the extended tile ----
+#pragma unroll
+          for (int jj = 0; jj < 2; ++jj) {
+            const int rr = warp * 2 + jj;
+            const int rb = (rr + 1) * BX4 + 1 + lane;    // X box row of y, centre float4 of the lane
+            const int cb = xst[1] * SF4;
+            const float4 c = dsm4[cb + rb];
+            const float4 e = dsm4[cb + (rr + 1) * BX4 + (lane == 0 ? 0 : (TX + XH) / 4)];
+            float l = __shfl_up_sync(FULL, c.w, 1);
+            float r = __shfl_down_sync(FULL, c.x, 1);
+            if (lane == 0) l = e.w;
+            if (lane == 31) r = e.x;
+            if (pl) l = pick4(rsx, c, 0.0f);
+            if (pr) r = pick4(rex, c, 0.0f);
+            Win<1> w;
+            w.x[0] = l; w.x[1] = c.x; w.x[2] = c.y; w.x[3] = c.z; w.x[4] = c.w; w.x[5] = r;
+            set4(w.ym[0], dsm4[cb + rb + xm[jj]]);
+            set4(w.yp[0], dsm4[cb + rb + xq[jj]]);
+            set4(w.zm[0], dsm4[xst[0] * SF4 + rb]);
+            set4(w.zp[0], dsm4[xst[2] * SF4 + rb]);
+            const float4 pw = make_float4(0.f, 0.f, 0.f, 0.f);
+            float4 v;
+            v.x = eval<K2_WSTAR, 1, 0>(p, w, pw, 0, 0, 0);
+            v.y = eval<K2_WSTAR, 1, 1>(p, w, pw, 0, 0, 0);
+            v.z = eval<K2_WSTAR, 1, 2>(p, w, pw, 0, 0, 0);
+            v.w = eval<K2_WSTAR, 1, 3>(p, w, pw, 0, 0, 0);
+            ysm[ys * T2_YF4 + rr * TX4 + lane] = v;
+          }
+        }
+        // X plane yz-1 is done
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&empty[xst[0]]);
+        xst[0] = xst[1];
+        xst[1] = xst[2];
+        yreal[0] = yreal[1];
+        yreal[1] = yreal[2];
+        yreal[2] = inside ? ys : -1;
+        named_bar_sync(1, NCONS);
+        if (i < 2) continue;
+        // ---- step 2: X_{t+2} plane oz = yz - 1 from X_{t+1} planes oz-1..oz+1 ----
+        const int oz = yz - 1;
+        // ring slots with the pad of X_{t+1} in z (a plane outside the grid
+        // aliases the remapped plane, which is one of the three)
+#pragma unroll
+        for (int k = 0; k < 3; ++k) {
+          const int gzk = oz - 1 + k;
+          int src = k;
+          if (gzk < 0 || gzk >= gnz) src = (int)pad_remap(gzk, gnz, kz) - (oz - 1);
+          yslot[k] = (src == 0 ? yreal[0] : (src == 1 ? yreal[1] : yreal[2]));
+        }
+        float* op = out + ((int64_t)(oz - p.z_off) + p.ghost) * p.plane;
+#pragma unroll
+        for (int jj = 0; jj < 2; ++jj) {
+          const int rr = warp * 2 + jj, gy = y0 - 1 + rr;
+          const int rb = rr * TX4 + lane;
+          const float4 c = ysm[yslot[1] * T2_YF4 + rb];
+          float l = __shfl_up_sync(FULL, c.w, 1);
+          float r = __shfl_down_sync(FULL, c.x, 1);
+          if (pl) l = pick4(rsx, c, 0.0f);
+          if (pr) r = pick4(rex, c, 0.0f);
+          Win<1> w;
+          w.x[0] = l; w.x[1] = c.x; w.x[2] = c.y; w.x[3] = c.z; w.x[4] = c.w; w.x[5] = r;
+          set4(w.ym[0], ysm[yslot[1] * T2_YF4 + rb + ym_[jj]]);
+          set4(w.yp[0], ysm[yslot[1] * T2_YF4 + rb + yq[jj]]);
+          set4(w.zm[0], ysm[yslot[0] * T2_YF4 + rb]);
+          set4(w.zp[0], ysm[yslot[2] * T2_YF4 + rb]);
+          const float4 pw = make_float4(0.f, 0.f, 0.f, 0.f);
+          float4 v;
+          v.x = eval<K2_WSTAR, 1, 0>(p, w, pw, 0, 0, 0);
+          v.y = eval<K2_WSTAR, 1, 1>(p, w, pw, 0, 0, 0);
+          v.z = eval<K2_WSTAR, 1, 2>(p, w, pw, 0, 0, 0);
+          v.w = eval<K2_WSTAR, 1, 3>(p, w, pw, 0, 0, 0);
+          const bool ok = lane >= 1 && lane <= 30 && rr >= 1 && rr <= T2_TYO && xo < nx && gy < ny;
+          if (ok) stg128(op + (int64_t)gy * nx + xo, v);
+        }
+      }
+      // the chunk's last two X planes are still held
+      __syncwarp();
+      if (lane == 0) {
+        mbar_arrive(&empty[xst[0]]);
+        mbar_arrive(&empty[xst[1]]);
+      }
+    }
+  }
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    __threadfence();
+    const unsigned prev = atomicAdd(&g_done[slot], 1u);
+    if (prev == gridDim.x - 1) {
+      g_ticket[slot] = 0;
+      g_done[slot] = 0;
+      __threadfence();
+    }
+  }
+}
+
+// ---------------------------------------------------------------------------
 // host side
 // ---------------------------------------------------------------------------
 bool star_weights(const StencilParams& p, int R) {
@@ -716,6 +955,56 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   int slot = (int)(g_slot.fetch_add(1) % kTickets);
   void* args[] = {(void*)&p, (void*)&map, (void*)&pwmap, (void*)&slid, (void*)&out,
                   &ntx_i, &nty_i, &zc_i, &nch_i, &slot};
+  return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
+}
+
+}  // namespace lift
+
+namespace lift {
+
+bool sweep3d_t2_supported(const StencilParams& p) {
+  if (p.op != OP_WEIGHTED || p.radius != 1 || !sweep3d_supported(p)) return false;
+  if (!star_weights(p, 1)) return false;
+  for (int d = 0; d < 3; ++d)
+    if (p.kind[d] != PAD_CLAMP && p.kind[d] != PAD_MIRROR && p.kind[d] != PAD_REFLECT) return false;
+  if (p.put_lo || p.put_hi || p.fused_step) return false;
+  if (p.slab && p.ghost < 2) return false;        // X_{t+1} of the planes next to the slab edge
+  return true;
+}
+
+cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* out, cudaStream_t stream, int num_sms,
+                              std::string* err) {
+  const int64_t nz_reg = p.reg1 - p.reg0;
+  if (nz_reg <= 0) return cudaSuccess;
+  constexpr int S = 5;
+  static Launcher L{};
+  static std::once_flag once;
+  std::call_once(once, [] {
+    auto fn = k2t_sweep<S>;
+    cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, CfgT2<S>::SMEM);
+    int occ = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, NCONS + 32, CfgT2<S>::SMEM) != cudaSuccess) occ = 1;
+    cudaGetLastError();
+    L = Launcher{reinterpret_cast<const void*>(fn), CfgT2<S>::SMEM, T2_TYO, occ > 0 ? occ : 1};
+  });
+  CUtensorMap map;
+  if (!get_map(in, p.n[2], p.n[1], p.n[0] + 2 * p.ghost, BX, T2_BY, &map, err)) return cudaErrorInvalidValue;
+  const int ntx = (int)((p.n[2] + T2_TXO - 1) / T2_TXO);
+  const int nty = (int)((p.n[1] + T2_TYO - 1) / T2_TYO);
+  const int64_t tiles = (int64_t)ntx * nty;
+  const int64_t slots = (int64_t)num_sms * L.ctas_per_sm;
+  const int64_t work = nz_reg * tiles;
+  int64_t zc = (work + 8 * slots - 1) / (8 * slots);
+  const int64_t zmin = std::min<int64_t>(16, std::max<int64_t>(2, (work + 2 * slots - 1) / (2 * slots)));
+  if (zc < zmin) zc = zmin;
+  if (zc > nz_reg) zc = nz_reg;
+  const int64_t nchunk = (nz_reg + zc - 1) / zc;
+  const int64_t items = tiles * nchunk;
+  if (items > 0x7fffffff) return cudaErrorInvalidConfiguration;
+  int64_t grid = slots < items ? slots : items;
+  int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk;
+  int slot = (int)(g_slot.fetch_add(1) % kTickets);
+  void* args[] = {(void*)&p, (void*)&map, (void*)&out, &ntx_i, &nty_i, &zc_i, &nch_i, &slot};
   return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
 }
 

@@ -84,6 +84,13 @@ class Plan:
     def set_variant(self, variant):
         L.stencil_plan_set_variant(self.handle, VARIANTS[variant] if isinstance(variant, str) else int(variant))
 
+    def set_time_block(self, steps: int):
+        L.stencil_plan_set_time_block(self.handle, steps)
+
+    @property
+    def time_block(self) -> int:
+        return L.stencil_plan_time_block(self.handle)
+
     @property
     def variant(self) -> int:
         return L.stencil_plan_variant(self.handle)

@@ -344,3 +344,34 @@ def test_poisson19_and_heat7(lift):
     check(lift, spec(x.shape, 3, si.weights_poisson19(), MIRROR), [x])
     _, plan = check(lift, spec(x.shape, 3, si.weights_heat7(), CLAMP), [x])
     assert plan.variant == 2
+
+
+# ------------------------------------------- temporal blocking (NEXT-3) ----
+@pytest.mark.parametrize("kind", [CLAMP, MIRROR, REFLECT])
+@pytest.mark.parametrize("shape", [(37, 70, 260), (3, 15, 124), (1, 14, 120), (2, 29, 244), (40, 8, 516)])
+def test_time_block2_bitwise_equal_single_steps(lift, kind, shape):
+    """Two steps per pass (K2T) give exactly the bits of single steps."""
+    x = rnd(shape, 60)
+    sp = spec(shape, 3, si.weights_j3d7(), kind)
+    res = {}
+    for tb in (1, 2):
+        plan = lift.Plan.from_spec(sp)
+        plan.set_time_block(tb)
+        assert plan.time_block == tb
+        a = torch.from_numpy(x).cuda()
+        b = torch.empty_like(a)
+        ri = plan.iterate([a, b], 7)
+        res[tb] = (a, b)[ri].cpu().numpy()
+    np.testing.assert_array_equal(res[2], res[1])
+    ref = orc.iterate(sp, [x], [], 7)[0]
+    assert np.max(np.abs(res[2] - ref) / np.abs(ref)) <= TOL10
+
+
+def test_time_block_eligibility(lift):
+    for sp_, exp in [(spec((64, 64, 128), 3, si.weights_j3d7()), 2),
+                     (spec((64, 64, 128), 3, si.weights_j3d7(), WRAP), 1),
+                     (spec((64, 64, 128), 5, si.weights_j3d13()), 1)]:
+        plan = lift.Plan.from_spec(sp_)
+        assert plan.time_block == 1          # default: one step per pass
+        plan.set_time_block(2)
+        assert plan.time_block == exp
