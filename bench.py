@@ -40,7 +40,8 @@ sys.path.insert(0, ROOT)
 METRIC = "stencil Gpoints/s & achieved HBM GB/s vs 8 TB/s at 1/2/4/8 B200"
 
 # algorithmic (compulsory) HBM bytes per output point per launch
-BYTES_PER_POINT = {0: 8, 1: 12, 2: 8, 3: 12, 4: 12, 5: 12, 6: 8}
+# SRAD (full iteration): the q0 reduction reads I (4 B) + the fused pass reads I, writes I' (8 B)
+BYTES_PER_POINT = {0: 8, 1: 12, 2: 8, 3: 12, 4: 12, 5: 12, 6: 8, 7: 12}
 KERNEL_NAME = {"j3d7_512_clamp": "k2_sweep", "acoustic7_1024": "k2_sweep", "acoustic13_1024": "k2_sweep",
                "hotspot3d_8x512x512": "k2_sweep", "gauss5_8192_mirror": "k1_tile", "j2d5_256_clamp": "k1_tile",
                "srad1_4096": "k1_tile", "srad2_4096": "k1_tile"}
@@ -219,7 +220,7 @@ def main():
     steps_per_iter = w.steps
     spec = w.spec
     ext1 = spec.extents
-    iterable = spec.op in (si.WEIGHTED, si.HOTSPOT3D, si.ACOUSTIC) and steps_per_iter > 1
+    iterable = spec.op in (si.WEIGHTED, si.HOTSPOT3D, si.ACOUSTIC, si.SRAD) and steps_per_iter > 1
     slabbed = (world > 1 or (args.force_slab and use_pg)) and iterable and len(ext1) == 3
 
     # ---- inputs: seeded synthetic grids resident in HBM (host copies kept for e2e)
@@ -274,6 +275,8 @@ def main():
         # slab + NCCL: boundary low, boundary high, interior per time step;
         # slab + fused: one launch per time step
         launches_per_step = steps_per_iter * (3 if (slabbed and args.halo == "nccl") else 1)
+        if op == si.SRAD:
+            launches_per_step = steps_per_iter * 3        # q0 partials, q0, fused SRAD1+SRAD2
     else:
         out = plan.empty_output()
         launches_per_step = 1
@@ -340,7 +343,10 @@ def main():
     # launches of it on one stream (single GPU), so avg launch = step time / launches
     bpp = BYTES_PER_POINT[op]
     if not slabbed:
-        avg_launch_s = (t_ms * 1e-3) / (args.steps * launches_per_step)
+        # the step is back-to-back launches of the dominant kernel on one stream
+        # (SRAD: one iteration = reduction + fused pass, counted as one unit)
+        units = args.steps * (steps_per_iter if op == si.SRAD else launches_per_step)
+        avg_launch_s = (t_ms * 1e-3) / units
         alg_bytes = npts_local * bpp
     else:
         # time the owned-slab sweep alone (all planes in one launch) on this rank

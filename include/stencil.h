@@ -74,9 +74,14 @@ typedef enum {
   STENCIL_OP_HOTSPOT2D = 5,  /* Rodinia hotspot (A26, Table 1): inputs {T
                                 (slid), P (point-wise)}; params {step/Cap, 1/Rx,
                                 1/Ry, 1/Rz, amb}; 2D, size 3                       */
-  STENCIL_OP_GRADIENT = 6    /* Rawat et al. 2D gradient (A25, Table 1):
+  STENCIL_OP_GRADIENT = 6,   /* Rawat et al. 2D gradient (A25, Table 1):
                                 I + 1/sqrt(eps + sum of squared differences to
                                 the 4 neighbours); params {eps}; 2D, size 3        */
+  STENCIL_OP_SRAD = 7        /* one full SRAD iteration (A27, NEXT-2): q0^2 =
+                                var/mean^2 of the input (fp64 reduction on the
+                                device), c = SRAD1, I' = SRAD2 fused in one pass;
+                                input {I}; params {lambda}; 2D, size 3, reindexing
+                                pads; the plan owns a small device workspace      */
 } stencil_op;
 
 /* Which kernel family executes a plan (stencil_plan_variant). */
@@ -210,7 +215,7 @@ stencil_status stencil_wait_signals(const uint32_t* sig_a, const uint32_t* sig_b
  * iterate(in, f, n_steps) with the state rotation of reading A21:
  *   WEIGHTED  : state {X0, X1}            X_{t+1} = S(X_t), ping-pong
  *   HOTSPOT3D, HOTSPOT2D : state {T0, T1}, aux {P}   T_{t+1} = S(T_t, P)
- *   GRADIENT  : state {X0, X1}            ping-pong like WEIGHTED
+ *   GRADIENT, SRAD : state {X0, X1}       ping-pong like WEIGHTED
  *   ACOUSTIC  : state {prev, cur}         next overwrites prev; roles swap
  * *result_index receives the index into ``state`` holding the newest grid.
  * Requires output extents == input extents.

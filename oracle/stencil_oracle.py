@@ -42,7 +42,7 @@ from typing import Callable, List, Sequence, Tuple
 import numpy as np
 
 CLAMP, MIRROR, WRAP, CONSTANT, REFLECT = 0, 1, 2, 3, 4
-WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC, HOTSPOT2D, GRADIENT = 0, 1, 2, 3, 4, 5, 6
+WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC, HOTSPOT2D, GRADIENT, SRAD = 0, 1, 2, 3, 4, 5, 6, 7
 
 
 # ---------------------------------------------------------------------------
@@ -234,6 +234,31 @@ def f_srad2(Wc: Callable, WI: Callable, prm: Sequence[float]) -> Tuple:
     return Y, A
 
 
+def srad_q0sqr(I: np.ndarray) -> float:
+    """q0^2 = var(I) / mean(I)^2 over the whole image, fp64 (reading A18/A27)."""
+    x = np.asarray(I, np.float64)
+    m = x.mean()
+    return float(x.var() / (m * m))
+
+
+def srad_iteration(spec, I: np.ndarray):
+    """One full SRAD iteration (reading A27, NEXT-2): q0^2 from the current
+    image, c = SRAD1(I; q0^2), I' = SRAD2(c, I; lambda).  The diffusion
+    coefficient c is a grid like any other: SRAD2 reads it through the same
+    pad/slide (P:525).  Returns (I', A)."""
+    q0 = srad_q0sqr(I)
+    c, _ = apply(_with(spec, SRAD1, (q0,)), [I])
+    return apply(_with(spec, SRAD2, (spec.params[0],)), [c, I])
+
+
+def _with(spec, op, params):
+    import copy
+    s = copy.copy(spec)
+    s.op = op
+    s.params = tuple(params)
+    return s
+
+
 def f_hotspot2d(WT: Callable, WP: Callable, prm: Sequence[float]) -> Tuple:
     """Rodinia v3.1 hotspot (2D) update (reading A26; PARITY UNPINNED formula):
     T' = T + sdc*(P + (S + N - 2T)/Ry + (E + W - 2T)/Rx + (amb - T)/Rz),
@@ -309,7 +334,7 @@ def f_acoustic(W: Callable, prev_c, K, r: int, prm: Sequence[float]) -> Tuple:
 def _check_op_shape(spec):
     if spec.op in (HOTSPOT3D, ACOUSTIC):
         assert spec.ndim == 3
-    if spec.op in (SRAD1, SRAD2, HOTSPOT2D, GRADIENT):
+    if spec.op in (SRAD1, SRAD2, HOTSPOT2D, GRADIENT, SRAD):
         assert spec.ndim == 2
     if spec.op != WEIGHTED:
         assert all(s == 1 for s in spec.step)
@@ -333,6 +358,8 @@ def apply(spec, inputs: Sequence[np.ndarray]):
         Y, A = f_srad1(tapper(pad(inputs[0])), spec.params)
     elif spec.op == SRAD2:
         Y, A = f_srad2(tapper(pad(inputs[0])), tapper(pad(inputs[1])), spec.params)
+    elif spec.op == SRAD:
+        Y, A = srad_iteration(spec, inputs[0])
     elif spec.op == HOTSPOT2D:
         Y, A = f_hotspot2d(tapper(pad(inputs[0])), tapper(pad(inputs[1])), spec.params)
     elif spec.op == GRADIENT:
@@ -398,7 +425,7 @@ def iterate(spec, state: Sequence[np.ndarray], aux: Sequence[np.ndarray], n_step
     before feeding it back (not used by the parity tests: the oracle keeps
     fp64 state)."""
     cvt = (lambda a: a.astype(np.float32).astype(np.float64)) if round_fp32 else (lambda a: a)
-    if spec.op in (WEIGHTED, HOTSPOT3D, HOTSPOT2D, GRADIENT):
+    if spec.op in (WEIGHTED, HOTSPOT3D, HOTSPOT2D, GRADIENT, SRAD):
         X = np.asarray(state[0], np.float64)
         for _ in range(n_steps):
             X, _A = apply(spec, [X] + list(aux))

@@ -13,6 +13,7 @@
 #include "../../include/stencil.h"
 #include "common.cuh"
 #include "launch.hpp"
+#include "ops.cuh"
 
 using namespace lift;
 
@@ -25,6 +26,8 @@ struct stencil_plan_s {
   int32_t forced_variant = STENCIL_VARIANT_AUTO;
   int32_t time_block = 1;          // stencil_iterate: time steps per pass where K2T applies (opt-in, see DESIGN)
   int32_t last_variant = STENCIL_VARIANT_GENERIC;
+  // OP_SRAD: device workspace {partials of the q0 reduction, q0 constants}
+  void* srad_ws = nullptr;
   // stencil_run_host workspace (device)
   std::vector<float*> ws;
   size_t ws_elems = 0;
@@ -67,6 +70,7 @@ int op_arity(int op) {
     case OP_ACOUSTIC: return 2;
     case OP_HOTSPOT2D: return 2;
     case OP_GRADIENT: return 1;
+    case OP_SRAD: return 1;
     default: return -1;
   }
 }
@@ -81,6 +85,7 @@ int slid_mask(int op) {
     case OP_ACOUSTIC: return 2;       // prev point-wise, cur slid
     case OP_HOTSPOT2D: return 1;      // T slid, P point-wise
     case OP_GRADIENT: return 1;
+    case OP_SRAD: return 1;
     default: return 0;
   }
 }
@@ -106,8 +111,19 @@ int choose_variant(stencil_plan_s* pl, const float* in0, const float* in1, const
   return STENCIL_VARIANT_GENERIC;
 }
 
-stencil_status launch(stencil_plan_s* pl, const StencilParams& p, const float* in0, const float* in1,
+stencil_status launch(stencil_plan_s* pl, const StencilParams& p_in, const float* in0, const float* in1,
                       float* out, cudaStream_t stream) {
+  StencilParams p = p_in;
+  if (p.op == OP_SRAD) {
+    // q0^2 of the current image first (deterministic two-pass fp64 reduction)
+    if (!pl->srad_ws) {
+      cudaError_t e = cudaMalloc(&pl->srad_ws, srad_workspace_bytes(pl->num_sms));
+      if (e != cudaSuccess) return cuda_fail(e, "cudaMalloc (SRAD workspace)");
+    }
+    cudaError_t e = launch_srad_q0(in0, p.n[1] * p.n[2], pl->srad_ws, pl->num_sms, stream);
+    if (e != cudaSuccess) return cuda_fail(e, "SRAD q0 reduction");
+    p.srad_q0 = srad_q0_ptr(pl->srad_ws, pl->num_sms);
+  }
   const int v = choose_variant(pl, in0, in1, out);
   if (v < 0) return fail(STENCIL_E_UNSUPPORTED, "forced kernel variant cannot run this plan/pointers");
   pl->last_variant = v;
@@ -175,7 +191,7 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
   if (ndim < 1) return fail(STENCIL_E_INVALID, "ndim must be 1, 2 or 3");
   if (!extents || !size || !step || !pad_lo || !pad_hi || !kind)
     return fail(STENCIL_E_INVALID, "NULL array argument");
-  if (op < 0 || op > OP_GRADIENT) return fail(STENCIL_E_INVALID, "unknown op");
+  if (op < 0 || op > OP_SRAD) return fail(STENCIL_E_INVALID, "unknown op");
   if (n_params < 0 || n_params > kMaxParams || (n_params > 0 && !params))
     return fail(STENCIL_E_INVALID, "bad params");
 
@@ -292,15 +308,20 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
       if (n_params < 1) return fail(STENCIL_E_INVALID, "SRAD needs 1 param");
       if (op == OP_SRAD1) {
         if (!(params[0] > 0.0f)) return fail(STENCIL_E_INVALID, "SRAD1 needs q0sqr > 0");
-        const double q0 = params[0];                       // derived plan constants (A18b)
-        p.prm[1] = (float)(q0 / (1.0 + q0));
-        p.prm[2] = (float)(1.0 / (q0 * (1.0 + q0)));
+        srad1_constants(params[0], p.prm);                // derived plan constants (A18b)
       }
       p.radius = 1;
       break;
     case OP_HOTSPOT2D:
       if (ndim != 2 || !centred(1)) return fail(STENCIL_E_INVALID, "HOTSPOT2D needs ndim 2, size 3, pad 1, step 1");
       if (n_params < 5) return fail(STENCIL_E_INVALID, "HOTSPOT2D needs 5 params");
+      p.radius = 1;
+      break;
+    case OP_SRAD:
+      if (ndim != 2 || !centred(1)) return fail(STENCIL_E_INVALID, "SRAD needs ndim 2, size 3, pad 1, step 1");
+      if (n_params < 1) return fail(STENCIL_E_INVALID, "SRAD needs 1 param (lambda)");
+      if (kind[0] == PAD_CONSTANT || kind[1] == PAD_CONSTANT)
+        return fail(STENCIL_E_UNSUPPORTED, "SRAD iteration is built for reindexing pads");
       p.radius = 1;
       break;
     case OP_GRADIENT:
@@ -480,8 +501,8 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
   if (!state || n_state != 2) return fail(STENCIL_E_INVALID, "iterate needs 2 state buffers");
   if (!state[0] || !state[1] || state[0] == state[1]) return fail(STENCIL_E_INVALID, "bad state buffers");
   int ri = (p.op == OP_ACOUSTIC) ? 1 : 0;
-  if (p.op == OP_WEIGHTED || p.op == OP_GRADIENT) {
-    if (n_aux != 0) return fail(STENCIL_E_INVALID, "WEIGHTED/GRADIENT iterate takes no aux grids");
+  if (p.op == OP_WEIGHTED || p.op == OP_GRADIENT || p.op == OP_SRAD) {
+    if (n_aux != 0) return fail(STENCIL_E_INVALID, "WEIGHTED/GRADIENT/SRAD iterate takes no aux grids");
     int t = 0;
     // temporal blocking: two steps per pass (K2T) while at least two remain
     if (pl->time_block >= 2 && n_steps >= 2 && sweep3d_t2_supported(p) &&
@@ -565,7 +586,7 @@ stencil_status stencil_run_host(stencil_plan pl, const float* const* host_state,
   }
   const float* result = nullptr;
   const bool iterable = (p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D || p.op == OP_ACOUSTIC ||
-                         p.op == OP_HOTSPOT2D || p.op == OP_GRADIENT) && same_extents(p);
+                         p.op == OP_HOTSPOT2D || p.op == OP_GRADIENT || p.op == OP_SRAD) && same_extents(p);
   if (iterable && (p.op != OP_ACOUSTIC || n_state == 2)) {
     // WEIGHTED/HOTSPOT3D: state {X, scratch}; ACOUSTIC: state {prev, cur}
     float* state[2] = {pl->ws[0], pl->ws[1]};
@@ -591,9 +612,10 @@ stencil_status stencil_run_host(stencil_plan pl, const float* const* host_state,
 
 void stencil_plan_destroy(stencil_plan pl) {
   if (!pl) return;
-  if (!pl->ws.empty()) {
+  if (!pl->ws.empty() || pl->srad_ws) {
     DeviceGuard g(pl->device);
     for (float* b : pl->ws) cudaFree(b);
+    if (pl->srad_ws) cudaFree(pl->srad_ws);
   }
   delete pl;
 }

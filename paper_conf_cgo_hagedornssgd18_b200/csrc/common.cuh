@@ -12,7 +12,8 @@ namespace lift {
 
 enum PadKind : int { PAD_CLAMP = 0, PAD_MIRROR = 1, PAD_WRAP = 2, PAD_CONSTANT = 3, PAD_REFLECT = 4 };
 enum OpKind : int {
-  OP_WEIGHTED = 0, OP_HOTSPOT3D = 1, OP_SRAD1 = 2, OP_SRAD2 = 3, OP_ACOUSTIC = 4, OP_HOTSPOT2D = 5, OP_GRADIENT = 6
+  OP_WEIGHTED = 0, OP_HOTSPOT3D = 1, OP_SRAD1 = 2, OP_SRAD2 = 3, OP_ACOUSTIC = 4, OP_HOTSPOT2D = 5, OP_GRADIENT = 6,
+  OP_SRAD = 7
 };
 
 constexpr int kMaxTaps = 125;     // 5x5x5
@@ -62,6 +63,9 @@ struct StencilParams {
   // z-chunk) the producer waits until *wait_lo / *wait_hi >= wait_value
   // (acquire, system scope); the boundary chunks are scheduled first and the
   // neighbours' flags are raised as soon as their chunk is complete
+  // OP_SRAD (full iteration): device array {q0sqr, a, b} written by the q0
+  // reduction before the stencil launch (SRAD1's constants, op_srad1)
+  const float* srad_q0;
   const unsigned int* wait_lo;
   const unsigned int* wait_hi;
   unsigned int wait_value;

@@ -52,6 +52,21 @@ struct CentredAcc {
   }
 };
 
+// OP_SRAD: the diffusion coefficient c = SRAD1(I) at the padded position
+// (oy + DY, ox + DX) — c is read through the plan's pad like any grid (A27)
+struct SradCAcc {
+  const StencilParams& p;
+  const float* __restrict__ in;
+  Geo g;
+  template <int DZ, int DY, int DX>
+  __device__ __forceinline__ float at() const {
+    int64_t cy = g.oy + DY, cx = g.ox + DX;
+    if (cy < 0 || cy >= p.n[1]) cy = pad_remap(cy, p.n[1], p.kind[1]);
+    if (cx < 0 || cx >= p.n[2]) cx = pad_remap(cx, p.n[2], p.kind[2]);
+    return op_srad1(CentredAcc{p, in, Geo{g.oz, cy, cx}}, p.srad_q0);
+  }
+};
+
 __global__ void __launch_bounds__(256) k0_generic(const __grid_constant__ StencilParams p,
                                                   const float* __restrict__ in0,
                                                   const float* __restrict__ in1,
@@ -115,6 +130,9 @@ __global__ void __launch_bounds__(256) k0_generic(const __grid_constant__ Stenci
         break;
       case OP_GRADIENT:
         v = op_gradient(CentredAcc{p, in0, g}, p.prm);
+        break;
+      case OP_SRAD:
+        v = op_srad2(SradCAcc{p, in0, g}, CentredAcc{p, in0, g}, p.prm);
         break;
       case OP_ACOUSTIC: {
         // inputs: in0 = prev (point-wise), in1 = cur (slid)

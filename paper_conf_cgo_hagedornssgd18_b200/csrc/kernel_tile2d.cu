@@ -21,6 +21,7 @@
 #include <cuda_runtime.h>
 
 #include <cstdlib>
+#include <climits>
 #include <mutex>
 #include <string>
 
@@ -252,6 +253,150 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
   }
 }
 
+// ---------------------------------------------------------------------------
+// K1S: one full SRAD iteration fused into one tile pass:
+// I' = SRAD2(c, I) with c = SRAD1(I) computed on the fly for the tile's rows
+// plus one row below and one column to the right (the S and E taps of
+// SRAD2), never stored.  The I box is (128+8) x (TY+4) at (x0-4, y0-2); each
+// warp keeps 4 I x-windows and 3 c rows in registers while sweeping its rows.
+// c is a grid read through the same pad as I: out-of-grid c rows/columns
+// take the value at the remapped position.  Every value goes through
+// op_srad1 / op_srad2, so the result equals SRAD1 then SRAD2 bit for bit.
+// ---------------------------------------------------------------------------
+template <int RX, int I>
+struct RowsAcc {                 // rows[0..2] = I rows y-1, y, y+1 (x-windows with offsets -RX..)
+  const float* r0;
+  const float* r1;
+  const float* r2;
+  template <int DZ, int DY, int DX>
+  __device__ __forceinline__ float at() const {
+    static_assert(DZ == 0, "2D");
+    return DY < 0 ? r0[I + RX + DX] : (DY > 0 ? r2[I + RX + DX] : r1[I + RX + DX]);
+  }
+};
+
+template <int I>
+struct CRowsAcc {                // c at (y, x+i) = cy[i], (y+1, x+i) = cs[i]
+  const float* cy;
+  const float* cs;
+  template <int DZ, int DY, int DX>
+  __device__ __forceinline__ float at() const {
+    static_assert(DZ == 0 && DY >= 0 && DX >= 0, "SRAD2 reads c at C, S, E");
+    return DY > 0 ? cs[I + DX] : cy[I + DX];
+  }
+};
+
+template <int RPW, int S>
+__global__ void __launch_bounds__(NCONS + 32, 3)
+    k1_srad_fused(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap map0,
+                  const float* __restrict__ src0, float* __restrict__ out, int ntx, int nty) {
+  using C = Cfg<2, RPW, S, 1>;
+  constexpr int TY = C::TY;
+  constexpr int W = 8;            // x-window offsets -2 .. +5
+  constexpr int BX4 = BX / 4;
+  constexpr int SF4 = C::STAGE_FLOATS / 4;
+  extern __shared__ __align__(128) float4 dsm4[];
+  uint64_t* full = reinterpret_cast<uint64_t*>(dsm4 + S * SF4);
+  uint64_t* empty = full + S;
+  const int64_t ntiles = (int64_t)ntx * nty;
+  const int nt = (int)((ntiles - blockIdx.x + gridDim.x - 1) / gridDim.x);
+  if (nt <= 0) return;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  if (threadIdx.x == 0) {
+    for (int s = 0; s < S; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NW);
+    }
+    fence_mbar_init();
+  }
+  __syncthreads();
+  if (warp == NW) {
+    if (lane == 0) {
+      prefetch_tmap(&map0);
+      int s = 0;
+      uint32_t pass = 0;
+      for (int i = 0; i < nt; ++i) {
+        if (pass > 0) mbar_wait(&empty[s], (pass - 1) & 1);
+        const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
+        const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
+        mbar_arrive_expect_tx(&full[s], C::BOX_BYTES);
+        tma_load_3d(dsm4 + s * SF4, &map0, &full[s], x0 - XH, y0 - 2, 0);
+        if (++s == S) { s = 0; ++pass; }
+      }
+    }
+    return;
+  }
+  const int nx = (int)p.n[2], ny = (int)p.n[1];
+  const int kx = p.kind[2], ky = p.kind[1];
+  const float* q = p.srad_q0;
+  const int r0 = warp * RPW;
+  int s = 0;
+  uint32_t pass = 0;
+  for (int it = 0; it < nt; ++it) {
+    mbar_wait(&full[s], pass & 1);
+    const int64_t t = blockIdx.x + (int64_t)it * gridDim.x;
+    const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
+    const bool edge = (x0 == 0) || (x0 + TX + 2 > nx) || (y0 < 2) || (y0 + TY + 2 > ny);
+    if (edge) {
+      fixup_tile<2, 2, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + s * SF4), src0, 0, x0, y0,
+                                             threadIdx.x);
+      fence_proxy_async_smem();
+      named_bar_sync(1, NCONS);
+    }
+    const int xo = x0 + 4 * lane;
+    const bool x_ok = xo < nx;
+    // c column x+4 at the right grid edge takes the remapped column's value
+    const int ce = (xo + 4 == nx) ? (int)(pad_remap(nx, nx, kx) - xo) : 4;
+    const float4* box = dsm4 + s * SF4;
+    float iw[4][W];
+    float cr[3][5];
+    float* orow = out + ((int64_t)(y0 + r0) * nx + xo);
+    // box rows r0+1 .. r0+RPW+3  <->  I rows y0+r0-1 .. y0+r0+RPW+1
+    static_for<RPW + 3>([&](auto K) {
+      constexpr int k = decltype(K)::value;
+      load_row<2>(box + (r0 + 1 + k) * BX4, lane, iw[k % 4]);
+      if constexpr (k >= 2) {
+        // c for I row crow = y0 + r0 + k - 2 from I rows crow-1 .. crow+1
+        constexpr int cs_ = (k - 2) % 3;
+        const int crow = y0 + r0 + k - 2;
+        if (crow < ny) {
+          static_for<5>([&](auto II) {
+            constexpr int ii = decltype(II)::value;
+            cr[cs_][ii] = op_srad1(RowsAcc<2, ii>{iw[(k - 2) % 4], iw[(k - 1) % 4], iw[k % 4]}, q);
+          });
+          cr[cs_][4] = ce == 4 ? cr[cs_][4] : (ce == 3 ? cr[cs_][3] : (ce == 2 ? cr[cs_][2] : cr[cs_][1]));
+        } else if constexpr (k >= 3) {
+          // c row outside the grid: the remapped row (one or two above)
+          const int d = crow - (int)pad_remap(crow, ny, ky);
+#pragma unroll
+          for (int ii = 0; ii < 5; ++ii) {
+            if constexpr (k >= 4)
+              cr[cs_][ii] = d == 1 ? cr[(k - 3) % 3][ii] : cr[(k - 4) % 3][ii];
+            else
+              cr[cs_][ii] = cr[(k - 3) % 3][ii];
+          }
+        }
+      }
+      if constexpr (k >= 3) {
+        // output row o = k - 3 (I row y0 + r0 + o)
+        constexpr int o = k - 3;
+        if constexpr (o < RPW) {
+          float v[4];
+          static_for<4>([&](auto II) {
+            constexpr int ii = decltype(II)::value;
+            v[ii] = op_srad2(CRowsAcc<ii>{cr[o % 3], cr[(o + 1) % 3]},
+                             RowsAcc<2, ii>{iw[o % 4], iw[(o + 1) % 4], iw[(o + 2) % 4]}, p.prm);
+          });
+          if (x_ok && y0 + r0 + o < ny) stg128(orow + (int64_t)o * nx, make_float4(v[0], v[1], v[2], v[3]));
+        }
+      }
+    });
+    __syncwarp();
+    if (lane == 0) mbar_arrive(&empty[s]);
+    if (++s == S) { s = 0; ++pass; }
+  }
+}
+
 struct Launcher {
   const void* fn;
   int smem;
@@ -351,6 +496,30 @@ bool get_map(const float* base, int64_t nx, int64_t ny, int by, CUtensorMap* out
 
 }  // namespace
 
+cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* out, cudaStream_t stream,
+                              int num_sms, std::string* err) {
+  constexpr int RPW = 6, S = 2;
+  using C = Cfg<2, RPW, S, 1>;
+  static Launcher L{};
+  static std::once_flag once;
+  std::call_once(once, [] {
+    auto fn = k1_srad_fused<RPW, S>;
+    cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
+    int occ = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, NCONS + 32, C::SMEM) != cudaSuccess) occ = 1;
+    cudaGetLastError();
+    L = Launcher{reinterpret_cast<const void*>(fn), C::SMEM, C::TY, 2, 1, occ > 0 ? occ : 1};
+  });
+  CUtensorMap m0;
+  if (!get_map(in0, p.n[2], p.n[1], L.ty + 4, &m0, err)) return cudaErrorInvalidValue;
+  const int ntx = (int)((p.n[2] + TX - 1) / TX);
+  const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);
+  int64_t grid = (int64_t)num_sms * L.ctas_per_sm;
+  if (grid > (int64_t)ntx * nty) grid = (int64_t)ntx * nty;
+  void* args[] = {(void*)&p, (void*)&m0, (void*)&in0, (void*)&out, (void*)&ntx, (void*)&nty};
+  return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
+}
+
 bool tile2d_supported(const StencilParams& p) {
   // canonical 2D plan: dimension 0 is the dummy (extent 1, size 1, no pad)
   if (p.n[0] != 1 || p.size[0] != 1 || p.lo[0] != 0 || p.hi[0] != 0 || p.slab) return false;
@@ -358,7 +527,7 @@ bool tile2d_supported(const StencilParams& p) {
   for (int d = 1; d < 3; ++d)
     if (p.step[d] != 1 || p.hi[d] != p.lo[d] || p.size[d] != 2 * p.lo[d] + 1) return false;
   if (ry < 1 || ry > 2 || rx < 1 || rx > 2) return false;
-  if (p.op == OP_SRAD1 || p.op == OP_SRAD2 || p.op == OP_HOTSPOT2D || p.op == OP_GRADIENT) {
+  if (p.op == OP_SRAD1 || p.op == OP_SRAD2 || p.op == OP_HOTSPOT2D || p.op == OP_GRADIENT || p.op == OP_SRAD) {
     if (ry != 1 || rx != 1) return false;
   } else if (p.op != OP_WEIGHTED) {
     return false;
@@ -370,6 +539,7 @@ bool tile2d_supported(const StencilParams& p) {
 
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,
                           cudaStream_t stream, int num_sms, std::string* err) {
+  if (p.op == OP_SRAD) return launch_srad_fused(p, in0, out, stream, num_sms, err);
   Launcher L;
   if (!pick(p, &L)) {
     *err = "tile2d: no instantiation";

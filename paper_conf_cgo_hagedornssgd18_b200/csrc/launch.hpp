@@ -34,6 +34,12 @@ bool tile2d_supported(const StencilParams& p);
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,
                           cudaStream_t stream, int num_sms, std::string* err);
 
+// OP_SRAD: q0^2 = var/mean^2 of the image (fp64, deterministic) into the
+// workspace, as SRAD1's constants {q0, a, b}
+size_t srad_workspace_bytes(int num_sms);
+const float* srad_q0_ptr(void* ws, int num_sms);
+cudaError_t launch_srad_q0(const float* img, int64_t n, void* ws, int num_sms, cudaStream_t stream);
+
 // wait (one thread, acquire.sys) until *a >= value and *b >= value (NULL = skip)
 cudaError_t launch_wait_signals(const unsigned int* a, const unsigned int* b, unsigned int value,
                                 cudaStream_t stream);

@@ -92,6 +92,14 @@ __device__ __forceinline__ float op_srad1(const Acc& I, const float* prm) {
   return c;
 }
 
+// SRAD1's constants {q0, a, b} from q0 (the same derivation as the plan's)
+__host__ __device__ inline void srad1_constants(float q0f, float* out3) {
+  const double q0 = q0f;
+  out3[0] = q0f;
+  out3[1] = (float)(q0 / (1.0 + q0));
+  out3[2] = (float)(1.0 / (q0 * (1.0 + q0)));
+}
+
 // ---- SRAD kernel 2: (c, I) -> I' (Rodinia v3.1 srad; A18) --------
 template <class AccC, class AccI>
 __device__ __forceinline__ float op_srad2(const AccC& C, const AccI& I, const float* prm) {

@@ -18,7 +18,8 @@ from . import _lib as L
 KINDS = {"clamp": L.PAD_CLAMP, "mirror": L.PAD_MIRROR, "symmetric": L.PAD_MIRROR, "wrap": L.PAD_WRAP,
          "constant": L.PAD_CONSTANT, "zero": L.PAD_CONSTANT, "reflect": L.PAD_REFLECT}
 OPS = {"weighted": L.OP_WEIGHTED, "hotspot3d": L.OP_HOTSPOT3D, "srad1": L.OP_SRAD1, "srad2": L.OP_SRAD2,
-       "acoustic": L.OP_ACOUSTIC, "hotspot2d": L.OP_HOTSPOT2D, "gradient": L.OP_GRADIENT}
+       "acoustic": L.OP_ACOUSTIC, "hotspot2d": L.OP_HOTSPOT2D, "gradient": L.OP_GRADIENT,
+       "srad": L.OP_SRAD}
 VARIANTS = {"auto": L.VARIANT_AUTO, "generic": L.VARIANT_GENERIC, "tile2d": L.VARIANT_TILE2D,
             "sweep3d": L.VARIANT_SWEEP3D}
 

@@ -28,12 +28,13 @@ KIND_NAMES = {CLAMP: "clamp", MIRROR: "mirror", WRAP: "wrap",
               CONSTANT: "constant", REFLECT: "reflect"}
 
 # Ops — numeric values are the C-ABI enum ``stencil_op``.
-WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC, HOTSPOT2D, GRADIENT = 0, 1, 2, 3, 4, 5, 6
+WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC, HOTSPOT2D, GRADIENT, SRAD = 0, 1, 2, 3, 4, 5, 6, 7
 OP_NAMES = {WEIGHTED: "weighted", HOTSPOT3D: "hotspot3d", SRAD1: "srad1",
-            SRAD2: "srad2", ACOUSTIC: "acoustic", HOTSPOT2D: "hotspot2d", GRADIENT: "gradient"}
+            SRAD2: "srad2", ACOUSTIC: "acoustic", HOTSPOT2D: "hotspot2d", GRADIENT: "gradient",
+            SRAD: "srad"}
 
 # Number of input grids per op (zip arity).
-N_INPUTS = {WEIGHTED: 1, HOTSPOT3D: 2, SRAD1: 1, SRAD2: 2, ACOUSTIC: 2, HOTSPOT2D: 2, GRADIENT: 1}
+N_INPUTS = {WEIGHTED: 1, HOTSPOT3D: 2, SRAD1: 1, SRAD2: 2, ACOUSTIC: 2, HOTSPOT2D: 2, GRADIENT: 1, SRAD: 1}
 
 
 @dataclass
@@ -352,6 +353,13 @@ _WORKLOADS = {
     "acoustic13_1024": _c5b,
 }
 
+def _srad_iter():
+    return Workload("srad_iter_4096", _spec((4096, 4096), 3, op=SRAD, params=params_srad2()), (1006,), ((0.0, 1.0),),
+                    20, transform=("exp",),
+                    note="NEXT-2: full SRAD iterations (q0 reduction + fused SRAD1/SRAD2), clamp, 20 iterations")
+
+
+_WORKLOADS["srad_iter_4096"] = _srad_iter
 _WORKLOADS.update(_TABLE1)
 WORKLOAD_NAMES = tuple(_WORKLOADS)
 TABLE1_NAMES = tuple(_TABLE1)

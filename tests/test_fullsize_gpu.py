@@ -162,3 +162,16 @@ def test_table1_paper_sizes(lift, name):
     xs, spec = si.make_workload_inputs(w)
     y, plan = gpu_apply(lift, spec, xs)
     check_points(spec, xs, y, samples(spec.extents, 200, 16))
+
+
+def test_srad_iteration_4096(lift):
+    w = si.workload("srad_iter_4096")
+    xs, spec = si.make_workload_inputs(w)
+    y, plan = gpu_apply(lift, spec, xs)
+    assert plan.variant == 1
+    # the q0 statistic is global: compare sampled points with the oracle's full iteration
+    Y, A = orc.apply(spec, xs)
+    pts = samples(spec.extents, 2000, 17)
+    g = y.cpu().numpy()
+    err = max(abs(float(g[p]) - Y[p]) / max(abs(Y[p]), A[p]) for p in pts)
+    assert err <= 1e-5

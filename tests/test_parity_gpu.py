@@ -375,3 +375,23 @@ def test_time_block_eligibility(lift):
         assert plan.time_block == 1          # default: one step per pass
         plan.set_time_block(2)
         assert plan.time_block == exp
+
+
+# ---------------------------------------- full SRAD iteration (NEXT-2) -----
+@pytest.mark.parametrize("kind", [CLAMP, MIRROR, REFLECT])
+def test_srad_iteration(lift, kind):
+    """q0 reduction + SRAD1/SRAD2 fused in one pass (K1S) vs the oracle's
+    SRAD1-then-SRAD2 with q0 of the current image; K1S == K0 bitwise."""
+    I = np.exp(rnd((150, 388), 61, 0.0, 1.0)).astype(np.float32)
+    sp = spec(I.shape, 3, op=si.SRAD, params=si.params_srad2(), kind=kind)
+    y, plan = check(lift, sp, [I])
+    assert plan.variant == 1
+    y0, _ = run_gpu(lift, sp, [I], "generic")
+    np.testing.assert_array_equal(y, y0)
+    # 10 iterations
+    a = torch.from_numpy(I).cuda()
+    b = torch.empty_like(a)
+    ri = plan.iterate([a, b], 10)
+    g = (a, b)[ri].cpu().numpy()
+    ref = orc.iterate(sp, [I], [], 10)[0]
+    assert np.max(np.abs(g - ref) / np.abs(ref)) <= TOL10
