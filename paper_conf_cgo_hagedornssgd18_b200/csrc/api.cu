@@ -101,7 +101,8 @@ int choose_variant(stencil_plan_s* pl, const float* in0, const float* in1, const
   const bool ptr_ok = aligned16(in0) && (in1 == nullptr || aligned16(in1)) && aligned16(out);
   auto want = [&](int v) {
     if (v == STENCIL_VARIANT_SWEEP3D) return ptr_ok && sweep3d_supported(p);
-    if (v == STENCIL_VARIANT_TILE2D) return ptr_ok && tile2d_supported(p);
+    // K1 fills its tiles with cp.async when TMA cannot (unaligned / nx % 4 != 0)
+    if (v == STENCIL_VARIANT_TILE2D) return tile2d_supported(p) && (p.op != OP_SRAD || ptr_ok);
     return v == STENCIL_VARIANT_GENERIC;
   };
   if (pl->forced_variant != STENCIL_VARIANT_AUTO)

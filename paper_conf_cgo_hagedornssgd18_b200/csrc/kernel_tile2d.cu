@@ -85,7 +85,7 @@ struct RingAcc {
   }
 };
 
-template <int OP, int RY, int RX, int RPW, int S, int NIN, int MINB>
+template <int OP, int RY, int RX, int RPW, int S, int NIN, int MINB, bool LDG>
 __global__ void __launch_bounds__(NCONS + 32, MINB)
     k1_tile(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap map0,
             const __grid_constant__ CUtensorMap map1, const float* __restrict__ src0,
@@ -120,7 +120,7 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
   __syncthreads();
 
   if (warp == NW) {
-    if (lane == 0) {
+    if (!LDG && lane == 0) {
       prefetch_tmap(&map0);
       if (NIN > 1) prefetch_tmap(&map1);
       int s = 0;
@@ -141,12 +141,9 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
   const int nx = (int)p.n[2], ny = (int)p.n[1];
   const bool zero_fill_ok = p.pad_value == 0.0f && p.kind[1] == PAD_CONSTANT && p.kind[2] == PAD_CONSTANT;
   const int r0 = warp * RPW;   // first output row of this warp (tile-relative)
-  int s = 0;
-  uint32_t pass = 0;
-  for (int i = 0; i < nt; ++i) {
-    mbar_wait(&full[s], pass & 1);
-    const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
-    const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
+  // 128-bit stores need 16-B aligned rows (nx % 4 == 0 and an aligned base)
+  const bool vec = (nx % 4 == 0) && ((reinterpret_cast<uintptr_t>(out) & 15u) == 0);
+  auto fixup = [&](int s, int x0, int y0) {
     const bool edge = (x0 == 0) || (x0 + TX + RX > nx) || (y0 < RY) || (y0 + TY + RY > ny);
     if (edge && !zero_fill_ok) {
       fixup_tile<RY, RX, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + s * SF4), src0, 0, x0, y0,
@@ -157,12 +154,22 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
       fence_proxy_async_smem();
       named_bar_sync(1, NCONS);
     }
+  };
+  auto compute = [&](int s, int x0, int y0) {
     const int xo = x0 + 4 * lane;
     const bool x_ok = xo < nx;
     const float4* box0 = dsm4 + s * SF4 + r0 * BX4;     // box row r0 = output row r0 - RY
     float* orow = out + ((int64_t)(y0 + r0) * nx + xo);
     auto store = [&](int o, const float (&v)[4]) {
-      if (x_ok && y0 + r0 + o < ny) stg128(orow + (int64_t)o * nx, make_float4(v[0], v[1], v[2], v[3]));
+      if (!(x_ok && y0 + r0 + o < ny)) return;
+      float* dst = orow + (int64_t)o * nx;
+      if (vec) {
+        stg128(dst, make_float4(v[0], v[1], v[2], v[3]));
+      } else {
+#pragma unroll
+        for (int q = 0; q < 4; ++q)
+          if (xo + q < nx) dst[q] = v[q];
+      }
     };
 
     if constexpr (OP == K1_WBOX || OP == K1_WSTAR || OP == K1_WSEP) {
@@ -247,9 +254,56 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
         }
       });
     }
-    __syncwarp();
-    if (lane == 0) mbar_arrive(&empty[s]);
-    if (++s == S) { s = 0; ++pass; }
+  };
+
+  if constexpr (!LDG) {
+    int s = 0;
+    uint32_t pass = 0;
+    for (int i = 0; i < nt; ++i) {
+      mbar_wait(&full[s], pass & 1);
+      const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
+      const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
+      fixup(s, x0, y0);
+      compute(s, x0, y0);
+      __syncwarp();
+      if (lane == 0) mbar_arrive(&empty[s]);
+      if (++s == S) { s = 0; ++pass; }
+    }
+  } else {
+    // rows that TMA cannot describe (nx % 4 != 0 or an unaligned base): the
+    // consumers fill a double-buffered box with 4-byte cp.async copies
+    // (out-of-grid cells are zero, as TMA's fill) while computing the other
+    static_assert(S == 2, "LDG variant double-buffers");
+    auto fill = [&](int s, int64_t t) {
+      const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
+      float* base = reinterpret_cast<float*>(dsm4 + s * SF4);
+      for (int idx = threadIdx.x; idx < NIN * C::BY * BX; idx += NCONS) {
+        const int b = idx / (C::BY * BX), rem = idx % (C::BY * BX);
+        const int r = rem / BX, c = rem % BX;
+        const int gy = y0 - RY + r, gx = x0 - XH + c;
+        float* dst = base + b * C::BOX_FLOATS + r * BX + c;
+        if (gy >= 0 && gy < ny && gx >= 0 && gx < nx)
+          cp_async4(dst, (b == 0 ? src0 : src1) + (int64_t)gy * nx + gx);
+        else
+          *dst = 0.0f;
+      }
+      cp_async_commit();
+    };
+    fill(0, blockIdx.x);
+    for (int i = 0; i < nt; ++i) {
+      const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
+      if (i + 1 < nt) {
+        fill((i + 1) & 1, t + gridDim.x);
+        cp_async_wait<1>();
+      } else {
+        cp_async_wait<0>();
+      }
+      named_bar_sync(1, NCONS);
+      const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
+      fixup(i & 1, x0, y0);
+      compute(i & 1, x0, y0);
+      named_bar_sync(1, NCONS);       // the next fill reuses this stage
+    }
   }
 }
 
@@ -406,13 +460,13 @@ struct Launcher {
   int ctas_per_sm;
 };
 
-template <int OP, int RY, int RX, int RPW, int S, int NIN, int MINB = 3>
+template <int OP, int RY, int RX, int RPW, int S, int NIN, int MINB = 3, bool LDG = false>
 Launcher get_launcher() {
   static Launcher L{};
   static std::once_flag once;
   std::call_once(once, [] {
     using C = Cfg<RY, RPW, S, NIN>;
-    auto fn = k1_tile<OP, RY, RX, RPW, S, NIN, MINB>;
+    auto fn = k1_tile<OP, RY, RX, RPW, S, NIN, MINB, LDG>;
     cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
     int occ = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, NCONS + 32, C::SMEM) != cudaSuccess) occ = 1;
@@ -430,9 +484,10 @@ bool star2d(const StencilParams& p, int RY, int RX) {
   return true;
 }
 
-#define K1_PICK(OPV, RYV, RXV, NINV) get_launcher<OPV, RYV, RXV, 6, 2, NINV>()
+#define K1_PICK(OPV, RYV, RXV, NINV) \
+  (ldg ? get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, true>() : get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, false>())
 
-bool pick(const StencilParams& p, Launcher* L) {
+bool pick(const StencilParams& p, bool ldg, Launcher* L) {
   const int ry = p.lo[1], rx = p.lo[2];
   if (p.op == OP_WEIGHTED) {
     const int mode = p.sep ? K1_WSEP : (star2d(p, ry, rx) ? K1_WSTAR : K1_WBOX);
@@ -440,7 +495,7 @@ bool pick(const StencilParams& p, Launcher* L) {
     // selects alternative (rows per warp, stages, CTAs per SM) for the
     // separable radius-2 case; the default is the tuned one
     static const int tv = [] { const char* e = getenv("LIFT_K1_VARIANT"); return e ? atoi(e) : 0; }();
-    if (mode == K1_WSEP && ry == 2 && rx == 2 && tv != 0) {
+    if (mode == K1_WSEP && ry == 2 && rx == 2 && tv != 0 && !ldg) {
       switch (tv) {
         case 1: *L = get_launcher<K1_WSEP, 2, 2, 8, 2, 1, 3>(); return true;
         case 2: *L = get_launcher<K1_WSEP, 2, 2, 4, 2, 1, 4>(); return true;
@@ -532,25 +587,30 @@ bool tile2d_supported(const StencilParams& p) {
   } else if (p.op != OP_WEIGHTED) {
     return false;
   }
-  if (p.n[2] % 4 != 0) return false;
-  if (p.n[2] >= (1ll << 31) || p.n[1] >= (1ll << 31)) return false;
+  if (p.op == OP_SRAD && p.n[2] % 4 != 0) return false;   // the fused SRAD pass is TMA-only
+  if (p.n[2] * p.n[1] >= (1ll << 31)) return false;
   return true;
 }
 
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,
                           cudaStream_t stream, int num_sms, std::string* err) {
   if (p.op == OP_SRAD) return launch_srad_fused(p, in0, out, stream, num_sms, err);
+  // TMA needs 16-B aligned bases and row pitches; otherwise cp.async fills the box
+  const bool ldg = (p.n[2] % 4 != 0) || (reinterpret_cast<uintptr_t>(in0) & 15u) ||
+                   (in1 && (reinterpret_cast<uintptr_t>(in1) & 15u));
   Launcher L;
-  if (!pick(p, &L)) {
+  if (!pick(p, ldg, &L)) {
     *err = "tile2d: no instantiation";
     return cudaErrorNotSupported;
   }
-  CUtensorMap m0, m1;
-  if (!get_map(in0, p.n[2], p.n[1], L.ty + 2 * L.ry, &m0, err)) return cudaErrorInvalidValue;
-  if (L.nin > 1) {
-    if (!get_map(in1, p.n[2], p.n[1], L.ty + 2 * L.ry, &m1, err)) return cudaErrorInvalidValue;
-  } else {
-    m1 = m0;
+  CUtensorMap m0{}, m1{};
+  if (!ldg) {
+    if (!get_map(in0, p.n[2], p.n[1], L.ty + 2 * L.ry, &m0, err)) return cudaErrorInvalidValue;
+    if (L.nin > 1) {
+      if (!get_map(in1, p.n[2], p.n[1], L.ty + 2 * L.ry, &m1, err)) return cudaErrorInvalidValue;
+    } else {
+      m1 = m0;
+    }
   }
   const int ntx = (int)((p.n[2] + TX - 1) / TX);
   const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);

@@ -395,3 +395,63 @@ def test_srad_iteration(lift, kind):
     g = (a, b)[ri].cpu().numpy()
     ref = orc.iterate(sp, [I], [], 10)[0]
     assert np.max(np.abs(g - ref) / np.abs(ref)) <= TOL10
+
+
+def test_cuda_graph_capture_replay(lift):
+    """apply / iterate allocate nothing and are stream-ordered: captured into a
+    CUDA graph, replays give the same bits as eager calls (stencil.h)."""
+    x = rnd((24, 40, 136), 62)
+    sp = spec(x.shape, 3, si.weights_j3d7(), CLAMP)
+    plan = lift.Plan.from_spec(sp)
+    a = torch.from_numpy(x).cuda()
+    b = torch.empty_like(a)
+    c = torch.empty_like(a)
+    s = torch.cuda.Stream()
+    s.wait_stream(torch.cuda.current_stream())
+    with torch.cuda.stream(s):
+        plan.apply(a, out=b)                       # warm-up (TMA descriptors, function attributes)
+    torch.cuda.current_stream().wait_stream(s)
+    g = torch.cuda.CUDAGraph()
+    with torch.cuda.graph(g):
+        plan.apply(a, out=b)
+        plan.iterate([b, c], 4)
+    for _ in range(3):
+        g.replay()
+    torch.cuda.synchronize()
+    e1 = plan.apply(a)
+    e2 = torch.empty_like(a)
+    ri = plan.iterate([e1, e2], 4)
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal((b, c)[ri].cpu().numpy(), (e1, e2)[ri].cpu().numpy())
+
+
+# --------------------------- K1 with cp.async fill (nx % 4 != 0, unaligned) --
+@pytest.mark.parametrize("shape", [(67, 301), (45, 258), (50, 4098 // 8 + 1)])
+def test_tile2d_unaligned_widths(lift, shape):
+    x = rnd(shape, 63)
+    I = np.exp(rnd(shape, 64, 0, 1)).astype(np.float32)
+    cases = [(spec(shape, 3, si.weights_j2d5(), MIRROR), [x]),
+             (spec(shape, 5, si.weights_gauss5(), CLAMP), [x]),
+             (spec(shape, 3, si.weights_j2d9(), WRAP), [x]),
+             (spec(shape, 3, op=si.SRAD1, params=si.params_srad1(si.srad_q0sqr(I))), [I]),
+             (spec(shape, 3, op=si.HOTSPOT2D, params=si.params_hotspot2d(512, 512)), [x * 300, x * 1e-2]),
+             (spec(shape, 3, op=si.GRADIENT, params=si.params_gradient()), [x])]
+    for sp_, xs in cases:
+        y, plan = check(lift, sp_, xs)
+        assert plan.variant == 1, sp_
+        y0, _ = run_gpu(lift, sp_, xs, "generic")
+        np.testing.assert_array_equal(y, y0)
+
+
+def test_tile2d_unaligned_pointer(lift):
+    shape = (70, 264)
+    big = torch.from_numpy(rnd((70 * 264 + 1,), 65)).cuda()
+    xin = big[1:].view(*shape)                      # 4-byte aligned only
+    sp = spec(shape, 5, si.weights_gauss5(), MIRROR)
+    plan = lift.Plan.from_spec(sp)
+    out_big = torch.empty(70 * 264 + 3, device="cuda")
+    out = out_big[3:].view(*shape)
+    plan.apply(xin, out=out)
+    torch.cuda.synchronize()
+    Y, A = orc.apply(sp, [xin.cpu().numpy()])
+    assert orc.max_rel_err(out.cpu().numpy(), Y, A) <= TOL1
