@@ -42,10 +42,6 @@ METRIC = "stencil Gpoints/s & achieved HBM GB/s vs 8 TB/s at 1/2/4/8 B200"
 # algorithmic (compulsory) HBM bytes per output point per launch
 # SRAD (full iteration): the q0 reduction reads I (4 B) + the fused pass reads I, writes I' (8 B)
 BYTES_PER_POINT = {0: 8, 1: 12, 2: 8, 3: 12, 4: 12, 5: 12, 6: 8, 7: 12}
-KERNEL_NAME = {"j3d7_512_clamp": "k2_sweep", "acoustic7_1024": "k2_sweep", "acoustic13_1024": "k2_sweep",
-               "hotspot3d_8x512x512": "k2_sweep", "gauss5_8192_mirror": "k1_tile", "j2d5_256_clamp": "k1_tile",
-               "srad1_4096": "k1_tile", "srad2_4096": "k1_tile"}
-
 
 def env_int(k, d):
     try:

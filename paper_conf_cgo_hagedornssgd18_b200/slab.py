@@ -115,7 +115,7 @@ class SlabPlan:
     def __init__(self, global_extents: Sequence[int], rank: int, world: int, size=3, pad=None, kind="clamp",
                  pad_value: float = 0.0, op="weighted", weights=None, params=(), group=None,
                  device: Optional[int] = None, exchange=None, exchange_factory=None):
-        from .plan import Plan, KINDS, _kind
+        from .plan import Plan
         self.global_extents = tuple(int(e) for e in global_extents)
         self.rank, self.world = rank, world
         self.z0, self.z1 = partition(self.global_extents[0], world)[rank]

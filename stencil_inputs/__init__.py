@@ -17,8 +17,8 @@ Weights/constants are the readings A13, A14, A16, A18, A19, A20 of DESIGN.md
 """
 from __future__ import annotations
 
-from dataclasses import dataclass, field
-from typing import Dict, List, Optional, Sequence, Tuple
+from dataclasses import dataclass
+from typing import List, Optional, Sequence, Tuple
 
 import numpy as np
 
