@@ -255,6 +255,10 @@ def main():
         host = [torch.from_numpy(x).pin_memory() for x in xs]
         bufs = [x.to(dev, non_blocking=True) for x in host]
     torch.cuda.synchronize()
+    if use_pg:
+        # a collective first: NCCL point-to-point batches then run on an
+        # initialised communicator (torch's batch_isend_irecv requirement)
+        dist.barrier()
 
     # state/aux layout per op
     op = spec.op
