@@ -183,6 +183,9 @@ def main():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--no-graph", action="store_true", help="launch single sweeps eagerly instead of a CUDA graph")
+    ap.add_argument("--scaling", default="weak", choices=["weak", "strong"],
+                    help="multi-GPU iterated sweeps: weak = the single-GPU grid per rank (default), "
+                         "strong = the single-GPU grid split over the ranks")
     ap.add_argument("--force-slab", action="store_true",
                     help="run the slab (multi-GPU) path even at world size 1 (launch under torchrun)")
     ap.add_argument("--halo", default="nccl", choices=["nccl", "fused"],
@@ -222,10 +225,17 @@ def main():
     # ---- inputs: seeded synthetic grids resident in HBM (host copies kept for e2e)
     local_ext = ext1
     if slabbed:
-        # weak scaling: the per-rank slab is the single-GPU workload
-        gext = (ext1[0] * world,) + tuple(ext1[1:])
+        from paper_conf_cgo_hagedornssgd18_b200.slab import partition
         ws = si.workload(args.workload)
-        ws.spec.extents = ext1
+        if args.scaling == "weak":
+            # weak scaling: the per-rank slab is the single-GPU workload
+            gext = (ext1[0] * world,) + tuple(ext1[1:])
+            ws.spec.extents = ext1
+        else:
+            # strong scaling: the single-GPU grid is split over the ranks
+            gext = tuple(ext1)
+            z0, z1 = partition(ext1[0], world)[rank]
+            ws.spec.extents = (z1 - z0,) + tuple(ext1[1:])
         seeds = tuple(s + 7919 * rank for s in ws.seeds)
         ws.seeds = seeds
         xs, spec = si.make_workload_inputs(ws)
@@ -423,9 +433,10 @@ def main():
     if rank == 0:
         line = {
             "metric": METRIC, "value": value, "unit": "Gpoints/s", "n_gpus": world, "steps": args.steps,
-            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "weak",
+            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True,
+            "scaling": args.scaling if slabbed else "weak",
             "vs_baseline": None, "dtype": "f32", "data": "synthetic",
-            "config": {"workload": args.workload, "extents_per_gpu": list(ext1),
+            "config": {"workload": args.workload, "extents_per_gpu": list(spec.extents),
                        "global_extents": list(gext) if slabbed else list(ext1),
                        "time_steps_per_bench_step": steps_per_iter if iterable else 1,
                        "op": si.OP_NAMES[op], "boundary": [si.KIND_NAMES[k] for k in spec.kind],
