@@ -38,6 +38,7 @@
 #include <cstdlib>
 #include <mutex>
 #include <string>
+#include <type_traits>
 
 #include "common.cuh"
 #include "halo.cuh"
@@ -134,7 +135,7 @@ __device__ __forceinline__ float pick4(int s, const float4& c, float pv) {
 }
 
 template <int OP, int R, int RPW, int S, bool ZC, bool FZ>
-__global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
+__global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW == 1)) ? 3 : 2)
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
              const __grid_constant__ CUtensorMap pwmap, const float* __restrict__ src, float* out, int ntx,
              int nty, int zc, int nchunk, int slot) {
@@ -225,11 +226,13 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
           const int64_t lz = done ? -1 : plane_of(p, p.z_off + zs - R + i);
           if (i == 0) stage_item[s] = done ? -1 : item;
           stage_const[s] = lz < 0;
-          if (lz >= 0) {
+          if (!done && (lz >= 0 || !ZC)) {
+            // a zero value-pad plane (kind CONSTANT, pad_value 0, !ZC) is loaded at
+            // z = -1: entirely out of bounds, so TMA fills it with zeros (no HBM bytes)
             mbar_arrive_expect_tx(&full[s], C::TX_BYTES);
-            tma_load_3d(dsm4 + s * SF4, &tmap, &full[s], x0 - XH, y0 - R, (int)lz);
+            tma_load_3d(dsm4 + s * SF4, &tmap, &full[s], x0 - XH, y0 - R, lz >= 0 ? (int)lz : -1);
           } else {
-            mbar_arrive(&full[s]);   // constant plane (value pad) or end marker: nothing to load
+            mbar_arrive(&full[s]);   // non-zero constant plane (ZC) or end marker: nothing to load
           }
           if (++s == S) { s = 0; ++pass; }
         }
@@ -268,17 +271,16 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
     // into row offsets (y) and register selects (x)
     const bool wrap_fix = (kx == PAD_WRAP || ky == PAD_WRAP) ||
                           ((kx == PAD_CONSTANT || ky == PAD_CONSTANT) && pv != 0.0f);
-    // float4 offsets (within a stage) of this thread's first row: centre column, halo column
+    // float4 offset (within a stage) of this thread's first row, centre column
     const int roff4 = (warp * RPW + R) * BX4 + XH / 4 + lane;
-    const int eoff4 = (warp * RPW + R) * BX4 + (lane == 0 ? 0 : (TX + XH) / 4);
-    // out-of-grid x taps for CLAMP/MIRROR/REFLECT/CONSTANT come from the lane's
-    // own float4 (R <= 2 < 4 <= nx): source element per halo slot, -1 = pad_value
-    int sl[R], sr[R];
-#pragma unroll
-    for (int k = 1; k <= R; ++k) {
-      sl[k - 1] = kx == PAD_CONSTANT ? -1 : (int)pad_remap(-k, nx, kx);          // -1: zero (TMA fill)
-      sr[k - 1] = kx == PAD_CONSTANT ? -1 : (int)(pad_remap(nx - 1 + k, nx, kx) - (nx - 4));
-    }
+    // CLAMP / MIRROR / REFLECT in x: out-of-grid x taps are read from the
+    // remapped in-grid column of the same row (address folded in per item)
+    const bool x_remap = !wrap_fix && kx != PAD_CONSTANT;
+    const float* dsf = reinterpret_cast<const float*>(dsm4);
+    // Acoustic interior constants: x part of K when all 4 x-neighbour sets are
+    // in the domain, and the centre coefficient 2 - l2*K at K = 6R
+    constexpr int kx_full = (2 * R) * 0x1111;
+    const float a_int = __fsub_rn(2.0f, __fmul_rn(p.prm[0], (float)(6 * R)));
     int sn = 0;            // stage of the next load to wait for
     uint32_t pn = 0;       // its pass (barrier phase parity)
     int psc = 0;           // point-wise ring slot of the current output plane
@@ -299,10 +301,29 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
       const int xo = x0 + 4 * lane;
       const bool x_ok = xo < nx;
       const bool y_edge = (y0 < R) || (y0 + TY + R > ny);
-      const bool fix = wrap_fix && ((x0 == 0) || (x0 + TX + R > nx) || y_edge);
-      const bool pl = !wrap_fix && kx != PAD_CONSTANT && x0 == 0 && lane == 0;   // left x-halo out of grid
-      const bool pr = !wrap_fix && kx != PAD_CONSTANT && xo + 4 == nx;           // right x-halo out of grid
+      const bool x_edge = (x0 == 0) || (x0 + TX + R > nx);
+      const bool fix = wrap_fix && (x_edge || y_edge);
       const bool yr = !wrap_fix && ky != PAD_CONSTANT && y_edge;
+      // Edge items (the tile or its halo touches the grid boundary) run the
+      // general loop body; interior items a specialised copy with compile-time
+      // row offsets, no pad logic and no store predicates.
+      // x halo taps: lanes 1..31 take x-1..x-R from the lane below by shuffle,
+      // x+1..x+R from the lane above.  Interior: lane 0 / lane 31 take them from
+      // the halo float4 of the row.  Edge: lane 0 reads them from shared memory
+      // at lrel (floats, relative to its centre element), lane 31 and the lane
+      // holding the last in-grid column at rrel — for CLAMP / MIRROR / REFLECT
+      // the remapped in-grid column of the same row; lanes that do not use the
+      // read get lane 0's / lane 31's address (a broadcast).
+      const bool x_last = x_remap && xo + 4 == nx;
+      const bool use_r = lane == 31 || x_last;
+      int lrel[R], rrel[R];
+#pragma unroll
+      for (int k = 1; k <= R; ++k) {
+        lrel[k - 1] = (x_remap && x0 == 0 && lane == 0) ? (int)pad_remap(-k, nx, kx) : -k - 4 * lane;
+        rrel[k - 1] = x_last ? (int)pad_remap(nx - 1 + k, nx, kx) - xo : TX - 1 + k - 4 * lane;
+      }
+      // float4 offset of the halo float4 of a row relative to the lane's centre float4
+      const int eo4 = (lane == 0 ? 0 : (XH + TX) / 4) - XH / 4 - lane;
       // Acoustic: x part of the in-domain neighbour count of the lane's 4
       // outputs, packed 4 bits each (computed once per item)
       int kxp = 0;
@@ -315,26 +336,23 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
           kxp |= kxi << (4 * i);
         }
       }
-      // float4 offsets of rows y-k / y+k relative to row y (pad redirect folded in)
-      int om[RPW][R], oq[RPW][R];
+      // float4 offset of the warp's row d - R (d = 0 .. RPW-1+2R) relative to
+      // its first row, with the y pad redirect folded in (edge items)
+      int rowo[RPW + 2 * R];
 #pragma unroll
-      for (int jj = 0; jj < RPW; ++jj) {
-        const int rr = warp * RPW + jj, gy = y0 + rr;
-#pragma unroll
-        for (int k = 1; k <= R; ++k) {
-          om[jj][k - 1] = -k * BX4;
-          oq[jj][k - 1] = k * BX4;
-          if (yr) {
-            if (gy - k < 0)
-              om[jj][k - 1] = (min(max((int)pad_remap(gy - k, ny, ky) - y0 + R, 0), C::BY - 1) - (rr + R)) * BX4;
-            if (gy + k >= ny)
-              oq[jj][k - 1] = (min(max((int)pad_remap(gy + k, ny, ky) - y0 + R, 0), C::BY - 1) - (rr + R)) * BX4;
-          }
-        }
+      for (int d = 0; d < RPW + 2 * R; ++d) {
+        const int gy = y0 + warp * RPW + d - R;
+        rowo[d] = (d - R) * BX4;
+        if (yr && (gy < 0 || gy >= ny))
+          rowo[d] = (min(max((int)pad_remap(gy, ny, ky) - y0 + R, 0), C::BY - 1) - (warp * RPW + R)) * BX4;
       }
       // Stages of the 2R+1 planes around the current output plane z: zst[k]
-      // holds plane z - R + k (stage index, or -1 for a constant value plane).
+      // holds plane z - R + k as the float4 offset of its stage (sn * SF4), or
+      // -1 - sn * SF4 for a non-zero constant value plane (ZC; zero planes are
+      // TMA out-of-bounds fills and read like any other stage)
       int zst[2 * R + 1];
+      auto zenc = [&](int st) { return (ZC && stage_const[st]) ? -1 - st * SF4 : st * SF4; };
+      auto zdec = [&](int v) { return (v < 0 ? -1 - v : v) / SF4; };
       // WRAP / non-zero constant: rewrite a plane's out-of-grid halo cells as
       // soon as it arrives (no warp has read that stage since its TMA landed),
       // so every plane of a window — not only the centre — is complete
@@ -347,192 +365,261 @@ __global__ void __launch_bounds__(NCONS + 32, (R == 1 || RPW == 1 ? 3 : 2))
                                                plane_of(p, gzp), x0, y0, threadIdx.x);
         fence_proxy_async_smem();
       };
-#pragma unroll
-      for (int k = 0; k < 2 * R; ++k) {
-        if (k > 0) mbar_wait(&full[sn], pn & 1);
-        zst[k] = (ZC && stage_const[sn]) ? -1 - sn : sn;
-        if constexpr (FIX_ON_ARRIVAL) {
-          if (fix) fix_plane(sn, p.z_off + zs - R + k);
-        }
-        if (++sn == S) { sn = 0; ++pn; }
-      }
-      if constexpr (FIX_ON_ARRIVAL) {
-        if (fix) named_bar_sync(1, NCONS);
-      }
       float* orow = out + ((zs + p.ghost) * p.plane + (int64_t)(y0 + warp * RPW) * nx + xo);
 
-      for (int j = 0; j < nzc; ++j) {
-        mbar_wait(&full[sn], pn & 1);
-        zst[2 * R] = (ZC && stage_const[sn]) ? -1 - sn : sn;
-        const int64_t z = zs + j;                  // local output plane
-        const int gz = (int)(p.z_off + z);
-        if constexpr (FIX_ON_ARRIVAL) {
-          if (fix) {
-            fix_plane(sn, p.z_off + z + R);
-            named_bar_sync(1, NCONS);
-          }
-        }
-        if (++sn == S) { sn = 0; ++pn; }
-        const int cbase = zst[R] * SF4;             // the centre plane is inside the grid
-        if constexpr (!FIX_ON_ARRIVAL) {
-          if (fix) {
-            // all warps are past the previous plane (which read this stage as its
-            // z+1 neighbour, including the padding lanes/rows of ragged tiles)
-            named_bar_sync(1, NCONS);
-            fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + cbase), src,
-                                                   plane_of(p, (int64_t)gz), x0, y0, threadIdx.x);
-            fence_proxy_async_smem();
-            named_bar_sync(1, NCONS);
-          }
-        }
-        // point-wise input of this output plane: its own TMA ring (no halo)
-        if constexpr (PW) mbar_wait(&pwfull[psc], ppc & 1);
+      auto plane_loop = [&](auto edge_tag) {
+        constexpr bool EDGE = decltype(edge_tag)::value;
+        auto RO = [&](int d) { return EDGE ? rowo[d] : (d - R) * BX4; };
+        // the x-window (offsets -R .. 3+R) of the row whose centre float4 is at
+        // a (c = its value; cz: a constant value plane)
+        auto xwin = [&](int a, const float4& c, bool cz, float (&xw)[4 + 2 * R]) {
+          const float cv[4] = {c.x, c.y, c.z, c.w};
+          float4 e = pv4;
+          if (!EDGE && !(ZC && cz)) e = dsm4[a + eo4];
+          const float ev[4] = {e.x, e.y, e.z, e.w};
 #pragma unroll
-        for (int jj = 0; jj < RPW; ++jj) {
-          const int rr = warp * RPW + jj;
-          const int gy = y0 + rr;
-          const bool ok = x_ok && gy < ny;
-          float4 pw = make_float4(0.f, 0.f, 0.f, 0.f);
-          if constexpr (PW) pw = dsm4[S * SF4 + psc * PWF4 + (warp * RPW + jj) * (TX / 4) + lane];
-          const int rb = roff4 + jj * BX4;          // row offset within a stage
-          const float4 c = dsm4[cbase + rb];
-          const float4 e = dsm4[cbase + eoff4 + jj * BX4];
-          float xw[4 + 2 * R];                      // centre row, x offsets -R .. 3+R
-          {
-            const float cv[4] = {c.x, c.y, c.z, c.w};
-            const float ev[4] = {e.x, e.y, e.z, e.w};
-#pragma unroll
-            for (int k = 1; k <= R; ++k) {
-              float l = __shfl_up_sync(FULL, cv[4 - k], 1);
-              float r = __shfl_down_sync(FULL, cv[k - 1], 1);
+          for (int k = 1; k <= R; ++k) {
+            float l = __shfl_up_sync(FULL, cv[4 - k], 1);
+            float r = __shfl_down_sync(FULL, cv[k - 1], 1);
+            if constexpr (EDGE) {
+              const float hl = (ZC && cz) ? pv : dsf[a * 4 + lrel[k - 1]];
+              const float hr = (ZC && cz) ? pv : dsf[a * 4 + rrel[k - 1]];
+              if (lane == 0) l = hl;
+              if (use_r) r = hr;
+            } else {
               if (lane == 0) l = ev[4 - k];
               if (lane == 31) r = ev[k - 1];
-              if (pl) l = pick4(sl[k - 1], c, 0.0f);
-              if (pr) r = pick4(sr[k - 1], c, 0.0f);
-              xw[R - k] = l;
-              xw[R + 3 + k] = r;
+            }
+            xw[R - k] = l;
+            xw[R + 3 + k] = r;
+          }
+#pragma unroll
+          for (int i = 0; i < 4; ++i) xw[R + i] = cv[i];
+        };
+        // 3x3x3 box: running accumulators along z.  Each arriving plane q is read
+        // once (rows -1 .. RPW, one x-window each) and its taps go to three
+        // outputs: q-1 (kz = 2, completes it), q (kz = 1) and q+1 (kz = 0, starts
+        // it).  Every output's FMA chain still runs over its 27 taps in
+        // row-major (kz, ky, kx) order from 0 — K0's order, so the bits agree.
+        float P1[RPW][4], P0[RPW][4];     // partial sums of outputs q and q+1
+        if constexpr (OP == K2_WBOX) {
+#pragma unroll
+          for (int jj = 0; jj < RPW; ++jj)
+#pragma unroll
+            for (int i = 0; i < 4; ++i) P1[jj][i] = P0[jj][i] = 0.0f;
+        }
+        auto box_plane = [&](int az, float (&O)[RPW][4]) {
+          const bool cz = ZC && az < 0;
+          const int sb = cz ? 0 : az;
+          float N1[RPW][4], N0[RPW][4];
+#pragma unroll
+          for (int jj = 0; jj < RPW; ++jj)
+#pragma unroll
+            for (int i = 0; i < 4; ++i) {
+              O[jj][i] = P1[jj][i];
+              N1[jj][i] = P0[jj][i];
+              N0[jj][i] = 0.0f;
             }
 #pragma unroll
-            for (int i = 0; i < 4; ++i) xw[R + i] = cv[i];
-          }
-          auto zrow = [&](int k) -> float4 {       // centre float4 of plane z + k
-            const int a = zst[R + k];
-            if constexpr (ZC) return a < 0 ? pv4 : dsm4[a * SF4 + rb];
-            return dsm4[a * SF4 + rb];
-          };
-          float4 res;
-          if constexpr (OP == K2_WBOX) {
-            // 3x3x3 box: every (plane, row) of the window is an x-window; taps
-            // are added in row-major (kz, ky, kx) order — K0's order
-            float acc[4] = {0.f, 0.f, 0.f, 0.f};
+          for (int d = 0; d < RPW + 2; ++d) {
+            const int a = sb + roff4 + RO(d);
+            const float4 c2 = cz ? pv4 : dsm4[a];
+            float w6[4 + 2 * R];
+            xwin(a, c2, cz, w6);
 #pragma unroll
-            for (int kz = 0; kz < 3; ++kz) {
-              const int a = zst[kz];
-              const bool cz = ZC && a < 0;
-              const int sb = (cz ? 0 : a) * SF4;
+            for (int jj = 0; jj < RPW; ++jj) {
+              const int kyy = d - jj;
+              if (kyy < 0 || kyy > 2) continue;
 #pragma unroll
-              for (int kyy = 0; kyy < 3; ++kyy) {
-                const int ro = rb + (kyy == 0 ? om[jj][0] : (kyy == 2 ? oq[jj][0] : 0));
-                const float4 c2 = cz ? pv4 : dsm4[sb + ro];
-                const float4 e2 = cz ? pv4 : dsm4[sb + ro - rb + eoff4 + jj * BX4];
-                float l = __shfl_up_sync(FULL, c2.w, 1);
-                float r = __shfl_down_sync(FULL, c2.x, 1);
-                if (lane == 0) l = e2.w;
-                if (lane == 31) r = e2.x;
-                if (pl && !cz) l = pick4(sl[0], c2, 0.0f);
-                if (pr && !cz) r = pick4(sr[0], c2, 0.0f);
-                const float w6[6] = {l, c2.x, c2.y, c2.z, c2.w, r};
+              for (int kxx = 0; kxx < 3; ++kxx) {
+                const float w2 = p.wbox[(2 * 3 + kyy) * 3 + kxx];
+                const float w1 = p.wbox[(1 * 3 + kyy) * 3 + kxx];
+                const float w0 = p.wbox[(0 * 3 + kyy) * 3 + kxx];
 #pragma unroll
-                for (int kxx = 0; kxx < 3; ++kxx) {
-                  const float wt = p.wbox[(kz * 3 + kyy) * 3 + kxx];
-#pragma unroll
-                  for (int i = 0; i < 4; ++i) acc[i] = __fmaf_rn(wt, w6[i + kxx], acc[i]);
+                for (int i = 0; i < 4; ++i) {
+                  O[jj][i] = __fmaf_rn(w2, w6[i + kxx], O[jj][i]);
+                  N1[jj][i] = __fmaf_rn(w1, w6[i + kxx], N1[jj][i]);
+                  N0[jj][i] = __fmaf_rn(w0, w6[i + kxx], N0[jj][i]);
                 }
               }
             }
-            res = make_float4(acc[0], acc[1], acc[2], acc[3]);
-          } else if constexpr (OP == K2_ACOUSTIC) {
-            // ordered neighbour sum (acoustic_sum's row-major order), accumulated
-            // as the taps are loaded: z-R..z-1, y-R..y-1, x-R..x-1, x+1..x+R,
-            // y+1..y+R, z+1..z+R
-            float sm[4];
-            bool first = true;
-            auto add4 = [&](const float4& v) {
-              const float vv[4] = {v.x, v.y, v.z, v.w};
+          }
 #pragma unroll
-              for (int i = 0; i < 4; ++i) sm[i] = first ? vv[i] : __fadd_rn(sm[i], vv[i]);
-              first = false;
+          for (int jj = 0; jj < RPW; ++jj)
+#pragma unroll
+            for (int i = 0; i < 4; ++i) {
+              P1[jj][i] = N1[jj][i];
+              P0[jj][i] = N0[jj][i];
+            }
+        };
+        // the first 2R planes of the chunk
+#pragma unroll
+        for (int k = 0; k < 2 * R; ++k) {
+          if (k > 0) mbar_wait(&full[sn], pn & 1);
+          zst[k] = zenc(sn);
+          if constexpr (FIX_ON_ARRIVAL && EDGE) {
+            if (fix) {
+              fix_plane(sn, p.z_off + zs - R + k);
+              named_bar_sync(1, NCONS);
+            }
+          }
+          if (++sn == S) { sn = 0; ++pn; }
+          if constexpr (OP == K2_WBOX) {
+            float O[RPW][4];
+            box_plane(zst[k], O);          // O: not an output yet
+          }
+        }
+        for (int j = 0; j < nzc; ++j) {
+          mbar_wait(&full[sn], pn & 1);
+          zst[2 * R] = zenc(sn);
+          const int64_t z = zs + j;                  // local output plane
+          const int gz = (int)(p.z_off + z);
+          if constexpr (FIX_ON_ARRIVAL && EDGE) {
+            if (fix) {
+              fix_plane(sn, p.z_off + z + R);
+              named_bar_sync(1, NCONS);
+            }
+          }
+          if (++sn == S) { sn = 0; ++pn; }
+          const int cbase = zst[R];                   // the centre plane is inside the grid
+          if constexpr (!FIX_ON_ARRIVAL && EDGE) {
+            if (fix) {
+              // all warps are past the previous plane (which read this stage as its
+              // z+1 neighbour, including the padding lanes/rows of ragged tiles)
+              named_bar_sync(1, NCONS);
+              fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + cbase), src,
+                                                     plane_of(p, (int64_t)gz), x0, y0, threadIdx.x);
+              fence_proxy_async_smem();
+              named_bar_sync(1, NCONS);
+            }
+          }
+          // point-wise input of this output plane: its own TMA ring (no halo)
+          if constexpr (PW) mbar_wait(&pwfull[psc], ppc & 1);
+          // box: plane z+1 completes output z
+          float BO[RPW][4];
+          if constexpr (OP == K2_WBOX) box_plane(zst[2], BO);
+          // star ops: rows -R .. RPW-1+R of the centre plane, each read once
+          float4 cr[RPW + 2 * R];
+          if constexpr (OP != K2_WBOX) {
+#pragma unroll
+            for (int d = 0; d < RPW + 2 * R; ++d) cr[d] = dsm4[cbase + roff4 + RO(d)];
+          }
+#pragma unroll
+          for (int jj = 0; jj < RPW; ++jj) {
+            const int rr = warp * RPW + jj;
+            const int gy = y0 + rr;
+            const bool ok = EDGE ? (x_ok && gy < ny) : true;
+            float4 pw = make_float4(0.f, 0.f, 0.f, 0.f);
+            if constexpr (PW) pw = dsm4[S * SF4 + psc * PWF4 + (warp * RPW + jj) * (TX / 4) + lane];
+            const int rb = roff4 + jj * BX4;          // natural row offset within a stage
+            auto zrow = [&](int k) -> float4 {       // centre float4 of plane z + k
+              const int a = zst[R + k];
+              if constexpr (ZC) return a < 0 ? pv4 : dsm4[a + rb];
+              return dsm4[a + rb];
             };
+            float4 res;
+            if constexpr (OP == K2_WBOX) {
+              res = make_float4(BO[jj][0], BO[jj][1], BO[jj][2], BO[jj][3]);
+            } else {
+              float xw[4 + 2 * R];                    // centre row, x offsets -R .. 3+R
+              xwin(cbase + roff4 + RO(jj + R), cr[jj + R], false, xw);
+              if constexpr (OP == K2_ACOUSTIC) {
+                // ordered neighbour sum (acoustic_sum's row-major order), accumulated
+                // as the taps are loaded: z-R..z-1, y-R..y-1, x-R..x-1, x+1..x+R,
+                // y+1..y+R, z+1..z+R
+                float sm[4];
+                bool first = true;
+                auto add4 = [&](const float4& v) {
+                  const float vv[4] = {v.x, v.y, v.z, v.w};
 #pragma unroll
-            for (int k = R; k >= 1; --k) add4(zrow(-k));
+                  for (int i = 0; i < 4; ++i) sm[i] = first ? vv[i] : __fadd_rn(sm[i], vv[i]);
+                  first = false;
+                };
 #pragma unroll
-            for (int k = R; k >= 1; --k) add4(dsm4[cbase + rb + om[jj][k - 1]]);
+                for (int k = R; k >= 1; --k) add4(zrow(-k));
 #pragma unroll
-            for (int k = R; k >= 1; --k) add4(make_float4(xw[0 + R - k], xw[1 + R - k], xw[2 + R - k], xw[3 + R - k]));
+                for (int k = R; k >= 1; --k) add4(cr[jj + R - k]);
 #pragma unroll
-            for (int k = 1; k <= R; ++k) add4(make_float4(xw[0 + R + k], xw[1 + R + k], xw[2 + R + k], xw[3 + R + k]));
+                for (int k = R; k >= 1; --k) add4(make_float4(xw[0 + R - k], xw[1 + R - k], xw[2 + R - k], xw[3 + R - k]));
 #pragma unroll
-            for (int k = 1; k <= R; ++k) add4(dsm4[cbase + rb + oq[jj][k - 1]]);
+                for (int k = 1; k <= R; ++k) add4(make_float4(xw[0 + R + k], xw[1 + R + k], xw[2 + R + k], xw[3 + R + k]));
 #pragma unroll
-            for (int k = 1; k <= R; ++k) add4(zrow(k));
-            const int Kzy = [&] {
-              int K = 0;
+                for (int k = 1; k <= R; ++k) add4(cr[jj + R + k]);
 #pragma unroll
-              for (int o = 1; o <= R; ++o)
-                K += (gz - o >= 0) + (gz + o < (int)p.gnz) + (gy - o >= 0) + (gy + o < ny);
-              return K;
-            }();
-            const float pwv[4] = {pw.x, pw.y, pw.z, pw.w};
-            float rv[4];
+                for (int k = 1; k <= R; ++k) add4(zrow(k));
+                const int Kzy = [&] {
+                  int K = 0;
 #pragma unroll
-            for (int i = 0; i < 4; ++i)
-              rv[i] = acoustic_combine<R>(sm[i], xw[R + i], pwv[i], Kzy + ((kxp >> (4 * i)) & 15), p.prm);
-            res = make_float4(rv[0], rv[1], rv[2], rv[3]);
-          } else {
-            Win<R> w;
+                  for (int o = 1; o <= R; ++o)
+                    K += (gz - o >= 0) + (gz + o < (int)p.gnz) + (gy - o >= 0) + (gy + o < ny);
+                  return K;
+                }();
+                const float pwv[4] = {pw.x, pw.y, pw.z, pw.w};
+                float rv[4];
+                if (Kzy == 4 * R && kxp == kx_full) {
+                  // all 4 points interior (K = 6R): cf1 = cf2 = 1 and 2 - l2*K is a
+                  // per-launch constant; the operations left are acoustic_combine's
+                  // (the product by cf1 = 1 is exact), so the bits are unchanged
 #pragma unroll
-            for (int i = 0; i < 4 + 2 * R; ++i) w.x[i] = xw[i];
+                  for (int i = 0; i < 4; ++i) {
+                    float t = __fmul_rn(a_int, xw[R + i]);
+                    t = __fmaf_rn(p.prm[0], sm[i], t);
+                    rv[i] = __fmaf_rn(-1.0f, pwv[i], t);
+                  }
+                } else {
 #pragma unroll
-            for (int k = 1; k <= R; ++k) {
-              set4(w.ym[k - 1], dsm4[cbase + rb + om[jj][k - 1]]);
-              set4(w.yp[k - 1], dsm4[cbase + rb + oq[jj][k - 1]]);
-              set4(w.zm[k - 1], zrow(-k));
-              set4(w.zp[k - 1], zrow(k));
+                  for (int i = 0; i < 4; ++i)
+                    rv[i] = acoustic_combine<R>(sm[i], xw[R + i], pwv[i], Kzy + ((kxp >> (4 * i)) & 15), p.prm);
+                }
+                res = make_float4(rv[0], rv[1], rv[2], rv[3]);
+              } else {
+                Win<R> w;
+#pragma unroll
+                for (int i = 0; i < 4 + 2 * R; ++i) w.x[i] = xw[i];
+#pragma unroll
+                for (int k = 1; k <= R; ++k) {
+                  set4(w.ym[k - 1], cr[jj + R - k]);
+                  set4(w.yp[k - 1], cr[jj + R + k]);
+                  set4(w.zm[k - 1], zrow(-k));
+                  set4(w.zp[k - 1], zrow(k));
+                }
+                res.x = eval<OP, R, 0>(p, w, pw, gz, gy, xo);
+                res.y = eval<OP, R, 1>(p, w, pw, gz, gy, xo);
+                res.z = eval<OP, R, 2>(p, w, pw, gz, gy, xo);
+                res.w = eval<OP, R, 3>(p, w, pw, gz, gy, xo);
+              }
             }
-            res.x = eval<OP, R, 0>(p, w, pw, gz, gy, xo);
-            res.y = eval<OP, R, 1>(p, w, pw, gz, gy, xo);
-            res.z = eval<OP, R, 2>(p, w, pw, gz, gy, xo);
-            res.w = eval<OP, R, 3>(p, w, pw, gz, gy, xo);
-          }
-          if (ok) {
-            stg128(orow + jj * nx, res);
-            if constexpr (FZ) {
-              // fused halo put: boundary planes also go to the neighbour's ghosts
-              if (z < p.ghost && p.put_lo) stg128(p.put_lo + z * p.plane + (int64_t)gy * nx + xo, res);
-              if (z >= p.n[0] - p.ghost && p.put_hi)
-                stg128(p.put_hi + (z - (p.n[0] - p.ghost)) * p.plane + (int64_t)gy * nx + xo, res);
+            if (ok) {
+              stg128(orow + jj * nx, res);
+              if constexpr (FZ) {
+                // fused halo put: boundary planes also go to the neighbour's ghosts
+                if (z < p.ghost && p.put_lo) stg128(p.put_lo + z * p.plane + (int64_t)gy * nx + xo, res);
+                if (z >= p.n[0] - p.ghost && p.put_hi)
+                  stg128(p.put_hi + (z - (p.n[0] - p.ghost)) * p.plane + (int64_t)gy * nx + xo, res);
+              }
             }
           }
-        }
-        orow += p.plane;
-        // plane z - R is no longer needed (pre-chunk planes included)
-        __syncwarp();
-        if (lane == 0) {
-          const int t = zst[0] < 0 ? -1 - zst[0] : zst[0];
-          mbar_arrive(&empty[t]);
-          if constexpr (PW) mbar_arrive(&pwempty[psc]);
-        }
-        if constexpr (PW) {
-          if (++psc == PS) { psc = 0; ++ppc; }
-        }
+          orow += p.plane;
+          // plane z - R is no longer needed (pre-chunk planes included)
+          __syncwarp();
+          if (lane == 0) {
+            mbar_arrive(&empty[zdec(zst[0])]);
+            if constexpr (PW) mbar_arrive(&pwempty[psc]);
+          }
+          if constexpr (PW) {
+            if (++psc == PS) { psc = 0; ++ppc; }
+          }
 #pragma unroll
-        for (int k = 0; k < 2 * R; ++k) zst[k] = zst[k + 1];
-      }
+          for (int k = 0; k < 2 * R; ++k) zst[k] = zst[k + 1];
+        }
+      };
+      if (x_edge || y_edge) plane_loop(std::true_type{});
+      else plane_loop(std::false_type{});
       // the chunk's last 2R planes (z_end - R .. z_end + R - 1) are still held
       __syncwarp();
       if (lane == 0) {
 #pragma unroll
-        for (int k = 0; k < 2 * R; ++k) mbar_arrive(&empty[zst[k] < 0 ? -1 - zst[k] : zst[k]]);
+        for (int k = 0; k < 2 * R; ++k) mbar_arrive(&empty[zdec(zst[k])]);
         // fused step: when every warp of every tile of a boundary chunk is done,
         // publish its peer stores and raise that neighbour's flag
         if (FZ && p.fused_step) {
@@ -862,7 +949,8 @@ Launcher get_launcher_zf(bool zc, bool fz) {
 
 Launcher pick(const StencilParams& p) {
   const int R = p.radius;
-  const bool zc = p.kind[0] == PAD_CONSTANT;   // value-pad planes in z are possible
+  // non-zero value-pad planes in z are possible (zero ones are TMA out-of-bounds fills)
+  const bool zc = p.kind[0] == PAD_CONSTANT && p.pad_value != 0.0f;
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;   // fused halo launch
   if (p.op == OP_WEIGHTED) {
     if (R == 1 && !star_weights(p, 1)) return get_launcher_zf<K2_WBOX, 1, 2, 7>(zc, fz);
