@@ -71,7 +71,10 @@ def ncu_traffic(workload):
 
 
 class ClockSampler:
-    """nvidia-smi clocks + throttle reasons sampled during the timed region."""
+    """SM clock + throttle reasons sampled during the timed region.
+
+    NVML (the library nvidia-smi reads) every 20 ms, so even a ~1 s timed
+    region gets dozens of samples; falls back to nvidia-smi if NVML is absent."""
 
     Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
          "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
@@ -82,7 +85,29 @@ class ClockSampler:
         self.stop = threading.Event()
         self.t = threading.Thread(target=self.run, daemon=True)
 
+    def run_nvml(self):
+        import pynvml as nv
+        nv.nvmlInit()
+        try:
+            vis = os.environ.get("CUDA_VISIBLE_DEVICES")
+            idx = int(vis.split(",")[self.idx]) if vis and vis.split(",")[self.idx].isdigit() else self.idx
+            h = nv.nvmlDeviceGetHandleByIndex(idx)
+            mx = nv.nvmlDeviceGetMaxClockInfo(h, nv.NVML_CLOCK_SM)
+            bits = [0x8, 0x40, 0x20, 0x4]    # hw_slowdown, hw_thermal, sw_thermal, sw_power_cap
+            while not self.stop.is_set():
+                sm = nv.nvmlDeviceGetClockInfo(h, nv.NVML_CLOCK_SM)
+                rs = nv.nvmlDeviceGetCurrentClocksEventReasons(h)
+                self.samples.append([str(sm), str(mx)] + ["Active" if rs & b else "Not Active" for b in bits])
+                self.stop.wait(0.02)
+        finally:
+            nv.nvmlShutdown()
+
     def run(self):
+        try:
+            self.run_nvml()
+            return
+        except Exception:
+            pass
         while not self.stop.is_set():
             try:
                 r = subprocess.run(["nvidia-smi", "-i", str(self.idx), f"--query-gpu={self.Q}",
@@ -290,6 +315,12 @@ def main():
     else:
         out = plan.empty_output()
         launches_per_step = 1
+    # a bench step of a single-sweep workload is a CUDA graph of `sweeps` full
+    # sweeps (each reads the whole input and writes the whole output): small
+    # grids (J2D5 256^2) take microseconds per sweep, so one graph launch per
+    # sweep would time the host, not the kernel
+    sweeps = 1 if iterable else int(min(1000, max(1, (1 << 26) // max(1, npts_local))))
+    launches_per_step *= sweeps
 
     stream = torch.cuda.current_stream()
 
@@ -298,13 +329,15 @@ def main():
             if slabbed:
                 return sp.iterate(state, steps_per_iter, aux, fused=fused)
             return plan.iterate(state, steps_per_iter, aux)
-        plan.apply(*bufs, out=out)
+        for _ in range(sweeps):
+            plan.apply(*bufs, out=out)
         return 0
 
-    # single-sweep workloads are launch-latency bound at small sizes: capture the
-    # step (the same C-ABI call, graph-capturable by design) into a CUDA graph
+    # single-GPU steps are captured once into a CUDA graph (the C-ABI calls are
+    # graph-capturable by design: stream-ordered, no allocation, no sync) and
+    # replayed; the slab path keeps its stream launches (NCCL + side streams)
     graph = None
-    if not iterable and not args.no_graph:
+    if not slabbed and not args.no_graph:
         side = torch.cuda.Stream()
         side.wait_stream(torch.cuda.current_stream())
         with torch.cuda.stream(side):
@@ -346,7 +379,7 @@ def main():
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
         t_max = float(tt.item())
     ms_per_step = t_max / args.steps
-    points = npts_local * world * steps_per_iter * args.steps
+    points = npts_local * world * steps_per_iter * sweeps * args.steps
     value = points / (t_max * 1e-3) / 1e9
 
     # per-launch kernel duration of the dominant kernel: a step is back-to-back
@@ -439,6 +472,7 @@ def main():
             "config": {"workload": args.workload, "extents_per_gpu": list(spec.extents),
                        "global_extents": list(gext) if slabbed else list(ext1),
                        "time_steps_per_bench_step": steps_per_iter if iterable else 1,
+                       "sweeps_per_bench_step": steps_per_iter if iterable else sweeps,
                        "op": si.OP_NAMES[op], "boundary": [si.KIND_NAMES[k] for k in spec.kind],
                        "window": list(spec.size),
                        "halo": (args.halo if slabbed else None),
@@ -447,7 +481,8 @@ def main():
                        "l2": "inputs larger than L2 (no flush needed)" if npts_local * 4 > 126e6
                        else "L2-resident working set (no flush; reported as such)",
                        "variant": {0: "K0 generic", 1: "K1 tile2d (TMA)", 2: "K2 sweep3d (TMA)"}[plan.variant],
-                       "launch": "cuda graph replay" if graph is not None else "stream launches"},
+                       "launch": (f"cuda graph replay ({launches_per_step} launches per graph)" if graph is not None
+                                  else "stream launches")},
             "hbm_gbs_per_gpu_whole_step": value * bpp / world,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": ncu_traffic(args.workload),

@@ -112,4 +112,21 @@ __host__ __device__ __forceinline__ int64_t plane_of(const StencilParams& p, int
   return gz - p.z_off + p.ghost;
 }
 
+// Programmatic dependent launch (sm_90+): a kernel launched with the
+// programmatic-stream-serialization attribute may be scheduled while the
+// previous kernel of the stream is still draining; it runs its prologue
+// (mbarrier init, tensor-map prefetch), then waits here for the previous
+// grid's completion and memory flush before touching global memory.  Both are
+// no-ops for an ordinary launch.
+__device__ __forceinline__ void pdl_wait() {
+#if defined(__CUDA_ARCH__)
+  asm volatile("griddepcontrol.wait;" ::: "memory");
+#endif
+}
+__device__ __forceinline__ void pdl_launch_dependents() {
+#if defined(__CUDA_ARCH__)
+  asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+#endif
+}
+
 }  // namespace lift

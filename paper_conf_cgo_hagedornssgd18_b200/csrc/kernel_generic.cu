@@ -71,6 +71,8 @@ __global__ void __launch_bounds__(256) k0_generic(const __grid_constant__ Stenci
                                                   const float* __restrict__ in0,
                                                   const float* __restrict__ in1,
                                                   float* __restrict__ out) {
+  pdl_launch_dependents();
+  pdl_wait();
   const int64_t o1 = p.o[1], o2 = p.o[2];
   const int64_t per_plane = o1 * o2;
   const int64_t total = (p.reg1 - p.reg0) * per_plane;
@@ -164,8 +166,10 @@ cudaError_t launch_generic(const StencilParams& p, const float* in0, const float
   int64_t blocks = (total + threads - 1) / threads;
   const int64_t cap = (int64_t)num_sms * 8 * 4;   // grid-stride beyond a few waves
   if (blocks > cap) blocks = cap;
-  k0_generic<<<(unsigned)blocks, threads, 0, stream>>>(p, in0, in1, out);
-  return cudaGetLastError();
+  const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
+  void* args[] = {(void*)&p, (void*)&in0, (void*)&in1, (void*)&out};
+  return launch_kernel(reinterpret_cast<const void*>(&k0_generic), dim3((unsigned)blocks), dim3(threads), args, 0,
+                       stream, !fz);
 }
 
 }  // namespace lift

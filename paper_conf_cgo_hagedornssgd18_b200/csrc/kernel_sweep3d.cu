@@ -180,6 +180,8 @@ __global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW =
     fence_mbar_init();
   }
   __syncthreads();
+  pdl_launch_dependents();   // PDL: let the next launch ramp up now
+  pdl_wait();                // ... and wait for the previous one before any global access
 
   if (warp == NW) {
     // ---------------- producers ----------------
@@ -717,6 +719,8 @@ __global__ void __launch_bounds__(NCONS + 32, 2)
     fence_mbar_init();
   }
   __syncthreads();
+  pdl_launch_dependents();   // PDL: let the next launch ramp up now
+  pdl_wait();                // ... and wait for the previous one before any global access
 
   if (warp == NW) {
     if (lane == 0) {
@@ -1043,7 +1047,8 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   int slot = (int)(g_slot.fetch_add(1) % kTickets);
   void* args[] = {(void*)&p, (void*)&map, (void*)&pwmap, (void*)&slid, (void*)&out,
                   &ntx_i, &nty_i, &zc_i, &nch_i, &slot};
-  return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
+  const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
+  return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, !fz);
 }
 
 }  // namespace lift
@@ -1093,7 +1098,7 @@ cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* ou
   int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk;
   int slot = (int)(g_slot.fetch_add(1) % kTickets);
   void* args[] = {(void*)&p, (void*)&map, (void*)&out, &ntx_i, &nty_i, &zc_i, &nch_i, &slot};
-  return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
+  return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, true);
 }
 
 }  // namespace lift

@@ -118,6 +118,8 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
     fence_mbar_init();
   }
   __syncthreads();
+  pdl_launch_dependents();   // PDL: let the next launch ramp up now
+  pdl_wait();                // ... and wait for the previous one before any global access
 
   if (warp == NW) {
     if (!LDG && lane == 0) {
@@ -364,6 +366,8 @@ __global__ void __launch_bounds__(NCONS + 32, 3)
     fence_mbar_init();
   }
   __syncthreads();
+  pdl_launch_dependents();   // PDL: let the next launch ramp up now
+  pdl_wait();                // ... and wait for the previous one before any global access
   if (warp == NW) {
     if (lane == 0) {
       prefetch_tmap(&map0);
@@ -484,10 +488,14 @@ bool star2d(const StencilParams& p, int RY, int RX) {
   return true;
 }
 
-#define K1_PICK(OPV, RYV, RXV, NINV) \
-  (ldg ? get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, true>() : get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, false>())
+// small grids (fewer 128 x 48 tiles than SMs, e.g. J2D5 256^2, SRAD 504x458)
+// take 128 x 8 tiles: 6x the CTAs, each a sixth of the latency chain
+#define K1_PICK(OPV, RYV, RXV, NINV)                                                   \
+  (ldg ? get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, true>()                            \
+       : (small ? get_launcher<OPV, RYV, RXV, 1, 2, NINV, 4, false>()                  \
+                : get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, false>()))
 
-bool pick(const StencilParams& p, bool ldg, Launcher* L) {
+bool pick(const StencilParams& p, bool ldg, bool small, Launcher* L) {
   const int ry = p.lo[1], rx = p.lo[2];
   if (p.op == OP_WEIGHTED) {
     const int mode = p.sep ? K1_WSEP : (star2d(p, ry, rx) ? K1_WSTAR : K1_WBOX);
@@ -502,6 +510,10 @@ bool pick(const StencilParams& p, bool ldg, Launcher* L) {
         case 3: *L = get_launcher<K1_WSEP, 2, 2, 2, 4, 1, 4>(); return true;
         case 4: *L = get_launcher<K1_WSEP, 2, 2, 8, 3, 1, 2>(); return true;
         case 5: *L = get_launcher<K1_WSEP, 2, 2, 4, 3, 1, 3>(); return true;
+        case 6: *L = get_launcher<K1_WSEP, 2, 2, 6, 3, 1, 2>(); return true;
+        case 7: *L = get_launcher<K1_WSEP, 2, 2, 4, 4, 1, 2>(); return true;
+        case 8: *L = get_launcher<K1_WSEP, 2, 2, 12, 2, 1, 2>(); return true;
+        case 9: *L = get_launcher<K1_WSEP, 2, 2, 3, 5, 1, 2>(); return true;
         default: break;
       }
     }
@@ -572,7 +584,7 @@ cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* o
   int64_t grid = (int64_t)num_sms * L.ctas_per_sm;
   if (grid > (int64_t)ntx * nty) grid = (int64_t)ntx * nty;
   void* args[] = {(void*)&p, (void*)&m0, (void*)&in0, (void*)&out, (void*)&ntx, (void*)&nty};
-  return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
+  return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, true);
 }
 
 bool tile2d_supported(const StencilParams& p) {
@@ -598,8 +610,9 @@ cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float*
   // TMA needs 16-B aligned bases and row pitches; otherwise cp.async fills the box
   const bool ldg = (p.n[2] % 4 != 0) || (reinterpret_cast<uintptr_t>(in0) & 15u) ||
                    (in1 && (reinterpret_cast<uintptr_t>(in1) & 15u));
+  const bool small = ((p.n[2] + TX - 1) / TX) * ((p.n[1] + 6 * NW - 1) / (6 * NW)) < num_sms;
   Launcher L;
-  if (!pick(p, ldg, &L)) {
+  if (!pick(p, ldg, small, &L)) {
     *err = "tile2d: no instantiation";
     return cudaErrorNotSupported;
   }
@@ -619,7 +632,7 @@ cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float*
   if (grid > ntiles) grid = ntiles;
   const float* s1 = L.nin > 1 ? in1 : in0;
   void* args[] = {(void*)&p, (void*)&m0, (void*)&m1, (void*)&in0, (void*)&s1, (void*)&out, (void*)&ntx, (void*)&nty};
-  return cudaLaunchKernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream);
+  return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, true);
 }
 
 }  // namespace lift

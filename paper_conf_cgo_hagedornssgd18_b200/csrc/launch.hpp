@@ -4,11 +4,39 @@
 #include <cuda_runtime.h>
 
 #include <cstdint>
+#include <cstdlib>
 #include <string>
 
 #include "common.cuh"
 
 namespace lift {
+
+// Whether stencil kernels are launched with programmatic dependent launch
+// (overlaps a launch's ramp-up with the previous kernel's tail; every such
+// kernel calls pdl_wait() before its first global access).  LIFT_PDL=0 turns
+// it off (A/B measurement).
+inline bool pdl_enabled() {
+  static const bool on = [] {
+    const char* e = getenv("LIFT_PDL");
+    return !(e && e[0] == '0');
+  }();
+  return on;
+}
+
+inline cudaError_t launch_kernel(const void* fn, dim3 grid, dim3 block, void** args, size_t smem,
+                                 cudaStream_t stream, bool pdl) {
+  cudaLaunchConfig_t cfg{};
+  cfg.gridDim = grid;
+  cfg.blockDim = block;
+  cfg.dynamicSmemBytes = smem;
+  cfg.stream = stream;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+  at[0].val.programmaticStreamSerializationAllowed = (pdl && pdl_enabled()) ? 1 : 0;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  return cudaLaunchKernelExC(&cfg, fn, args);
+}
 
 // K0 — generic remap kernel (any plan).
 cudaError_t launch_generic(const StencilParams& p, const float* in0, const float* in1, float* out,
