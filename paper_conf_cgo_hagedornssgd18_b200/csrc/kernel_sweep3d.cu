@@ -74,13 +74,13 @@ __device__ __forceinline__ void spin_until(const unsigned int* f, unsigned int v
 
 enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2, K2_WBOX = 3 };
 
-template <int R, int RPW, int S, bool PW>
+template <int R, int RPW, int S, int PSN>
 struct Cfg {
   static constexpr int TY = NW * RPW;
   static constexpr int BY = TY + 2 * R;
   static constexpr int TX_BYTES = BX * BY * 4;
   static constexpr int STAGE_FLOATS = ((TX_BYTES + 127) / 128) * 128 / 4;
-  static constexpr int PS = PW ? 3 : 0;                 // point-wise ring slots
+  static constexpr int PS = PSN;                        // point-wise ring slots (0: no point-wise grid)
   static constexpr int PW_BYTES = TX * TY * 4;
   static constexpr int PW_FLOATS = TX * TY;
   static constexpr int SMEM = S * STAGE_FLOATS * 4 + PS * PW_BYTES + 2 * (S + PS + 4) * 8 + (2 * S + 4) * 4 + 256;
@@ -134,12 +134,12 @@ __device__ __forceinline__ float pick4(int s, const float4& c, float pv) {
   return s < 0 ? pv : (s == 0 ? c.x : (s == 1 ? c.y : (s == 2 ? c.z : c.w)));
 }
 
-template <int OP, int R, int RPW, int S, bool ZC, bool FZ>
+template <int OP, int R, int RPW, int S, bool ZC, bool FZ, int PSN>
 __global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW == 1)) ? 3 : 2)
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
              const __grid_constant__ CUtensorMap pwmap, const float* __restrict__ src, float* out, int ntx,
              int nty, int zc, int nchunk, int slot) {
-  using C = Cfg<R, RPW, S, (OP == K2_HOTSPOT || OP == K2_ACOUSTIC)>;
+  using C = Cfg<R, RPW, S, (OP == K2_HOTSPOT || OP == K2_ACOUSTIC) ? PSN : 0>;
   constexpr bool PW = OP == K2_HOTSPOT || OP == K2_ACOUSTIC;           // a point-wise zipped grid (Hotspot P, Acoustic prev)
   constexpr int PS = C::PS;                     // point-wise ring slots
   constexpr int QN = 4;                         // item queue between the two producer lanes
@@ -929,13 +929,13 @@ struct Launcher {
   int ctas_per_sm;
 };
 
-template <int OP, int R, int RPW, int S, bool ZC, bool FZ>
+template <int OP, int R, int RPW, int S, bool ZC, bool FZ, int PSN>
 Launcher get_launcher() {
   static Launcher L{};
   static std::once_flag once;
   std::call_once(once, [] {
-    using C = Cfg<R, RPW, S, (OP == K2_HOTSPOT || OP == K2_ACOUSTIC)>;
-    auto fn = k2_sweep<OP, R, RPW, S, ZC, FZ>;
+    using C = Cfg<R, RPW, S, (OP == K2_HOTSPOT || OP == K2_ACOUSTIC) ? PSN : 0>;
+    auto fn = k2_sweep<OP, R, RPW, S, ZC, FZ, PSN>;
     cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
     int occ = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, NCONS + 32, C::SMEM) != cudaSuccess) occ = 1;
@@ -945,10 +945,10 @@ Launcher get_launcher() {
   return L;
 }
 
-template <int OP, int R, int RPW, int S>
+template <int OP, int R, int RPW, int S, int PSN = 3>
 Launcher get_launcher_zf(bool zc, bool fz) {
-  if (fz) return zc ? get_launcher<OP, R, RPW, S, true, true>() : get_launcher<OP, R, RPW, S, false, true>();
-  return zc ? get_launcher<OP, R, RPW, S, true, false>() : get_launcher<OP, R, RPW, S, false, false>();
+  if (fz) return zc ? get_launcher<OP, R, RPW, S, true, true, PSN>() : get_launcher<OP, R, RPW, S, false, true, PSN>();
+  return zc ? get_launcher<OP, R, RPW, S, true, false, PSN>() : get_launcher<OP, R, RPW, S, false, false, PSN>();
 }
 
 Launcher pick(const StencilParams& p) {
@@ -957,13 +957,24 @@ Launcher pick(const StencilParams& p) {
   const bool zc = p.kind[0] == PAD_CONSTANT && p.pad_value != 0.0f;
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;   // fused halo launch
   if (p.op == OP_WEIGHTED) {
-    if (R == 1 && !star_weights(p, 1)) return get_launcher_zf<K2_WBOX, 1, 2, 7>(zc, fz);
-    if (R == 1) return get_launcher_zf<K2_WSTAR, 1, 2, 7>(zc, fz);
-    return get_launcher_zf<K2_WSTAR, 2, 2, 8>(zc, fz);
+    if (R == 1 && !star_weights(p, 1)) return get_launcher_zf<K2_WBOX, 1, 2, 7, 0>(zc, fz);
+    if (R == 1) return get_launcher_zf<K2_WSTAR, 1, 2, 7, 0>(zc, fz);
+    return get_launcher_zf<K2_WSTAR, 2, 2, 8, 0>(zc, fz);
   }
-  if (p.op == OP_HOTSPOT3D) return get_launcher_zf<K2_HOTSPOT, 1, 2, 5>(zc, fz);
-  if (R == 1) return get_launcher_zf<K2_ACOUSTIC, 1, 2, 5>(zc, fz);
-  return get_launcher_zf<K2_ACOUSTIC, 2, 2, 8>(zc, fz);
+  // point-wise ring depth tuning hook (LIFT_K2_PW: 1 = the round-1 (S, 3) rings)
+  const char* e = getenv("LIFT_K2_PW");
+  const int pv = e ? atoi(e) : 0;
+  if (p.op == OP_HOTSPOT3D) {
+    if (pv == 1) return get_launcher_zf<K2_HOTSPOT, 1, 2, 5, 3>(zc, fz);
+    return get_launcher_zf<K2_HOTSPOT, 1, 2, 5, 5>(zc, fz);
+  }
+  if (R == 1) {
+    if (pv == 1) return get_launcher_zf<K2_ACOUSTIC, 1, 2, 5, 3>(zc, fz);
+    return get_launcher_zf<K2_ACOUSTIC, 1, 2, 5, 5>(zc, fz);
+  }
+  if (pv == 1) return get_launcher_zf<K2_ACOUSTIC, 2, 2, 8, 3>(zc, fz);
+  if (pv == 2) return get_launcher_zf<K2_ACOUSTIC, 2, 2, 7, 4>(zc, fz);
+  return get_launcher_zf<K2_ACOUSTIC, 2, 2, 6, 5>(zc, fz);
 }
 
 struct MapEntry {
@@ -1037,6 +1048,21 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   int64_t zc = (work + 8 * slots - 1) / (8 * slots);
   const int64_t zmin = std::min<int64_t>(16, std::max<int64_t>(2, (work + 2 * slots - 1) / (2 * slots)));
   if (zc < zmin) zc = zmin;
+  if (work < 16 * slots) {
+    // small (L2-resident, latency-bound) grids, e.g. Hotspot3D's 8 planes: the
+    // step takes about (waves of items) x (planes loaded per item), so pick
+    // the chunk that minimises ceil(items / slots) * (zc + 2R)
+    int64_t best = -1;
+    for (int64_t z = 1; z <= nz_reg; ++z) {
+      const int64_t it = tiles * ((nz_reg + z - 1) / z);
+      const int64_t cost = ((it + slots - 1) / slots) * (z + 2 * R);
+      if (best < 0 || cost < best) {
+        best = cost;
+        zc = z;
+      }
+    }
+  }
+  if (const char* e = getenv("LIFT_K2_ZC")) zc = std::max<int64_t>(1, atoll(e));   // tuning hook
   if (p.fused_step && zc < p.ghost) zc = p.ghost;     // boundary planes stay in the first / last chunk
   if (zc > nz_reg) zc = nz_reg;
   const int64_t nchunk = (nz_reg + zc - 1) / zc;

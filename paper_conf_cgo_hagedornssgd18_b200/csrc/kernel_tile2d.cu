@@ -488,35 +488,31 @@ bool star2d(const StencilParams& p, int RY, int RX) {
   return true;
 }
 
-// small grids (fewer 128 x 48 tiles than SMs, e.g. J2D5 256^2, SRAD 504x458)
-// take 128 x 8 tiles: 6x the CTAs, each a sixth of the latency chain
-#define K1_PICK(OPV, RYV, RXV, NINV)                                                   \
-  (ldg ? get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, true>()                            \
-       : (small ? get_launcher<OPV, RYV, RXV, 1, 2, NINV, 4, false>()                  \
-                : get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, false>()))
+// Tile shape per launch: small grids (fewer 128 x 48 tiles than SMs, e.g.
+// J2D5 256^2, SRAD 504x458) take 128 x 8 tiles (6x the CTAs, each a sixth
+// of the latency chain); otherwise (rows per warp, stages, CTAs per SM) =
+// (4, 4, 2) for the separable Gaussian — a 4-deep ring of 128 x 32 tiles
+// keeps more bytes in flight — and (6, 2, 3) for SRAD (measured per op,
+// profiles/r01_sweep_k1_shapes_k3.txt); LIFT_K1_SHAPE overrides
+// (1 = (6, 2, 3), 2 = (4, 3, 3), 3 = (8, 3, 2), 4 = (4, 4, 2))
+template <int OPV, int RYV, int RXV, int NINV>
+Launcher pick_k1(bool ldg, bool small) {
+  if (ldg) return get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, true>();
+  if (small) return get_launcher<OPV, RYV, RXV, 1, 2, NINV, 4, false>();
+  const char* e = getenv("LIFT_K1_SHAPE");
+  switch (e ? atoi(e) : (OPV == K1_WSEP ? 4 : 1)) {
+    case 2: return get_launcher<OPV, RYV, RXV, 4, 3, NINV, 3, false>();
+    case 3: return get_launcher<OPV, RYV, RXV, 8, 3, NINV, 2, false>();
+    case 4: return get_launcher<OPV, RYV, RXV, 4, 4, NINV, 2, false>();
+    default: return get_launcher<OPV, RYV, RXV, 6, 2, NINV, 3, false>();
+  }
+}
+#define K1_PICK(OPV, RYV, RXV, NINV) pick_k1<OPV, RYV, RXV, NINV>(ldg, small)
 
 bool pick(const StencilParams& p, bool ldg, bool small, Launcher* L) {
   const int ry = p.lo[1], rx = p.lo[2];
   if (p.op == OP_WEIGHTED) {
     const int mode = p.sep ? K1_WSEP : (star2d(p, ry, rx) ? K1_WSTAR : K1_WBOX);
-    // tile-shape sweep hook (NEXT-4 / ATF role): LIFT_K1_VARIANT
-    // selects alternative (rows per warp, stages, CTAs per SM) for the
-    // separable radius-2 case; the default is the tuned one
-    static const int tv = [] { const char* e = getenv("LIFT_K1_VARIANT"); return e ? atoi(e) : 0; }();
-    if (mode == K1_WSEP && ry == 2 && rx == 2 && tv != 0 && !ldg) {
-      switch (tv) {
-        case 1: *L = get_launcher<K1_WSEP, 2, 2, 8, 2, 1, 3>(); return true;
-        case 2: *L = get_launcher<K1_WSEP, 2, 2, 4, 2, 1, 4>(); return true;
-        case 3: *L = get_launcher<K1_WSEP, 2, 2, 2, 4, 1, 4>(); return true;
-        case 4: *L = get_launcher<K1_WSEP, 2, 2, 8, 3, 1, 2>(); return true;
-        case 5: *L = get_launcher<K1_WSEP, 2, 2, 4, 3, 1, 3>(); return true;
-        case 6: *L = get_launcher<K1_WSEP, 2, 2, 6, 3, 1, 2>(); return true;
-        case 7: *L = get_launcher<K1_WSEP, 2, 2, 4, 4, 1, 2>(); return true;
-        case 8: *L = get_launcher<K1_WSEP, 2, 2, 12, 2, 1, 2>(); return true;
-        case 9: *L = get_launcher<K1_WSEP, 2, 2, 3, 5, 1, 2>(); return true;
-        default: break;
-      }
-    }
 #define K1_CASE(RYV, RXV)                                                     \
   if (ry == RYV && rx == RXV) {                                              \
     if (mode == K1_WSEP) *L = K1_PICK(K1_WSEP, RYV, RXV, 1);                 \
@@ -607,10 +603,12 @@ bool tile2d_supported(const StencilParams& p) {
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,
                           cudaStream_t stream, int num_sms, std::string* err) {
   if (p.op == OP_SRAD) return launch_srad_fused(p, in0, out, stream, num_sms, err);
+  const bool small = ((p.n[2] + TX - 1) / TX) * ((p.n[1] + 6 * NW - 1) / (6 * NW)) < num_sms;
+  // per-warp streaming sweeps (K3) where they measured faster than the tiles
+  if (wsweep2d_supported(p, in0, in1, small)) return launch_wsweep2d(p, in0, in1, out, stream, num_sms, err);
   // TMA needs 16-B aligned bases and row pitches; otherwise cp.async fills the box
   const bool ldg = (p.n[2] % 4 != 0) || (reinterpret_cast<uintptr_t>(in0) & 15u) ||
                    (in1 && (reinterpret_cast<uintptr_t>(in1) & 15u));
-  const bool small = ((p.n[2] + TX - 1) / TX) * ((p.n[1] + 6 * NW - 1) / (6 * NW)) < num_sms;
   Launcher L;
   if (!pick(p, ldg, small, &L)) {
     *err = "tile2d: no instantiation";

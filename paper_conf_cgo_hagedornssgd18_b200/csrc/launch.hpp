@@ -62,6 +62,11 @@ bool tile2d_supported(const StencilParams& p);
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,
                           cudaStream_t stream, int num_sms, std::string* err);
 
+// K3 — 2D per-warp TMA y-sweeps (the K1 ops; TMA-describable rows, x pad not WRAP).
+bool wsweep2d_supported(const StencilParams& p, const float* in0, const float* in1, bool small);
+cudaError_t launch_wsweep2d(const StencilParams& p, const float* in0, const float* in1, float* out,
+                            cudaStream_t stream, int num_sms, std::string* err);
+
 // OP_SRAD: q0^2 = var/mean^2 of the image (fp64, deterministic) into the
 // workspace, as SRAD1's constants {q0, a, b}
 size_t srad_workspace_bytes(int num_sms);

@@ -455,3 +455,43 @@ def test_tile2d_unaligned_pointer(lift):
     torch.cuda.synchronize()
     Y, A = orc.apply(sp, [xin.cpu().numpy()])
     assert orc.max_rel_err(out.cpu().numpy(), Y, A) <= TOL1
+
+
+# ------------------------------------------------- K3 per-warp sweeps ------
+@pytest.mark.parametrize("case", ["j2d5", "gauss", "box", "srad1", "srad2", "hot2d", "grad"])
+@pytest.mark.parametrize("kind", [CLAMP, MIRROR, REFLECT, CONSTANT, WRAP])
+def test_wsweep2d_bitwise_vs_k1_k0(lift, case, kind, monkeypatch):
+    """K3 (per-warp y-sweeps) against K1 (tiles) and K0 (generic), bitwise, for
+    several rows-per-item values (one group, several sweep blocks, a ragged
+    last chunk) and ragged strips; WRAP in y runs K3 with remapped rows."""
+    shape = (203, 392)          # 4 strips, the last 8 columns wide
+    kinds = (kind, CLAMP if kind == WRAP else kind)     # WRAP in x runs on K1
+    if case == "j2d5":
+        sp, xs = spec(shape, 3, si.weights_j2d5(), kinds, value=0.75), [rnd(shape, 60)]
+    elif case == "gauss":
+        sp, xs = spec(shape, 5, si.weights_gauss5(), kinds, value=0.75), [rnd(shape, 61)]
+    elif case == "box":
+        w = np.random.default_rng(62).standard_normal((5, 3)).astype(np.float32)
+        sp, xs = spec(shape, (5, 3), w, kinds, value=-0.5), [rnd(shape, 63)]
+    elif case == "srad1":
+        I = np.exp(rnd(shape, 64, 0, 1)).astype(np.float32)
+        sp, xs = spec(shape, 3, op=si.SRAD1, params=si.params_srad1(si.srad_q0sqr(I)), kind=kinds, value=1.5), [I]
+    elif case == "srad2":
+        I = np.exp(rnd(shape, 65, 0, 1)).astype(np.float32)
+        sp, xs = spec(shape, 3, op=si.SRAD2, params=si.params_srad2(), kind=kinds, value=0.5), [rnd(shape, 66, 0, 1), I]
+    elif case == "hot2d":
+        sp = spec(shape, 3, op=si.HOTSPOT2D, params=si.params_hotspot2d(*shape), kind=kinds, value=320.0)
+        xs = [rnd(shape, 67, 300, 350), rnd(shape, 68, 0, 1e-2)]
+    else:
+        sp, xs = spec(shape, 3, op=si.GRADIENT, params=si.params_gradient(), kind=kinds, value=0.5), [rnd(shape, 69)]
+    y0, plan = run_gpu(lift, sp, xs, "generic")
+    monkeypatch.setenv("LIFT_K3", "0")
+    y1, _ = run_gpu(lift, sp, xs, "tile2d")
+    np.testing.assert_array_equal(y1, y0)
+    monkeypatch.setenv("LIFT_K3", "1")
+    for hc in ("1", "6", "14", "61", "203", "512"):
+        monkeypatch.setenv("LIFT_K3_HC", hc)
+        y, plan = run_gpu(lift, sp, xs, "tile2d")
+        np.testing.assert_array_equal(y, y0, err_msg=f"hc={hc}")
+    Y, A = orc.apply(sp, xs)
+    assert orc.max_rel_err(y0, Y, A) <= TOL1
