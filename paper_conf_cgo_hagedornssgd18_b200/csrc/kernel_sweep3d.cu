@@ -961,7 +961,11 @@ Launcher pick(const StencilParams& p) {
     if (R == 1) return get_launcher_zf<K2_WSTAR, 1, 2, 7, 0>(zc, fz);
     return get_launcher_zf<K2_WSTAR, 2, 2, 8, 0>(zc, fz);
   }
-  // point-wise ring depth tuning hook (LIFT_K2_PW: 1 = the round-1 (S, 3) rings)
+  // the point-wise grid's TMA ring was the top stall of Acoustic-13 (16.6% of
+  // samples waiting on it with 3 slots): radius 1 takes 5 slots (Acoustic-7
+  // 484 -> 506, Hotspot3D 276 -> 305 Gpts/s).  LIFT_K2_PW=1: the round-1
+  // (S, 3) rings.  (Reading it with global loads two planes ahead instead of
+  // a ring measured 20% slower: register spills.)
   const char* e = getenv("LIFT_K2_PW");
   const int pv = e ? atoi(e) : 0;
   if (p.op == OP_HOTSPOT3D) {
@@ -972,9 +976,11 @@ Launcher pick(const StencilParams& p) {
     if (pv == 1) return get_launcher_zf<K2_ACOUSTIC, 1, 2, 5, 3>(zc, fz);
     return get_launcher_zf<K2_ACOUSTIC, 1, 2, 5, 5>(zc, fz);
   }
+  // radius 2: the 5 live planes need a deep plane ring too; (7 plane stages,
+  // 4 point-wise slots) fits 2 CTAs per SM (Acoustic-13 1024^3: 451 Gpts/s
+  // vs 448 for (8, 3) and 411 for (6, 5))
   if (pv == 1) return get_launcher_zf<K2_ACOUSTIC, 2, 2, 8, 3>(zc, fz);
-  if (pv == 2) return get_launcher_zf<K2_ACOUSTIC, 2, 2, 7, 4>(zc, fz);
-  return get_launcher_zf<K2_ACOUSTIC, 2, 2, 6, 5>(zc, fz);
+  return get_launcher_zf<K2_ACOUSTIC, 2, 2, 7, 4>(zc, fz);
 }
 
 struct MapEntry {
