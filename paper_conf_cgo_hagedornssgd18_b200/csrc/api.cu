@@ -26,8 +26,17 @@ struct stencil_plan_s {
   int32_t forced_variant = STENCIL_VARIANT_AUTO;
   int32_t time_block = 1;          // stencil_iterate: time steps per pass where K2T applies (opt-in, see DESIGN)
   int32_t last_variant = STENCIL_VARIANT_GENERIC;
-  // OP_SRAD: device workspace {partials of the q0 reduction, q0 constants}
+  // OP_SRAD: device workspace {2 x partials of the q0 reduction, q0 constants}
   void* srad_ws = nullptr;
+  // OP_SRAD inside stencil_iterate: the fused pass left the statistics of the
+  // image it wrote (srad_chain_img) in partials buffer srad_chain_buf
+  // (srad_chain_n entries), so the next pass skips the reduction over I.
+  // Only set while stencil_iterate runs (between API calls the caller may
+  // rewrite any buffer).
+  bool srad_chain = false;
+  const float* srad_chain_img = nullptr;
+  int srad_chain_buf = 0;
+  int srad_chain_n = 0;
   // stencil_run_host workspace (device)
   std::vector<float*> ws;
   size_t ws_elems = 0;
@@ -115,19 +124,48 @@ int choose_variant(stencil_plan_s* pl, const float* in0, const float* in1, const
 stencil_status launch(stencil_plan_s* pl, const StencilParams& p_in, const float* in0, const float* in1,
                       float* out, cudaStream_t stream) {
   StencilParams p = p_in;
+  const int v = choose_variant(pl, in0, in1, out);
+  if (v < 0) return fail(STENCIL_E_UNSUPPORTED, "forced kernel variant cannot run this plan/pointers");
+  pl->last_variant = v;
   if (p.op == OP_SRAD) {
-    // q0^2 of the current image first (deterministic two-pass fp64 reduction)
     if (!pl->srad_ws) {
       cudaError_t e = cudaMalloc(&pl->srad_ws, srad_workspace_bytes(pl->num_sms));
       if (e != cudaSuccess) return cuda_fail(e, "cudaMalloc (SRAD workspace)");
     }
-    cudaError_t e = launch_srad_q0(in0, p.n[1] * p.n[2], pl->srad_ws, pl->num_sms, stream);
+    const int64_t npts = p.n[1] * p.n[2];
+    if (v == STENCIL_VARIANT_TILE2D) {
+      // K1S: q0 from partials of in0 (reduced inside the pass), which also
+      // writes the partials of out; the image is read for q0 only when no
+      // earlier pass of this iterate chain left its statistics
+      int src = 0, n_in = 0;
+      if (pl->srad_chain && pl->srad_chain_img == in0 && pl->srad_chain_n > 0) {
+        src = pl->srad_chain_buf;
+        n_in = pl->srad_chain_n;
+      } else {
+        cudaError_t e = launch_srad_partials(in0, npts, srad_partials_ptr(pl->srad_ws, pl->num_sms, 0), pl->num_sms,
+                                             stream, &n_in);
+        if (e != cudaSuccess) return cuda_fail(e, "SRAD q0 partials");
+      }
+      p.srad_part_in = srad_partials_ptr(pl->srad_ws, pl->num_sms, src);
+      p.srad_nparts = n_in;
+      p.srad_part_out = srad_partials_ptr(pl->srad_ws, pl->num_sms, 1 - src);
+      std::string err;
+      int n_out = 0;
+      cudaError_t e = launch_srad_fused(p, in0, out, stream, pl->num_sms, &err, &n_out);
+      if (e != cudaSuccess)
+        return fail(STENCIL_E_CUDA, std::string("kernel launch failed: ") + cudaGetErrorString(e) + " " + err);
+      if (pl->srad_chain) {
+        pl->srad_chain_img = out;
+        pl->srad_chain_buf = 1 - src;
+        pl->srad_chain_n = n_out;
+      }
+      return STENCIL_OK;
+    }
+    // generic kernel: q0^2 of the current image first (deterministic fp64 reduction)
+    cudaError_t e = launch_srad_q0(in0, npts, pl->srad_ws, pl->num_sms, stream);
     if (e != cudaSuccess) return cuda_fail(e, "SRAD q0 reduction");
     p.srad_q0 = srad_q0_ptr(pl->srad_ws, pl->num_sms);
   }
-  const int v = choose_variant(pl, in0, in1, out);
-  if (v < 0) return fail(STENCIL_E_UNSUPPORTED, "forced kernel variant cannot run this plan/pointers");
-  pl->last_variant = v;
   std::string err;
   cudaError_t e;
   switch (v) {
@@ -519,6 +557,18 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
         ri = 1 - ri;
       }
     }
+    // SRAD: each fused pass hands the statistics of its output to the next
+    struct ChainGuard {
+      stencil_plan_s* pl;
+      ~ChainGuard() {
+        pl->srad_chain = false;
+        pl->srad_chain_img = nullptr;
+        pl->srad_chain_n = 0;
+      }
+    } chain_guard{pl};
+    pl->srad_chain = p.op == OP_SRAD;
+    pl->srad_chain_img = nullptr;
+    pl->srad_chain_n = 0;
     for (; t < n_steps; ++t) {
       const float* in[1] = {state[ri]};
       stencil_status s = stencil_apply(pl, in, 1, state[1 - ri], stream);

@@ -8,6 +8,8 @@
 #pragma once
 #include <cstdint>
 
+#include <vector_types.h>
+
 namespace lift {
 
 enum PadKind : int { PAD_CLAMP = 0, PAD_MIRROR = 1, PAD_WRAP = 2, PAD_CONSTANT = 3, PAD_REFLECT = 4 };
@@ -59,13 +61,20 @@ struct StencilParams {
   unsigned int* sig_lo;
   unsigned int* sig_hi;
   unsigned int sig_value;
+  // OP_SRAD (full iteration): device array {q0sqr, a, b} written by the q0
+  // reduction before the stencil launch (SRAD1's constants, op_srad1)
+  const float* srad_q0;
+  // OP_SRAD, fused pass (K1S): q0 from srad_nparts fp64 (sum, sum of squares)
+  // partials of the input image (reduced in-kernel, fixed order), and this
+  // launch's own output statistics, one partial per CTA, into srad_part_out
+  // (so the next iteration needs no reduction pass over I)
+  const double2* srad_part_in;
+  double2* srad_part_out;
+  int32_t srad_nparts;
   // single-launch fused step: before loading ghost planes (first / last
   // z-chunk) the producer waits until *wait_lo / *wait_hi >= wait_value
   // (acquire, system scope); the boundary chunks are scheduled first and the
   // neighbours' flags are raised as soon as their chunk is complete
-  // OP_SRAD (full iteration): device array {q0sqr, a, b} written by the q0
-  // reduction before the stencil launch (SRAD1's constants, op_srad1)
-  const float* srad_q0;
   const unsigned int* wait_lo;
   const unsigned int* wait_hi;
   unsigned int wait_value;

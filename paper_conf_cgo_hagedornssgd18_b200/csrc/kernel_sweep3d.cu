@@ -72,7 +72,10 @@ __device__ __forceinline__ void spin_until(const unsigned int* f, unsigned int v
   while ((int)(ld_acquire_sys(f) - v) < 0) __nanosleep(32);
 }
 
-enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2, K2_WBOX = 3 };
+enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2, K2_WBOX = 3, K2_WBOX19 = 4 };
+// 3x3x3 box weights; K2_WBOX19: the 8 corner taps are zero (Poisson 19-point)
+// and are skipped at compile time (19 instead of 27 FMAs per point)
+constexpr bool is_box(int op) { return op == K2_WBOX || op == K2_WBOX19; }
 
 template <int R, int RPW, int S, int PSN>
 struct Cfg {
@@ -135,7 +138,7 @@ __device__ __forceinline__ float pick4(int s, const float4& c, float pv) {
 }
 
 template <int OP, int R, int RPW, int S, bool ZC, bool FZ, int PSN>
-__global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW == 1)) ? 3 : 2)
+__global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 1)) ? 3 : 2)
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
              const __grid_constant__ CUtensorMap pwmap, const float* __restrict__ src, float* out, int ntx,
              int nty, int zc, int nchunk, int slot) {
@@ -360,7 +363,7 @@ __global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW =
       // so every plane of a window — not only the centre — is complete
       // (box windows read the halo of every plane: fix each plane on arrival;
       // star windows read only the centre plane's halo: fix the centre)
-      constexpr bool FIX_ON_ARRIVAL = OP == K2_WBOX;
+      constexpr bool FIX_ON_ARRIVAL = is_box(OP);
       auto fix_plane = [&](int stage, int64_t gzp) {
         if (stage_const[stage]) return;
         fixup_tile<R, R, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + stage * SF4), src,
@@ -404,7 +407,7 @@ __global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW =
         // it).  Every output's FMA chain still runs over its 27 taps in
         // row-major (kz, ky, kx) order from 0 — K0's order, so the bits agree.
         float P1[RPW][4], P0[RPW][4];     // partial sums of outputs q and q+1
-        if constexpr (OP == K2_WBOX) {
+        if constexpr (is_box(OP)) {
 #pragma unroll
           for (int jj = 0; jj < RPW; ++jj)
 #pragma unroll
@@ -437,11 +440,13 @@ __global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW =
                 const float w2 = p.wbox[(2 * 3 + kyy) * 3 + kxx];
                 const float w1 = p.wbox[(1 * 3 + kyy) * 3 + kxx];
                 const float w0 = p.wbox[(0 * 3 + kyy) * 3 + kxx];
+                // corner taps (kz, ky, kx all off-centre) of the 19-point pattern
+                const bool corner = OP == K2_WBOX19 && kyy != 1 && kxx != 1;
 #pragma unroll
                 for (int i = 0; i < 4; ++i) {
-                  O[jj][i] = __fmaf_rn(w2, w6[i + kxx], O[jj][i]);
+                  if (!corner) O[jj][i] = __fmaf_rn(w2, w6[i + kxx], O[jj][i]);
                   N1[jj][i] = __fmaf_rn(w1, w6[i + kxx], N1[jj][i]);
-                  N0[jj][i] = __fmaf_rn(w0, w6[i + kxx], N0[jj][i]);
+                  if (!corner) N0[jj][i] = __fmaf_rn(w0, w6[i + kxx], N0[jj][i]);
                 }
               }
             }
@@ -466,7 +471,7 @@ __global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW =
             }
           }
           if (++sn == S) { sn = 0; ++pn; }
-          if constexpr (OP == K2_WBOX) {
+          if constexpr (is_box(OP)) {
             float O[RPW][4];
             box_plane(zst[k], O);          // O: not an output yet
           }
@@ -499,10 +504,10 @@ __global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW =
           if constexpr (PW) mbar_wait(&pwfull[psc], ppc & 1);
           // box: plane z+1 completes output z
           float BO[RPW][4];
-          if constexpr (OP == K2_WBOX) box_plane(zst[2], BO);
+          if constexpr (is_box(OP)) box_plane(zst[2], BO);
           // star ops: rows -R .. RPW-1+R of the centre plane, each read once
           float4 cr[RPW + 2 * R];
-          if constexpr (OP != K2_WBOX) {
+          if constexpr (!is_box(OP)) {
 #pragma unroll
             for (int d = 0; d < RPW + 2 * R; ++d) cr[d] = dsm4[cbase + roff4 + RO(d)];
           }
@@ -520,7 +525,7 @@ __global__ void __launch_bounds__(NCONS + 32, (OP != K2_WBOX && (R == 1 || RPW =
               return dsm4[a + rb];
             };
             float4 res;
-            if constexpr (OP == K2_WBOX) {
+            if constexpr (is_box(OP)) {
               res = make_float4(BO[jj][0], BO[jj][1], BO[jj][2], BO[jj][3]);
             } else {
               float xw[4 + 2 * R];                    // centre row, x offsets -R .. 3+R
@@ -957,8 +962,23 @@ Launcher pick(const StencilParams& p) {
   const bool zc = p.kind[0] == PAD_CONSTANT && p.pad_value != 0.0f;
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;   // fused halo launch
   if (p.op == OP_WEIGHTED) {
-    if (R == 1 && !star_weights(p, 1)) return get_launcher_zf<K2_WBOX, 1, 2, 7, 0>(zc, fz);
+    if (R == 1 && !star_weights(p, 1)) {
+      bool corners = false;
+      for (int kz = 0; kz < 3; kz += 2)
+        for (int ky = 0; ky < 3; ky += 2)
+          for (int kx = 0; kx < 3; kx += 2) corners |= p.wbox[(kz * 3 + ky) * 3 + kx] != 0.0f;
+      if (!corners) {
+        const char* eb = getenv("LIFT_K2_BOX");      // A/B: (rows per warp, stages)
+        if (eb && atoi(eb) == 1) return get_launcher_zf<K2_WBOX19, 1, 1, 8, 0>(zc, fz);
+        if (eb && atoi(eb) == 2) return get_launcher_zf<K2_WBOX19, 1, 3, 6, 0>(zc, fz);
+        return get_launcher_zf<K2_WBOX19, 1, 2, 7, 0>(zc, fz);
+      }
+      return get_launcher_zf<K2_WBOX, 1, 2, 7, 0>(zc, fz);
+    }
     if (R == 1) return get_launcher_zf<K2_WSTAR, 1, 2, 7, 0>(zc, fz);
+    const char* e2 = getenv("LIFT_K2_R2");            // A/B: (rows per warp, stages)
+    if (e2 && atoi(e2) == 1) return get_launcher_zf<K2_WSTAR, 2, 1, 8, 0>(zc, fz);
+    if (e2 && atoi(e2) == 2) return get_launcher_zf<K2_WSTAR, 2, 3, 6, 0>(zc, fz);
     return get_launcher_zf<K2_WSTAR, 2, 2, 8, 0>(zc, fz);
   }
   // the point-wise grid's TMA ring was the top stall of Acoustic-13 (16.6% of

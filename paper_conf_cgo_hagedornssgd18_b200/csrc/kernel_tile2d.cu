@@ -38,6 +38,7 @@ constexpr int TX = 128;
 constexpr int XH = 4;
 constexpr int BX = TX + 2 * XH;
 constexpr int NW = 8;
+constexpr int kSradMaxParts = 2048;     // q0 partials one K1S pass can reduce (8 per consumer thread)
 constexpr int NCONS = NW * 32;
 constexpr unsigned FULL = 0xffffffffu;
 
@@ -342,8 +343,8 @@ struct CRowsAcc {                // c at (y, x+i) = cy[i], (y+1, x+i) = cs[i]
   }
 };
 
-template <int RPW, int S>
-__global__ void __launch_bounds__(NCONS + 32, 3)
+template <int RPW, int S, int MINB>
+__global__ void __launch_bounds__(NCONS + 32, MINB)
     k1_srad_fused(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap map0,
                   const float* __restrict__ src0, float* __restrict__ out, int ntx, int nty) {
   using C = Cfg<2, RPW, S, 1>;
@@ -386,7 +387,44 @@ __global__ void __launch_bounds__(NCONS + 32, 3)
   }
   const int nx = (int)p.n[2], ny = (int)p.n[1];
   const int kx = p.kind[2], ky = p.kind[1];
-  const float* q = p.srad_q0;
+  // q0 of the input image: reduce the previous pass's (or k_sum2's) fp64
+  // partials here, in a fixed order (so every CTA gets the same bits), while
+  // the producer's first TMA loads are already in flight
+  __shared__ double2 s_red[NW];
+  float q[3];                      // SRAD1's constants {q0, a, b} in registers
+  if (!p.srad_part_in) {
+#pragma unroll
+    for (int k = 0; k < 3; ++k) q[k] = p.srad_q0[k];
+  } else {
+    constexpr int K = kSradMaxParts / NCONS;
+    double2 v[K];
+#pragma unroll
+    for (int k = 0; k < K; ++k) {
+      const int i = threadIdx.x + k * NCONS;
+      v[k] = i < p.srad_nparts ? p.srad_part_in[i] : make_double2(0.0, 0.0);
+    }
+    double a = 0.0, b = 0.0;
+#pragma unroll
+    for (int k = 0; k < K; ++k) {
+      a += v[k].x;
+      b += v[k].y;
+    }
+    for (int o = 16; o > 0; o >>= 1) {
+      a += __shfl_down_sync(0xffffffffu, a, o);
+      b += __shfl_down_sync(0xffffffffu, b, o);
+    }
+    if (lane == 0) s_red[warp] = make_double2(a, b);
+    named_bar_sync(1, NCONS);
+    a = b = 0.0;
+#pragma unroll
+    for (int w = 0; w < NW; ++w) {
+      a += s_red[w].x;
+      b += s_red[w].y;
+    }
+    srad1_constants(srad_q0sqr(a, b, p.n[1] * p.n[2]), q);
+    named_bar_sync(1, NCONS);      // s_red is reused for this pass's own statistics
+  }
+  double st_s = 0.0, st_ss = 0.0;  // statistics of the written image (next iteration's q0)
   const int r0 = warp * RPW;
   int s = 0;
   uint32_t pass = 0;
@@ -445,13 +483,37 @@ __global__ void __launch_bounds__(NCONS + 32, 3)
             v[ii] = op_srad2(CRowsAcc<ii>{cr[o % 3], cr[(o + 1) % 3]},
                              RowsAcc<2, ii>{iw[o % 4], iw[(o + 1) % 4], iw[(o + 2) % 4]}, p.prm);
           });
-          if (x_ok && y0 + r0 + o < ny) stg128(orow + (int64_t)o * nx, make_float4(v[0], v[1], v[2], v[3]));
+          if (x_ok && y0 + r0 + o < ny) {
+            stg128(orow + (int64_t)o * nx, make_float4(v[0], v[1], v[2], v[3]));
+#pragma unroll
+            for (int ii = 0; ii < 4; ++ii) {
+              const double d = v[ii];
+              st_s += d;
+              st_ss = fma(d, d, st_ss);
+            }
+          }
         }
       }
     });
     __syncwarp();
     if (lane == 0) mbar_arrive(&empty[s]);
     if (++s == S) { s = 0; ++pass; }
+  }
+  if (p.srad_part_out) {
+    for (int o = 16; o > 0; o >>= 1) {
+      st_s += __shfl_down_sync(0xffffffffu, st_s, o);
+      st_ss += __shfl_down_sync(0xffffffffu, st_ss, o);
+    }
+    if (lane == 0) s_red[warp] = make_double2(st_s, st_ss);
+    named_bar_sync(1, NCONS);
+    if (threadIdx.x == 0) {
+      double a = 0.0, b = 0.0;
+      for (int w = 0; w < NW; ++w) {
+        a += s_red[w].x;
+        b += s_red[w].y;
+      }
+      p.srad_part_out[blockIdx.x] = make_double2(a, b);
+    }
   }
 }
 
@@ -559,26 +621,45 @@ bool get_map(const float* base, int64_t nx, int64_t ny, int by, CUtensorMap* out
 
 }  // namespace
 
-cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* out, cudaStream_t stream,
-                              int num_sms, std::string* err) {
-  constexpr int RPW = 6, S = 2;
-  using C = Cfg<2, RPW, S, 1>;
+template <int RPW, int S, int MINB>
+Launcher srad_fused_launcher() {
   static Launcher L{};
   static std::once_flag once;
   std::call_once(once, [] {
-    auto fn = k1_srad_fused<RPW, S>;
+    using C = Cfg<2, RPW, S, 1>;
+    auto fn = k1_srad_fused<RPW, S, MINB>;
     cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
     int occ = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, NCONS + 32, C::SMEM) != cudaSuccess) occ = 1;
     cudaGetLastError();
     L = Launcher{reinterpret_cast<const void*>(fn), C::SMEM, C::TY, 2, 1, occ > 0 ? occ : 1};
   });
+  return L;
+}
+
+cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* out, cudaStream_t stream,
+                              int num_sms, std::string* err, int* nparts_out) {
+  // (rows per warp, stages, min CTAs/SM); LIFT_SRAD_SHAPE overrides (A/B sweeps)
+  const char* env = getenv("LIFT_SRAD_SHAPE");
+  Launcher L;
+  switch (env ? atoi(env) : 0) {
+    case 1: L = srad_fused_launcher<6, 2, 2>(); break;
+    case 2: L = srad_fused_launcher<4, 3, 2>(); break;
+    case 3: L = srad_fused_launcher<6, 3, 2>(); break;
+    case 4: L = srad_fused_launcher<4, 2, 3>(); break;
+    default: L = srad_fused_launcher<6, 2, 3>(); break;
+  }
   CUtensorMap m0;
   if (!get_map(in0, p.n[2], p.n[1], L.ty + 4, &m0, err)) return cudaErrorInvalidValue;
   const int ntx = (int)((p.n[2] + TX - 1) / TX);
   const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);
   int64_t grid = (int64_t)num_sms * L.ctas_per_sm;
   if (grid > (int64_t)ntx * nty) grid = (int64_t)ntx * nty;
+  if (p.srad_part_in && p.srad_nparts > kSradMaxParts) {
+    *err = "SRAD: too many q0 partials";
+    return cudaErrorInvalidValue;
+  }
+  if (nparts_out) *nparts_out = (int)grid;
   void* args[] = {(void*)&p, (void*)&m0, (void*)&in0, (void*)&out, (void*)&ntx, (void*)&nty};
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, true);
 }
@@ -602,7 +683,7 @@ bool tile2d_supported(const StencilParams& p) {
 
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,
                           cudaStream_t stream, int num_sms, std::string* err) {
-  if (p.op == OP_SRAD) return launch_srad_fused(p, in0, out, stream, num_sms, err);
+  if (p.op == OP_SRAD) return launch_srad_fused(p, in0, out, stream, num_sms, err, nullptr);
   const bool small = ((p.n[2] + TX - 1) / TX) * ((p.n[1] + 6 * NW - 1) / (6 * NW)) < num_sms;
   // per-warp streaming sweeps (K3) where they measured faster than the tiles
   if (wsweep2d_supported(p, in0, in1, small)) return launch_wsweep2d(p, in0, in1, out, stream, num_sms, err);

@@ -70,8 +70,17 @@ cudaError_t launch_wsweep2d(const StencilParams& p, const float* in0, const floa
 // OP_SRAD: q0^2 = var/mean^2 of the image (fp64, deterministic) into the
 // workspace, as SRAD1's constants {q0, a, b}
 size_t srad_workspace_bytes(int num_sms);
+int srad_partials_cap(int num_sms);
+double2* srad_partials_ptr(void* ws, int num_sms, int which);     // which = 0 / 1 (ping-pong)
 const float* srad_q0_ptr(void* ws, int num_sms);
 cudaError_t launch_srad_q0(const float* img, int64_t n, void* ws, int num_sms, cudaStream_t stream);
+// (sum, sum of squares) partials of the image only (first iteration of a fused chain)
+cudaError_t launch_srad_partials(const float* img, int64_t n, double2* partials, int num_sms, cudaStream_t stream,
+                                 int* nparts);
+// K1S: the fused SRAD pass; p.srad_part_in/srad_nparts/srad_part_out set;
+// *nparts_out = partials written (one per CTA)
+cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* out, cudaStream_t stream,
+                              int num_sms, std::string* err, int* nparts_out);
 
 // wait (one thread, acquire.sys) until *a >= value and *b >= value (NULL = skip)
 cudaError_t launch_wait_signals(const unsigned int* a, const unsigned int* b, unsigned int value,

@@ -120,6 +120,14 @@ __host__ __device__ inline void srad1_constants(float q0f, float* out3) {
   out3[2] = (float)(1.0 / (q0 * (1.0 + q0)));
 }
 
+// q0^2 = var(I) / mean(I)^2 from fp64 (sum, sum of squares) over n points
+// (Rodinia SRAD's per-iteration statistic; A27)
+__host__ __device__ inline float srad_q0sqr(double s, double ss, int64_t n) {
+  const double mean = s / (double)n;
+  const double var = ss / (double)n - mean * mean;
+  return (float)(var / (mean * mean));
+}
+
 // ---- SRAD kernel 2: (c, I) -> I' (Rodinia v3.1 srad; A18) --------
 template <class AccC, class AccI>
 __device__ __forceinline__ float op_srad2(const AccC& C, const AccI& I, const float* prm) {

@@ -176,7 +176,8 @@ def _variants(plan_nd):
 
 
 @pytest.mark.parametrize("case", ["j2d5", "gauss", "j3d7", "j3d13", "hotspot", "acoustic13", "srad1", "srad2",
-                                  "box27_wrap", "box27_const", "box27_mirror"])
+                                  "box27_wrap", "box27_const", "box27_mirror", "box19_wrap", "box19_const",
+                                  "box19_clamp"])
 def test_kernel_families_bitwise_equal(lift, case):
     """Tiling independence: every kernel family gives the same bits."""
     rng = np.random.default_rng(24)
@@ -194,9 +195,11 @@ def test_kernel_families_bitwise_equal(lift, case):
     elif case == "acoustic13":
         sp = spec((19, 37, 136), 5, op=si.ACOUSTIC, params=si.params_acoustic(13), kind=CONSTANT)
         xs = [rnd((19, 37, 136), 31, -1, 1), rnd((19, 37, 136), 32, -1, 1)]
-    elif case.startswith("box27"):
-        k = {"wrap": WRAP, "const": CONSTANT, "mirror": MIRROR}[case.split("_")[1]]
+    elif case.startswith("box"):
+        k = {"wrap": WRAP, "const": CONSTANT, "mirror": MIRROR, "clamp": CLAMP}[case.split("_")[1]]
         w = np.random.default_rng(54).standard_normal((3, 3, 3)).astype(np.float32)
+        if case.startswith("box19"):        # zero corners: the 19-point kernel (corner taps skipped)
+            w[::2, ::2, ::2] = 0.0
         sp, xs = spec((19, 37, 264), 3, w, (k, k, k), value=0.7), [rnd((19, 37, 264), 55)]
     elif case == "srad1":
         I = np.exp(rnd((130, 264), 33, 0, 1)).astype(np.float32)
@@ -394,6 +397,30 @@ def test_srad_iteration(lift, kind):
     ri = plan.iterate([a, b], 10)
     g = (a, b)[ri].cpu().numpy()
     ref = orc.iterate(sp, [I], [], 10)[0]
+    assert np.max(np.abs(g - ref) / np.abs(ref)) <= TOL10
+
+
+@pytest.mark.parametrize("shape", [(2500, 2052), (97, 260)])
+def test_srad_iterate_chain(lift, shape):
+    """stencil_iterate hands each fused pass's q0 statistics (per-CTA fp64
+    partials of the image it wrote) to the next pass instead of re-reducing
+    the image: the chain agrees with step-by-step applies (each reducing its
+    own input) to fp64-sum rounding, and with the oracle after 6 iterations.
+    (2500, 2052): more tiles than resident CTAs, ragged in y."""
+    I = np.exp(rnd(shape, 63, 0.0, 1.0)).astype(np.float32)
+    sp = spec(I.shape, 3, op=si.SRAD, params=si.params_srad2(), kind=CLAMP)
+    plan = lift.Plan.from_spec(sp)
+    a = torch.from_numpy(I).cuda()
+    b = torch.empty_like(a)
+    ri = plan.iterate([a, b], 6)
+    assert plan.variant == 1
+    g = (a, b)[ri].cpu().numpy()
+    x = torch.from_numpy(I).cuda()
+    for _ in range(6):
+        x = plan.apply(x)
+    h = x.cpu().numpy()
+    assert np.max(np.abs(g - h) / np.abs(h)) <= 1e-6
+    ref = orc.iterate(sp, [I], [], 6)[0]
     assert np.max(np.abs(g - ref) / np.abs(ref)) <= TOL10
 
 
