@@ -216,6 +216,10 @@ stencil_status stencil_wait_signals(const uint32_t* sig_a, const uint32_t* sig_b
  *   WEIGHTED  : state {X0, X1}            X_{t+1} = S(X_t), ping-pong
  *   HOTSPOT3D, HOTSPOT2D : state {T0, T1}, aux {P}   T_{t+1} = S(T_t, P)
  *   GRADIENT, SRAD : state {X0, X1}       ping-pong like WEIGHTED
+ *     (SRAD: each fused pass also writes the fp64 q0 statistics of the image
+ *     it produced to the plan's workspace and the next pass of this call
+ *     reduces those instead of re-reading the image; only the first pass
+ *     reads X0 once more for its q0)
  *   ACOUSTIC  : state {prev, cur}         next overwrites prev; roles swap
  * *result_index receives the index into ``state`` holding the newest grid.
  * Requires output extents == input extents.

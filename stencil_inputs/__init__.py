@@ -372,3 +372,49 @@ def make_workload_inputs(w: Workload) -> Tuple[List[np.ndarray], StencilSpec]:
     if spec.op == SRAD1:
         spec.params = params_srad1(srad_q0sqr(xs[0]))
     return xs, spec
+
+
+# ---- counter-based grids for sizes too large to draw on the host ----------
+# value(i) = 1 + (h(i) >> 9) * 2^-23 in [1, 2), exact in fp32, where h is a
+# 32-bit integer hash of the linear index i.  The device side evaluates the
+# same integer formula with torch int64 ops (hash_grid_torch); the oracle side
+# reads single points through HashGrid[...] (no arithmetic of the method).
+_M32 = 0xFFFFFFFF
+
+
+def _hash32(i: int, seed: int) -> int:
+    h = (i * 2654435761 + seed) & _M32
+    h ^= h >> 15
+    h = (h * 2246822519) & _M32
+    h ^= h >> 13
+    return h
+
+
+class HashGrid:
+    """Read-only fp32 grid of the given extents whose element at linear index i
+    is ``1 + (hash32(i, seed) >> 9) * 2**-23``; indexable by index tuples."""
+
+    def __init__(self, extents: Sequence[int], seed: int):
+        self.shape = tuple(int(e) for e in extents)
+        self.seed = int(seed)
+        self.strides = tuple(int(np.prod(self.shape[d + 1:])) for d in range(len(self.shape)))
+
+    def __getitem__(self, idx) -> np.float32:
+        lin = sum(int(i) * s for i, s in zip(idx, self.strides))
+        return np.float32(1.0 + (_hash32(lin, self.seed) >> 9) * 2.0 ** -23)
+
+
+def hash_grid_torch(extents: Sequence[int], seed: int, device, chunk: int = 1 << 26):
+    """The HashGrid values materialised on ``device`` (torch int64 arithmetic
+    in chunks; int64 products wrap mod 2^64, so the low 32 bits are exact)."""
+    import torch
+    n = int(np.prod(extents))
+    out = torch.empty(n, dtype=torch.float32, device=device)
+    for a in range(0, n, chunk):
+        b = min(n, a + chunk)
+        h = (torch.arange(a, b, dtype=torch.int64, device=device) * 2654435761 + seed) & _M32
+        h ^= h >> 15
+        h = (h * 2246822519) & _M32
+        h ^= h >> 13
+        out[a:b] = ((h >> 9).to(torch.float32) * 2.0 ** -23) + 1.0
+    return out.view(*extents)

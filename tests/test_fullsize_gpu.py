@@ -175,3 +175,24 @@ def test_srad_iteration_4096(lift):
     g = y.cpu().numpy()
     err = max(abs(float(g[p]) - Y[p]) / max(abs(Y[p]), A[p]) for p in pts)
     assert err <= 1e-5
+
+
+@pytest.mark.parametrize("kind", [si.CLAMP, si.WRAP])
+def test_beyond_2pow31_elements_3d(lift, kind):
+    """Maximum sizes: a (2050, 1024, 1024) grid (2.15e9 elements, 8.6 GB per
+    buffer) — linear offsets past 2^31 in the 3D sweep (K2); J3D7 weights,
+    counter-based input (stencil_inputs.HashGrid), sampled points including
+    the last planes, checked one by one against the oracle."""
+    ext = (2050, 1024, 1024)
+    w = si.weights_j3d7()
+    spec = si.StencilSpec(ext, (3, 3, 3), (1, 1, 1), (1, 1, 1), (1, 1, 1), (kind,) * 3, 0.0, si.WEIGHTED, w, ())
+    x = si.hash_grid_torch(ext, 2024, "cuda")
+    plan = lift.Plan.from_spec(spec)
+    y = plan.apply(x)
+    torch.cuda.synchronize()
+    assert plan.variant == 2
+    del x
+    pts = samples(ext, 300, 19) + [(ext[0] - 1 - k, 1023 - k, 1023 - 3 * k) for k in range(8)]
+    check_points(spec, [si.HashGrid(ext, 2024)], y, pts)
+    del y
+    torch.cuda.empty_cache()
