@@ -68,6 +68,14 @@ __device__ __forceinline__ int chunk_of(int c, int nchunk, bool fused) {
   return c == 0 ? 0 : (c == 1 ? nchunk - 1 : c - 1);
 }
 
+// first plane (relative to reg0) of z-chunk c: the first n1 chunks hold zc
+// planes, the rest zc2 (guided schedule: the last waves of items are short,
+// so the launch's tail — CTAs still finishing their last item while the
+// others idle — is short too)
+__device__ __forceinline__ int64_t chunk_z0(int c, int zc, int n1, int zc2) {
+  return c < n1 ? (int64_t)c * zc : (int64_t)n1 * zc + (int64_t)(c - n1) * zc2;
+}
+
 __device__ __forceinline__ void spin_until(const unsigned int* f, unsigned int v) {
   while ((int)(ld_acquire_sys(f) - v) < 0) __nanosleep(32);
 }
@@ -141,7 +149,7 @@ template <int OP, int R, int RPW, int S, bool ZC, bool FZ, int PSN>
 __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 1)) ? 3 : 2)
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
              const __grid_constant__ CUtensorMap pwmap, const float* __restrict__ src, float* out, int ntx,
-             int nty, int zc, int nchunk, int slot) {
+             int nty, int zc, int nchunk, int slot, int n1, int zc2) {
   using C = Cfg<R, RPW, S, (OP == K2_HOTSPOT || OP == K2_ACOUSTIC) ? PSN : 0>;
   constexpr bool PW = OP == K2_HOTSPOT || OP == K2_ACOUSTIC;           // a point-wise zipped grid (Hotspot P, Acoustic prev)
   constexpr int PS = C::PS;                     // point-wise ring slots
@@ -213,8 +221,8 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
           const int chunk = chunk_of(item / ntile, nchunk, FZ && p.fused_step), tile = item % ntile;
           x0 = (tile % ntx) * TX;
           y0 = (tile / ntx) * TY;
-          zs = p.reg0 + (int64_t)chunk * zc;
-          const int64_t ze = min(zs + (int64_t)zc, p.reg1);
+          zs = p.reg0 + chunk_z0(chunk, zc, n1, zc2);
+          const int64_t ze = min(zs + (int64_t)(chunk < n1 ? zc : zc2), p.reg1);
           nload = (int)(ze - zs) + 2 * R;
           // fused step: the ghost planes of this chunk must hold the neighbours'
           // previous step before the TMA reads them
@@ -255,8 +263,8 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
         if (item < 0) break;
         const int chunk = chunk_of(item / ntile, nchunk, FZ && p.fused_step), tile = item % ntile;
         const int x0 = (tile % ntx) * TX, y0 = (tile / ntx) * TY;
-        const int64_t zs = p.reg0 + (int64_t)chunk * zc;
-        const int nzc = (int)(min(zs + (int64_t)zc, p.reg1) - zs);
+        const int64_t zs = p.reg0 + chunk_z0(chunk, zc, n1, zc2);
+        const int nzc = (int)(min(zs + (int64_t)(chunk < n1 ? zc : zc2), p.reg1) - zs);
         for (int j = 0; j < nzc; ++j) {
           if (ppass > 0) mbar_wait(&pwempty[ps], (ppass - 1) & 1);
           mbar_arrive_expect_tx(&pwfull[ps], C::PW_BYTES);
@@ -301,8 +309,8 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
       const int chunk = chunk_of(item / ntile, nchunk, FZ && p.fused_step), tile = item % ntile;
       const int x0 = (tile % ntx) * TX;
       const int y0 = (tile / ntx) * TY;
-      const int64_t zs = p.reg0 + (int64_t)chunk * zc;
-      const int nzc = (int)(min(zs + (int64_t)zc, p.reg1) - zs);
+      const int64_t zs = p.reg0 + chunk_z0(chunk, zc, n1, zc2);
+      const int nzc = (int)(min(zs + (int64_t)(chunk < n1 ? zc : zc2), p.reg1) - zs);
       const int xo = x0 + 4 * lane;
       const bool x_ok = xo < nx;
       const bool y_edge = (y0 < R) || (y0 + TY + R > ny);
@@ -1088,17 +1096,53 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
       }
     }
   }
+  // Large grids, measured per kernel family (profiles/r01_sweep_zchunk.txt):
+  // the memory-bound radius-1 sweeps (7-point weighted star, Acoustic-7) run
+  // fastest with short chunks — CTAs in flight then stay within a narrow z
+  // window (halo planes and rows are L2 hits) and the launch's tail is short:
+  // J3D7 512^3 766 -> 825 Gpts/s at 6 planes (~20 planes' worth of items in
+  // flight for the weighted star, ~40 for Acoustic, whose items carry a
+  // point-wise grid); the instruction-heavier radius-2 and box sweeps keep
+  // long chunks (their 2R warm-up planes per chunk cost issue slots) and only
+  // shorten the chunks of the last waves (guided tail).
+  int64_t tail_zc = 0;
+  if (work >= 16 * slots && !p.fused_step) {
+    const bool box = p.op == OP_WEIGHTED && !star_weights(p, 1);
+    if (R == 1 && !box && (p.op == OP_WEIGHTED || p.op == OP_ACOUSTIC)) {
+      const int64_t k = p.op == OP_ACOUSTIC ? 40 : 20;
+      zc = std::min<int64_t>(64, std::max<int64_t>(4, (k * tiles + slots / 2) / slots));
+    } else {
+      tail_zc = p.op == OP_ACOUSTIC ? 16 : 8;
+    }
+  }
   if (const char* e = getenv("LIFT_K2_ZC")) zc = std::max<int64_t>(1, atoll(e));   // tuning hook
   if (p.fused_step && zc < p.ghost) zc = p.ghost;     // boundary planes stay in the first / last chunk
   if (zc > nz_reg) zc = nz_reg;
-  const int64_t nchunk = (nz_reg + zc - 1) / zc;
+  int64_t nchunk = (nz_reg + zc - 1) / zc;
+  // guided tail: the last ~tailw waves of items take zc2-plane chunks
+  int64_t n1 = nchunk, zc2 = zc;
+  {
+    const char* e2 = getenv("LIFT_K2_ZC2");
+    const char* ew = getenv("LIFT_K2_TAILW");
+    const int64_t want = e2 ? atoll(e2) : tail_zc;
+    const int64_t tailw = ew ? std::max<int64_t>(1, atoll(ew)) : 2;
+    if (want > 0 && want < zc && !p.fused_step && work >= 16 * slots) {
+      const int64_t nsmall = (tailw * slots + tiles - 1) / tiles;      // small chunks per tile column
+      const int64_t z2 = nsmall * want;
+      if (z2 < nz_reg) {
+        n1 = (nz_reg - z2) / zc;
+        zc2 = want;
+        nchunk = n1 + (nz_reg - n1 * zc + zc2 - 1) / zc2;
+      }
+    }
+  }
   const int64_t items = tiles * nchunk;
   if (items > 0x7fffffff) return cudaErrorInvalidConfiguration;
   int64_t grid = slots < items ? slots : items;
-  int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk;
+  int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk, n1_i = (int)n1, zc2_i = (int)zc2;
   int slot = (int)(g_slot.fetch_add(1) % kTickets);
   void* args[] = {(void*)&p, (void*)&map, (void*)&pwmap, (void*)&slid, (void*)&out,
-                  &ntx_i, &nty_i, &zc_i, &nch_i, &slot};
+                  &ntx_i, &nty_i, &zc_i, &nch_i, &slot, &n1_i, &zc2_i};
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, !fz);
 }
