@@ -363,6 +363,11 @@ def main():
     for _ in range(args.warmup):
         step()
     barrier()
+    # K4 (persistent iterate of a small L2-resident 3D grid): one launch per step
+    persist = (not slabbed) and iterable and plan.last_variant == 3
+    if persist:
+        launches_per_step = 1
+    variant_id = 3 if persist else plan.variant
 
     # timed region: exactly K steps, barrier + sync on both sides, events on the launching stream
     ev0 = torch.cuda.Event(enable_timing=True)
@@ -391,6 +396,8 @@ def main():
         # the step is back-to-back launches of the dominant kernel on one stream
         # (SRAD: one iteration = one fused pass; the first iteration's q0 pass is in the time)
         units = args.steps * (steps_per_iter if op == si.SRAD else launches_per_step)
+        if persist:   # K4: one launch per bench step runs all time steps; time per time step
+            units = args.steps * steps_per_iter
         avg_launch_s = (t_ms * 1e-3) / units
         alg_bytes = npts_local * bpp
     else:
@@ -482,13 +489,14 @@ def main():
                        (f"replicas x{world}" if world > 1 else "single"),
                        "l2": "inputs larger than L2 (no flush needed)" if npts_local * 4 > 126e6
                        else "L2-resident working set (no flush; reported as such)",
-                       "variant": {0: "K0 generic", 1: "K1 tile2d (TMA)", 2: "K2 sweep3d (TMA)"}[plan.variant],
+                       "variant": {0: "K0 generic", 1: "K1 tile2d (TMA)", 2: "K2 sweep3d (TMA)",
+                                   3: "K4 persistent iterate (cooperative)"}[variant_id],
                        "launch": (f"cuda graph replay ({launches_per_step} launches per graph)" if graph is not None
                                   else "stream launches")},
             "hbm_gbs_per_gpu_whole_step": value * bpp / world,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": ncu_traffic(args.workload),
-                         "kernel": {0: "k0_generic", 1: "k1_tile", 2: "k2_sweep"}[plan.variant],
+                         "kernel": {0: "k0_generic", 1: "k1_tile", 2: "k2_sweep", 3: "k4_iterate"}[variant_id],
                          "peak_source": peak_src,
                          "alg_bytes_per_launch": alg_bytes, "avg_launch_us": avg_launch_s * 1e6,
                          "frac_of_8TBs": achieved / 8000.0},

@@ -89,7 +89,11 @@ typedef enum {
   STENCIL_VARIANT_AUTO = -1,
   STENCIL_VARIANT_GENERIC = 0,   /* K0: one thread per output, remapped loads  */
   STENCIL_VARIANT_TILE2D = 1,    /* K1: TMA halo tile, 2D                       */
-  STENCIL_VARIANT_SWEEP3D = 2    /* K2: TMA plane ring, 2.5D sweep along z      */
+  STENCIL_VARIANT_SWEEP3D = 2,   /* K2: TMA plane ring, 2.5D sweep along z      */
+  STENCIL_VARIANT_PERSIST3D = 3  /* K4: all n steps of stencil_iterate in one
+                                    persistent cooperative launch (small,
+                                    L2-resident 3D radius-1 star / Hotspot3D
+                                    grids; AUTO only — reported, not forceable) */
 } stencil_variant;
 
 /*
@@ -154,6 +158,9 @@ int32_t stencil_plan_time_block(stencil_plan plan);
 stencil_status stencil_plan_set_variant(stencil_plan plan, int32_t variant);
 /* The family AUTO (or the forced one) selects for the given pointers. */
 int32_t stencil_plan_variant(stencil_plan plan);
+/* The family that ran the plan's most recent apply / iterate launch
+ * (STENCIL_VARIANT_PERSIST3D after a K4 iterate; GENERIC before any launch). */
+int32_t stencil_plan_last_variant(stencil_plan plan);
 
 /*
  * out = map(f, slide(pad(inputs))) — one application.

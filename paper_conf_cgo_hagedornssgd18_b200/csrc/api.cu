@@ -435,6 +435,8 @@ int32_t stencil_plan_time_block(stencil_plan pl) {
   return (pl->time_block >= 2 && sweep3d_t2_supported(pl->p)) ? 2 : 1;
 }
 
+int32_t stencil_plan_last_variant(stencil_plan pl) { return pl ? pl->last_variant : -1; }
+
 int32_t stencil_plan_variant(stencil_plan pl) {
   if (!pl) return -1;
   if (pl->forced_variant != STENCIL_VARIANT_AUTO) return pl->forced_variant;
@@ -540,6 +542,22 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
   if (!state || n_state != 2) return fail(STENCIL_E_INVALID, "iterate needs 2 state buffers");
   if (!state[0] || !state[1] || state[0] == state[1]) return fail(STENCIL_E_INVALID, "bad state buffers");
   int ri = (p.op == OP_ACOUSTIC) ? 1 : 0;
+  // small L2-resident 3D grids: all steps in one persistent launch (K4)
+  if ((p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D) && n_steps >= 2 && pl->ndim == 3 && pl->time_block < 2 &&
+      pl->forced_variant == STENCIL_VARIANT_AUTO &&
+      (p.op == OP_WEIGHTED ? n_aux == 0 : (n_aux == 1 && aux && aux[0])) &&
+      persist3d_supported(p, state[0], state[1], p.op == OP_HOTSPOT3D ? aux[0] : nullptr)) {
+    DeviceGuard g(pl->device);
+    if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+    std::string err;
+    cudaError_t e = launch_persist3d(p, state[0], state[1], p.op == OP_HOTSPOT3D ? aux[0] : nullptr, n_steps,
+                                     (cudaStream_t)stream, pl->num_sms, &err);
+    if (e != cudaSuccess)
+      return fail(STENCIL_E_CUDA, std::string("K4 launch failed: ") + cudaGetErrorString(e) + " " + err);
+    pl->last_variant = STENCIL_VARIANT_PERSIST3D;
+    if (result_index) *result_index = n_steps % 2;
+    return STENCIL_OK;
+  }
   if (p.op == OP_WEIGHTED || p.op == OP_GRADIENT || p.op == OP_SRAD) {
     if (n_aux != 0) return fail(STENCIL_E_INVALID, "WEIGHTED/GRADIENT/SRAD iterate takes no aux grids");
     int t = 0;

@@ -82,6 +82,13 @@ cudaError_t launch_srad_partials(const float* img, int64_t n, double2* partials,
 cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* out, cudaStream_t stream,
                               int num_sms, std::string* err, int* nparts_out);
 
+// K4 — n steps of a small (L2-resident) 3D radius-1 star stencil (weighted
+// star, Hotspot3D) in one persistent cooperative launch with grid barriers;
+// the result is in s0 when n_steps is even, else in s1.
+bool persist3d_supported(const StencilParams& p, const float* s0, const float* s1, const float* aux);
+cudaError_t launch_persist3d(const StencilParams& p, float* s0, float* s1, const float* aux, int n_steps,
+                             cudaStream_t stream, int num_sms, std::string* err);
+
 // wait (one thread, acquire.sys) until *a >= value and *b >= value (NULL = skip)
 cudaError_t launch_wait_signals(const unsigned int* a, const unsigned int* b, unsigned int value,
                                 cudaStream_t stream);

@@ -21,7 +21,7 @@ OPS = {"weighted": L.OP_WEIGHTED, "hotspot3d": L.OP_HOTSPOT3D, "srad1": L.OP_SRA
        "acoustic": L.OP_ACOUSTIC, "hotspot2d": L.OP_HOTSPOT2D, "gradient": L.OP_GRADIENT,
        "srad": L.OP_SRAD}
 VARIANTS = {"auto": L.VARIANT_AUTO, "generic": L.VARIANT_GENERIC, "tile2d": L.VARIANT_TILE2D,
-            "sweep3d": L.VARIANT_SWEEP3D}
+            "sweep3d": L.VARIANT_SWEEP3D, "persist3d": L.VARIANT_PERSIST3D}
 
 
 def _tuple(v, nd):
@@ -95,6 +95,11 @@ class Plan:
     @property
     def variant(self) -> int:
         return L.stencil_plan_variant(self.handle)
+
+    @property
+    def last_variant(self) -> int:
+        """Kernel family of the most recent apply / iterate launch."""
+        return L.stencil_plan_last_variant(self.handle)
 
     def _check(self, t: torch.Tensor, shape, name):
         if not isinstance(t, torch.Tensor) or not t.is_cuda:

@@ -286,6 +286,12 @@ def _c4a():
                     (1004, 1005), ((300.0, 350.0), (0.0, 1e-2)), 1, note="C4a: Rodinia Hotspot3D, clamp")
 
 
+def _c4a100():
+    return Workload("hotspot3d_8x512x512_x100", _spec((8, 512, 512), 3, op=HOTSPOT3D, params=params_hotspot3d()),
+                    (1004, 1005), ((300.0, 350.0), (0.0, 1e-2)), 100,
+                    note="C4a iterated (SURVEY §8(d)): Rodinia Hotspot3D, clamp, 100 time steps")
+
+
 def _c4b1():
     return Workload("srad1_4096", _spec((4096, 4096), 3, op=SRAD1), (1006,), ((0.0, 1.0),), 1,
                     transform=("exp",), note="C4b: Rodinia SRAD1 (I -> c), clamp; q0sqr from the input")
@@ -360,6 +366,7 @@ def _srad_iter():
 
 
 _WORKLOADS["srad_iter_4096"] = _srad_iter
+_WORKLOADS["hotspot3d_8x512x512_x100"] = _c4a100
 _WORKLOADS.update(_TABLE1)
 WORKLOAD_NAMES = tuple(_WORKLOADS)
 TABLE1_NAMES = tuple(_TABLE1)

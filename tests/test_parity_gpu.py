@@ -424,6 +424,42 @@ def test_srad_iterate_chain(lift, shape):
     assert np.max(np.abs(g - ref) / np.abs(ref)) <= TOL10
 
 
+@pytest.mark.parametrize("case,steps", [("clamp", 10), ("wrap", 7), ("const", 10), ("mirror", 3), ("hotspot", 10),
+                                        ("hotspot_reflect", 5), ("ragged", 6)])
+def test_persistent_iterate_bitwise(lift, case, steps, monkeypatch):
+    """K4 — all time steps of a small (L2-resident) 3D grid in one cooperative
+    launch with grid barriers — gives the bits of step-by-step K2 launches,
+    and matches the oracle after the steps (odd counts: result in state[1])."""
+    monkeypatch.setenv("LIFT_K4", "1")          # K4 is opt-in (measured slower than K2 steps)
+    shape = (11, 13, 52) if case == "ragged" else (12, 36, 136)
+    if case == "ragged":
+        case = "clamp"
+    if case.startswith("hotspot"):
+        kind = REFLECT if case.endswith("reflect") else CLAMP
+        sp = spec(shape, 3, op=si.HOTSPOT3D, params=si.params_hotspot3d(), kind=kind)
+        xs, aux = [rnd(shape, 71, 300, 350)], [rnd(shape, 72, 0, 1e-2)]
+    else:
+        k = {"clamp": CLAMP, "wrap": WRAP, "const": CONSTANT, "mirror": MIRROR}[case]
+        sp = spec(shape, 3, si.weights_j3d7(), k, value=0.3)
+        xs, aux = [rnd(shape, 73)], []
+    outs = []
+    for variant, fam in [(None, 3), ("sweep3d", 2)]:
+        plan = lift.Plan.from_spec(sp)
+        if variant:
+            plan.set_variant(variant)
+        a = torch.from_numpy(xs[0].copy()).cuda()
+        b = torch.empty_like(a)
+        dev_aux = [torch.from_numpy(x).cuda() for x in aux]
+        ri = plan.iterate([a, b], steps, aux=dev_aux)
+        torch.cuda.synchronize()
+        assert plan.last_variant == fam
+        assert ri == steps % 2
+        outs.append((a, b)[ri].cpu().numpy())
+    np.testing.assert_array_equal(outs[0], outs[1])
+    ref = orc.iterate(sp, xs, aux, steps)[0]
+    assert np.max(np.abs(outs[0] - ref) / np.maximum(np.abs(ref), 1e-3)) <= TOL10
+
+
 def test_cuda_graph_capture_replay(lift):
     """apply / iterate allocate nothing and are stream-ordered: captured into a
     CUDA graph, replays give the same bits as eager calls (stencil.h)."""
