@@ -17,12 +17,14 @@ import stencil_inputs as si  # noqa: E402
 BPP = {0: 8, 1: 12, 2: 8, 3: 12, 4: 12, 5: 12, 6: 8, 7: 8}
 WORKLOADS = sys.argv[1:] or ["j3d7_512_clamp", "gauss5_8192_mirror", "acoustic7_1024", "acoustic13_1024",
                              "srad1_4096", "srad2_4096", "t1_hotspot2d_8192", "t1_gradient_8192",
-                             "t1_jacobi3d13_512", "t1_poisson19_512", "t1_stencil2d_4098", "srad_iter_4096"]
+                             "t1_jacobi3d13_512", "t1_poisson19_512", "t1_stencil2d_4098", "srad_iter_4096",
+                             "t1_jacobi2d5_8192", "t1_jacobi2d9_8192", "t1_heat7_512", "hotspot3d_8x512x512",
+                             "hotspot3d_8x512x512_x100", "j2d5_256_clamp"]
 out = {}
 for wl in WORKLOADS:
     w = si.workload(wl)
     npts = int(np.prod(w.spec.out_extents()))
-    kern = "regex:k1_srad|k1_tile|k2_sweep|k2t|k0_generic"
+    kern = "regex:k1_srad|k1_tile|k2_sweep|k2t|k0_generic|k3_wsweep|k4_iterate"
     skip = "6" if w.steps > 1 else "2"     # single sweeps: 3 warm-up + 1 timed launch
     cmd = ["ncu", "--metrics", "dram__bytes_read.sum,dram__bytes_write.sum,gpu__time_duration.sum",
            "--clock-control", "none", "-k", kern, "-s", skip, "-c", "2", "--csv",
@@ -55,3 +57,13 @@ for wl in WORKLOADS:
                "duration_ns_cold": t, "dram_gbs_cold": (rd + wr) / t}
     print(wl, json.dumps(out[wl]), flush=True)
 json.dump(out, open("gpurun_out/ncu_bytes.json", "w"), indent=1)
+# the per-launch traffic bench.py reports as roofline.traffic
+traffic = {"_source": "ncu --metrics dram__bytes_read.sum,dram__bytes_write.sum --clock-control none: median of 2 "
+                      "launches of the dominant kernel after warm-up (scripts/ncu_bytes.py); "
+                      "dram_bytes_per_launch = read + write"}
+for wl, d in out.items():
+    if "error" not in d:
+        traffic[wl] = {"kernel": d["kernel"], "dram_bytes_per_launch": int(d["dram_read_bytes"] + d["dram_write_bytes"]),
+                       "dram_bytes_per_point": round(d["dram_bytes_per_point"], 3),
+                       "compulsory_bytes_per_point": d["compulsory_bytes_per_point"]}
+json.dump(traffic, open("gpurun_out/ncu_traffic.json", "w"), indent=1)
