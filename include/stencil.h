@@ -90,10 +90,14 @@ typedef enum {
   STENCIL_VARIANT_GENERIC = 0,   /* K0: one thread per output, remapped loads  */
   STENCIL_VARIANT_TILE2D = 1,    /* K1: TMA halo tile, 2D                       */
   STENCIL_VARIANT_SWEEP3D = 2,   /* K2: TMA plane ring, 2.5D sweep along z      */
-  STENCIL_VARIANT_PERSIST3D = 3  /* K4: all n steps of stencil_iterate in one
+  STENCIL_VARIANT_PERSIST3D = 3, /* K4: all n steps of stencil_iterate in one
                                     persistent cooperative launch (small,
                                     L2-resident 3D radius-1 star / Hotspot3D
                                     grids; AUTO only — reported, not forceable) */
+  STENCIL_VARIANT_GATHER = 4     /* K5: WEIGHTED plans the TMA families do not
+                                    take (step > 1, even / asymmetric windows,
+                                    1D, wide boxes, unaligned 3D) through
+                                    shared-memory tiles of the input box        */
 } stencil_variant;
 
 /*

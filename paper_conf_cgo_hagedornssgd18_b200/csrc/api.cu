@@ -112,12 +112,16 @@ int choose_variant(stencil_plan_s* pl, const float* in0, const float* in1, const
     if (v == STENCIL_VARIANT_SWEEP3D) return ptr_ok && sweep3d_supported(p);
     // K1 fills its tiles with cp.async when TMA cannot (unaligned / nx % 4 != 0)
     if (v == STENCIL_VARIANT_TILE2D) return tile2d_supported(p) && (p.op != OP_SRAD || ptr_ok);
+    if (v == STENCIL_VARIANT_GATHER) return gather_supported(p);
     return v == STENCIL_VARIANT_GENERIC;
   };
   if (pl->forced_variant != STENCIL_VARIANT_AUTO)
     return want(pl->forced_variant) ? pl->forced_variant : -1;
   if (pl->ndim == 3 && want(STENCIL_VARIANT_SWEEP3D)) return STENCIL_VARIANT_SWEEP3D;
   if (pl->ndim == 2 && want(STENCIL_VARIANT_TILE2D)) return STENCIL_VARIANT_TILE2D;
+  // WEIGHTED plans the TMA families do not take (strided, asymmetric, 1D, wide
+  // boxes, unaligned 3D): shared-memory tiles (K5) instead of K0's per-tap loads
+  if (want(STENCIL_VARIANT_GATHER)) return STENCIL_VARIANT_GATHER;
   return STENCIL_VARIANT_GENERIC;
 }
 
@@ -171,6 +175,9 @@ stencil_status launch(stencil_plan_s* pl, const StencilParams& p_in, const float
   switch (v) {
     case STENCIL_VARIANT_SWEEP3D:
       e = launch_sweep3d(p, in0, in1, out, stream, pl->num_sms, &err);
+      break;
+    case STENCIL_VARIANT_GATHER:
+      e = launch_gather(p, in0, out, stream, pl->num_sms, &err);
       break;
     case STENCIL_VARIANT_TILE2D:
       e = launch_tile2d(p, in0, in1, out, stream, pl->num_sms, &err);
@@ -413,8 +420,10 @@ stencil_status stencil_plan_set_slab(stencil_plan pl, int64_t z_offset, int64_t 
 
 stencil_status stencil_plan_set_variant(stencil_plan pl, int32_t variant) {
   if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
-  if (variant < STENCIL_VARIANT_AUTO || variant > STENCIL_VARIANT_SWEEP3D)
-    return fail(STENCIL_E_INVALID, "unknown variant");
+  if (variant < STENCIL_VARIANT_AUTO || variant > STENCIL_VARIANT_GATHER || variant == STENCIL_VARIANT_PERSIST3D)
+    return fail(STENCIL_E_INVALID, "unknown or non-forceable variant");
+  if (variant == STENCIL_VARIANT_GATHER && !gather_supported(pl->p))
+    return fail(STENCIL_E_UNSUPPORTED, "GATHER cannot run this plan");
   if (variant == STENCIL_VARIANT_SWEEP3D && !sweep3d_supported(pl->p))
     return fail(STENCIL_E_UNSUPPORTED, "SWEEP3D cannot run this plan");
   if (variant == STENCIL_VARIANT_TILE2D && !tile2d_supported(pl->p))
@@ -443,6 +452,7 @@ int32_t stencil_plan_variant(stencil_plan pl) {
   const StencilParams& p = pl->p;
   if (pl->ndim == 3 && sweep3d_supported(p)) return STENCIL_VARIANT_SWEEP3D;
   if (pl->ndim == 2 && tile2d_supported(p)) return STENCIL_VARIANT_TILE2D;
+  if (gather_supported(p)) return STENCIL_VARIANT_GATHER;
   return STENCIL_VARIANT_GENERIC;
 }
 

@@ -1,0 +1,295 @@
+// kernel_gather.cu — K5: WEIGHTED stencils of any shape through shared-memory
+// tiles: strided slides (step > 1), even or asymmetric
+// windows, 1D grids, wide boxes — every plan the TMA families (K1/K2/K3) do
+// not take and K0 would otherwise run tap by tap from global memory.
+//
+// slide(size, step) of an output tile of OT = (OTZ, OTY, OTX)
+// points reads the input box ((OT_d - 1) * step_d + size_d) per dimension —
+// for a 2D 3x3 step-2 slide of a 16 x 128 tile, 33 x 257 floats, each read
+// from HBM once instead of (size/step)^2 times.  The warps fill the box with
+// coalesced 4-byte cp.async row copies, double-buffered so the next tile's box
+// streams in while this one is evaluated (pad, is applied while
+// loading: remapped index or the constant, so no padded copy exists); every thread
+// evaluates its outputs from shared memory with the plan's non-zero taps in
+// row-major order (or the separable row/column form) — exactly K0's sequence,
+// so the two agree bitwise.  Slab mode (global z offset, ghost planes) and
+// output regions along dimension 0 behave as in K0.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <climits>
+#include <cstdlib>
+#include <mutex>
+#include <string>
+
+#include "common.cuh"
+#include "launch.hpp"
+#include "ops.cuh"
+#include "tma.cuh"
+
+namespace lift {
+namespace {
+
+constexpr int kThreads = 256;
+constexpr int NJ = 4;                          // outputs per thread per pass
+constexpr int NP = 2;                          // passes: tiles hold at most NP * NJ * kThreads outputs
+constexpr int kMaxSmemFloats = 48 * 1024;     // 192 KiB box limit
+constexpr int kMaxRows = 1024;                 // box rows (bz * by)
+
+struct Tile {
+  int otz, oty, otx;      // outputs per tile
+  int bz, by, bx;         // input box
+};
+
+__host__ __device__ inline Tile tile_of(const StencilParams& p, int otz, int oty, int otx) {
+  Tile t{otz, oty, otx, 0, 0, 0};
+  t.bz = (otz - 1) * p.step[0] + p.size[0];
+  t.by = (oty - 1) * p.step[1] + p.size[1];
+  t.bx = (otx - 1) * p.step[2] + p.size[2];
+  return t;
+}
+
+// unpadded index -> in-grid index, or -1 for the constant (y / x dimensions)
+__device__ __forceinline__ int64_t remap_or_const(int64_t i, int64_t n, int kind) {
+  if (i >= 0 && i < n) return i;
+  if (kind == PAD_CONSTANT) return -1;
+  return pad_remap(i, n, kind);
+}
+
+// fill one box with 4-byte cp.async copies.  Warp w copies box rows w, w + 8,
+// ...; pad per row is resolved first, one row per lane (element
+// offset of the row's x origin in the input, or -1 for the constant), and
+// handed to the copying lanes by shuffles — no shared table, no CTA barrier;
+// x is remapped per element only on tiles touching the x edges.
+__device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, const float* __restrict__ in,
+                                         float* dst_box, int64_t gz0, int64_t gy0, int64_t gx0, int warp,
+                                         int lane) {
+  constexpr int NWARP = kThreads / 32;
+  const int nrows = T.bz * T.by;
+  const bool x_inside = gx0 >= 0 && gx0 + T.bx <= p.n[2];
+  for (int base = warp; base < nrows; base += NWARP * 32) {
+    const int r = base + lane * NWARP;
+    int64_t off = -1;
+    if (r < nrows) {
+      const int bzi = r / T.by, byi = r - bzi * T.by;
+      const int64_t lz = plane_of(p, gz0 + bzi);
+      const int64_t iy = remap_or_const(gy0 + byi, p.n[1], p.kind[1]);
+      if (lz >= 0 && iy >= 0) off = lz * p.plane + iy * p.row + (x_inside ? gx0 : 0);
+    }
+    const int cnt = min(32, (nrows - base + NWARP - 1) / NWARP);
+    for (int i = 0; i < cnt; ++i) {
+      const int64_t o = __shfl_sync(0xffffffffu, off, i);
+      float* dst = dst_box + (base + i * NWARP) * T.bx;
+      if (o < 0) {
+        for (int b = lane; b < T.bx; b += 32) dst[b] = p.pad_value;
+      } else if (x_inside) {
+        const float* s0 = in + o;
+        for (int b = lane; b < T.bx; b += 32) cp_async4(dst + b, s0 + b);
+      } else {
+        for (int b = lane; b < T.bx; b += 32) {
+          const int64_t ix = remap_or_const(gx0 + b, p.n[2], p.kind[2]);
+          if (ix < 0) dst[b] = p.pad_value;
+          else cp_async4(dst + b, in + o + ix);
+        }
+      }
+    }
+  }
+}
+
+// nbuf = 2: the next tile's box streams in (cp.async) while this one is evaluated
+__global__ void __launch_bounds__(kThreads) k5_gather(const __grid_constant__ StencilParams p, Tile T,
+                                                      const float* __restrict__ in, float* __restrict__ out,
+                                                      int64_t ntz, int64_t nty, int64_t ntx, int nbuf) {
+  extern __shared__ __align__(16) float box[];
+  __shared__ int toff[kMaxTaps];
+  pdl_launch_dependents();
+  const int BYX = T.by * T.bx;
+  const int box_floats = T.bz * BYX;
+  for (int t = threadIdx.x; t < p.ntaps; t += kThreads)
+    toff[t] = p.tap[t][0] * BYX + p.tap[t][1] * T.bx + p.tap[t][2];
+  pdl_wait();
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int64_t oz_n = p.reg1 - p.reg0, oy_n = p.o[1], ox_n = p.o[2];
+  const int64_t out_plane = p.o[1] * p.o[2];
+  const int64_t ntiles = ntz * nty * ntx;
+  const int nout = T.otz * T.oty * T.otx;
+  auto origin = [&](int64_t tile, int64_t& oz0, int64_t& oy0, int64_t& ox0) {
+    // 32-bit division: ntiles < 2^31 (checked at launch)
+    const uint32_t t32 = (uint32_t)tile, r = t32 / (uint32_t)ntx;
+    const uint32_t tx = t32 - r * (uint32_t)ntx;
+    const uint32_t tz = r / (uint32_t)nty, ty = r - tz * (uint32_t)nty;
+    oz0 = p.reg0 + tz * T.otz;
+    oy0 = ty * T.oty;
+    ox0 = tx * T.otx;
+  };
+  auto fill = [&](int64_t tile, int buf) {
+    int64_t oz0, oy0, ox0;
+    origin(tile, oz0, oy0, ox0);
+    // unpadded coordinates of the box origin (global z)
+    fill_box(p, T, in, box + buf * box_floats, p.z_off + oz0 * p.step[0] - p.lo[0], oy0 * p.step[1] - p.lo[1],
+             ox0 * p.step[2] - p.lo[2], warp, lane);
+    cp_async_commit();
+  };
+  // this thread's outputs within a tile (tile-invariant: no per-tile division):
+  // k = tid + (pass * NJ + j) * kThreads, at most NP passes (nout <= NP*NJ*kThreads)
+  int woff[NP * NJ], kxs[NP * NJ], kys[NP * NJ], kzs[NP * NJ];
+#pragma unroll
+  for (int q = 0; q < NP * NJ; ++q) {
+    const int k = threadIdx.x + q * kThreads;
+    const int kx = k % T.otx, kr = k / T.otx;
+    const int ky = kr % T.oty, kz = kr / T.oty;
+    const bool v = k < nout;
+    kxs[q] = kx;
+    kys[q] = ky;
+    kzs[q] = v ? kz : INT32_MAX / 2;     // invalid slots fail the range check below
+    woff[q] = v ? kz * p.step[0] * BYX + ky * p.step[1] * T.bx + kx * p.step[2] : 0;
+  }
+  int cur = 0;
+  if ((int64_t)blockIdx.x < ntiles) fill(blockIdx.x, 0);
+  for (int64_t tile = blockIdx.x; tile < ntiles; tile += gridDim.x) {
+    const int64_t next = tile + gridDim.x;
+    float* bcur = box + cur * box_floats;
+    if (nbuf == 2) {
+      if (next < ntiles) fill(next, cur ^ 1);
+      else cp_async_commit();
+      cp_async_wait<1>();
+    } else {
+      cp_async_wait<0>();
+    }
+    __syncthreads();
+    int64_t oz0, oy0, ox0;
+    origin(tile, oz0, oy0, ox0);
+    // each thread evaluates NJ outputs per pass: the tap loop's index / weight
+    // loads are shared by NJ independent FMA chains
+#pragma unroll
+    for (int ps = 0; ps < NP; ++ps) {
+      if (threadIdx.x + ps * NJ * kThreads >= nout) break;
+      int64_t oidx[NJ];
+      bool ok[NJ];
+#pragma unroll
+      for (int j = 0; j < NJ; ++j) {
+        const int q = ps * NJ + j;
+        const int64_t oz = oz0 + kzs[q], oy = oy0 + kys[q], ox = ox0 + kxs[q];
+        ok[j] = oz - p.reg0 < oz_n && oy < oy_n && ox < ox_n;
+        oidx[j] = (oz + p.ghost) * out_plane + oy * ox_n + ox;
+      }
+      float acc[NJ];
+#pragma unroll
+      for (int j = 0; j < NJ; ++j) acc[j] = 0.0f;
+      if (p.sep) {
+        // separable 2D weights: rows first (x taps in order), then the column (K0's order)
+        for (int a = 0; a < p.size[1]; ++a) {
+          float h[NJ];
+#pragma unroll
+          for (int j = 0; j < NJ; ++j) h[j] = 0.0f;
+          for (int b = 0; b < p.size[2]; ++b) {
+            const float wv = p.sv[b];
+            const int o = a * T.bx + b;
+#pragma unroll
+            for (int j = 0; j < NJ; ++j) h[j] = __fmaf_rn(wv, bcur[woff[ps * NJ + j] + o], h[j]);
+          }
+          const float wu = p.su[a];
+#pragma unroll
+          for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wu, h[j], acc[j]);
+        }
+      } else {
+        for (int t = 0; t < p.ntaps; ++t) {
+          const float wv = p.w[t];
+          const int o = toff[t];
+#pragma unroll
+          for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wv, bcur[woff[ps * NJ + j] + o], acc[j]);
+        }
+      }
+#pragma unroll
+      for (int j = 0; j < NJ; ++j)
+        if (ok[j]) out[oidx[j]] = acc[j];
+    }
+    __syncthreads();     // bcur is refilled two tiles from now
+    if (nbuf == 2) {
+      cur ^= 1;
+    } else if (next < ntiles) {
+      fill(next, 0);
+    }
+  }
+}
+
+struct Shape {
+  int otz, oty, otx;
+};
+
+// output tile per dimensionality: 3D (2, 4, 128), 2D (1, 16, 128), 1D (1, 1, 1024),
+// halved (largest first) until the box fits
+bool choose(const StencilParams& p, Tile* T) {
+  const bool d3 = p.o[0] > 1 || p.size[0] > 1;
+  const bool d2 = p.o[1] > 1 || p.size[1] > 1;
+  // 3D: long box rows amortise the per-row work of the fill (measured on 512^3
+  // step-2 slides: (2, 4, 128) 1217 GB/s vs (4, 8, 32) 903 GB/s for 3x3x3)
+  Shape s = d3 ? Shape{2, 4, 128} : (d2 ? Shape{1, 16, 128} : Shape{1, 1, 1024});
+  if (d3) {
+    if (const char* e = getenv("LIFT_K5_3D")) {     // A/B hook: 1 = (2, 8, 64), 2 = (1, 8, 128), 3 = (4, 8, 32)
+      const int v = atoi(e);
+      if (v == 1) s = Shape{2, 8, 64};
+      if (v == 2) s = Shape{1, 8, 128};
+      if (v == 3) s = Shape{4, 8, 32};
+    }
+  }
+  for (int it = 0; it < 16; ++it) {
+    const Tile t = tile_of(p, s.otz, s.oty, s.otx);
+    if ((int64_t)t.bz * t.by * t.bx <= kMaxSmemFloats && s.otz * s.oty * s.otx <= NP * NJ * kThreads &&
+        t.bz * t.by <= kMaxRows) {
+      *T = t;
+      return true;
+    }
+    if (s.otx >= 2 * s.oty && s.otx > 1) s.otx /= 2;
+    else if (s.oty > 1) s.oty /= 2;
+    else if (s.otz > 1) s.otz /= 2;
+    else if (s.otx > 1) s.otx /= 2;
+    else return false;
+  }
+  return false;
+}
+
+}  // namespace
+
+bool gather_supported(const StencilParams& p) {
+  if (p.op != OP_WEIGHTED || p.ntaps < 1) return false;
+  Tile t;
+  return choose(p, &t);
+}
+
+cudaError_t launch_gather(const StencilParams& p, const float* in0, float* out, cudaStream_t stream, int num_sms,
+                          std::string* err) {
+  Tile T;
+  if (!choose(p, &T)) {
+    *err = "gather: window box exceeds shared memory";
+    return cudaErrorInvalidConfiguration;
+  }
+  const int64_t oz_n = p.reg1 - p.reg0;
+  if (oz_n <= 0 || p.o[1] <= 0 || p.o[2] <= 0) return cudaSuccess;
+  const int64_t ntz = (oz_n + T.otz - 1) / T.otz, nty = (p.o[1] + T.oty - 1) / T.oty;
+  const int64_t ntx = (p.o[2] + T.otx - 1) / T.otx;
+  const size_t box_bytes = (size_t)T.bz * T.by * T.bx * sizeof(float);
+  const int nbuf = 2 * box_bytes <= (size_t)kMaxSmemFloats * 4 ? 2 : 1;
+  const size_t smem = nbuf * box_bytes;
+  static std::once_flag once;
+  std::call_once(once, [] {
+    cudaFuncSetAttribute(k5_gather, cudaFuncAttributeMaxDynamicSharedMemorySize, kMaxSmemFloats * 4);
+  });
+  int occ = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k5_gather, kThreads, smem) != cudaSuccess || occ < 1) occ = 1;
+  cudaGetLastError();
+  int64_t grid = (int64_t)num_sms * occ;
+  const int64_t ntiles = ntz * nty * ntx;
+  if (ntiles >= (1ll << 31)) {
+    *err = "gather: too many tiles";
+    return cudaErrorInvalidConfiguration;
+  }
+  if (grid > ntiles) grid = ntiles;
+  const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
+  int nb = nbuf;
+  void* args[] = {(void*)&p, (void*)&T, (void*)&in0, (void*)&out, (void*)&ntz, (void*)&nty, (void*)&ntx, (void*)&nb};
+  return launch_kernel(reinterpret_cast<const void*>(&k5_gather), dim3((unsigned)grid), dim3(kThreads), args, smem,
+                       stream, !fz);
+}
+
+}  // namespace lift

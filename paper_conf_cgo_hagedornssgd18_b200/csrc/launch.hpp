@@ -82,6 +82,11 @@ cudaError_t launch_srad_partials(const float* img, int64_t n, double2* partials,
 cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* out, cudaStream_t stream,
                               int num_sms, std::string* err, int* nparts_out);
 
+// K5 — WEIGHTED plans of any shape through shared-memory input boxes.
+bool gather_supported(const StencilParams& p);
+cudaError_t launch_gather(const StencilParams& p, const float* in0, float* out, cudaStream_t stream, int num_sms,
+                          std::string* err);
+
 // K4 — n steps of a small (L2-resident) 3D radius-1 star stencil (weighted
 // star, Hotspot3D) in one persistent cooperative launch with grid barriers;
 // the result is in s0 when n_steps is even, else in s1.

@@ -21,7 +21,8 @@ OPS = {"weighted": L.OP_WEIGHTED, "hotspot3d": L.OP_HOTSPOT3D, "srad1": L.OP_SRA
        "acoustic": L.OP_ACOUSTIC, "hotspot2d": L.OP_HOTSPOT2D, "gradient": L.OP_GRADIENT,
        "srad": L.OP_SRAD}
 VARIANTS = {"auto": L.VARIANT_AUTO, "generic": L.VARIANT_GENERIC, "tile2d": L.VARIANT_TILE2D,
-            "sweep3d": L.VARIANT_SWEEP3D, "persist3d": L.VARIANT_PERSIST3D}
+            "sweep3d": L.VARIANT_SWEEP3D, "persist3d": L.VARIANT_PERSIST3D,
+            "gather": L.VARIANT_GATHER}
 
 
 def _tuple(v, nd):

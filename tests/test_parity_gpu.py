@@ -228,12 +228,63 @@ def test_variant_selection(lift):
              (spec((64, 128), 5, si.weights_gauss5(), MIRROR), "tile2d"),
              (spec((64, 128), 3, op=si.SRAD1, params=(0.1,)), "tile2d"),
              (spec((64, 128), 3, op=si.SRAD2, params=(0.5,)), "tile2d"),
-             (spec((64, 64, 130), 3, si.weights_j3d7()), "generic"),
+             (spec((64, 64, 130), 3, si.weights_j3d7()), "gather"),
              (spec((64, 64, 128), 3, np.ones((3, 3, 3), np.float32)), "sweep3d"),
-             (spec((64, 64, 128), 5, np.ones((5, 5, 5), np.float32)), "generic")]
+             (spec((64, 64, 128), 5, np.ones((5, 5, 5), np.float32)), "gather"),
+             (spec((64, 128), 3, si.weights_j2d5(), step=(2, 2)), "gather"),
+             (spec((1000,), 3, [1, 2, 3]), "gather")]
     for sp, v in cases:
         plan = lift.Plan.from_spec(sp)
         assert plan.variant == lift.plan.VARIANTS[v], (sp, v)
+
+
+def _gather_cases():
+    r = np.random.default_rng(81)
+    w = lambda *shape: r.standard_normal(shape).astype(np.float32)
+    return {
+        "1d_s2": (spec((1001,), 5, w(5), MIRROR, lo=(3,), hi=(1,), step=(2,)), [rnd((1001,), 82)]),
+        "1d_wide_pad": (spec((7,), 4, w(4), WRAP, lo=(9,), hi=(6,)), [rnd((7,), 83)]),
+        "2d_3x3_s2_clamp": (spec((257, 390), 3, w(3, 3), CLAMP, step=(2, 2)), [rnd((257, 390), 84)]),
+        "2d_2x2_s2_const": (spec((130, 260), 2, w(2, 2), CONSTANT, lo=(0, 0), hi=(1, 1), step=(2, 2), value=0.4),
+                            [rnd((130, 260), 85)]),
+        "2d_5x5_s3_reflect": (spec((200, 300), 5, w(5, 5), REFLECT, step=(3, 3)), [rnd((200, 300), 86)]),
+        "2d_gauss_sep_s2": (spec((300, 520), 5, si.weights_gauss5(), MIRROR, step=(2, 2)), [rnd((300, 520), 87)]),
+        "2d_mixed_s21": (spec((99, 333), 3, w(3, 3), (WRAP, CLAMP), step=(2, 1)), [rnd((99, 333), 88)]),
+        "3d_3x3x3_s2": (spec((33, 40, 70), 3, w(3, 3, 3), CLAMP, step=(2, 2, 2)), [rnd((33, 40, 70), 89)]),
+        "3d_2x2x2_s2_wrap": (spec((32, 34, 64), 2, w(2, 2, 2), WRAP, lo=(0, 0, 0), hi=(1, 1, 1), step=(2, 2, 2)),
+                             [rnd((32, 34, 64), 90)]),
+        "3d_box5": (spec((20, 30, 68), 5, w(5, 5, 5), MIRROR), [rnd((20, 30, 68), 91)]),
+        "3d_odd_width": (spec((20, 30, 66), 3, si.weights_j3d7(), CONSTANT, value=-0.5), [rnd((20, 30, 66), 92)]),
+        "3d_asym": (spec((21, 22, 64), (3, 2, 4), w(3, 2, 4), REFLECT, lo=(2, 0, 1), hi=(0, 1, 2)),
+                    [rnd((21, 22, 64), 93)]),
+    }
+
+
+@pytest.mark.parametrize("case", list(_gather_cases()))
+def test_gather_kernel(lift, case):
+    """K5 (shared-memory input boxes) for WEIGHTED plans the TMA families do
+    not take: parity with the oracle and bitwise equality with K0."""
+    sp, xs = _gather_cases()[case]
+    y, plan = check(lift, sp, xs)
+    assert plan.variant == lift.plan.VARIANTS["gather"]
+    y0, p0 = run_gpu(lift, sp, xs, "generic")
+    assert p0.variant == 0
+    np.testing.assert_array_equal(y, y0)
+
+
+def test_gather_apply_region_pieces(lift):
+    x = rnd((41, 36, 70), 94)
+    sp = spec(x.shape, 3, np.random.default_rng(95).standard_normal((3, 3, 3)).astype(np.float32), MIRROR,
+              step=(2, 1, 2))
+    full, plan = run_gpu(lift, sp, [x])
+    assert plan.variant == lift.plan.VARIANTS["gather"]
+    xd = torch.from_numpy(x).cuda()
+    o = sp.out_extents()
+    out = torch.full(o, float("nan"), device="cuda")
+    for a, b in [(0, 1), (1, 6), (6, 20), (20, o[0])]:
+        plan.apply_region(xd, out=out, begin=a, end=b)
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(out.cpu().numpy(), full)
 
 
 def test_apply_region_pieces_bitwise(lift):
