@@ -58,6 +58,21 @@ def test_virtual_slab_weighted_bitwise(lift, kind, world):
     np.testing.assert_array_equal(got.cpu().numpy(), ref)
 
 
+@pytest.mark.parametrize("kind", [si.CLAMP, si.WRAP, si.CONSTANT])
+def test_virtual_slab_gather_bitwise(lift, kind):
+    """Slabs on the K5 gather kernel (nx % 4 != 0 rules out TMA; a 5x5x5 box):
+    ghost planes, global-z pad and output regions as in the single plan."""
+    from paper_conf_cgo_hagedornssgd18_b200.slab import virtual_slab_iterate
+    ext = (26, 20, 66)
+    w = np.random.default_rng(96).standard_normal((5, 5, 5)).astype(np.float32) * 0.01
+    sp = si.StencilSpec(ext, (5,) * 3, (1,) * 3, (2,) * 3, (2,) * 3, (kind,) * 3, 0.25, si.WEIGHTED, w, ())
+    assert lift.Plan.from_spec(sp).variant == lift.plan.VARIANTS["gather"]
+    x = si.uniform(ext, 97, 0.5, 1.5)
+    ref = single_iterate(lift, sp, [x], [], 3)[0]
+    got = virtual_slab_iterate(ext, 3, [torch.from_numpy(x).cuda()], 3, **kw(sp))[0]
+    np.testing.assert_array_equal(got.cpu().numpy(), ref)
+
+
 @pytest.mark.parametrize("pts,sz", [(7, 3), (13, 5)])
 def test_virtual_slab_acoustic_bitwise(lift, pts, sz):
     from paper_conf_cgo_hagedornssgd18_b200.slab import virtual_slab_iterate
