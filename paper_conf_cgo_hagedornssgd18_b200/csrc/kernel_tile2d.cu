@@ -447,6 +447,23 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
     float iw[4][W];
     float cr[3][5];
     float* orow = out + ((int64_t)(y0 + r0) * nx + xo);
+    // c at the tile's right halo column x0 + 128 (SRAD2's E tap of lane 31)
+    // for this warp's RPW + 1 c rows, one row per lane (lanes 0..RPW): every
+    // other lane's column x + 4 is its right neighbour's column x (shuffle),
+    // so each lane evaluates SRAD1 for 4 columns instead of 5
+    float halo_c;
+    {
+      const int j = lane < RPW + 1 ? lane : RPW;
+      const float* bf = reinterpret_cast<const float*>(box) + (r0 + j + 1) * BX + TX + XH - 1;
+      float a0[3], a1[3], a2[3];
+#pragma unroll
+      for (int d = 0; d < 3; ++d) {
+        a0[d] = bf[d];
+        a1[d] = bf[BX + d];
+        a2[d] = bf[2 * BX + d];
+      }
+      halo_c = op_srad1(RowsAcc<1, 0>{a0, a1, a2}, q);
+    }
     // box rows r0+1 .. r0+RPW+3  <->  I rows y0+r0-1 .. y0+r0+RPW+1
     static_for<RPW + 3>([&](auto K) {
       constexpr int k = decltype(K)::value;
@@ -456,10 +473,13 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
         constexpr int cs_ = (k - 2) % 3;
         const int crow = y0 + r0 + k - 2;
         if (crow < ny) {
-          static_for<5>([&](auto II) {
+          static_for<4>([&](auto II) {
             constexpr int ii = decltype(II)::value;
             cr[cs_][ii] = op_srad1(RowsAcc<2, ii>{iw[(k - 2) % 4], iw[(k - 1) % 4], iw[k % 4]}, q);
           });
+          const float right = __shfl_down_sync(0xffffffffu, cr[cs_][0], 1);
+          const float hcol = __shfl_sync(0xffffffffu, halo_c, k - 2);
+          cr[cs_][4] = lane == 31 ? hcol : right;
           cr[cs_][4] = ce == 4 ? cr[cs_][4] : (ce == 3 ? cr[cs_][3] : (ce == 2 ? cr[cs_][2] : cr[cs_][1]));
         } else if constexpr (k >= 3) {
           // c row outside the grid: the remapped row (one or two above)
