@@ -1006,7 +1006,8 @@ Launcher pick(const StencilParams& p) {
   }
   // radius 2: the 5 live planes need a deep plane ring too; (7 plane stages,
   // 4 point-wise slots) fits 2 CTAs per SM (Acoustic-13 1024^3: 451 Gpts/s
-  // vs 448 for (8, 3) and 411 for (6, 5))
+  // vs 448 for (8, 3) and 411 for (6, 5); 8-row tiles at 3 CTAs/SM and
+  // 24-row tiles measured 379 / 371 vs 466, profiles/r01_sweep_acoustic13_shapes.txt)
   if (pv == 1) return get_launcher_zf<K2_ACOUSTIC, 2, 2, 8, 3>(zc, fz);
   return get_launcher_zf<K2_ACOUSTIC, 2, 2, 7, 4>(zc, fz);
 }
