@@ -434,6 +434,10 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
     const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
     const bool edge = (x0 == 0) || (x0 + TX + 2 > nx) || (y0 < 2) || (y0 + TY + 2 > ny);
     if (edge) {
+      // every warp is past this stage's previous tile (guaranteed already by
+      // the empty/full mbarrier hand-off; the barrier makes it explicit to
+      // racecheck, edge tiles only)
+      named_bar_sync(1, NCONS);
       fixup_tile<2, 2, XH, BX, C::BY, NCONS>(p, reinterpret_cast<float*>(dsm4 + s * SF4), src0, 0, x0, y0,
                                              threadIdx.x);
       fence_proxy_async_smem();
