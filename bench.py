@@ -44,6 +44,7 @@ METRIC = "stencil Gpoints/s & achieved HBM GB/s vs 8 TB/s at 1/2/4/8 B200"
 # q0 statistics of I' for the next iteration; only the first iteration of a
 # stencil_iterate chain reads I once more for its q0 (timed, not counted)
 BYTES_PER_POINT = {0: 8, 1: 12, 2: 8, 3: 12, 4: 12, 5: 12, 6: 8, 7: 8}
+L2_BYTES = 126e6     # B200 L2 (the flush writes 2x this before each timed step of an L2-resident workload)
 
 def env_int(k, d):
     try:
@@ -209,6 +210,8 @@ def main():
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
+    ap.add_argument("--no-flush", action="store_true",
+                    help="L2-resident workloads: time L2-warm back-to-back sweeps instead of cold flushed steps")
     ap.add_argument("--no-graph", action="store_true", help="launch single sweeps eagerly instead of a CUDA graph")
     ap.add_argument("--scaling", default="weak", choices=["weak", "strong"],
                     help="multi-GPU iterated sweeps: weak = the single-GPU grid per rank (default), "
@@ -369,17 +372,71 @@ def main():
         launches_per_step = 1
     variant_id = 3 if persist else plan.variant
 
+    # L2-resident working sets (one sweep's algorithmic bytes < 2 x L2): the
+    # timed steps are cold — a 2 x L2 buffer is written before every step,
+    # outside the step's event pair — and single-sweep workloads time ONE
+    # sweep per step; the hot number (graph of back-to-back sweeps, L2-warm)
+    # is reported beside it as "hot"
+    bpp = BYTES_PER_POINT[op]
+    cold = (not slabbed) and npts_local * bpp < 2 * L2_BYTES and not args.no_flush
+    hot = None
+    if cold:
+        def time_hot():
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            barrier()
+            e0.record(stream)
+            for _ in range(args.steps):
+                step()
+            e1.record(stream)
+            barrier()
+            th = e0.elapsed_time(e1)
+            return {"value": npts_local * steps_per_iter * sweeps * args.steps / (th * 1e-3) / 1e9,
+                    "sweeps_per_step": steps_per_iter if iterable else sweeps,
+                    "ms_per_step": th / args.steps, "l2": "warm (back-to-back sweeps, no flush)"}
+        hot = time_hot()
+        flush = torch.empty(int(2 * L2_BYTES) // 4, dtype=torch.int32, device=dev)
+        if not iterable:
+            one = None
+            if graph is not None:
+                one = torch.cuda.CUDAGraph()
+                side = torch.cuda.Stream()
+                side.wait_stream(torch.cuda.current_stream())
+                with torch.cuda.stream(side):
+                    plan.apply(*bufs, out=out)
+                torch.cuda.current_stream().wait_stream(side)
+                with torch.cuda.graph(one):
+                    plan.apply(*bufs, out=out)
+
+            def step():  # noqa: F811  (one cold sweep)
+                if one is not None:
+                    one.replay()
+                else:
+                    plan.apply(*bufs, out=out)
+                return 0
+            launches_per_step //= sweeps
+            sweeps = 1
+            for _ in range(2):
+                step()
     # timed region: exactly K steps, barrier + sync on both sides, events on the launching stream
     ev0 = torch.cuda.Event(enable_timing=True)
     ev1 = torch.cuda.Event(enable_timing=True)
     with ClockSampler(local) as clk:
         barrier()
-        ev0.record(stream)
-        for _ in range(args.steps):
-            step()
-        ev1.record(stream)
+        if cold:
+            pairs = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
+                     for _ in range(args.steps)]
+            for k in range(args.steps):
+                flush.fill_(k)              # evict the working set from L2 (not timed)
+                pairs[k][0].record(stream)
+                step()
+                pairs[k][1].record(stream)
+        else:
+            ev0.record(stream)
+            for _ in range(args.steps):
+                step()
+            ev1.record(stream)
         barrier()
-    t_ms = ev0.elapsed_time(ev1)
+    t_ms = sum(a.elapsed_time(b) for a, b in pairs) if cold else ev0.elapsed_time(ev1)
     t_max = t_ms
     if use_pg:
         tt = torch.tensor([t_ms], device=dev)
@@ -391,7 +448,6 @@ def main():
 
     # per-launch kernel duration of the dominant kernel: a step is back-to-back
     # launches of it on one stream (single GPU), so avg launch = step time / launches
-    bpp = BYTES_PER_POINT[op]
     if not slabbed:
         # the step is back-to-back launches of the dominant kernel on one stream
         # (SRAD: one iteration = one fused pass; the first iteration's q0 pass is in the time)
@@ -487,8 +543,11 @@ def main():
                        "halo": (args.halo if slabbed else None),
                        "parallelism": f"slab-z x{world}" if slabbed else
                        (f"replicas x{world}" if world > 1 else "single"),
-                       "l2": "inputs larger than L2 (no flush needed)" if npts_local * 4 > 126e6
-                       else "L2-resident working set (no flush; reported as such)",
+                       "l2": ("L2 flushed (2 x L2 write) before every timed step; one sweep per step"
+                              if cold and not iterable else
+                              "L2 flushed (2 x L2 write) before every timed step" if cold else
+                              "inputs larger than L2 (no flush needed)" if npts_local * bpp >= 2 * L2_BYTES
+                              else "L2-resident working set, not flushed (--no-flush)"),
                        "variant": {0: "K0 generic", 1: "K1 tile2d (TMA)", 2: "K2 sweep3d (TMA)",
                                    3: "K4 persistent iterate (cooperative)"}[variant_id],
                        "launch": (f"cuda graph replay ({launches_per_step} launches per graph)" if graph is not None
@@ -501,6 +560,7 @@ def main():
                          "alg_bytes_per_launch": alg_bytes, "avg_launch_us": avg_launch_s * 1e6,
                          "frac_of_8TBs": achieved / 8000.0},
             "cpu_baseline": cpu,
+            "hot": hot,
             "e2e": e2e,
             "gpu_launches": int(args.steps * launches_per_step),
             "clocks": clocks,
