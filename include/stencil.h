@@ -55,7 +55,13 @@ typedef enum {
   STENCIL_PAD_MIRROR = 1,     /* symmetric, edge repeated (numpy 'symmetric')  A2 */
   STENCIL_PAD_WRAP = 2,       /* ((i mod n) + n) mod n                         A3 */
   STENCIL_PAD_CONSTANT = 3,   /* value variant of pad: pad_value              A4 */
-  STENCIL_PAD_REFLECT = 4     /* edge not repeated (numpy 'reflect')          A2 */
+  STENCIL_PAD_REFLECT = 4,    /* edge not repeated (numpy 'reflect')          A2 */
+  STENCIL_PAD_DAMPEN = 5      /* "dampening boundary conditions where the
+                                 out-of-bound value decreases with the distance
+                                 to the boundary", reading A29: the
+                                 cell d steps outside holds the nearest element
+                                 times decay^d (stencil_plan_set_pad_decay);
+                                 WEIGHTED only; decay 1 = CLAMP, 0 = zeros    */
 } stencil_pad;
 
 /* Neighbourhood functions f of map (A13-A20). */
@@ -162,6 +168,10 @@ int32_t stencil_plan_time_block(stencil_plan plan);
 stencil_status stencil_plan_set_variant(stencil_plan plan, int32_t variant);
 /* The family AUTO (or the forced one) selects for the given pointers. */
 int32_t stencil_plan_variant(stencil_plan plan);
+/* PAD_DAMPEN dimensions: the factor per cell of distance outside the grid,
+ * decay in [0, 1] (default 1).  E_INVALID outside that range.  Applies to
+ * subsequent launches. */
+stencil_status stencil_plan_set_pad_decay(stencil_plan plan, float decay);
 /* The family that ran the plan's most recent apply / iterate launch
  * (STENCIL_VARIANT_PERSIST3D after a K4 iterate; GENERIC before any launch). */
 int32_t stencil_plan_last_variant(stencil_plan plan);

@@ -41,7 +41,7 @@ from typing import Callable, List, Sequence, Tuple
 
 import numpy as np
 
-CLAMP, MIRROR, WRAP, CONSTANT, REFLECT = 0, 1, 2, 3, 4
+CLAMP, MIRROR, WRAP, CONSTANT, REFLECT, DAMPEN = 0, 1, 2, 3, 4, 5
 WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC, HOTSPOT2D, GRADIENT, SRAD = 0, 1, 2, 3, 4, 5, 6, 7
 
 
@@ -86,13 +86,30 @@ H = {CLAMP: h_clamp, MIRROR: h_mirror, WRAP: h_wrap, REFLECT: h_reflect}
 # ---------------------------------------------------------------------------
 # pad and pad_n
 # ---------------------------------------------------------------------------
-def pad1(x: np.ndarray, axis: int, l: int, r: int, kind: int, value: float = 0.0) -> np.ndarray:
+def dampen_distance(i, n):
+    """Distance of unpadded index i outside [0, n): -i left, i-n+1 right, 0 inside."""
+    i = np.asarray(i)
+    return np.where(i < 0, -i, np.where(i >= n, i - n + 1, 0))
+
+
+def pad1(x: np.ndarray, axis: int, l: int, r: int, kind: int, value: float = 0.0,
+         decay: float = 1.0) -> np.ndarray:
     """1D pad applied along ``axis``: type [T]_n -> [T]_{l+n+r}.
 
     Reindexing variant: padded index j in [0, l+n+r) reads x[h(j - l, n)]
     (h receives i - l in [-l, n+r), reading A1).  Value variant:
-    positions outside [l, l+n) hold ``value`` (CONSTANT, reading A4)."""
+    positions outside [l, l+n) hold ``value`` (CONSTANT, reading A4).
+    DAMPEN ("dampening boundary conditions where the out-of-bound value
+    decreases with the distance to the boundary"; reading A29):
+    the cell at distance d >= 1 outside the array holds the nearest element
+    times decay**d."""
     n = x.shape[axis]
+    if kind == DAMPEN:
+        i = np.arange(-l, n + r)
+        out = np.take(np.asarray(x, np.float64), h_clamp(i, n), axis=axis)
+        shape = [1] * out.ndim
+        shape[axis] = l + n + r
+        return out * (np.float64(decay) ** dampen_distance(i, n)).reshape(shape)
     if kind == CONSTANT:
         shape = list(x.shape)
         shape[axis] = l + n + r
@@ -106,13 +123,13 @@ def pad1(x: np.ndarray, axis: int, l: int, r: int, kind: int, value: float = 0.0
 
 
 def pad_n(x: np.ndarray, pad_lo: Sequence[int], pad_hi: Sequence[int],
-          kind: Sequence[int], value: float = 0.0) -> np.ndarray:
+          kind: Sequence[int], value: float = 0.0, decay: float = 1.0) -> np.ndarray:
     """pad_n(l, r, h, input) = map_{n-1}(pad(l, r, h), pad_{n-1}(l, r, h, input))
     (P:537-539): pad the outer dimension(s) first, then the inner ones.  A
     per-dimension h is allowed (reading A10)."""
     P = np.asarray(x, dtype=np.float64)
     for d in range(P.ndim):
-        P = pad1(P, d, pad_lo[d], pad_hi[d], kind[d], value)
+        P = pad1(P, d, pad_lo[d], pad_hi[d], kind[d], value, decay)
     return P
 
 
@@ -347,7 +364,7 @@ def apply(spec, inputs: Sequence[np.ndarray]):
     """One application of the stencil: returns (Y, A) as fp64 arrays of the
     output extents; A is the absolute-term error scale (reading A22)."""
     _check_op_shape(spec)
-    pad = lambda x: pad_n(x, spec.pad_lo, spec.pad_hi, spec.kind, spec.pad_value)
+    pad = lambda x: pad_n(x, spec.pad_lo, spec.pad_hi, spec.kind, spec.pad_value, getattr(spec, "pad_decay", 1.0))
     tapper = lambda P: (lambda k: slide_tap(P, k, spec.size, spec.step))
     outs = spec.out_extents()
     if spec.op == WEIGHTED:
@@ -385,16 +402,25 @@ def apply_point(spec, inputs: Sequence[np.ndarray], o: Sequence[int]):
     _check_op_shape(spec)
 
     def fetch(x, k):
-        idx = []
-        for d in range(spec.ndim):
+        # pad_n pads the outer dimension first, so the cell seen
+        # through an inner pad is resolved first: walk the dimensions innermost
+        # first — a CONSTANT dimension outside ends the walk with the value,
+        # DAMPEN contributes decay^distance (reading A29)
+        idx = [0] * spec.ndim
+        factor = np.float64(1.0)
+        for d in reversed(range(spec.ndim)):
             i = int(o[d]) * spec.step[d] + k[d] - spec.pad_lo[d]
             n = spec.extents[d]
             if i < 0 or i >= n:
                 if spec.kind[d] == CONSTANT:
-                    return np.float64(spec.pad_value)
-                i = int(H[spec.kind[d]](i, n))
-            idx.append(i)
-        return np.float64(x[tuple(idx)])
+                    return np.float64(spec.pad_value) * factor
+                if spec.kind[d] == DAMPEN:
+                    factor *= np.float64(getattr(spec, "pad_decay", 1.0)) ** int(dampen_distance(i, n))
+                    i = int(h_clamp(i, n))
+                else:
+                    i = int(H[spec.kind[d]](i, n))
+            idx[d] = i
+        return np.float64(x[tuple(idx)]) * factor
 
     tap = lambda x: (lambda k: fetch(x, k))
     if spec.op == WEIGHTED:

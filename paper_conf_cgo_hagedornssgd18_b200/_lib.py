@@ -23,7 +23,7 @@ _lib = C.CDLL(LIB_PATH)
 
 # status / enums (include/stencil.h)
 STENCIL_OK, STENCIL_E_INVALID, STENCIL_E_UNSUPPORTED, STENCIL_E_CUDA, STENCIL_E_NOMEM = range(5)
-PAD_CLAMP, PAD_MIRROR, PAD_WRAP, PAD_CONSTANT, PAD_REFLECT = range(5)
+PAD_CLAMP, PAD_MIRROR, PAD_WRAP, PAD_CONSTANT, PAD_REFLECT, PAD_DAMPEN = range(6)
 OP_WEIGHTED, OP_HOTSPOT3D, OP_SRAD1, OP_SRAD2, OP_ACOUSTIC, OP_HOTSPOT2D, OP_GRADIENT, OP_SRAD = range(8)
 VARIANT_AUTO, VARIANT_GENERIC, VARIANT_TILE2D, VARIANT_SWEEP3D, VARIANT_PERSIST3D, VARIANT_GATHER = -1, 0, 1, 2, 3, 4
 OP_ARITY = {OP_WEIGHTED: 1, OP_HOTSPOT3D: 2, OP_SRAD1: 1, OP_SRAD2: 2, OP_ACOUSTIC: 2, OP_HOTSPOT2D: 2, OP_GRADIENT: 1, OP_SRAD: 1}
@@ -49,6 +49,7 @@ _set_slab = _sig("stencil_plan_set_slab", C.c_int, [_P, C.c_int64, C.c_int64, C.
 _set_variant = _sig("stencil_plan_set_variant", C.c_int, [_P, C.c_int32])
 _variant = _sig("stencil_plan_variant", C.c_int32, [_P])
 _last_variant = _sig("stencil_plan_last_variant", C.c_int32, [_P])
+_set_decay = _sig("stencil_plan_set_pad_decay", C.c_int, [_P, C.c_float])
 _set_tb = _sig("stencil_plan_set_time_block", C.c_int, [_P, C.c_int32])
 _tb = _sig("stencil_plan_time_block", C.c_int32, [_P])
 _apply = _sig("stencil_apply", C.c_int, [_P, _FPP, C.c_int32, _P, _P])
@@ -67,6 +68,7 @@ _version = _sig("stencil_version", C.c_char_p, [])
 
 EXPORTED = ("stencil_plan_create", "stencil_plan_output_extents", "stencil_plan_set_slab",
             "stencil_plan_set_variant", "stencil_plan_variant", "stencil_plan_last_variant",
+            "stencil_plan_set_pad_decay",
             "stencil_plan_set_time_block",
             "stencil_plan_time_block", "stencil_apply", "stencil_apply_region",
             "stencil_apply_region_put", "stencil_slab_step_fused", "stencil_wait_signals",
@@ -141,6 +143,10 @@ def stencil_plan_set_variant(plan: int, variant: int):
 
 def stencil_plan_variant(plan: int) -> int:
     return int(_variant(plan))
+
+
+def stencil_plan_set_pad_decay(plan: int, decay: float):
+    _check(_set_decay(plan, float(decay)), "stencil_plan_set_pad_decay")
 
 
 def stencil_plan_last_variant(plan: int) -> int:

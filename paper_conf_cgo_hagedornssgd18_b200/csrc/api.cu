@@ -249,7 +249,9 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
   for (int d = 0; d < ndim; ++d) {
     if (extents[d] < 1 || size[d] < 1 || step[d] < 1 || pad_lo[d] < 0 || pad_hi[d] < 0)
       return fail(STENCIL_E_INVALID, "extents/size/step must be >= 1 and pads >= 0");
-    if (kind[d] < PAD_CLAMP || kind[d] > PAD_REFLECT) return fail(STENCIL_E_INVALID, "unknown pad kind");
+    if (kind[d] < PAD_CLAMP || kind[d] > PAD_DAMPEN) return fail(STENCIL_E_INVALID, "unknown pad kind");
+    if (kind[d] == PAD_DAMPEN && op != OP_WEIGHTED)
+      return fail(STENCIL_E_UNSUPPORTED, "DAMPEN pads are built for WEIGHTED stencils");
     if (extents[d] + pad_lo[d] + pad_hi[d] < size[d])
       return fail(STENCIL_E_INVALID, "n + l + r < size: slide yields no window");
     if (extents[d] > (int64_t)1 << 40 || size[d] > 4096 || pad_lo[d] > (1 << 20) || pad_hi[d] > (1 << 20))
@@ -265,6 +267,7 @@ stencil_status stencil_plan_create(stencil_plan* out, int device, int ndim, cons
   p.row = p.n[2];
   p.plane = p.n[1] * p.n[2];
   p.pad_value = pad_value;
+  p.pad_decay = 1.0f;
   p.op = op;
   p.z_off = 0;
   p.gnz = p.n[0];
@@ -445,6 +448,13 @@ int32_t stencil_plan_time_block(stencil_plan pl) {
 }
 
 int32_t stencil_plan_last_variant(stencil_plan pl) { return pl ? pl->last_variant : -1; }
+
+stencil_status stencil_plan_set_pad_decay(stencil_plan pl, float decay) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  if (!(decay >= 0.0f && decay <= 1.0f)) return fail(STENCIL_E_INVALID, "pad decay must be in [0, 1]");
+  pl->p.pad_decay = decay;
+  return STENCIL_OK;
+}
 
 int32_t stencil_plan_variant(stencil_plan pl) {
   if (!pl) return -1;

@@ -12,7 +12,7 @@
 
 namespace lift {
 
-enum PadKind : int { PAD_CLAMP = 0, PAD_MIRROR = 1, PAD_WRAP = 2, PAD_CONSTANT = 3, PAD_REFLECT = 4 };
+enum PadKind : int { PAD_CLAMP = 0, PAD_MIRROR = 1, PAD_WRAP = 2, PAD_CONSTANT = 3, PAD_REFLECT = 4, PAD_DAMPEN = 5 };
 enum OpKind : int {
   OP_WEIGHTED = 0, OP_HOTSPOT3D = 1, OP_SRAD1 = 2, OP_SRAD2 = 3, OP_ACOUSTIC = 4, OP_HOTSPOT2D = 5, OP_GRADIENT = 6,
   OP_SRAD = 7
@@ -32,6 +32,7 @@ struct StencilParams {
   int32_t size[3], step[3], lo[3], hi[3];
   int32_t kind[3];
   float pad_value;
+  float pad_decay;       // PAD_DAMPEN: factor per cell of distance outside the grid (reading A29)
   int32_t op;
   int32_t radius;        // star/box radius for non-WEIGHTED ops and fast kernels
   // slab mode along z (ghost == 0 and z_off == 0 and gnz == n[0] otherwise)
@@ -87,6 +88,7 @@ struct StencilParams {
 __host__ __device__ __forceinline__ int64_t pad_remap(int64_t i, int64_t n, int kind) {
   switch (kind) {
     case PAD_CLAMP:
+    case PAD_DAMPEN:     // the nearest element (scaled by the caller, dampen_pow)
       return i < 0 ? 0 : (i >= n ? n - 1 : i);
     case PAD_MIRROR: {
       if (i < 0) i = -1 - i;               // now i >= 0
@@ -108,6 +110,23 @@ __host__ __device__ __forceinline__ int64_t pad_remap(int64_t i, int64_t n, int 
     default:
       return i;
   }
+}
+
+// PAD_DAMPEN (reading A29): a cell d steps outside the grid holds the nearest
+// element times decay^d, per dimension in pad_n's order, so a
+// window element crossing k DAMPEN cells in total (over the dimensions inside
+// the innermost out-of-range CONSTANT one) is x (or the constant) times
+// decay^k — computed as a sequential product, identical in every kernel.
+__host__ __device__ __forceinline__ int64_t outside_dist(int64_t i, int64_t n) {
+  return i < 0 ? -i : (i >= n ? i - n + 1 : 0);
+}
+__device__ __forceinline__ float dampen_pow(float g, int64_t k) {
+  float f = 1.0f;
+  for (; k > 0; --k) f = __fmul_rn(f, g);
+  return f;
+}
+__host__ __device__ __forceinline__ bool has_dampen(const StencilParams& p) {
+  return p.kind[0] == PAD_DAMPEN || p.kind[1] == PAD_DAMPEN || p.kind[2] == PAD_DAMPEN;
 }
 
 // Local plane index (within a buffer of n0 + 2*ghost planes) of the input

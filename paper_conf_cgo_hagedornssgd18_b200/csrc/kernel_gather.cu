@@ -58,38 +58,80 @@ __device__ __forceinline__ int64_t remap_or_const(int64_t i, int64_t n, int kind
 
 // fill one box with 4-byte cp.async copies.  Warp w copies box rows w, w + 8,
 // ...; pad per row is resolved first, one row per lane (element
-// offset of the row's x origin in the input, or -1 for the constant), and
-// handed to the copying lanes by shuffles — no shared table, no CTA barrier;
-// x is remapped per element only on tiles touching the x edges.
+// offset of the row's x origin in the input, or -1 for a value row, and the
+// DAMPEN cells the row's y / z indices crossed), and handed to the copying
+// lanes by shuffles — no shared table, no CTA barrier; x is remapped per
+// element only on tiles touching the x edges.  Dimensions resolve innermost
+// first, as in K0's fetch (x, then y, then z; reading A29 for DAMPEN), so the
+// two kernels give the same bits.
 __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, const float* __restrict__ in,
                                          float* dst_box, int64_t gz0, int64_t gy0, int64_t gx0, int warp,
                                          int lane) {
   constexpr int NWARP = kThreads / 32;
   const int nrows = T.bz * T.by;
   const bool x_inside = gx0 >= 0 && gx0 + T.bx <= p.n[2];
+  const bool damp = has_dampen(p);
   for (int base = warp; base < nrows; base += NWARP * 32) {
     const int r = base + lane * NWARP;
     int64_t off = -1;
+    int nrow = 0;
     if (r < nrows) {
       const int bzi = r / T.by, byi = r - bzi * T.by;
-      const int64_t lz = plane_of(p, gz0 + bzi);
-      const int64_t iy = remap_or_const(gy0 + byi, p.n[1], p.kind[1]);
-      if (lz >= 0 && iy >= 0) off = lz * p.plane + iy * p.row + (x_inside ? gx0 : 0);
+      int64_t iy = gy0 + byi;
+      bool vrow = false;
+      if (iy < 0 || iy >= p.n[1]) {
+        if (p.kind[1] == PAD_CONSTANT) vrow = true;
+        else {
+          if (p.kind[1] == PAD_DAMPEN) nrow += (int)outside_dist(iy, p.n[1]);
+          iy = pad_remap(iy, p.n[1], p.kind[1]);
+        }
+      }
+      if (!vrow) {
+        const int64_t gz = gz0 + bzi;
+        const int64_t lz = plane_of(p, gz);
+        if (lz >= 0) {
+          if (p.kind[0] == PAD_DAMPEN) nrow += (int)outside_dist(gz, p.gnz);
+          off = lz * p.plane + iy * p.row + (x_inside ? gx0 : 0);
+        }
+      } else {
+        nrow = 0;       // the y value cell: only x's DAMPEN cells (inside it) count
+      }
     }
     const int cnt = min(32, (nrows - base + NWARP - 1) / NWARP);
     for (int i = 0; i < cnt; ++i) {
       const int64_t o = __shfl_sync(0xffffffffu, off, i);
+      const int nr = __shfl_sync(0xffffffffu, nrow, i);
       float* dst = dst_box + (base + i * NWARP) * T.bx;
-      if (o < 0) {
-        for (int b = lane; b < T.bx; b += 32) dst[b] = p.pad_value;
-      } else if (x_inside) {
-        const float* s0 = in + o;
-        for (int b = lane; b < T.bx; b += 32) cp_async4(dst + b, s0 + b);
+      if (!damp) {
+        if (o < 0) {
+          for (int b = lane; b < T.bx; b += 32) dst[b] = p.pad_value;
+        } else if (x_inside) {
+          const float* s0 = in + o;
+          for (int b = lane; b < T.bx; b += 32) cp_async4(dst + b, s0 + b);
+        } else {
+          for (int b = lane; b < T.bx; b += 32) {
+            const int64_t ix = remap_or_const(gx0 + b, p.n[2], p.kind[2]);
+            if (ix < 0) dst[b] = p.pad_value;
+            else cp_async4(dst + b, in + o + ix);
+          }
+        }
       } else {
+        // DAMPEN plans: values computed directly (decay^k scaling)
         for (int b = lane; b < T.bx; b += 32) {
-          const int64_t ix = remap_or_const(gx0 + b, p.n[2], p.kind[2]);
-          if (ix < 0) dst[b] = p.pad_value;
-          else cp_async4(dst + b, in + o + ix);
+          int64_t ix = gx0 + b;
+          int k = nr;
+          float v;
+          if ((ix < 0 || ix >= p.n[2]) && p.kind[2] == PAD_CONSTANT) {
+            v = p.pad_value;
+            k = 0;
+          } else {
+            if (ix < 0 || ix >= p.n[2]) {
+              if (p.kind[2] == PAD_DAMPEN) k += (int)outside_dist(ix, p.n[2]);
+              ix = pad_remap(ix, p.n[2], p.kind[2]);
+            }
+            v = o < 0 ? p.pad_value : __ldg(in + o + (x_inside ? ix - gx0 : ix));
+          }
+          dst[b] = k ? __fmul_rn(v, dampen_pow(p.pad_decay, k)) : v;
         }
       }
     }
@@ -97,7 +139,7 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
 }
 
 // nbuf = 2: the next tile's box streams in (cp.async) while this one is evaluated
-__global__ void __launch_bounds__(kThreads) k5_gather(const __grid_constant__ StencilParams p, Tile T,
+__global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__ StencilParams p, Tile T,
                                                       const float* __restrict__ in, float* __restrict__ out,
                                                       int64_t ntz, int64_t nty, int64_t ntx, int nbuf) {
   extern __shared__ __align__(16) float box[];
@@ -163,7 +205,7 @@ __global__ void __launch_bounds__(kThreads) k5_gather(const __grid_constant__ St
     // loads are shared by NJ independent FMA chains
 #pragma unroll
     for (int ps = 0; ps < NP; ++ps) {
-      if (threadIdx.x + ps * NJ * kThreads >= nout) break;
+      if (threadIdx.x + ps * NJ * kThreads >= nout) continue;   // (no break: keeps the loop fully unrolled)
       int64_t oidx[NJ];
       bool ok[NJ];
 #pragma unroll

@@ -21,20 +21,27 @@ struct Geo {
 };
 
 // padded-grid read for one input: window element at unpadded coordinates
-// (gz global plane, iy, ix)
+// (gz global plane, iy, ix).  Dimensions resolve innermost first (pad_n pads
+// the outer dimension first, so an inner pad sees the outer one's
+// cells): a CONSTANT dimension out of range gives the value, DAMPEN counts
+// its distance (reading A29), the others remap.
 __device__ __forceinline__ float fetch(const StencilParams& p, const float* __restrict__ in,
                                        int64_t gz, int64_t iy, int64_t ix) {
-  const int64_t lz = plane_of(p, gz);
-  if (lz < 0) return p.pad_value;
-  if (iy < 0 || iy >= p.n[1]) {
-    if (p.kind[1] == PAD_CONSTANT) return p.pad_value;
-    iy = pad_remap(iy, p.n[1], p.kind[1]);
-  }
+  int64_t nd = 0;
   if (ix < 0 || ix >= p.n[2]) {
     if (p.kind[2] == PAD_CONSTANT) return p.pad_value;
+    if (p.kind[2] == PAD_DAMPEN) nd += outside_dist(ix, p.n[2]);
     ix = pad_remap(ix, p.n[2], p.kind[2]);
   }
-  return __ldg(in + lz * p.plane + iy * p.row + ix);
+  if (iy < 0 || iy >= p.n[1]) {
+    if (p.kind[1] == PAD_CONSTANT) return nd ? __fmul_rn(p.pad_value, dampen_pow(p.pad_decay, nd)) : p.pad_value;
+    if (p.kind[1] == PAD_DAMPEN) nd += outside_dist(iy, p.n[1]);
+    iy = pad_remap(iy, p.n[1], p.kind[1]);
+  }
+  if (p.kind[0] == PAD_DAMPEN) nd += outside_dist(gz, p.gnz);
+  const int64_t lz = plane_of(p, gz);
+  const float v = lz < 0 ? p.pad_value : __ldg(in + lz * p.plane + iy * p.row + ix);
+  return nd ? __fmul_rn(v, dampen_pow(p.pad_decay, nd)) : v;
 }
 
 // Accessor for centred ops: at<DZ,DY,DX>() is the window element at offset D

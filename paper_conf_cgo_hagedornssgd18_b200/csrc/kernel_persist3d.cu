@@ -217,7 +217,7 @@ bool persist3d_supported(const StencilParams& p, const float* s0, const float* s
   // Hotspot3D 8x512x512 (267 vs 303 Gpts/s)
   const char* e = getenv("LIFT_K4");
   if (!(e && e[0] == '1')) return false;
-  if (p.slab || p.n[0] < 1) return false;
+  if (p.slab || p.n[0] < 1 || has_dampen(p)) return false;
   if (p.op != OP_WEIGHTED && p.op != OP_HOTSPOT3D) return false;
   for (int d = 0; d < 3; ++d)
     if (p.size[d] != 3 || p.lo[d] != 1 || p.hi[d] != 1 || p.step[d] != 1) return false;

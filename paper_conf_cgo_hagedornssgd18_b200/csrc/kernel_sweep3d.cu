@@ -1041,6 +1041,7 @@ std::atomic<unsigned> g_slot{0};
 }  // namespace
 
 bool sweep3d_supported(const StencilParams& p) {
+  if (has_dampen(p)) return false;     // DAMPEN pads run on K5 / K0
   const int R = p.radius;
   if (R != 1 && R != 2) return false;
   for (int d = 0; d < 3; ++d)

@@ -689,6 +689,7 @@ cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* o
 }
 
 bool tile2d_supported(const StencilParams& p) {
+  if (has_dampen(p)) return false;     // DAMPEN pads run on K5 / K0
   // canonical 2D plan: dimension 0 is the dummy (extent 1, size 1, no pad)
   if (p.n[0] != 1 || p.size[0] != 1 || p.lo[0] != 0 || p.hi[0] != 0 || p.slab) return false;
   const int ry = p.lo[1], rx = p.lo[2];

@@ -16,7 +16,7 @@ import torch
 from . import _lib as L
 
 KINDS = {"clamp": L.PAD_CLAMP, "mirror": L.PAD_MIRROR, "symmetric": L.PAD_MIRROR, "wrap": L.PAD_WRAP,
-         "constant": L.PAD_CONSTANT, "zero": L.PAD_CONSTANT, "reflect": L.PAD_REFLECT}
+         "constant": L.PAD_CONSTANT, "zero": L.PAD_CONSTANT, "reflect": L.PAD_REFLECT, "dampen": L.PAD_DAMPEN}
 OPS = {"weighted": L.OP_WEIGHTED, "hotspot3d": L.OP_HOTSPOT3D, "srad1": L.OP_SRAD1, "srad2": L.OP_SRAD2,
        "acoustic": L.OP_ACOUSTIC, "hotspot2d": L.OP_HOTSPOT2D, "gradient": L.OP_GRADIENT,
        "srad": L.OP_SRAD}
@@ -74,8 +74,16 @@ class Plan:
     @classmethod
     def from_spec(cls, spec, device: Optional[int] = None) -> "Plan":
         """Build from a stencil_inputs.StencilSpec-like object (duck-typed)."""
-        return cls(spec.extents, spec.size, spec.step, spec.pad_lo, spec.pad_hi, list(spec.kind),
+        plan = cls(spec.extents, spec.size, spec.step, spec.pad_lo, spec.pad_hi, list(spec.kind),
                    spec.pad_value, spec.op, spec.weights, spec.params, device)
+        decay = getattr(spec, "pad_decay", 1.0)
+        if decay != 1.0:
+            plan.set_pad_decay(decay)
+        return plan
+
+    def set_pad_decay(self, decay: float):
+        """DAMPEN dimensions: factor per cell of distance outside the grid (A29)."""
+        L.stencil_plan_set_pad_decay(self.handle, decay)
 
     def set_slab(self, z_offset: int, global_n0: int, ghost: int):
         L.stencil_plan_set_slab(self.handle, z_offset, global_n0, ghost)

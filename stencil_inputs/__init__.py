@@ -23,9 +23,9 @@ from typing import List, Optional, Sequence, Tuple
 import numpy as np
 
 # Boundary kinds — numeric values are the C-ABI enum ``stencil_pad``.
-CLAMP, MIRROR, WRAP, CONSTANT, REFLECT = 0, 1, 2, 3, 4
+CLAMP, MIRROR, WRAP, CONSTANT, REFLECT, DAMPEN = 0, 1, 2, 3, 4, 5
 KIND_NAMES = {CLAMP: "clamp", MIRROR: "mirror", WRAP: "wrap",
-              CONSTANT: "constant", REFLECT: "reflect"}
+              CONSTANT: "constant", REFLECT: "reflect", DAMPEN: "dampen"}
 
 # Ops — numeric values are the C-ABI enum ``stencil_op``.
 WEIGHTED, HOTSPOT3D, SRAD1, SRAD2, ACOUSTIC, HOTSPOT2D, GRADIENT, SRAD = 0, 1, 2, 3, 4, 5, 6, 7
@@ -51,6 +51,7 @@ class StencilSpec:
     op: int = WEIGHTED
     weights: Optional[np.ndarray] = None    # float32, shape == size (WEIGHTED)
     params: Tuple[float, ...] = ()          # float32 op constants
+    pad_decay: float = 1.0                  # DAMPEN dimensions: decay per cell of distance (reading A29)
 
     @property
     def ndim(self) -> int:

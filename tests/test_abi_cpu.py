@@ -132,3 +132,22 @@ def test_product_package_does_not_import_oracle():
             if f.endswith((".py", ".cu", ".cuh", ".hpp", ".cpp", ".h")):
                 txt = open(os.path.join(dirpath, f)).read()
                 assert not pat.search(txt), f
+
+
+def test_dampen_pad_validation(lib):
+    """DAMPEN (reading A29) is a WEIGHTED pad kind; its decay lies in [0, 1]."""
+    with pytest.raises(lib.StencilError) as e:
+        lib.stencil_plan_create(0, [8, 8], [3, 3], [1, 1], [1, 1], [1, 1], [si.DAMPEN, 0], 0.0, si.SRAD1, None, (0.1,))
+    assert e.value.status == 2
+    with pytest.raises(lib.StencilError) as e:
+        lib.stencil_plan_create(0, [8, 8], [3, 3], [1, 1], [1, 1], [1, 1], [6, 0], 0.0, 0, np.ones((3, 3), np.float32))
+    assert e.value.status == 1
+    h = lib.stencil_plan_create(0, [8, 8], [3, 3], [1, 1], [1, 1], [1, 1], [si.DAMPEN, si.DAMPEN], 0.0, 0,
+                                np.ones((3, 3), np.float32))
+    lib.stencil_plan_set_pad_decay(h, 0.25)
+    for bad in (-0.1, 1.5, float("nan")):
+        with pytest.raises(lib.StencilError):
+            lib.stencil_plan_set_pad_decay(h, bad)
+    # DAMPEN plans never take the TMA families
+    assert lib.stencil_plan_variant(h) == lib._lib.VARIANT_GATHER
+    lib.stencil_plan_destroy(h)

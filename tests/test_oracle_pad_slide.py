@@ -205,3 +205,55 @@ def test_slide_tap_is_window_element():
     W = slide_n(P, (3, 2), (2, 3))
     for k in np.ndindex(3, 2):
         np.testing.assert_array_equal(slide_tap(P, k, (3, 2), (2, 3)), W[..., k[0], k[1]])
+
+
+# ------------------------------------- DAMPEN value pad (reading A29) ------
+def test_dampen_special_cases_are_edge_and_zero_padding():
+    """decay 1 is numpy 'edge' (CLAMP), decay 0 is zero padding."""
+    from oracle.stencil_oracle import DAMPEN
+    rng = np.random.default_rng(41)
+    for n in range(1, 7):
+        x = rng.random(n)
+        for l, r in itertools.product(range(4), range(4)):
+            np.testing.assert_array_equal(pad1(x, 0, l, r, DAMPEN, decay=1.0), np.pad(x, (l, r), mode="edge"))
+            np.testing.assert_array_equal(pad1(x, 0, l, r, DAMPEN, decay=0.0), np.pad(x, (l, r)))
+
+
+def test_dampen_brute_force_2d_and_mixed_with_constant():
+    """Per cell: the nearest element times decay^(cells outside), summed over
+    the DAMPEN dimensions; a CONSTANT dimension outside gives c times decay^
+    (cells outside in the dimensions padded after it, pad_n's order P:537-539)."""
+    from oracle.stencil_oracle import DAMPEN
+    x = np.arange(12, dtype=np.float64).reshape(3, 4) + 1.0
+    g, c = 0.5, 7.0
+    dist = lambda i, n: -i if i < 0 else (i - n + 1 if i >= n else 0)
+    cl = lambda i, n: min(max(i, 0), n - 1)
+    P = pad_n(x, (2, 1), (1, 3), (DAMPEN, DAMPEN), decay=g)
+    for a, b in itertools.product(range(6), range(8)):
+        i, j = a - 2, b - 1
+        assert P[a, b] == x[cl(i, 3), cl(j, 4)] * g ** (dist(i, 3) + dist(j, 4))
+    Q = pad_n(x, (2, 1), (1, 3), (CONSTANT, DAMPEN), value=c, decay=g)
+    for a, b in itertools.product(range(6), range(8)):
+        i, j = a - 2, b - 1
+        base = c if not 0 <= i < 3 else x[i, cl(j, 4)]
+        assert Q[a, b] == base * g ** dist(j, 4)
+    R = pad_n(x, (2, 1), (1, 3), (DAMPEN, CONSTANT), value=c, decay=g)
+    for a, b in itertools.product(range(6), range(8)):
+        i, j = a - 2, b - 1
+        assert R[a, b] == (c if not 0 <= j < 4 else x[cl(i, 3), j] * g ** dist(i, 3))
+
+
+def test_dampen_apply_point_equals_apply():
+    import stencil_inputs as si
+    from oracle import stencil_oracle as orc
+    rng = np.random.default_rng(42)
+    for kinds in [(si.DAMPEN, si.DAMPEN, si.DAMPEN), (si.CONSTANT, si.DAMPEN, si.WRAP),
+                  (si.DAMPEN, si.CONSTANT, si.DAMPEN), (si.MIRROR, si.DAMPEN, si.CONSTANT)]:
+        x = rng.random((5, 6, 7))
+        w = rng.standard_normal((3, 4, 3)).astype(np.float32)
+        sp = si.StencilSpec((5, 6, 7), (3, 4, 3), (2, 1, 2), (2, 3, 1), (1, 2, 2), kinds, 0.375, si.WEIGHTED,
+                            w, (), pad_decay=0.625)
+        Y, A = orc.apply(sp, [x])
+        for o in np.ndindex(*Y.shape):
+            y, a = orc.apply_point(sp, [x], o)
+            assert y == pytest.approx(Y[o], rel=1e-13, abs=1e-13)

@@ -257,7 +257,21 @@ def _gather_cases():
         "3d_odd_width": (spec((20, 30, 66), 3, si.weights_j3d7(), CONSTANT, value=-0.5), [rnd((20, 30, 66), 92)]),
         "3d_asym": (spec((21, 22, 64), (3, 2, 4), w(3, 2, 4), REFLECT, lo=(2, 0, 1), hi=(0, 1, 2)),
                     [rnd((21, 22, 64), 93)]),
+        # DAMPEN pads (reading A29): decay^distance, alone and mixed with CONSTANT / reindexing
+        "2d_dampen": (dampen(spec((130, 264), 5, si.weights_gauss5(), si.DAMPEN), 0.5), [rnd((130, 264), 98)]),
+        "2d_dampen_const": (dampen(spec((99, 140), 3, w(3, 3), (CONSTANT, si.DAMPEN), value=0.3, step=(2, 1)),
+                                   0.75), [rnd((99, 140), 99)]),
+        "3d_dampen_mixed": (dampen(spec((20, 26, 68), 3, w(3, 3, 3), (si.DAMPEN, CONSTANT, si.DAMPEN),
+                                        lo=(2, 1, 3), hi=(1, 2, 2), value=-0.2), 0.6), [rnd((20, 26, 68), 100)]),
+        "3d_dampen_star": (dampen(spec((24, 40, 136), 3, si.weights_j3d7(), (si.DAMPEN, WRAP, si.DAMPEN)), 0.9),
+                           [rnd((24, 40, 136), 101)]),
+        "1d_dampen": (dampen(spec((500,), 5, w(5), si.DAMPEN, lo=(4,), hi=(3,)), 0.3), [rnd((500,), 102)]),
     }
+
+
+def dampen(sp, decay):
+    sp.pad_decay = decay
+    return sp
 
 
 @pytest.mark.parametrize("case", list(_gather_cases()))
