@@ -138,7 +138,9 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
   }
 }
 
-// nbuf = 2: the next tile's box streams in (cp.async) while this one is evaluated
+// nbuf = 2: the next tile's box streams in (cp.async) while this one is evaluated.
+// SZ, SY, SX > 0: compile-time window (all taps non-zero, or separable 2D)
+template <int SZ, int SY, int SX>
 __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__ StencilParams p, Tile T,
                                                       const float* __restrict__ in, float* __restrict__ out,
                                                       int64_t ntz, int64_t nty, int64_t ntx, int nbuf) {
@@ -218,7 +220,43 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
       float acc[NJ];
 #pragma unroll
       for (int j = 0; j < NJ; ++j) acc[j] = 0.0f;
-      if (p.sep) {
+      const float* wj[NJ];
+#pragma unroll
+      for (int j = 0; j < NJ; ++j) wj[j] = bcur + woff[ps * NJ + j];
+      if constexpr (SZ > 0) {
+        // compile-time window (dense weights or separable 2D): unrolled taps,
+        // immediate x offsets, the same operation order as the tap list
+        if (p.sep) {
+#pragma unroll
+          for (int a = 0; a < SY; ++a) {
+            float h[NJ];
+#pragma unroll
+            for (int j = 0; j < NJ; ++j) h[j] = 0.0f;
+#pragma unroll
+            for (int b = 0; b < SX; ++b) {
+              const float wv = p.sv[b];
+#pragma unroll
+              for (int j = 0; j < NJ; ++j) h[j] = __fmaf_rn(wv, wj[j][a * T.bx + b], h[j]);
+            }
+            const float wu = p.su[a];
+#pragma unroll
+            for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wu, h[j], acc[j]);
+          }
+        } else {
+#pragma unroll
+          for (int kz = 0; kz < SZ; ++kz)
+#pragma unroll
+            for (int ky = 0; ky < SY; ++ky) {
+              const int ro = kz * BYX + ky * T.bx;
+#pragma unroll
+              for (int kx = 0; kx < SX; ++kx) {
+                const float wv = p.w[(kz * SY + ky) * SX + kx];
+#pragma unroll
+                for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wv, wj[j][ro + kx], acc[j]);
+              }
+            }
+        }
+      } else if (p.sep) {
         // separable 2D weights: rows first (x taps in order), then the column (K0's order)
         for (int a = 0; a < p.size[1]; ++a) {
           float h[NJ];
@@ -313,12 +351,28 @@ cudaError_t launch_gather(const StencilParams& p, const float* in0, float* out, 
   const size_t box_bytes = (size_t)T.bz * T.by * T.bx * sizeof(float);
   const int nbuf = 2 * box_bytes <= (size_t)kMaxSmemFloats * 4 ? 2 : 1;
   const size_t smem = nbuf * box_bytes;
+  // compile-time windows for the common shapes when every tap is non-zero
+  // (the unrolled loop then runs the tap list's order) or the weights are separable
+  const int sz = p.size[0], sy = p.size[1], sx = p.size[2];
+  const bool dense = p.ntaps == sz * sy * sx;
+  const bool ok = (dense || p.sep) && !getenv("LIFT_K5_GENERIC");
+  const void* fn = reinterpret_cast<const void*>(&k5_gather<0, 0, 0>);
+  if (ok && sz == 1 && sy == 3 && sx == 3) fn = reinterpret_cast<const void*>(&k5_gather<1, 3, 3>);
+  else if (ok && sz == 1 && sy == 5 && sx == 5) fn = reinterpret_cast<const void*>(&k5_gather<1, 5, 5>);
+  else if (ok && sz == 1 && sy == 2 && sx == 2) fn = reinterpret_cast<const void*>(&k5_gather<1, 2, 2>);
+  else if (dense && !getenv("LIFT_K5_GENERIC") && sz == 3 && sy == 3 && sx == 3)
+    fn = reinterpret_cast<const void*>(&k5_gather<3, 3, 3>);
+  else if (dense && !getenv("LIFT_K5_GENERIC") && sz == 2 && sy == 2 && sx == 2)
+    fn = reinterpret_cast<const void*>(&k5_gather<2, 2, 2>);
   static std::once_flag once;
   std::call_once(once, [] {
-    cudaFuncSetAttribute(k5_gather, cudaFuncAttributeMaxDynamicSharedMemorySize, kMaxSmemFloats * 4);
+    for (const void* f : {reinterpret_cast<const void*>(&k5_gather<0, 0, 0>), reinterpret_cast<const void*>(&k5_gather<1, 3, 3>),
+                          reinterpret_cast<const void*>(&k5_gather<1, 5, 5>), reinterpret_cast<const void*>(&k5_gather<1, 2, 2>),
+                          reinterpret_cast<const void*>(&k5_gather<3, 3, 3>), reinterpret_cast<const void*>(&k5_gather<2, 2, 2>)})
+      cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, kMaxSmemFloats * 4);
   });
   int occ = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k5_gather, kThreads, smem) != cudaSuccess || occ < 1) occ = 1;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, kThreads, smem) != cudaSuccess || occ < 1) occ = 1;
   cudaGetLastError();
   int64_t grid = (int64_t)num_sms * occ;
   const int64_t ntiles = ntz * nty * ntx;
@@ -330,8 +384,7 @@ cudaError_t launch_gather(const StencilParams& p, const float* in0, float* out, 
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
   int nb = nbuf;
   void* args[] = {(void*)&p, (void*)&T, (void*)&in0, (void*)&out, (void*)&ntz, (void*)&nty, (void*)&ntx, (void*)&nb};
-  return launch_kernel(reinterpret_cast<const void*>(&k5_gather), dim3((unsigned)grid), dim3(kThreads), args, smem,
-                       stream, !fz);
+  return launch_kernel(fn, dim3((unsigned)grid), dim3(kThreads), args, smem, stream, !fz);
 }
 
 }  // namespace lift
