@@ -196,3 +196,22 @@ def test_beyond_2pow31_elements_3d(lift, kind):
     check_points(spec, [si.HashGrid(ext, 2024)], y, pts)
     del y
     torch.cuda.empty_cache()
+
+
+def test_strided_and_dampen_full_size(lift):
+    """K5 at full size: an 8192^2 5x5 step-2 slide with DAMPEN pads (A29) and a
+    512^3 3x3x3 step-2 slide, sampled points one by one against the oracle."""
+    w2 = np.random.default_rng(131).standard_normal((5, 5)).astype(np.float32)
+    sp2 = si.StencilSpec((8192, 8192), (5, 5), (2, 2), (2, 2), (2, 2), (si.DAMPEN, si.MIRROR), 0.0, si.WEIGHTED,
+                         w2, (), pad_decay=0.7)
+    x2 = si.uniform((8192, 8192), 132, 0.5, 1.5)
+    y2, plan2 = gpu_apply(lift, sp2, [x2])
+    assert plan2.variant == lift.plan.VARIANTS["gather"]
+    check_points(sp2, [x2], y2, samples(sp2.out_extents(), 300, 133))
+    w3 = np.random.default_rng(134).standard_normal((3, 3, 3)).astype(np.float32)
+    sp3 = si.StencilSpec((512, 512, 512), (3, 3, 3), (2, 2, 2), (1, 1, 1), (1, 1, 1), (si.CLAMP,) * 3, 0.0,
+                         si.WEIGHTED, w3, ())
+    x3 = si.uniform((512, 512, 512), 135, 0.5, 1.5)
+    y3, plan3 = gpu_apply(lift, sp3, [x3])
+    assert plan3.variant == lift.plan.VARIANTS["gather"]
+    check_points(sp3, [x3], y3, samples(sp3.out_extents(), 300, 136))
