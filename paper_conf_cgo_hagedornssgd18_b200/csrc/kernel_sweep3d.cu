@@ -1108,12 +1108,12 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   // long chunks (their 2R warm-up planes per chunk cost issue slots) and only
   // shorten the chunks of the last waves (guided tail).
   int64_t tail_zc = 0;
-  if (work >= 16 * slots && !p.fused_step) {
+  if (work >= 16 * slots) {
     const bool box = p.op == OP_WEIGHTED && !star_weights(p, 1);
     if (R == 1 && !box && (p.op == OP_WEIGHTED || p.op == OP_ACOUSTIC)) {
       const int64_t k = p.op == OP_ACOUSTIC ? 40 : 20;
       zc = std::min<int64_t>(64, std::max<int64_t>(4, (k * tiles + slots / 2) / slots));
-    } else {
+    } else if (!p.fused_step) {       // (the fused step keeps uniform chunks: boundary chunks first)
       tail_zc = p.op == OP_ACOUSTIC ? 16 : 8;
     }
   }
