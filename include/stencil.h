@@ -99,7 +99,9 @@ typedef enum {
   STENCIL_VARIANT_PERSIST3D = 3, /* K4: all n steps of stencil_iterate in one
                                     persistent cooperative launch (small,
                                     L2-resident 3D radius-1 star / Hotspot3D
-                                    grids; AUTO only — reported, not forceable) */
+                                    grids; opt-in with LIFT_K4=1 — measured
+                                    slower than K2 steps; reported by
+                                    stencil_plan_last_variant, not forceable)  */
   STENCIL_VARIANT_GATHER = 4     /* K5: WEIGHTED plans the TMA families do not
                                     take (step > 1, even / asymmetric windows,
                                     1D, wide boxes, unaligned 3D) through
