@@ -13,9 +13,16 @@ per-time-step halo exchange (NCCL send/recv) overlapped with interior compute
 (weak scaling).  Inputs (512 MiB per grid) are larger than L2 (126 MB), so no
 L2 flush is needed between timed iterations.
 
-Other single-GPU workloads (--workload): the remaining BASELINE.json configs
-(gauss5_8192_mirror, j2d5_256_clamp, hotspot3d_8x512x512, srad1_4096,
-srad2_4096, acoustic7_1024, acoustic13_1024).
+Other workloads (--workload, stencil_inputs.WORKLOAD_NAMES): the remaining
+BASELINE.json configs (gauss5_8192_mirror, j2d5_256_clamp,
+hotspot3d_8x512x512[_x100], srad1_4096, srad2_4096, srad_iter_4096,
+acoustic7_1024, acoustic13_1024) and the Table-1 workloads (t1_*).
+Workloads whose per-sweep bytes are below 2 x L2 are timed cold: a 2 x L2
+buffer is written before every timed step (outside its event pair) and a
+single-sweep workload's step is one sweep; the warm number is reported as
+"hot" (--no-flush times warm).  --scaling strong splits the single-GPU grid
+over the ranks (Acoustic 1024^3 over 1/2/4/8 GPUs); --halo fused exchanges
+ghosts by peer stores from the boundary kernel instead of NCCL.
 
 Metric: stencil Gpoints/s = output points x time steps / time (PAPER.md
 P:958-959 "elements updated per second"); roofline: algorithmic HBM bytes per
