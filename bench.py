@@ -555,7 +555,11 @@ def main():
                               "L2 flushed (2 x L2 write) before every timed step" if cold else
                               "inputs larger than L2 (no flush needed)" if npts_local * bpp >= 2 * L2_BYTES
                               else "L2-resident working set, not flushed (--no-flush)"),
-                       "variant": {0: "K0 generic", 1: "K1 tile2d (TMA)", 2: "K2 sweep3d (TMA)",
+                       "variant": {0: "K0 generic",
+                                   1: ("K1 tile2d (TMA)" if ext1[-1] % 4 == 0 else
+                                       "K1 tile2d (cp.async 8-B pair fill)" if ext1[-1] % 2 == 0 else
+                                       "K1 tile2d (cp.async 4-B fill)"),
+                                   2: "K2 sweep3d (TMA)",
                                    3: "K4 persistent iterate (cooperative)"}[variant_id],
                        "launch": (f"cuda graph replay ({launches_per_step} launches per graph)" if graph is not None
                                   else "stream launches")},

@@ -277,9 +277,28 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
     // consumers fill a double-buffered box with 4-byte cp.async copies
     // (out-of-grid cells are zero, as TMA's fill) while computing the other
     static_assert(S == 2, "LDG variant double-buffers");
+    static_assert(BX % 2 == 0 && XH % 2 == 0 && TX % 2 == 0 && C::BOX_FLOATS % 2 == 0, "pair fill");
+    // even nx and 8-B aligned bases (e.g. SHOC's 4098-wide rows): the box is
+    // filled in 8-byte pairs; x0 - XH is even, so a pair is wholly in or out
+    const bool pairs = (nx % 2 == 0) && ((reinterpret_cast<uintptr_t>(src0) | reinterpret_cast<uintptr_t>(src1)) & 7u) == 0;
     auto fill = [&](int s, int64_t t) {
       const int x0 = (int)(t % ntx) * TX, y0 = (int)(t / ntx) * TY;
       float* base = reinterpret_cast<float*>(dsm4 + s * SF4);
+      if (pairs) {
+        constexpr int BX2 = BX / 2;
+        for (int idx = threadIdx.x; idx < NIN * C::BY * BX2; idx += NCONS) {
+          const int b = idx / (C::BY * BX2), rem = idx % (C::BY * BX2);
+          const int r = rem / BX2, c = 2 * (rem % BX2);
+          const int gy = y0 - RY + r, gx = x0 - XH + c;
+          float* dst = base + b * C::BOX_FLOATS + r * BX + c;
+          if (gy >= 0 && gy < ny && gx >= 0 && gx < nx)
+            cp_async8(dst, (b == 0 ? src0 : src1) + (int64_t)gy * nx + gx);
+          else
+            *reinterpret_cast<float2*>(dst) = make_float2(0.0f, 0.0f);
+        }
+        cp_async_commit();
+        return;
+      }
       for (int idx = threadIdx.x; idx < NIN * C::BY * BX; idx += NCONS) {
         const int b = idx / (C::BY * BX), rem = idx % (C::BY * BX);
         const int r = rem / BX, c = rem % BX;
