@@ -571,16 +571,20 @@ def test_tile2d_unaligned_widths(lift, shape):
         np.testing.assert_array_equal(y, y0)
 
 
-def test_tile2d_unaligned_pointer(lift):
-    shape = (70, 264)
-    big = torch.from_numpy(rnd((70 * 264 + 1,), 65)).cuda()
-    xin = big[1:].view(*shape)                      # 4-byte aligned only
-    sp = spec(shape, 5, si.weights_gauss5(), MIRROR)
+@pytest.mark.parametrize("off,shape,kind", [(1, (70, 264), MIRROR),      # 4-byte aligned only: 4-B fill
+                                             (2, (70, 264), MIRROR),      # 8-byte aligned: pair fill
+                                             (2, (37, 4098 // 16 * 2 + 2), CONSTANT)])
+def test_tile2d_unaligned_pointer(lift, off, shape, kind):
+    n = shape[0] * shape[1]
+    big = torch.from_numpy(rnd((n + off,), 65)).cuda()
+    xin = big[off:].view(*shape)
+    sp = spec(shape, 5, si.weights_gauss5(), kind, value=-0.25)
     plan = lift.Plan.from_spec(sp)
-    out_big = torch.empty(70 * 264 + 3, device="cuda")
+    out_big = torch.empty(n + 3, device="cuda")
     out = out_big[3:].view(*shape)
     plan.apply(xin, out=out)
     torch.cuda.synchronize()
+    assert plan.variant == 1
     Y, A = orc.apply(sp, [xin.cpu().numpy()])
     assert orc.max_rel_err(out.cpu().numpy(), Y, A) <= TOL1
 
