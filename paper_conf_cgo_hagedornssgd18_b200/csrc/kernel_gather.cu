@@ -38,14 +38,18 @@ constexpr int kMaxRows = 1024;                 // box rows (bz * by)
 
 struct Tile {
   int otz, oty, otx;      // outputs per tile
-  int bz, by, bx;         // input box
+  int bz, by, bx;         // input box; bx is the row pitch: the x extent wx + 3, rounded up to 4
+  int wx;                 // x extent of the box the outputs read
 };
 
 __host__ __device__ inline Tile tile_of(const StencilParams& p, int otz, int oty, int otx) {
-  Tile t{otz, oty, otx, 0, 0, 0};
+  Tile t{otz, oty, otx, 0, 0, 0, 0};
   t.bz = (otz - 1) * p.step[0] + p.size[0];
   t.by = (oty - 1) * p.step[1] + p.size[1];
-  t.bx = (otx - 1) * p.step[2] + p.size[2];
+  // box rows start at the tile's x origin rounded down to a multiple of 4
+  // (up to 3 leading columns), so interior rows are copied in 16-byte pieces
+  t.wx = (otx - 1) * p.step[2] + p.size[2];
+  t.bx = (t.wx + 3 + 3) & ~3;
   return t;
 }
 
@@ -69,7 +73,12 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
                                          int lane) {
   constexpr int NWARP = kThreads / 32;
   const int nrows = T.bz * T.by;
-  const bool x_inside = gx0 >= 0 && gx0 + T.bx <= p.n[2];
+  // row element b holds x = gxa + b: the origin gx0 rounded down to a multiple of 4
+  const int sh = (int)(gx0 & 3);
+  const int64_t gxa = gx0 - sh;
+  const bool x_inside = gx0 >= 0 && gx0 + T.wx <= p.n[2];
+  const int ncopy = sh + T.wx;      // columns the outputs read
+  const bool quads = (p.n[2] % 4 == 0) && (reinterpret_cast<uintptr_t>(in) & 15u) == 0;
   const bool damp = has_dampen(p);
   for (int base = warp; base < nrows; base += NWARP * 32) {
     const int r = base + lane * NWARP;
@@ -91,7 +100,7 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
         const int64_t lz = plane_of(p, gz);
         if (lz >= 0) {
           if (p.kind[0] == PAD_DAMPEN) nrow += (int)outside_dist(gz, p.gnz);
-          off = lz * p.plane + iy * p.row + (x_inside ? gx0 : 0);
+          off = lz * p.plane + iy * p.row + (x_inside ? gxa : 0);
         }
       } else {
         nrow = 0;       // the y value cell: only x's DAMPEN cells (inside it) count
@@ -107,10 +116,15 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
           for (int b = lane; b < T.bx; b += 32) dst[b] = p.pad_value;
         } else if (x_inside) {
           const float* s0 = in + o;
-          for (int b = lane; b < T.bx; b += 32) cp_async4(dst + b, s0 + b);
+          if (quads && (reinterpret_cast<uintptr_t>(s0) & 15u) == 0) {
+            // gxa and nx are multiples of 4 and gx0 + wx <= nx: the last quad ends in the row
+            for (int b = 4 * lane; b < ncopy; b += 128) cp_async16(dst + b, s0 + b);
+          } else {
+            for (int b = lane; b < ncopy; b += 32) cp_async4(dst + b, s0 + b);
+          }
         } else {
           for (int b = lane; b < T.bx; b += 32) {
-            const int64_t ix = remap_or_const(gx0 + b, p.n[2], p.kind[2]);
+            const int64_t ix = remap_or_const(gxa + b, p.n[2], p.kind[2]);
             if (ix < 0) dst[b] = p.pad_value;
             else cp_async4(dst + b, in + o + ix);
           }
@@ -118,7 +132,7 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
       } else {
         // DAMPEN plans: values computed directly (decay^k scaling)
         for (int b = lane; b < T.bx; b += 32) {
-          int64_t ix = gx0 + b;
+          int64_t ix = gxa + b;
           int k = nr;
           float v;
           if ((ix < 0 || ix >= p.n[2]) && p.kind[2] == PAD_CONSTANT) {
@@ -129,7 +143,7 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
               if (p.kind[2] == PAD_DAMPEN) k += (int)outside_dist(ix, p.n[2]);
               ix = pad_remap(ix, p.n[2], p.kind[2]);
             }
-            v = o < 0 ? p.pad_value : __ldg(in + o + (x_inside ? ix - gx0 : ix));
+            v = o < 0 ? p.pad_value : __ldg(in + o + (x_inside ? ix - gxa : ix));
           }
           dst[b] = k ? __fmul_rn(v, dampen_pow(p.pad_decay, k)) : v;
         }
@@ -203,6 +217,7 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
     __syncthreads();
     int64_t oz0, oy0, ox0;
     origin(tile, oz0, oy0, ox0);
+    const int xsh = (int)((ox0 * p.step[2] - p.lo[2]) & 3);   // leading columns of the aligned box rows
     // each thread evaluates NJ outputs per pass: the tap loop's index / weight
     // loads are shared by NJ independent FMA chains
 #pragma unroll
@@ -222,7 +237,7 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
       for (int j = 0; j < NJ; ++j) acc[j] = 0.0f;
       const float* wj[NJ];
 #pragma unroll
-      for (int j = 0; j < NJ; ++j) wj[j] = bcur + woff[ps * NJ + j];
+      for (int j = 0; j < NJ; ++j) wj[j] = bcur + xsh + woff[ps * NJ + j];
       if constexpr (SZ > 0) {
         // compile-time window (dense weights or separable 2D): unrolled taps,
         // immediate x offsets, the same operation order as the tap list
@@ -266,7 +281,7 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
             const float wv = p.sv[b];
             const int o = a * T.bx + b;
 #pragma unroll
-            for (int j = 0; j < NJ; ++j) h[j] = __fmaf_rn(wv, bcur[woff[ps * NJ + j] + o], h[j]);
+            for (int j = 0; j < NJ; ++j) h[j] = __fmaf_rn(wv, wj[j][o], h[j]);
           }
           const float wu = p.su[a];
 #pragma unroll
@@ -277,7 +292,7 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
           const float wv = p.w[t];
           const int o = toff[t];
 #pragma unroll
-          for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wv, bcur[woff[ps * NJ + j] + o], acc[j]);
+          for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wv, wj[j][o], acc[j]);
         }
       }
 #pragma unroll
