@@ -258,18 +258,41 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
             for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wu, h[j], acc[j]);
           }
         } else {
+          // even x step: every output's window starts at the same parity (xsh's), so
+          // tap pairs starting on an even column load as one 8-byte LDS; the FMA
+          // order is the tap list's either way
+          auto dense = [&](auto PARC) {
+            constexpr int PAR = decltype(PARC)::value;
 #pragma unroll
-          for (int kz = 0; kz < SZ; ++kz)
+            for (int kz = 0; kz < SZ; ++kz)
 #pragma unroll
-            for (int ky = 0; ky < SY; ++ky) {
-              const int ro = kz * BYX + ky * T.bx;
+              for (int ky = 0; ky < SY; ++ky) {
+                const int ro = kz * BYX + ky * T.bx;
+                static_for<SX>([&](auto KX) {
+                  constexpr int kx = decltype(KX)::value;
+                  const float* wr = p.w + (kz * SY + ky) * SX;
+                  if constexpr (PAR >= 0 && (kx + PAR) % 2 == 0 && kx + 1 < SX) {
 #pragma unroll
-              for (int kx = 0; kx < SX; ++kx) {
-                const float wv = p.w[(kz * SY + ky) * SX + kx];
+                    for (int j = 0; j < NJ; ++j) {
+                      const float2 v = *reinterpret_cast<const float2*>(wj[j] + ro + kx);
+                      acc[j] = __fmaf_rn(wr[kx], v.x, acc[j]);
+                      acc[j] = __fmaf_rn(wr[kx + 1], v.y, acc[j]);
+                    }
+                  } else if constexpr (PAR >= 0 && (kx + PAR) % 2 == 1 && kx > 0) {
+                    // second tap of a pair: done above
+                  } else {
 #pragma unroll
-                for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wv, wj[j][ro + kx], acc[j]);
+                    for (int j = 0; j < NJ; ++j) acc[j] = __fmaf_rn(wr[kx], wj[j][ro + kx], acc[j]);
+                  }
+                });
               }
-            }
+          };
+          if (p.step[2] % 2 == 0) {
+            if (xsh & 1) dense(std::integral_constant<int, 1>{});
+            else dense(std::integral_constant<int, 0>{});
+          } else {
+            dense(std::integral_constant<int, -1>{});
+          }
         }
       } else if (p.sep) {
         // separable 2D weights: rows first (x taps in order), then the column (K0's order)
