@@ -29,11 +29,16 @@ Pins (tests/test_oracle_*.py): brute force vs ``numpy.pad`` modes and
 linear field under the Laplacian, Gaussian separability, wrap translation
 equivariance, mirror symmetry, linearity).
 
-PARITY UNPINNED (the paper prints no formula or values, the definitions are
-external readings, A16/A18/A19/A25/A26): the Hotspot3D and
-Hotspot2D point functions, the SRAD1/SRAD2 point functions, the Gradient point
-function and the Acoustic constants.  For these only
-structural properties are pinned (fixed points, ranges, brute-force K count).
+The non-linear point functions are EXTERNAL READINGS (the paper prints no
+formula or values, A16/A18/A19/A25/A26): Hotspot3D, Hotspot2D,
+SRAD1/SRAD2, Gradient and the Acoustic constants.  Given the reading, each is
+pinned independently of this file: Hotspot3D/2D, SRAD2 and Gradient by
+independently written scalar Rodinia-style loops; SRAD1 by hand-derived closed
+forms (isolated spike q = eps^2, face neighbour 7eps^2/(16(1+eps/4)^2), ramp
+q = b^2/I^2, c = q0(1+q0)/(q0^2+q)); q0^2 by closed-form images; the
+Acoustic grid roles by the leapfrog identity u' = 2u^n - u^{n-1} on a linear
+u^n with random u^{n-1} and by the locality of each grid; K by brute force.
+What stays unpinned is only whether the readings are the paper's intent.
 """
 from __future__ import annotations
 
@@ -193,7 +198,8 @@ def _star(r: int, nd: int, d: int, off: int) -> Tuple[int, ...]:
 
 
 def f_hotspot3d(W: Callable, Pc, prm: Sequence[float]) -> Tuple:
-    """Rodinia v3.1 hotspot3D update (reading A16; PARITY UNPINNED formula):
+    """Rodinia v3.1 hotspot3D update (reading A16, external; pinned by
+    an independent scalar loop in tests/test_oracle_map.py):
     T' = cc*C + cn*N + cs*S + ce*E + cw*W + ct*T + cb*B + sdc*P + ct*amb,
     N=y-1, S=y+1, W=x-1, E=x+1, B=z-1, T=z+1 (clamped through the pad)."""
     cc, cn, cs, ce, cw, ct, cb, sdc, amb = (np.float64(v) for v in prm)
@@ -210,7 +216,8 @@ def f_hotspot3d(W: Callable, Pc, prm: Sequence[float]) -> Tuple:
 
 
 def f_srad1(W: Callable, prm: Sequence[float]) -> Tuple:
-    """Rodinia v3.1 SRAD first kernel, I -> c (reading A18; PARITY UNPINNED):
+    """Rodinia v3.1 SRAD first kernel, I -> c (reading A18, external; pinned by
+    hand-derived closed forms: spike, face neighbour, ramp):
     dX = I_X - I_c;  G2 = sum dX^2 / I_c^2;  L = sum dX / I_c;
     num = 0.5*G2 - L^2/16;  den = 1 + 0.25*L;  q = num/den^2;
     d = (q - q0)/(q0*(1+q0));  c = clamp(1/(1+d), 0, 1)."""
@@ -277,7 +284,8 @@ def _with(spec, op, params):
 
 
 def f_hotspot2d(WT: Callable, WP: Callable, prm: Sequence[float]) -> Tuple:
-    """Rodinia v3.1 hotspot (2D) update (reading A26; PARITY UNPINNED formula):
+    """Rodinia v3.1 hotspot (2D) update (reading A26, external; pinned by
+    an independent scalar loop):
     T' = T + sdc*(P + (S + N - 2T)/Ry + (E + W - 2T)/Rx + (amb - T)/Rz),
     with params (sdc, 1/Rx, 1/Ry, 1/Rz, amb); N=y-1, S=y+1, W=x-1, E=x+1."""
     sdc, rx1, ry1, rz1, amb = (np.float64(v) for v in prm)
@@ -294,7 +302,8 @@ def f_hotspot2d(WT: Callable, WP: Callable, prm: Sequence[float]) -> Tuple:
 
 
 def f_gradient(W: Callable, prm: Sequence[float]) -> Tuple:
-    """Rawat et al. [36] 2D gradient (reading A25; PARITY UNPINNED formula):
+    """Rawat et al. [36] 2D gradient (reading A25, external; pinned by
+    an independent scalar loop):
     out = I + 1/sqrt(eps + (I-N)^2 + (I-S)^2 + (I-W)^2 + (I-E)^2)."""
     eps = np.float64(prm[0])
     Ic = W((1, 1))
@@ -318,7 +327,8 @@ def acoustic_neighbours(o: Sequence, extents: Sequence[int], r: int):
 
 def f_acoustic(W: Callable, prev_c, K, r: int, prm: Sequence[float]) -> Tuple:
     """Listing 3 with the physics reading A19 (slid grid = u^n,
-    point-wise grid = u^{n-1}, output = u^{n+1}; PARITY UNPINNED constants):
+    point-wise grid = u^{n-1}, output = u^{n+1}; the constants are proposed;
+    roles pinned by the leapfrog identity and per-grid locality):
     u' = cf(K, l1) * ((2 - l2*K) * u_c + l2 * sum_nbr u - cf(K, l2loss) * prev),
     getCF(K, x, 1.0) = (K < K_max) ? x : 1.0."""
     l2, loss1, loss2 = (np.float64(v) for v in prm)
