@@ -176,9 +176,10 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
     const uint32_t t32 = (uint32_t)tile, r = t32 / (uint32_t)ntx;
     const uint32_t tx = t32 - r * (uint32_t)ntx;
     const uint32_t tz = r / (uint32_t)nty, ty = r - tz * (uint32_t)nty;
-    oz0 = p.reg0 + tz * T.otz;
-    oy0 = ty * T.oty;
-    ox0 = tx * T.otx;
+    // widen before multiplying: a 1D plan's x extent may exceed 2^32
+    oz0 = p.reg0 + (int64_t)tz * T.otz;
+    oy0 = (int64_t)ty * T.oty;
+    ox0 = (int64_t)tx * T.otx;
   };
   auto fill = [&](int64_t tile, int buf) {
     int64_t oz0, oy0, ox0;

@@ -464,8 +464,11 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
     }
     const int xo = x0 + 4 * lane;
     const bool x_ok = xo < nx;
-    // c column x+4 at the right grid edge takes the remapped column's value
-    const int ce = (xo + 4 == nx) ? (int)(pad_remap(nx, nx, kx) - xo) : 4;
+    // c column x+4 at the right grid edge takes the remapped column's value;
+    // under WRAP the fixed-up box already holds I's wrapped columns, so the
+    // value SRAD1 computes there IS c(0) (the remap would point at
+    // column -xo)
+    const int ce = (xo + 4 == nx && kx != PAD_WRAP) ? (int)(pad_remap(nx, nx, kx) - xo) : 4;
     const float4* box = dsm4 + s * SF4;
     float iw[4][W];
     float cr[3][5];
@@ -495,7 +498,9 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
         // c for I row crow = y0 + r0 + k - 2 from I rows crow-1 .. crow+1
         constexpr int cs_ = (k - 2) % 3;
         const int crow = y0 + r0 + k - 2;
-        if (crow < ny) {
+        // c rows past the bottom edge: WRAP computes them from the box's
+        // wrapped I rows (= c(crow - ny)); the others copy the remapped row
+        if (crow < ny || ky == PAD_WRAP) {
           static_for<4>([&](auto II) {
             constexpr int ii = decltype(II)::value;
             cr[cs_][ii] = op_srad1(RowsAcc<2, ii>{iw[(k - 2) % 4], iw[(k - 1) % 4], iw[k % 4]}, q);

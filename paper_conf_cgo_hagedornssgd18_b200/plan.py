@@ -152,6 +152,14 @@ class Plan:
                  stream: Optional[torch.cuda.Stream] = None) -> np.ndarray:
         if out is None:
             out = np.empty(self.out_alloc_extents, np.float32)
+        # the C side copies whole grids: a wrongly sized host array would be
+        # over-read / over-written, so check every size here
+        n_in = int(np.prod(self.alloc_extents))
+        for a in list(host_state) + list(host_aux):
+            if np.asarray(a).size != n_in:
+                raise ValueError(f"run_host: input of {np.asarray(a).size} elements, plan needs {n_in}")
+        if out.size != int(np.prod(self.out_alloc_extents)):
+            raise ValueError(f"run_host: out has {out.size} elements, plan writes {int(np.prod(self.out_alloc_extents))}")
         L.stencil_run_host(self.handle, list(host_state), list(host_aux), n_steps, out, _stream_handle(stream))
         return out
 

@@ -446,7 +446,7 @@ def test_time_block_eligibility(lift):
 
 
 # ---------------------------------------- full SRAD iteration (NEXT-2) -----
-@pytest.mark.parametrize("kind", [CLAMP, MIRROR, REFLECT])
+@pytest.mark.parametrize("kind", [CLAMP, MIRROR, REFLECT, WRAP, (WRAP, CLAMP), (MIRROR, WRAP)])
 def test_srad_iteration(lift, kind):
     """q0 reduction + SRAD1/SRAD2 fused in one pass (K1S) vs the oracle's
     SRAD1-then-SRAD2 with q0 of the current image; K1S == K0 bitwise."""
