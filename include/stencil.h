@@ -235,6 +235,24 @@ stencil_status stencil_wait_signals(const uint32_t* sig_a, const uint32_t* sig_b
                                     void* stream);
 
 /*
+ * Bounded halo waits.  Every flag wait of the fused slab path (the producer
+ * of stencil_slab_step_fused, the kernel of stencil_wait_signals) gives up
+ * after a process-wide timeout instead of spinning forever on a neighbour
+ * that died or stalled: it records the fault in a host-visible word and lets
+ * the launch finish (its ghost planes are then stale).
+ *   stencil_set_wait_timeout_ms : the timeout for subsequent launches; 0 =
+ *       wait forever; default 10000 ms (environment LIFT_WAIT_TIMEOUT_MS).
+ *   stencil_device_fault : after the caller has synchronised the stream,
+ *       returns E_CUDA (detail in stencil_last_error: which neighbour) if a
+ *       wait timed out since the last check, and clears the record; OK
+ *       otherwise.  stencil_slab_step_fused, stencil_apply_region_put and
+ *       stencil_wait_signals also check it on entry and return E_CUDA
+ *       without launching.
+ */
+stencil_status stencil_set_wait_timeout_ms(uint32_t ms);
+stencil_status stencil_device_fault(void);
+
+/*
  * iterate(in, f, n_steps) with the state rotation of reading A21:
  *   WEIGHTED  : state {X0, X1}            X_{t+1} = S(X_t), ping-pong
  *   HOTSPOT3D, HOTSPOT2D : state {T0, T1}, aux {P}   T_{t+1} = S(T_t, P)

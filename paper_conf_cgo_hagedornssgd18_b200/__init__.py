@@ -9,6 +9,7 @@ tensors, ``slab`` adds the multi-GPU slab decomposition.
 from . import _lib
 from ._lib import (StencilError, stencil_apply, stencil_apply_region, stencil_apply_region_put,  # noqa: F401
                    stencil_iterate, stencil_slab_step_fused, stencil_wait_signals,
+                   stencil_set_wait_timeout_ms, stencil_device_fault,
                    stencil_last_error, stencil_plan_create, stencil_plan_destroy,
                    stencil_plan_output_extents, stencil_plan_set_slab, stencil_plan_set_time_block,
                    stencil_plan_set_variant, stencil_plan_time_block,

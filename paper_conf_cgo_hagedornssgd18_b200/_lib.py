@@ -60,6 +60,8 @@ _slab_step_fused = _sig("stencil_slab_step_fused", C.c_int, [_P, _FPP, C.c_int32
                                                             _P, _P, C.c_uint32, _P])
 _wait_signals = _sig("stencil_wait_signals", C.c_int, [_P, _P, C.c_uint32, _P])
 _iterate = _sig("stencil_iterate", C.c_int, [_P, _FPP, C.c_int32, _FPP, C.c_int32, C.c_int32, _P, _I32P])
+_set_wait_timeout = _sig("stencil_set_wait_timeout_ms", C.c_int, [C.c_uint32])
+_device_fault = _sig("stencil_device_fault", C.c_int, [])
 _run_host = _sig("stencil_run_host", C.c_int, [_P, _FPP, C.c_int32, _FPP, C.c_int32, C.c_int32, _P, _P])
 _destroy = _sig("stencil_plan_destroy", None, [_P])
 _status_string = _sig("stencil_status_string", C.c_char_p, [C.c_int])
@@ -72,6 +74,7 @@ EXPORTED = ("stencil_plan_create", "stencil_plan_output_extents", "stencil_plan_
             "stencil_plan_set_time_block",
             "stencil_plan_time_block", "stencil_apply", "stencil_apply_region",
             "stencil_apply_region_put", "stencil_slab_step_fused", "stencil_wait_signals",
+            "stencil_set_wait_timeout_ms", "stencil_device_fault",
             "stencil_iterate", "stencil_run_host", "stencil_plan_destroy", "stencil_status_string",
             "stencil_last_error", "stencil_version")
 
@@ -201,6 +204,16 @@ def stencil_iterate(plan: int, state: Sequence[int], aux: Sequence[int], n_steps
     _check(_iterate(plan, _ptrs(state), len(state), _ptrs(aux), len(aux), int(n_steps), C.c_void_p(int(stream)),
                     C.byref(ri)), "stencil_iterate")
     return ri.value
+
+
+def stencil_set_wait_timeout_ms(ms: int):
+    _check(_set_wait_timeout(int(ms)), "stencil_set_wait_timeout_ms")
+
+
+def stencil_device_fault():
+    """Raises StencilError (E_CUDA) if a bounded halo wait timed out since the
+    last check (call after synchronising the stream)."""
+    _check(_device_fault(), "stencil_device_fault")
 
 
 def stencil_run_host(plan: int, host_state: Sequence[np.ndarray], host_aux: Sequence[np.ndarray], n_steps: int,

@@ -5,7 +5,9 @@
 
 #include <cmath>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
+#include <mutex>
 #include <new>
 #include <string>
 #include <vector>
@@ -54,6 +56,56 @@ stencil_status fail(stencil_status s, const std::string& msg) {
 stencil_status cuda_fail(cudaError_t e, const char* what) {
   g_last_error = std::string(what) + ": " + cudaGetErrorString(e);
   return STENCIL_E_CUDA;
+}
+
+// ---- bounded halo waits (fused slab path) --------------------------------
+// One process-wide fault word in mapped pinned host memory: a wait that times
+// out ORs a code into it (device store, system scope) and the host reads it
+// without a device round trip.  The timeout is process-wide too.
+std::mutex g_fault_mu;
+unsigned int* g_fault = nullptr;          // host pointer == device pointer (UVA)
+unsigned long long g_wait_timeout_ns = [] {
+  const char* e = getenv("LIFT_WAIT_TIMEOUT_MS");
+  return (unsigned long long)(e ? strtoull(e, nullptr, 10) : 10000ull) * 1000000ull;
+}();
+
+unsigned int* fault_word(cudaError_t* err) {
+  std::lock_guard<std::mutex> lk(g_fault_mu);
+  if (!g_fault) {
+    void* h = nullptr;
+    *err = cudaHostAlloc(&h, 64, cudaHostAllocMapped | cudaHostAllocPortable);
+    if (*err != cudaSuccess) return nullptr;
+    std::memset(h, 0, 64);
+    g_fault = static_cast<unsigned int*>(h);
+  }
+  *err = cudaSuccess;
+  return g_fault;
+}
+
+// E_CUDA (and clears the word) if a kernel recorded a fault since the last check
+stencil_status take_fault() {
+  unsigned int f = 0;
+  {
+    std::lock_guard<std::mutex> lk(g_fault_mu);
+    if (!g_fault) return STENCIL_OK;
+    f = __atomic_exchange_n(g_fault, 0u, __ATOMIC_ACQ_REL);
+  }
+  if (!f) return STENCIL_OK;
+  std::string which = (f & kFaultWaitLo) && (f & kFaultWaitHi) ? "lower and upper"
+                      : (f & kFaultWaitLo) ? "lower" : "upper";
+  return fail(STENCIL_E_CUDA, "fused halo wait timed out after " + std::to_string(g_wait_timeout_ns / 1000000ull) +
+                                  " ms: the " + which +
+                                  " neighbour never raised its flag (dead or stalled rank); the step's ghost "
+                                  "planes are stale");
+}
+
+// Arms a launch's bounded waits.
+stencil_status arm_waits(StencilParams& p) {
+  cudaError_t e;
+  p.fault = fault_word(&e);
+  if (!p.fault) return cuda_fail(e, "cudaHostAlloc (fault word)");
+  p.wait_timeout_ns = g_wait_timeout_ns;
+  return STENCIL_OK;
 }
 
 // Saves/restores the caller's current device around library calls.
@@ -418,6 +470,10 @@ stencil_status stencil_plan_set_slab(stencil_plan pl, int64_t z_offset, int64_t 
   p.gnz = global_n0;
   p.ghost = ghost;
   p.slab = 1;
+  // allocate the fault word now, outside any graph capture (without a device
+  // this fails quietly; the fused launches retry and report it)
+  cudaError_t e;
+  (void)fault_word(&e);
   return STENCIL_OK;
 }
 
@@ -497,6 +553,8 @@ stencil_status stencil_apply_region_put(stencil_plan pl, const float* const* inp
   stencil_status s = check_inputs(pl, inputs, n_inputs, out);
   if (s != STENCIL_OK) return s;
   if (!pl->p.slab) return fail(STENCIL_E_INVALID, "fused halo put needs a slab plan (stencil_plan_set_slab)");
+  s = take_fault();
+  if (s != STENCIL_OK) return s;
   if (o0_begin < 0 || o0_end > pl->p.o[0] || o0_begin >= o0_end)
     return fail(STENCIL_E_INVALID, "region outside the output extents");
   if (choose_variant(pl, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out) != STENCIL_VARIANT_SWEEP3D)
@@ -522,6 +580,8 @@ stencil_status stencil_slab_step_fused(stencil_plan pl, const float* const* inpu
   stencil_status s = check_inputs(pl, inputs, n_inputs, out);
   if (s != STENCIL_OK) return s;
   if (!pl->p.slab) return fail(STENCIL_E_INVALID, "fused step needs a slab plan (stencil_plan_set_slab)");
+  s = take_fault();
+  if (s != STENCIL_OK) return s;
   if (choose_variant(pl, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out) != STENCIL_VARIANT_SWEEP3D)
     return fail(STENCIL_E_UNSUPPORTED, "fused step is built on the TMA sweep kernel only");
   DeviceGuard g(pl->device);
@@ -538,14 +598,29 @@ stencil_status stencil_slab_step_fused(stencil_plan pl, const float* const* inpu
   p.wait_hi = wait_hi;
   p.wait_value = wait_value;
   p.fused_step = 1;
+  s = arm_waits(p);
+  if (s != STENCIL_OK) return s;
   return launch(pl, p, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out, (cudaStream_t)stream);
 }
 
 stencil_status stencil_wait_signals(const uint32_t* sig_a, const uint32_t* sig_b, uint32_t value, void* stream) {
-  cudaError_t e = launch_wait_signals(sig_a, sig_b, value, (cudaStream_t)stream);
+  stencil_status s = take_fault();
+  if (s != STENCIL_OK) return s;
+  cudaError_t e;
+  unsigned int* fault = fault_word(&e);
+  if (!fault) return cuda_fail(e, "cudaHostAlloc (fault word)");
+  e = launch_wait_signals(sig_a, sig_b, value, g_wait_timeout_ns, fault, (cudaStream_t)stream);
   if (e != cudaSuccess) return cuda_fail(e, "wait kernel launch");
   return STENCIL_OK;
 }
+
+stencil_status stencil_set_wait_timeout_ms(uint32_t ms) {
+  std::lock_guard<std::mutex> lk(g_fault_mu);
+  g_wait_timeout_ns = (unsigned long long)ms * 1000000ull;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_device_fault(void) { return take_fault(); }
 
 stencil_status stencil_apply(stencil_plan pl, const float* const* inputs, int32_t n_inputs, float* out,
                              void* stream) {

@@ -80,7 +80,15 @@ struct StencilParams {
   const unsigned int* wait_hi;
   unsigned int wait_value;
   int32_t fused_step;
+  // bounded waits: give up after wait_timeout_ns (0 = never) and OR a fault
+  // code into *fault (host-mapped word, read by stencil_device_fault)
+  unsigned long long wait_timeout_ns;
+  unsigned int* fault;
 };
+
+// fault codes ORed into the host-visible fault word by a timed-out wait
+constexpr unsigned int kFaultWaitLo = 1u;   // flag of the lower neighbour never arrived
+constexpr unsigned int kFaultWaitHi = 2u;   // flag of the upper neighbour never arrived
 
 // h(i, n) of the reindexing pad (A1-A5).
 // i is the unpadded index (padded index minus l).  Only called when i is out

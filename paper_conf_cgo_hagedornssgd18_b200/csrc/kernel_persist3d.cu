@@ -30,17 +30,15 @@
 #include "common.cuh"
 #include "launch.hpp"
 #include "ops.cuh"
+#include "slots.cuh"
 
 namespace lift {
 namespace {
 
 constexpr int kThreads = 512;
-constexpr int kSlots = 64;
-
-// per-launch-slot barrier state: arrivals, generation, exits (reset by the last CTA)
-__device__ unsigned int g_k4_arrive[kSlots];
-__device__ unsigned int g_k4_gen[kSlots];
-__device__ unsigned int g_k4_exit[kSlots];
+// grid-barrier state, one slot per running launch (slots.cuh): c[0]
+// arrivals, c[1] generation, c[2] exits (reset by the last CTA)
+__device__ LaunchSlot g_launch[kLaunchSlots];
 
 enum K4Op { K4_WSTAR = 0, K4_HOTSPOT = 1 };
 
@@ -96,7 +94,7 @@ __device__ __forceinline__ float4 eval4(const StencilParams& p, const Star4& w, 
 // loaded once and reused as the z-1 / z+1 taps of the next / previous plane.
 template <int OP, int ZB>
 __global__ void __launch_bounds__(kThreads) k4_iterate(const __grid_constant__ StencilParams p, float* s0, float* s1,
-                                                       const float* __restrict__ aux, int n_steps, int slot) {
+                                                       const float* __restrict__ aux, int n_steps) {
   const int64_t nx = p.n[2], ny = p.n[1], nz = p.n[0];
   const uint32_t nx4 = (uint32_t)(nx >> 2);
   const uint32_t nzb = (uint32_t)((nz + ZB - 1) / ZB);
@@ -107,6 +105,8 @@ __global__ void __launch_bounds__(kThreads) k4_iterate(const __grid_constant__ S
   const float4 cv = make_float4(p.pad_value, p.pad_value, p.pad_value, p.pad_value);
   const float* in = s0;
   float* out = s1;
+  int slot = 0;                      // used by thread 0 only
+  if (threadIdx.x == 0 && n_steps > 1) slot = claim_launch_slot(g_launch);
   for (int t = 0; t < n_steps; ++t) {
     // warp-uniform loop (full-warp shuffles); units < 2^31 (L2-resident grids only)
     for (uint32_t u0 = blockIdx.x * blockDim.x + (threadIdx.x & ~31u); u0 < units; u0 += wstride) {
@@ -163,12 +163,12 @@ __global__ void __launch_bounds__(kThreads) k4_iterate(const __grid_constant__ S
       __syncthreads();
       if (threadIdx.x == 0) {
         __threadfence();
-        const unsigned int a = atomicAdd(&g_k4_arrive[slot], 1u);
+        const unsigned int a = atomicAdd(&g_launch[slot].c[0], 1u);
         if (a == (unsigned)(t + 1) * gridDim.x - 1) {
           __threadfence();
-          atomicExch(&g_k4_gen[slot], (unsigned)(t + 1));
+          atomicExch(&g_launch[slot].c[1], (unsigned)(t + 1));
         } else {
-          while (*reinterpret_cast<volatile unsigned int*>(&g_k4_gen[slot]) < (unsigned)(t + 1)) __nanosleep(20);
+          while (*reinterpret_cast<volatile unsigned int*>(&g_launch[slot].c[1]) < (unsigned)(t + 1)) __nanosleep(20);
         }
         __threadfence();
       }
@@ -180,12 +180,7 @@ __global__ void __launch_bounds__(kThreads) k4_iterate(const __grid_constant__ S
   }
   // the last CTA out resets the slot (every CTA has passed every barrier by then)
   if (threadIdx.x == 0 && n_steps > 1) {
-    if (atomicAdd(&g_k4_exit[slot], 1u) == gridDim.x - 1) {
-      g_k4_arrive[slot] = 0;
-      g_k4_gen[slot] = 0;
-      g_k4_exit[slot] = 0;
-      __threadfence();
-    }
+    if (atomicAdd(&g_launch[slot].c[2], 1u) == gridDim.x - 1) release_launch_slot(g_launch, slot);
   }
 }
 
@@ -207,8 +202,6 @@ Launcher get_launcher() {
   });
   return L;
 }
-
-std::atomic<unsigned> g_k4_slot{0};
 
 }  // namespace
 
@@ -253,8 +246,7 @@ cudaError_t launch_persist3d(const StencilParams& p, float* s0, float* s1, const
   int64_t grid = (int64_t)num_sms * L.blocks_per_sm;
   const int64_t need = (units + kThreads - 1) / kThreads;
   if (grid > need) grid = need;
-  int slot = (int)(g_k4_slot.fetch_add(1) % kSlots);
-  void* args[] = {(void*)&p, (void*)&s0, (void*)&s1, (void*)&aux, (void*)&n_steps, (void*)&slot};
+  void* args[] = {(void*)&p, (void*)&s0, (void*)&s1, (void*)&aux, (void*)&n_steps};
   // cooperative attribute: all CTAs co-resident or the launch fails (never a
   // silent deadlock in the grid barrier); capturable into CUDA graphs
   cudaLaunchConfig_t cfg{};

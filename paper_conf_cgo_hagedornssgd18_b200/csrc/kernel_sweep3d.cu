@@ -44,6 +44,7 @@
 #include "halo.cuh"
 #include "launch.hpp"
 #include "ops.cuh"
+#include "slots.cuh"
 #include "tma.cuh"
 
 namespace lift {
@@ -55,12 +56,9 @@ constexpr int BX = TX + 2 * XH;
 constexpr int NW = 8;          // consumer warps
 constexpr int NCONS = NW * 32;
 constexpr unsigned FULL = 0xffffffffu;
-constexpr int kTickets = 4096;
-
-// dynamic work counters (one per in-flight launch slot; reset by the last CTA)
-__device__ unsigned int g_ticket[kTickets];
-__device__ unsigned int g_done[kTickets];
-__device__ unsigned int g_bdone[kTickets][2];   // finished boundary-chunk items (fused step)
+// dynamic work counters, one slot per running launch (slots.cuh): c[0] item
+// ticket, c[1] CTAs done, c[2..3] finished boundary-chunk items (fused step)
+__device__ LaunchSlot g_launch[kLaunchSlots];
 
 // fused step: boundary chunks first (item order: chunk 0, chunk last, then the rest)
 __device__ __forceinline__ int chunk_of(int c, int nchunk, bool fused) {
@@ -74,10 +72,6 @@ __device__ __forceinline__ int chunk_of(int c, int nchunk, bool fused) {
 // others idle — is short too)
 __device__ __forceinline__ int64_t chunk_z0(int c, int zc, int n1, int zc2) {
   return c < n1 ? (int64_t)c * zc : (int64_t)n1 * zc + (int64_t)(c - n1) * zc2;
-}
-
-__device__ __forceinline__ void spin_until(const unsigned int* f, unsigned int v) {
-  while ((int)(ld_acquire_sys(f) - v) < 0) __nanosleep(32);
 }
 
 enum K2Op { K2_WSTAR = 0, K2_HOTSPOT = 1, K2_ACOUSTIC = 2, K2_WBOX = 3, K2_WBOX19 = 4 };
@@ -149,7 +143,7 @@ template <int OP, int R, int RPW, int S, bool ZC, bool FZ, int PSN>
 __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 1)) ? 3 : 2)
     k2_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap,
              const __grid_constant__ CUtensorMap pwmap, const float* __restrict__ src, float* out, int ntx,
-             int nty, int zc, int nchunk, int slot, int n1, int zc2) {
+             int nty, int zc, int nchunk, int n1, int zc2) {
   using C = Cfg<R, RPW, S, (OP == K2_HOTSPOT || OP == K2_ACOUSTIC) ? PSN : 0>;
   constexpr bool PW = OP == K2_HOTSPOT || OP == K2_ACOUSTIC;           // a point-wise zipped grid (Hotspot P, Acoustic prev)
   constexpr int PS = C::PS;                     // point-wise ring slots
@@ -170,6 +164,7 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
   int* stage_item = reinterpret_cast<int*>(itemempty + QN);
   int* stage_const = stage_item + S;
   int* item_q = stage_const + S;
+  int* slot_sm = item_q + QN;
 
   const int ntile = ntx * nty;
   const int nitems = ntile * nchunk;
@@ -189,8 +184,10 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
       mbar_init(&itemempty[s], 1);
     }
     fence_mbar_init();
+    *slot_sm = claim_launch_slot(g_launch);
   }
   __syncthreads();
+  const int slot = *slot_sm;
   pdl_launch_dependents();   // PDL: let the next launch ramp up now
   pdl_wait();                // ... and wait for the previous one before any global access
 
@@ -207,7 +204,7 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
       int q = 0;
       uint32_t qpass = 0;
       while (true) {
-        const int item = (int)atomicAdd(&g_ticket[slot], 1u);
+        const int item = (int)atomicAdd(&g_launch[slot].c[0], 1u);
         const bool done = item >= nitems;
         if constexpr (PW) {
           if (qpass > 0) mbar_wait(&itemempty[q], (qpass - 1) & 1);
@@ -228,8 +225,14 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
           // previous step before the TMA reads them
           if constexpr (FZ) {
             bool waited = false;
-            if (chunk == 0 && p.wait_lo) { spin_until(p.wait_lo, p.wait_value); waited = true; }
-            if (chunk == nchunk - 1 && p.wait_hi) { spin_until(p.wait_hi, p.wait_value); waited = true; }
+            if (chunk == 0 && p.wait_lo) {
+              spin_until_bounded(p.wait_lo, p.wait_value, p.wait_timeout_ns, p.fault, kFaultWaitLo);
+              waited = true;
+            }
+            if (chunk == nchunk - 1 && p.wait_hi) {
+              spin_until_bounded(p.wait_hi, p.wait_value, p.wait_timeout_ns, p.fault, kFaultWaitHi);
+              waited = true;
+            }
             if (waited) asm volatile("fence.proxy.async.global;" ::: "memory");
           }
         }
@@ -641,14 +644,14 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
           const unsigned need = (unsigned)ntile * NW;
           if (chunk == 0 && p.sig_lo) {
             __threadfence_system();
-            if (atomicAdd(&g_bdone[slot][0], 1u) == need - 1) {
+            if (atomicAdd(&g_launch[slot].c[2], 1u) == need - 1) {
               __threadfence_system();
               st_release_sys(p.sig_lo, p.sig_value);
             }
           }
           if (chunk == nchunk - 1 && p.sig_hi) {
             __threadfence_system();
-            if (atomicAdd(&g_bdone[slot][1], 1u) == need - 1) {
+            if (atomicAdd(&g_launch[slot].c[3], 1u) == need - 1) {
               __threadfence_system();
               st_release_sys(p.sig_hi, p.sig_value);
             }
@@ -664,18 +667,14 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
   __syncthreads();
   if (threadIdx.x == 0) {
     __threadfence();
-    const unsigned prev = atomicAdd(&g_done[slot], 1u);
+    const unsigned prev = atomicAdd(&g_launch[slot].c[1], 1u);
     if (prev == gridDim.x - 1) {
-      g_ticket[slot] = 0;
-      g_done[slot] = 0;
-      g_bdone[slot][0] = 0;
-      g_bdone[slot][1] = 0;
       if (puts && !p.fused_step) {
         __threadfence_system();
         if (p.sig_lo) st_release_sys(p.sig_lo, p.sig_value);
         if (p.sig_hi) st_release_sys(p.sig_hi, p.sig_value);
       }
-      __threadfence();
+      release_launch_slot(g_launch, slot);
     }
   }
 }
@@ -710,7 +709,7 @@ struct CfgT2 {
 template <int S>
 __global__ void __launch_bounds__(NCONS + 32, 2)
     k2t_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmap, float* out, int ntx,
-              int nty, int zc, int nchunk, int slot) {
+              int nty, int zc, int nchunk) {
   using C = CfgT2<S>;
   constexpr int SF4 = C::STAGE_FLOATS / 4;
   constexpr int BX4 = BX / 4;
@@ -720,6 +719,7 @@ __global__ void __launch_bounds__(NCONS + 32, 2)
   uint64_t* full = reinterpret_cast<uint64_t*>(ysm + 4 * T2_YF4);
   uint64_t* empty = full + S;
   int* stage_item = reinterpret_cast<int*>(empty + S);
+  int* slot_sm = stage_item + S;
 
   const int ntile = ntx * nty;
   const int nitems = ntile * nchunk;
@@ -730,8 +730,10 @@ __global__ void __launch_bounds__(NCONS + 32, 2)
       mbar_init(&empty[s], NW);
     }
     fence_mbar_init();
+    *slot_sm = claim_launch_slot(g_launch);
   }
   __syncthreads();
+  const int slot = *slot_sm;
   pdl_launch_dependents();   // PDL: let the next launch ramp up now
   pdl_wait();                // ... and wait for the previous one before any global access
 
@@ -741,7 +743,7 @@ __global__ void __launch_bounds__(NCONS + 32, 2)
       int s = 0;
       uint32_t pass = 0;
       while (true) {
-        const int item = (int)atomicAdd(&g_ticket[slot], 1u);
+        const int item = (int)atomicAdd(&g_launch[slot].c[0], 1u);
         const bool done = item >= nitems;
         int nload = 1, x0 = 0, y0 = 0;
         int64_t zs = 0;
@@ -912,11 +914,9 @@ __global__ void __launch_bounds__(NCONS + 32, 2)
   __syncthreads();
   if (threadIdx.x == 0) {
     __threadfence();
-    const unsigned prev = atomicAdd(&g_done[slot], 1u);
+    const unsigned prev = atomicAdd(&g_launch[slot].c[1], 1u);
     if (prev == gridDim.x - 1) {
-      g_ticket[slot] = 0;
-      g_done[slot] = 0;
-      __threadfence();
+      release_launch_slot(g_launch, slot);
     }
   }
 }
@@ -1036,7 +1036,6 @@ bool get_map(const float* base, int64_t nx, int64_t ny, int64_t nz, int bx, int 
   return true;
 }
 
-std::atomic<unsigned> g_slot{0};
 
 }  // namespace
 
@@ -1142,9 +1141,8 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   if (items > 0x7fffffff) return cudaErrorInvalidConfiguration;
   int64_t grid = slots < items ? slots : items;
   int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk, n1_i = (int)n1, zc2_i = (int)zc2;
-  int slot = (int)(g_slot.fetch_add(1) % kTickets);
   void* args[] = {(void*)&p, (void*)&map, (void*)&pwmap, (void*)&slid, (void*)&out,
-                  &ntx_i, &nty_i, &zc_i, &nch_i, &slot, &n1_i, &zc2_i};
+                  &ntx_i, &nty_i, &zc_i, &nch_i, &n1_i, &zc2_i};
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, !fz);
 }
@@ -1194,8 +1192,7 @@ cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* ou
   if (items > 0x7fffffff) return cudaErrorInvalidConfiguration;
   int64_t grid = slots < items ? slots : items;
   int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk;
-  int slot = (int)(g_slot.fetch_add(1) % kTickets);
-  void* args[] = {(void*)&p, (void*)&map, (void*)&out, &ntx_i, &nty_i, &zc_i, &nch_i, &slot};
+  void* args[] = {(void*)&p, (void*)&map, (void*)&out, &ntx_i, &nty_i, &zc_i, &nch_i};
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, true);
 }
 

@@ -35,6 +35,7 @@
 #include "common.cuh"
 #include "launch.hpp"
 #include "ops.cuh"
+#include "slots.cuh"
 #include "tma.cuh"
 
 namespace lift {
@@ -45,10 +46,9 @@ constexpr int XH = 4;
 constexpr int BX = TX + 2 * XH;
 constexpr int BX4 = BX / 4;
 constexpr unsigned FULL = 0xffffffffu;
-constexpr int kTk = 4096;
-
-__device__ unsigned int g_wticket[kTk];
-__device__ unsigned int g_wdone[kTk];
+// dynamic work counters, one slot per running launch (slots.cuh): c[0] item
+// ticket, c[1] CTAs done
+__device__ LaunchSlot g_launch[kLaunchSlots];
 
 enum K3Op { K3_WBOX = 0, K3_SRAD1 = 1, K3_SRAD2 = 2, K3_WSTAR = 3, K3_WSEP = 4, K3_HOT2D = 5, K3_GRAD = 6 };
 
@@ -143,7 +143,7 @@ template <int OP, int RY, int RX, int G, int S, int NIN, int WPC, int MINB>
 __global__ void __launch_bounds__(WPC * 32, MINB)
     k3_wsweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap map0,
               const __grid_constant__ CUtensorMap map1, const float* __restrict__ src0,
-              const float* __restrict__ src1, float* __restrict__ out, int nstrips, int hc, int nitems, int slot) {
+              const float* __restrict__ src1, float* __restrict__ out, int nstrips, int hc, int nitems) {
   using C = WCfg<G, S, NIN, WPC>;
   constexpr int SY = 2 * RY + 1, SX = 2 * RX + 1;
   constexpr int W = 4 + 2 * RX;
@@ -161,12 +161,15 @@ __global__ void __launch_bounds__(WPC * 32, MINB)
   float4* ring = dsm4 + warp * (S * SLOT4);
   uint64_t* bars = reinterpret_cast<uint64_t*>(dsm4 + WPC * (S * SLOT4)) + warp * S;
 
+  int slot = 0;
   if (lane == 0) {
     for (int s = 0; s < S; ++s) mbar_init(&bars[s], 1);
     fence_mbar_init();
     prefetch_tmap(&map0);
     if constexpr (NIN > 1) prefetch_tmap(&map1);
+    slot = claim_launch_slot(g_launch);    // the same slot in every warp of the launch
   }
+  slot = __shfl_sync(FULL, slot, 0);
   __syncwarp();
   pdl_launch_dependents();
   pdl_wait();
@@ -190,7 +193,7 @@ __global__ void __launch_bounds__(WPC * 32, MINB)
   };
   auto fetch = [&]() {
     int v = 0;
-    if (lane == 0) v = (int)atomicAdd(&g_wticket[slot], 1u);
+    if (lane == 0) v = (int)atomicAdd(&g_launch[slot].c[0], 1u);
     return __shfl_sync(FULL, v, 0);
   };
 
@@ -405,12 +408,8 @@ __global__ void __launch_bounds__(WPC * 32, MINB)
   __syncthreads();
   if (threadIdx.x == 0) {
     __threadfence();
-    const unsigned prev = atomicAdd(&g_wdone[slot], 1u);
-    if (prev == gridDim.x - 1) {
-      g_wticket[slot] = 0;
-      g_wdone[slot] = 0;
-      __threadfence();
-    }
+    const unsigned prev = atomicAdd(&g_launch[slot].c[1], 1u);
+    if (prev == gridDim.x - 1) release_launch_slot(g_launch, slot);
   }
 }
 
@@ -520,8 +519,6 @@ bool get_map(const float* base, int64_t nx, int64_t ny, int by, CUtensorMap* out
   return true;
 }
 
-std::atomic<unsigned> g_wslot{0};
-
 }  // namespace
 
 bool wsweep2d_supported(const StencilParams& p, const float* in0, const float* in1, bool small) {
@@ -581,8 +578,7 @@ cudaError_t launch_wsweep2d(const StencilParams& p, const float* in0, const floa
   const int64_t need = (nitems + L.wpc - 1) / L.wpc;
   if (grid > need) grid = need;
   int ns = nstrips, hci = (int)hc, ni = (int)nitems;
-  int slot = (int)(g_wslot.fetch_add(1) % kTk);
-  void* args[] = {(void*)&p, (void*)&m0, (void*)&m1, (void*)&in0, (void*)&s1, (void*)&out, &ns, &hci, &ni, &slot};
+  void* args[] = {(void*)&p, (void*)&m0, (void*)&m1, (void*)&in0, (void*)&s1, (void*)&out, &ns, &hci, &ni};
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(L.wpc * 32), args, (size_t)L.smem, stream, true);
 }
 

@@ -94,8 +94,9 @@ bool persist3d_supported(const StencilParams& p, const float* s0, const float* s
 cudaError_t launch_persist3d(const StencilParams& p, float* s0, float* s1, const float* aux, int n_steps,
                              cudaStream_t stream, int num_sms, std::string* err);
 
-// wait (one thread, acquire.sys) until *a >= value and *b >= value (NULL = skip)
+// wait (one thread, acquire.sys) until *a >= value and *b >= value (NULL =
+// skip); bounded by timeout_ns (0 = none), a timeout ORs into *fault
 cudaError_t launch_wait_signals(const unsigned int* a, const unsigned int* b, unsigned int value,
-                                cudaStream_t stream);
+                                unsigned long long timeout_ns, unsigned int* fault, cudaStream_t stream);
 
 }  // namespace lift

@@ -5,7 +5,8 @@
 // boundary-plane kernel, it orders that kernel's ghost reads after the
 // neighbours' peer stores (which their boundary kernel published with a
 // release store of the same step number).  Step numbers only grow, so there
-// is no ABA.
+// is no ABA.  The wait is bounded (stencil_set_wait_timeout_ms): a flag that
+// never arrives is reported through stencil_device_fault, not a hang.
 #include <cuda_runtime.h>
 
 #include "launch.hpp"
@@ -15,18 +16,18 @@ namespace lift {
 namespace {
 
 __global__ void k_wait_signals(const unsigned int* __restrict__ a, const unsigned int* __restrict__ b,
-                               unsigned int value) {
-  if (a)
-    while ((int)(ld_acquire_sys(a) - value) < 0) __nanosleep(64);
-  if (b)
-    while ((int)(ld_acquire_sys(b) - value) < 0) __nanosleep(64);
+                               unsigned int value, unsigned long long timeout_ns, unsigned int* fault) {
+  // bounded (tma.cuh): a neighbour that never signals records a fault
+  // instead of hanging the stream
+  if (a) spin_until_bounded(a, value, timeout_ns, fault, kFaultWaitLo);
+  if (b) spin_until_bounded(b, value, timeout_ns, fault, kFaultWaitHi);
 }
 
 }  // namespace
 
 cudaError_t launch_wait_signals(const unsigned int* a, const unsigned int* b, unsigned int value,
-                                cudaStream_t stream) {
-  k_wait_signals<<<1, 1, 0, stream>>>(a, b, value);
+                                unsigned long long timeout_ns, unsigned int* fault, cudaStream_t stream) {
+  k_wait_signals<<<1, 1, 0, stream>>>(a, b, value, timeout_ns, fault);
   return cudaGetLastError();
 }
 

@@ -6,8 +6,11 @@
 // concurrently on two streams, two plans on two streams) would skip or repeat
 // items.  A slot index chosen on the host and baked into a captured graph
 // cannot guarantee that, so each launch claims its slot on the device, keyed
-// by its grid id (%gridid: the context's temporal launch number, distinct for
-// every launch, graph replays included — tested): slot = (grid id + 1) mod K.
+// by its grid id (%gridid: the context's temporal launch number — distinct
+// for every eager launch and for every kernel node of every instantiated
+// graph; replays of ONE executable graph reuse its node ids, but CUDA
+// serialises the launches of one executable graph, so they never overlap;
+// profiles/r02_gridid_probe.txt): slot = (grid id + 1) mod K.
 // Every CTA of the launch computes the same slot; the first one to arrive
 // takes ownership (CAS 0 -> id), the last one out zeroes the counters and
 // then frees it.  Two launches share a slot only if their ids differ by a

@@ -128,6 +128,32 @@ __device__ __forceinline__ unsigned int ld_acquire_sys(const unsigned int* p) {
   return v;
 }
 
+__device__ __forceinline__ unsigned long long globaltimer_ns() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+  return t;
+}
+
+// Waits (acquire, system scope) until *f >= v in wrap-around order.  A
+// neighbour that never raises its flag (a dead or stalled rank) must not hang
+// the GPU: after timeout_ns (0 = no limit) the wait gives up, ORs ``code``
+// into the host-visible fault word (stencil_device_fault reports it) and
+// returns false; the launch then completes with stale ghost data.
+__device__ __forceinline__ bool spin_until_bounded(const unsigned int* f, unsigned int v,
+                                                   unsigned long long timeout_ns, unsigned int* fault,
+                                                   unsigned int code) {
+  if ((int)(ld_acquire_sys(f) - v) >= 0) return true;
+  const unsigned long long t0 = globaltimer_ns();
+  while ((int)(ld_acquire_sys(f) - v) < 0) {
+    if (timeout_ns && globaltimer_ns() - t0 > timeout_ns) {
+      if (fault) atomicOr_system(fault, code);
+      return false;
+    }
+    __nanosleep(64);
+  }
+  return true;
+}
+
 // 4-byte asynchronous global->shared copy (LDGSTS) and its group control
 __device__ __forceinline__ void cp_async4(float* smem_dst, const float* gsrc) {
   asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(smem_u32(smem_dst)), "l"(gsrc) : "memory");

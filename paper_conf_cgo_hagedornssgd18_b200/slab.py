@@ -329,7 +329,11 @@ def virtual_slab_iterate_fused(global_extents, world: int, state_global: Sequenc
     own CUDA stream, the boundary kernels store into the neighbour slabs'
     ghost planes and raise their flags, and the streams synchronise only
     through those flags (stencil_wait_signals) — the multi-GPU protocol with
-    device-local "peer" pointers."""
+    device-local "peer" pointers.  A protocol test for grids that do not fill
+    the GPU: with every slab's persistent grid on one device, a step t+1 grid
+    could occupy every SM while spinning on a flag that a not-yet-resident
+    step-t grid must raise; the waits are bounded, so that case ends in a
+    StencilError (stencil_device_fault) instead of a hang."""
     slabs = [SlabPlan(global_extents, r, world, exchange=_NoExchange(), **plan_kw) for r in range(world)]
     ex = LocalExchange(slabs)
     nst = len(state_global)
@@ -354,5 +358,7 @@ def virtual_slab_iterate_fused(global_extents, world: int, state_global: Sequenc
             fused_step(s, fhs[r], ins, b[dst], dst, s.epoch, streams[r])
         ri = dst
     torch.cuda.synchronize(dev)
+    from . import _lib as L
+    L.stencil_device_fault()          # a timed-out flag wait raises here
     order = [1 - ri, ri] if acoustic else [ri]
     return [torch.cat([s.owned(b[k]) for s, b in zip(slabs, bufs)], 0) for k in order]
