@@ -166,6 +166,7 @@ def oracle_sample_spec(workload):
 
 
 def time_oracle(workload, min_seconds=10.0, max_reps=50):
+    """The oracle on ONE core: repeated sweeps of the bounded sub-grid."""
     from oracle import stencil_oracle as orc
     xs, spec, sub = oracle_sample_spec(workload)
     pts = int(np.prod(spec.out_extents()))
@@ -182,27 +183,159 @@ def time_oracle(workload, min_seconds=10.0, max_reps=50):
     return gpts, sample, el
 
 
+def _oracle_worker_init():
+    # one single-threaded numpy per process (no BLAS / OpenMP threads)
+    for k in ("OMP_NUM_THREADS", "OPENBLAS_NUM_THREADS", "MKL_NUM_THREADS"):
+        os.environ[k] = "1"
+
+
+def _oracle_worker(task):
+    """One process of the all-core oracle run: ``reps`` sweeps of its own
+    sub-grid (an independent z-slab sample of the workload, seeded by its
+    index).  Returns (points computed, seconds)."""
+    workload, idx, reps = task
+    import stencil_inputs as si
+    from oracle import stencil_oracle as orc
+    xs, spec, sub = oracle_sample_spec(workload)
+    if idx:
+        xs = [np.roll(x, idx, axis=-1) for x in xs]     # a different slab's values, same shape and op
+    pts = int(np.prod(spec.out_extents()))
+    t0 = time.perf_counter()
+    for _ in range(reps):
+        orc.apply(spec, xs)
+    return pts * reps, time.perf_counter() - t0
+
+
+def cpu_model():
+    try:
+        out = subprocess.run(["lscpu"], capture_output=True, text=True, timeout=10).stdout
+        for ln in out.splitlines():
+            if ln.startswith("Model name:"):
+                return ln.split(":", 1)[1].strip()
+    except Exception:
+        pass
+    return None
+
+
+class OraclePool:
+    """The oracle on all host cores: one single-threaded process per core, each
+    sweeping its own bounded sub-grid of the workload (the work is
+    embarrassingly parallel over z-slabs, as the slab decomposition is)."""
+
+    def __init__(self, workload, max_procs=64):
+        import multiprocessing as mp
+        self.workload = workload
+        self.nproc = os.cpu_count() or 1
+        self.procs = max(1, min(self.nproc, max_procs))
+        self.pool = mp.get_context("spawn").Pool(self.procs, initializer=_oracle_worker_init)
+        # warm-up: every worker imports numpy/oracle and builds its inputs once
+        self.pool.map(_oracle_worker, [(workload, i, 0) for i in range(self.procs)])
+
+    def run(self, reps):
+        t0 = time.perf_counter()
+        res = self.pool.map(_oracle_worker, [(self.workload, i, reps) for i in range(self.procs)])
+        el = time.perf_counter() - t0
+        pts = sum(r[0] for r in res)
+        return pts / el / 1e9, el
+
+    def close(self):
+        self.pool.close()
+        self.pool.join()
+
+
+def cpu_baseline(workload, single_seconds=8.0, all_seconds=8.0):
+    """Oracle timed on one core and on all host cores (rank 0, N=1)."""
+    g1, sample1, el1 = time_oracle(workload, min_seconds=single_seconds, max_reps=20)
+    xs, spec, sub = oracle_sample_spec(workload)
+    per_rep = int(np.prod(spec.out_extents())) / (g1 * 1e9)      # seconds per sweep on one core
+    pool = OraclePool(workload)
+    try:
+        reps = max(1, int(all_seconds / max(per_rep, 1e-3)))
+        gall, elall = pool.run(reps)
+    finally:
+        pool.close()
+    return {"value": gall, "unit": "Gpoints/s", "cores": pool.procs, "nproc": pool.nproc, "kind": "oracle",
+            "cpu_model": cpu_model(),
+            "sample": f"{pool.procs} processes x {reps} sweeps of a {'x'.join(map(str, sub))} sub-grid of "
+                      f"{workload} each (numpy fp64 oracle, one single-threaded process per core)",
+            "single_core_value": g1, "single_core_sample": sample1}
+
+
 def reference_arm(args, workload):
     rank = env_int("RANK", 0)
     if rank != 0:
         return
-    per_step = []
-    gp_all = []
-    for _ in range(args.warmup):
-        time_oracle(workload, min_seconds=0.0, max_reps=1)
-    sample = ""
-    for _ in range(args.steps):
-        gp, sample, el = time_oracle(workload, min_seconds=2.0, max_reps=20)
-        gp_all.append(gp)
-        per_step.append(el)
+    # each step: one sweep of the bounded sub-grid in every process of the
+    # all-core oracle pool (one single-threaded process per host core)
+    pool = OraclePool(workload)
+    try:
+        for _ in range(args.warmup):
+            pool.run(1)
+        per_step, gp_all = [], []
+        for _ in range(args.steps):
+            gp, el = pool.run(1)
+            gp_all.append(gp)
+            per_step.append(el)
+    finally:
+        pool.close()
     gpts = statistics.median(gp_all)
+    xs, spec, sub = oracle_sample_spec(workload)
+    sample = (f"per step: {pool.procs} processes x one sweep of a {'x'.join(map(str, sub))} sub-grid of "
+              f"{workload} (numpy fp64 oracle, one single-threaded process per core)")
     line = {"impl": "reference", "metric": METRIC, "value": gpts, "unit": "Gpoints/s", "n_gpus": args.gpus,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * statistics.median(per_step),
             "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
             "config": {"workload": workload},
-            "cpu_baseline": {"value": gpts, "unit": "Gpoints/s", "cores": 1, "kind": "oracle", "sample": sample},
+            "cpu_baseline": {"value": gpts, "unit": "Gpoints/s", "cores": pool.procs, "nproc": pool.nproc,
+                             "cpu_model": cpu_model(), "kind": "oracle", "sample": sample},
             "e2e": {"value": gpts, "unit": "Gpoints/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
+
+
+# ----------------------------------------------------------------------------
+# launcher: --gpus N without torchrun re-executes through torch.distributed.run
+# ----------------------------------------------------------------------------
+def _free_port():
+    import socket
+    with socket.socket(socket.AF_INET, socket.SOCK_STREAM) as so:
+        so.bind(("127.0.0.1", 0))
+        return so.getsockname()[1]
+
+
+def launch_ranks(nprocs, argv):
+    """One process per GPU: ``python -m torch.distributed.run --nnodes=1
+    --nproc-per-node N --master-addr 127.0.0.1 --master-port P bench.py ...``
+    (the driver's own launch line).  NCCL_DEBUG=INFO (INIT subsystem) unless
+    set, so the communicator's nranks shows in the log.  Returns the exit code."""
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={nprocs}",
+           "--master-addr", "127.0.0.1", "--master-port", str(_free_port()), os.path.abspath(__file__)] + list(argv)
+    env = dict(os.environ)
+    env.setdefault("NCCL_DEBUG", "INFO")
+    env.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+    return subprocess.call(cmd, env=env)
+
+
+def launcher_selftest(args):
+    """--selftest-launch: each rank joins a gloo group and checks that the
+    world is exactly --gpus ranks (CPU test of the launcher path)."""
+    import torch
+    import torch.distributed as dist
+    world = env_int("WORLD_SIZE", 1)
+    if world != args.gpus:
+        raise SystemExit(f"bench.py: --gpus {args.gpus} but WORLD_SIZE={world}")
+    if world > 1:
+        dist.init_process_group("gloo")
+        assert dist.get_world_size() == args.gpus
+        t = torch.tensor([dist.get_rank()], dtype=torch.int64)
+        ranks = [torch.zeros_like(t) for _ in range(world)]
+        dist.all_gather(ranks, t)
+        ranks = [int(r.item()) for r in ranks]
+        dist.destroy_process_group()
+    else:
+        ranks = [0]
+    if env_int("RANK", 0) == 0:
+        print(json.dumps({"launcher_ok": True, "world": world, "ranks": ranks,
+                          "nccl_debug": os.environ.get("NCCL_DEBUG")}), flush=True)
 
 
 # ----------------------------------------------------------------------------
@@ -228,8 +361,27 @@ def main():
     ap.add_argument("--halo", default="nccl", choices=["nccl", "fused"],
                     help="multi-GPU ghost exchange: NCCL send/recv overlapped with the interior (default), or the "
                          "fused boundary kernel storing into the neighbours' ghosts over NVLink peer memory")
+    ap.add_argument("--halo-depth", type=int, default=1,
+                    help="slab path: ghost depth in time steps k (NEXT-3 deep halos): ghosts of r*k planes are "
+                         "exchanged every k time steps and the overlap is recomputed redundantly")
+    ap.add_argument("--selftest-launch", action="store_true", help=argparse.SUPPRESS)
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
+
+    # --gpus N without a torchrun environment: launch N ranks ourselves (the
+    # same launch line the driver uses), so `python bench.py --gpus N` is a
+    # real N-process run; N = 1 runs in this process (the same code path)
+    if args.gpus > 1 and "WORLD_SIZE" not in os.environ and args.impl == "ours":
+        if not args.selftest_launch:
+            import torch
+            have = torch.cuda.device_count()
+            if have < args.gpus:
+                print(f"bench.py: --gpus {args.gpus} needs {args.gpus} visible GPUs, found {have}", file=sys.stderr)
+                sys.exit(2)
+        sys.exit(launch_ranks(args.gpus, sys.argv[1:]))
+    if args.selftest_launch:
+        launcher_selftest(args)
+        return
 
     if args.impl == "reference":
         reference_arm(args, args.workload)
@@ -246,10 +398,18 @@ def main():
     sym, fused = None, None
     rank = env_int("RANK", 0)
     local = env_int("LOCAL_RANK", 0)
+    if world != args.gpus:
+        raise SystemExit(f"bench.py: --gpus {args.gpus} but the launch has WORLD_SIZE={world} ranks")
+    if torch.cuda.device_count() <= local:
+        raise SystemExit(f"bench.py: rank {rank} needs cuda:{local}, {torch.cuda.device_count()} GPUs visible")
     torch.cuda.set_device(local)
     use_pg = world > 1 or (args.force_slab and "MASTER_ADDR" in os.environ)
     if use_pg:
+        os.environ.setdefault("NCCL_DEBUG", "INFO")        # communicator nranks in the log
+        os.environ.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
         dist.init_process_group("nccl", device_id=torch.device(f"cuda:{local}"))
+        if dist.get_world_size() != args.gpus:
+            raise SystemExit(f"bench.py: process group has {dist.get_world_size()} ranks, --gpus {args.gpus}")
     dev = torch.device(f"cuda:{local}")
 
     w = si.workload(args.workload)
@@ -284,7 +444,7 @@ def main():
 
     if slabbed:
         sp = SlabPlan(gext, rank, world, spec.size, spec.pad_lo, list(spec.kind), spec.pad_value, spec.op,
-                      spec.weights, spec.params, device=local)
+                      spec.weights, spec.params, device=local, depth=args.halo_depth)
         plan = sp.plan
         host = [torch.from_numpy(x).pin_memory() for x in xs]
         bufs = []
@@ -321,7 +481,11 @@ def main():
             aux = []
         # slab + NCCL: boundary low, boundary high, interior per time step;
         # slab + fused: one launch per time step
-        launches_per_step = steps_per_iter * (3 if (slabbed and args.halo == "nccl") else 1)
+        launches_per_step = steps_per_iter
+        if slabbed and args.halo == "nccl":
+            # every block of k steps: k - 1 extended sweeps, then boundary low,
+            # boundary high and interior of its last step
+            launches_per_step = steps_per_iter + 2 * (-(-steps_per_iter // args.halo_depth))
         if op == si.SRAD:
             launches_per_step = steps_per_iter + 1        # q0 partials of the input, then one fused pass per iteration
     else:
@@ -480,6 +644,45 @@ def main():
     peak, peak_src = peaks()
     achieved = alg_bytes / avg_launch_s / 1e9
 
+    # ---- halo exchange (slab path): bytes per rank, exchange time, NVLink fraction
+    halo = None
+    if slabbed:
+        from paper_conf_cgo_hagedornssgd18_b200.slab import neighbours
+        lo_nb, hi_nb = neighbours(rank, world, sp.wrap)
+        n_nb = (lo_nb is not None) + (hi_nb is not None)
+        plane_bytes = int(np.prod(spec.extents[1:])) * 4
+        k = args.halo_depth
+        grids = 2 if (op == si.ACOUSTIC and k > 1) else 1      # grids exchanged per exchange
+        per_nb = sp.g * plane_bytes * grids                     # bytes to (and from) each neighbour per exchange
+        exchanges_per_step = -(-steps_per_iter // k) if args.halo == "nccl" else steps_per_iter
+        ex_us = None
+        if args.halo == "nccl" and world > 1:
+            # the exchange alone (no compute), posted like in the step, max over ranks
+            exb = [state[0]] + ([state[1]] if grids == 2 else [])
+            nrep = 20
+            x0, x1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            barrier()
+            x0.record(stream)
+            for _ in range(nrep):
+                sp._join(sp._on_comm(lambda: sp._post(exb)))
+            x1.record(stream)
+            barrier()
+            tt = torch.tensor([x0.elapsed_time(x1) / nrep], device=dev)
+            dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+            ex_us = float(tt.item()) * 1e3
+        nvl_gbs = per_nb / (ex_us * 1e-6) / 1e9 if ex_us else None
+        halo = {"path": args.halo, "depth_steps": k, "ghost_planes": sp.g, "grids_per_exchange": grids,
+                "neighbours": n_nb, "bytes_per_neighbour_per_exchange": per_nb,
+                "bytes_per_rank_per_time_step": per_nb * n_nb * exchanges_per_step / steps_per_iter,
+                "exchanges_per_bench_step": exchanges_per_step,
+                "exchanges_per_100_time_steps": -(-100 // k) if args.halo == "nccl" else 100,
+                "exchange_us": ex_us,
+                "nvlink_gbs_per_direction": nvl_gbs,
+                "nvlink_peak_gbs_per_direction": 900.0,
+                "nvlink_frac": (nvl_gbs / 900.0) if nvl_gbs else None,
+                "exchange_share_of_time_step": ((ex_us * 1e-3) * exchanges_per_step / ms_per_step) if ex_us else None,
+                "owned_sweep_gpts": npts_local / avg_launch_s / 1e9}
+
     # ---- e2e: the C-ABI call with HOST buffers (H2D + compute + D2H timed), single GPU path
     e2e = None
     if not args.no_e2e and not slabbed:
@@ -531,8 +734,7 @@ def main():
     # ---- cpu baseline: the oracle on a bounded sample (rank 0, N=1 only)
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu:
-        gp, sample, _ = time_oracle(args.workload, min_seconds=10.0, max_reps=20)
-        cpu = {"value": gp, "unit": "Gpoints/s", "cores": 1, "kind": "oracle", "sample": sample}
+        cpu = cpu_baseline(args.workload)
 
     clocks = clk.summary()
     if rank == 0:
@@ -548,6 +750,7 @@ def main():
                        "op": si.OP_NAMES[op], "boundary": [si.KIND_NAMES[k] for k in spec.kind],
                        "window": list(spec.size),
                        "halo": (args.halo if slabbed else None),
+                       "halo_depth": (args.halo_depth if slabbed else None),
                        "parallelism": f"slab-z x{world}" if slabbed else
                        (f"replicas x{world}" if world > 1 else "single"),
                        "l2": ("L2 flushed (2 x L2 write) before every timed step; one sweep per step"
@@ -571,6 +774,7 @@ def main():
                          "alg_bytes_per_launch": alg_bytes, "avg_launch_us": avg_launch_s * 1e6,
                          "frac_of_8TBs": achieved / 8000.0},
             "cpu_baseline": cpu,
+            "halo": halo,
             "hot": hot,
             "e2e": e2e,
             "gpu_launches": int(args.steps * launches_per_step),

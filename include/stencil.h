@@ -190,7 +190,12 @@ stencil_status stencil_apply(stencil_plan plan, const float* const* inputs,
 
 /* Same, restricted to output planes [o0_begin, o0_end) of dimension 0
  * (slab interior / boundary split).  Results are bitwise identical to the
- * corresponding planes of stencil_apply. */
+ * corresponding planes of stencil_apply.  Slab plans (stencil_plan_set_slab)
+ * may extend the region into the ghost planes, o0_begin >= -(ghost -
+ * pad_lo[0]) and o0_end <= n0_local + ghost - pad_hi[0]: the redundant
+ * overlap compute of deep halos (ghosts of r*k planes exchanged every k
+ * steps; P:739-791 overlapped tiling applied in time); output
+ * plane z < 0 is written to ghost plane ghost + z of ``out``. */
 stencil_status stencil_apply_region(stencil_plan plan, const float* const* inputs,
                                     int32_t n_inputs, float* out, int64_t o0_begin,
                                     int64_t o0_end, void* stream);

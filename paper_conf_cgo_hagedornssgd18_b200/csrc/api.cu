@@ -535,8 +535,16 @@ stencil_status stencil_apply_region(stencil_plan pl, const float* const* inputs,
     o0_begin = 0;            // canonical dimension 0 has extent 1
     o0_end = pl->p.o[0];
   }
-  if (o0_begin < 0 || o0_end > pl->p.o[0] || o0_begin > o0_end)
-    return fail(STENCIL_E_INVALID, "region outside the output extents");
+  // slab plans may extend the region into the ghost planes (deep halos,
+  // NEXT-3: the overlap of k time steps is recomputed redundantly) as far as
+  // the window's input planes stay inside the allocation
+  int64_t lo_lim = 0, hi_lim = pl->p.o[0];
+  if (pl->p.slab) {
+    lo_lim = -(int64_t)(pl->p.ghost - pl->p.lo[0]);
+    hi_lim = pl->p.o[0] + (pl->p.ghost - pl->p.hi[0]);
+  }
+  if (o0_begin < lo_lim || o0_end > hi_lim || o0_begin > o0_end)
+    return fail(STENCIL_E_INVALID, "region outside the output extents (slab: ghost planes minus the pad)");
   if (o0_begin == o0_end) return STENCIL_OK;
   DeviceGuard g(pl->device);
   if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");

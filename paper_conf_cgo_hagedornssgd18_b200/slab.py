@@ -106,6 +106,41 @@ def slab_step(compute: Callable[[int, int], None], exchange_post: Callable[[], l
     return works
 
 
+def deep_halo_iterate(n_steps: int, k: int, r: int, n: int, g: int, extension, compute, post, on_comm, join,
+                      acoustic: bool, ri: int, aux=()) -> int:
+    """The time-step schedule of a slab with ghosts of g = r*k planes (k = 1:
+    the plain per-step exchange).  ``compute(src, dst, a, b)`` writes output
+    planes [a, b) (slab-local, may reach into the ghosts) of state ``dst`` from
+    state ``src``; ``post(grids)`` posts the ghost exchange of the listed state
+    indices / tensors and returns its works; ``on_comm`` runs a post on the
+    side stream, ``join`` waits for its works; ``extension(e)`` is the output
+    range reaching e planes into the ghosts on the sides that have a
+    neighbour.  Returns the index of the newest state."""
+    first = [ri]
+    if k > 1:
+        first += [1 - ri] if acoustic else list(aux)
+    join(on_comm(lambda: post(first)))
+    t = 0
+    while t < n_steps:
+        kb = min(k, n_steps - t)
+        for j in range(1, kb + 1):
+            dst = 1 - ri
+            if j < kb:
+                a, b = extension((kb - j) * r)
+                compute(ri, dst, a, b)
+            else:
+                # the block's last step: exactly the owned planes, boundary
+                # first, then (exchange || interior); Acoustic with k > 1 also
+                # exchanges the new u^{n-1} (the grid just read as u^n)
+                grids = [dst, ri] if (acoustic and k > 1) else [dst]
+                src = ri
+                works = slab_step(lambda a, b: compute(src, dst, a, b), lambda: post(grids), n, g, on_comm=on_comm)
+                join(works)
+            ri = dst
+        t += kb
+    return ri
+
+
 class SlabPlan:
     """One rank's slab of a global 3D stencil (CUDA, libstencil.so).
 
@@ -114,7 +149,7 @@ class SlabPlan:
 
     def __init__(self, global_extents: Sequence[int], rank: int, world: int, size=3, pad=None, kind="clamp",
                  pad_value: float = 0.0, op="weighted", weights=None, params=(), group=None,
-                 device: Optional[int] = None, exchange=None, exchange_factory=None):
+                 device: Optional[int] = None, exchange=None, exchange_factory=None, depth: int = 1):
         from .plan import Plan
         self.global_extents = tuple(int(e) for e in global_extents)
         self.rank, self.world = rank, world
@@ -122,9 +157,15 @@ class SlabPlan:
         self.n = self.z1 - self.z0
         ext = (self.n,) + self.global_extents[1:]
         self.plan = Plan(ext, size, 1, pad, None, kind, pad_value, op, weights, params, device)
-        self.g = max(self.plan.pad_lo[0], self.plan.pad_hi[0])
+        # deep halos (NEXT-3): ghosts of r*depth planes, exchanged every depth steps
+        if depth < 1:
+            raise ValueError("halo depth must be >= 1")
+        self.r = max(self.plan.pad_lo[0], self.plan.pad_hi[0])
+        self.depth = depth
+        self.g = self.r * depth
         if self.n < max(self.g, 1):
             raise ValueError("slab thinner than the ghost width")
+        self.exchanges = 0      # ghost exchanges posted (each: every exchanged grid, both neighbours)
         self.plan.set_slab(self.z0, self.global_extents[0], self.g)
         self.wrap = self.plan.kind[0] == WRAP
         factory = exchange_factory if exchange_factory is not None else DistExchange
@@ -162,31 +203,58 @@ class SlabPlan:
             w.wait()                       # on the comm stream
         torch.cuda.current_stream().wait_stream(self.comm)
 
+    def _post(self, bufs):
+        self.exchanges += 1
+        works = []
+        for b in bufs:
+            works += self.exchange.post(b)
+        return works
+
+    def extension(self, e: int) -> Tuple[int, int]:
+        """Output plane range [lo, hi) of a step whose region reaches ``e``
+        planes into the ghosts on every side that has a neighbour (global,
+        non-periodic edges are never extended: pad is applied there)."""
+        lo_nb, hi_nb = neighbours(self.rank, self.world, self.wrap)
+        if self.world == 1 and self.wrap:
+            lo_nb = hi_nb = 0
+        return (-e if lo_nb is not None else 0), (self.n + e if hi_nb is not None else self.n)
+
     def iterate(self, state: Sequence[torch.Tensor], n_steps: int, aux: Sequence[torch.Tensor] = (),
                 fused: Optional[FusedHalo] = None) -> int:
         """n time steps with the rotation of stencil_iterate (DESIGN.md A21);
         returns the index of the state buffer holding the newest grid.  With
         ``fused`` the ghosts travel by peer stores from the boundary kernel
-        (stencil_apply_region_put) instead of NCCL."""
+        (stencil_apply_region_put) instead of NCCL.
+
+        Deep halos (``depth`` k > 1, NEXT-3; the overlapped-tiling rule of
+        P:739-791 applied in time): ghosts hold g = r*k planes; a block of
+        kb <= k steps starts from fully exchanged ghosts, step j of the block
+        computes the owned planes plus (kb - j)*r ghost planes on each side
+        that has a neighbour (the neighbour computes the same planes with the
+        same kernel code: bitwise identical), and the block's last step
+        computes exactly the owned planes, boundary first, with the exchange of
+        g planes overlapped with its interior.  Acoustic exchanges both of its
+        grids per block (its point-wise u^{n-1} is read in the extended
+        region); Hotspot's fixed grid P is exchanged once.  One exchange per k
+        time steps instead of one per step."""
         op = self.plan.op
         acoustic = op == 4
         ri = 1 if acoustic else 0
-        self._join(self._on_comm(lambda: self.exchange.post(state[ri])))
         if fused is not None:
+            if self.depth > 1:
+                raise ValueError("the fused halo path exchanges every step (depth 1)")
+            self._join(self._on_comm(lambda: self._post([state[ri]])))
             return self._iterate_fused(state, n_steps, aux, fused, ri, acoustic)
-        for _ in range(n_steps):
-            if acoustic:
-                dst = 1 - ri
-                ins = (state[dst], state[ri])
-            else:
-                dst = 1 - ri
-                ins = (state[ri],) + tuple(aux)
-            out = state[dst]
-            works = slab_step(lambda a, b: self.plan.apply_region(*ins, out=out, begin=a, end=b),
-                              lambda: self.exchange.post(out), self.n, self.g, on_comm=self._on_comm)
-            self._join(works)
-            ri = dst
-        return ri
+
+        def compute(src, dst, a, b):
+            ins = (state[dst], state[src]) if acoustic else (state[src],) + tuple(aux)
+            self.plan.apply_region(*ins, out=state[dst], begin=a, end=b)
+
+        def post(grids):
+            return self._post([state[i] if isinstance(i, int) else i for i in grids])
+
+        return deep_halo_iterate(n_steps, self.depth, self.r, self.n, self.g, self.extension, compute, post,
+                                 self._on_comm, self._join, acoustic, ri, aux)
 
 
 def _iterate_fused_impl(slab, state, n_steps, aux, fused, ri, acoustic):
@@ -291,26 +359,39 @@ class LocalExchange:
 
 
 def virtual_slab_iterate(global_extents, world: int, state_global: Sequence[torch.Tensor], n_steps: int,
-                         aux_global: Sequence[torch.Tensor] = (), **plan_kw) -> List[torch.Tensor]:
+                         aux_global: Sequence[torch.Tensor] = (), depth: int = 1, **plan_kw) -> List[torch.Tensor]:
     """Run G slabs on the current device (no process group) and return the
-    reassembled global state (newest grid last for ACOUSTIC, else [newest])."""
-    slabs = [SlabPlan(global_extents, r, world, exchange=_NoExchange(), **plan_kw) for r in range(world)]
+    reassembled global state (newest grid last for ACOUSTIC, else [newest]).
+    ``depth`` k > 1: deep halos (r*k ghost planes filled every k steps, the
+    overlap recomputed; the schedule of deep_halo_iterate in lockstep)."""
+    slabs = [SlabPlan(global_extents, r, world, exchange=_NoExchange(), depth=depth, **plan_kw)
+             for r in range(world)]
     ex = LocalExchange(slabs)
     nst = len(state_global)
     bufs = [[s.scatter(state_global[k]) if k < nst else s.empty() for k in range(2)] for s in slabs]
-    if nst == 1:
-        pass
     auxs = [[s.scatter(a) for a in aux_global] for s in slabs]
     acoustic = slabs[0].plan.op == 4
     ri = 1 if acoustic else 0
     ex.fill([b[ri] for b in bufs])
-    for _ in range(n_steps):
-        dst = 1 - ri
-        for s, b, a in zip(slabs, bufs, auxs):
-            ins = (b[dst], b[ri]) if acoustic else (b[ri],) + tuple(a)
-            s.plan.apply(*ins, out=b[dst])
-        ex.fill([b[dst] for b in bufs])
-        ri = dst
+    if depth > 1:
+        if acoustic:
+            ex.fill([b[1 - ri] for b in bufs])
+        for k in range(len(aux_global)):
+            ex.fill([a[k] for a in auxs])
+    t = 0
+    while t < n_steps:
+        kb = min(depth, n_steps - t)
+        for j in range(1, kb + 1):
+            dst = 1 - ri
+            for s, b, a in zip(slabs, bufs, auxs):
+                ins = (b[dst], b[ri]) if acoustic else (b[ri],) + tuple(a)
+                lo, hi = s.extension((kb - j) * s.r)
+                s.plan.apply_region(*ins, out=b[dst], begin=lo, end=hi)
+            ri = dst
+        ex.fill([b[ri] for b in bufs])
+        if acoustic and depth > 1:
+            ex.fill([b[1 - ri] for b in bufs])
+        t += kb
     out = []
     order = [1 - ri, ri] if acoustic else [ri]
     for k in order:

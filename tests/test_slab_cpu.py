@@ -128,3 +128,93 @@ def test_gloo_slab_radius2_ghosts():
     gext = (11, 6, 8)
     ref = orc.iterate(_spec(gext, si.REFLECT, 5), [si.uniform(gext, 2024, 0.5, 1.5)], [], 2, round_fp32=True)[0]
     np.testing.assert_array_equal(got, ref.astype(np.float32))
+
+
+# ------------------------------------------------ deep halos (NEXT-3) -------
+def _region_compute(spec, gext, rank, world, n, g, inp, out, a, b):
+    """Output planes [a, b) (slab-local; a < 0 / b > n reach into the ghosts)
+    from the ghost-extended buffer ``inp`` with the fp64 oracle; pad in z only
+    at a global, non-periodic edge."""
+    wrap = spec.kind[0] == si.WRAP
+    lo, hi = spec.pad_lo[0], spec.pad_hi[0]
+    first = rank == 0 and not wrap and a == 0
+    last = rank == world - 1 and not wrap and b == n
+    x = inp.numpy().astype(np.float64)
+    zlo = g + a if first else g + a - lo
+    zhi = g + b if last else g + b + hi
+    assert zlo >= 0 and zhi <= n + 2 * g, "region reads outside the ghost planes"
+    sp = si.StencilSpec((zhi - zlo,) + tuple(gext[1:]), spec.size, spec.step,
+                        (lo if first else 0,) + spec.pad_lo[1:], (hi if last else 0,) + spec.pad_hi[1:],
+                        spec.kind, spec.pad_value, spec.op, spec.weights, spec.params)
+    Y, _ = orc.apply(sp, [x[zlo:zhi]])
+    assert Y.shape[0] == b - a
+    out[g + a:g + b] = torch.from_numpy(Y.astype(np.float32))
+
+
+def _deep_worker(rank, world, port, kind, size, steps, depth, q):
+    from paper_conf_cgo_hagedornssgd18_b200.slab import deep_halo_iterate
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        gext = (23, 6, 8)
+        spec = _spec(gext, kind, size)
+        r = size // 2
+        g = r * depth
+        z0, z1 = partition(gext[0], world)[rank]
+        n = z1 - z0
+        wrap = kind == si.WRAP
+        xg = si.uniform(gext, 2025, 0.5, 1.5)
+        bufs = [torch.zeros((n + 2 * g,) + gext[1:]), torch.zeros((n + 2 * g,) + gext[1:])]
+        bufs[0][g:g + n] = torch.from_numpy(xg[z0:z1])
+        ex = DistExchange(rank, world, n, g, wrap)
+        lo_nb, hi_nb = neighbours(rank, world, wrap)
+        posts = []
+
+        def extension(e):
+            return (-e if lo_nb is not None else 0), (n + e if hi_nb is not None else n)
+
+        def compute(src, dst, a, b):
+            _region_compute(spec, gext, rank, world, n, g, bufs[src], bufs[dst], a, b)
+
+        def post(grids):
+            posts.append(len(grids))
+            works = []
+            for i in grids:
+                works += ex.post(bufs[i])
+            return works
+
+        def join(works):
+            for w in works:
+                w.wait()
+
+        ri = deep_halo_iterate(steps, depth, r, n, g, extension, compute, post, lambda f: f(), join, False, 0)
+        q.put((rank, z0, bufs[ri][g:g + n].numpy().copy(), len(posts)))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("depth", [2, 4])
+@pytest.mark.parametrize("world,kind,size", [(2, si.CLAMP, 3), (3, si.WRAP, 3), (2, si.MIRROR, 5),
+                                             (3, si.CONSTANT, 3)])
+def test_gloo_deep_halo_matches_global_oracle(world, kind, size, depth):
+    """Ghosts of r*k planes exchanged every k steps, the overlap recomputed:
+    bit-for-bit the oracle's global iterate (fp32 rounding per step), with
+    ceil(steps/k) + 1 exchanges (the first fills the initial ghosts)."""
+    steps = 7
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_deep_worker, args=(r, world, port, kind, size, steps, depth, q))
+             for r in range(world)]
+    for p in procs:
+        p.start()
+    res = sorted(q.get(timeout=240) for _ in range(world))
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    got = np.concatenate([r[2] for r in res], 0)
+    gext = (23, 6, 8)
+    ref = orc.iterate(_spec(gext, kind, size), [si.uniform(gext, 2025, 0.5, 1.5)], [], steps, round_fp32=True)[0]
+    np.testing.assert_array_equal(got, ref.astype(np.float32))
+    assert all(r[3] == -(-steps // depth) + 1 for r in res)

@@ -155,3 +155,54 @@ def test_apply_region_put_needs_slab(lift):
     with pytest.raises(lift.StencilError) as e:
         lift.stencil_apply_region_put(plan.handle, [x.data_ptr()], y.data_ptr(), 0, 1)
     assert e.value.status == 1
+
+
+# ------------------------------------------------ deep halos (NEXT-3) -------
+DEEP_CASES = {
+    "j3d7_clamp": lambda: (si.StencilSpec((40, 40, 136), (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.CLAMP,) * 3,
+                                          0.0, si.WEIGHTED, si.weights_j3d7(), ()), [si.uniform((40, 40, 136), 95)],
+                           []),
+    "j3d7_wrap": lambda: (si.StencilSpec((40, 40, 136), (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.WRAP,) * 3,
+                                         0.0, si.WEIGHTED, si.weights_j3d7(), ()), [si.uniform((40, 40, 136), 96)],
+                          []),
+    "j3d13_mirror": lambda: (si.StencilSpec((48, 40, 136), (5,) * 3, (1,) * 3, (2,) * 3, (2,) * 3,
+                                            (si.MIRROR,) * 3, 0.0, si.WEIGHTED, si.weights_j3d13(), ()),
+                             [si.uniform((48, 40, 136), 97)], []),
+    "acoustic13": lambda: (si.StencilSpec((48, 36, 132), (5,) * 3, (1,) * 3, (2,) * 3, (2,) * 3,
+                                          (si.CONSTANT,) * 3, 0.0, si.ACOUSTIC, None, si.params_acoustic(13)),
+                           [si.uniform((48, 36, 132), 98, -1, 1), si.uniform((48, 36, 132), 99, -1, 1)], []),
+    "hotspot3d": lambda: (si.StencilSpec((40, 64, 128), (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.CLAMP,) * 3,
+                                         0.0, si.HOTSPOT3D, None, si.params_hotspot3d()),
+                          [si.uniform((40, 64, 128), 100, 300, 350)], [si.uniform((40, 64, 128), 101, 0, 0.01)]),
+}
+
+
+@pytest.mark.parametrize("depth", [2, 4])
+@pytest.mark.parametrize("world", [1, 2, 3])
+@pytest.mark.parametrize("case", list(DEEP_CASES))
+def test_virtual_slab_deep_halo_bitwise(lift, case, world, depth):
+    """Deep halos: ghosts of r*k planes filled every k steps, the overlap of
+    the extended regions recomputed by apply_region into the ghost planes —
+    bitwise equal to the single-plan iterate (7 steps: a partial last block)."""
+    from paper_conf_cgo_hagedornssgd18_b200.slab import virtual_slab_iterate
+    sp, state, aux = DEEP_CASES[case]()
+    ref = single_iterate(lift, sp, state, aux, 7)
+    got = virtual_slab_iterate(sp.extents, world, [torch.from_numpy(x).cuda() for x in state], 7,
+                               [torch.from_numpy(x).cuda() for x in aux], depth=depth, **kw(sp))
+    for g_, r_ in zip(got, ref):
+        np.testing.assert_array_equal(g_.cpu().numpy(), r_)
+
+
+def test_apply_region_into_ghosts_validation(lift):
+    """A slab plan's region may reach ghost - pad planes into the ghosts, no
+    further; an unslabbed plan may not leave [0, n)."""
+    from paper_conf_cgo_hagedornssgd18_b200 import StencilError
+    from paper_conf_cgo_hagedornssgd18_b200.slab import SlabPlan, _NoExchange
+    s = SlabPlan((40, 40, 136), 1, 3, size=3, kind="clamp", weights=si.weights_j3d7(), exchange=_NoExchange(),
+                 depth=4)
+    a, b = s.empty().uniform_(), s.empty()
+    s.plan.apply_region(a, out=b, begin=-3, end=s.n + 3)
+    with pytest.raises(StencilError):
+        s.plan.apply_region(a, out=b, begin=-4, end=s.n)
+    with pytest.raises(StencilError):
+        s.plan.apply_region(a, out=b, begin=0, end=s.n + 4)

@@ -78,7 +78,7 @@ def _case(name):
     return sp, [si.uniform(ext, 92, -1, 1), si.uniform(ext, 93, -1, 1)], []
 
 
-def _worker(rank, world, port, name, steps, q):
+def _worker(rank, world, port, name, steps, q, depth=1):
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -89,13 +89,14 @@ def _worker(rank, world, port, name, steps, q):
         sp, state, aux = _case(name)
         slab = SlabPlan(sp.extents, rank, world, size=sp.size, pad=sp.pad_lo, kind=list(sp.kind),
                         pad_value=sp.pad_value, op=sp.op, weights=sp.weights, params=sp.params,
-                        exchange_factory=StagedExchange)
+                        exchange_factory=StagedExchange, depth=depth)
         bufs = [slab.scatter(torch.from_numpy(x).cuda()) for x in state]
         if len(bufs) == 1:
             bufs.append(slab.empty())
         ri = slab.iterate(bufs, steps)
         torch.cuda.synchronize()
         q.put((rank, slab.owned(bufs[ri]).cpu().numpy()))
+        q.put((100 + rank, slab.exchanges))
         if rank == 0:
             plan = lift.Plan.from_spec(sp)
             st = [torch.from_numpy(x).cuda() for x in state]
@@ -108,20 +109,24 @@ def _worker(rank, world, port, name, steps, q):
         dist.destroy_process_group()
 
 
-@pytest.mark.parametrize("name,world", [("j3d7_wrap", 2), ("j3d7_wrap", 3), ("j3d13_mirror", 2),
-                                        ("acoustic13", 3)])
-def test_multiprocess_slab_bitwise(name, world):
+@pytest.mark.parametrize("name,world,depth", [("j3d7_wrap", 2, 1), ("j3d7_wrap", 3, 1), ("j3d13_mirror", 2, 1),
+                                              ("acoustic13", 3, 1), ("j3d7_wrap", 2, 2), ("j3d7_wrap", 3, 4),
+                                              ("j3d13_mirror", 2, 2), ("acoustic13", 2, 2)])
+def test_multiprocess_slab_bitwise(name, world, depth):
+    """depth k > 1: deep halos (r*k ghost planes every k steps); the number of
+    exchanges per rank is ceil(6/k) + 1 (the first fills the initial ghosts)."""
     import __graft_entry__
     __graft_entry__.build()
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _port()
-    procs = [ctx.Process(target=_worker, args=(r, world, port, name, 6, q)) for r in range(world)]
+    procs = [ctx.Process(target=_worker, args=(r, world, port, name, 6, q, depth)) for r in range(world)]
     for p in procs:
         p.start()
-    res = dict(q.get(timeout=300) for _ in range(world + 1))
+    res = dict(q.get(timeout=300) for _ in range(2 * world + 1))
     for p in procs:
         p.join(timeout=120)
         assert p.exitcode == 0
     got = np.concatenate([res[r] for r in range(world)], 0)
     np.testing.assert_array_equal(got, res[-1])
+    assert all(res[100 + r] == -(-6 // depth) + 1 for r in range(world))
