@@ -305,13 +305,14 @@ def _free_port():
 def launch_ranks(nprocs, argv):
     """One process per GPU: ``python -m torch.distributed.run --nnodes=1
     --nproc-per-node N --master-addr 127.0.0.1 --master-port P bench.py ...``
-    (the driver's own launch line).  NCCL_DEBUG=INFO (INIT subsystem) unless
-    set, so the communicator's nranks shows in the log.  Returns the exit code."""
+    (the driver's own launch line).  NCCL_DEBUG=INFO unless set, written to
+    stderr, so the communicator's nranks shows in the log while stdout keeps
+    the one JSON line.  Returns the exit code."""
     cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={nprocs}",
            "--master-addr", "127.0.0.1", "--master-port", str(_free_port()), os.path.abspath(__file__)] + list(argv)
     env = dict(os.environ)
     env.setdefault("NCCL_DEBUG", "INFO")
-    env.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+    env.setdefault("NCCL_DEBUG_FILE", "/dev/stderr")    # keep stdout to the one JSON line
     return subprocess.call(cmd, env=env)
 
 
@@ -405,8 +406,8 @@ def main():
     torch.cuda.set_device(local)
     use_pg = world > 1 or (args.force_slab and "MASTER_ADDR" in os.environ)
     if use_pg:
-        os.environ.setdefault("NCCL_DEBUG", "INFO")        # communicator nranks in the log
-        os.environ.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+        os.environ.setdefault("NCCL_DEBUG", "INFO")        # communicator nranks in the log (stderr)
+        os.environ.setdefault("NCCL_DEBUG_FILE", "/dev/stderr")
         dist.init_process_group("nccl", device_id=torch.device(f"cuda:{local}"))
         if dist.get_world_size() != args.gpus:
             raise SystemExit(f"bench.py: process group has {dist.get_world_size()} ranks, --gpus {args.gpus}")
