@@ -452,6 +452,79 @@ def apply_point(spec, inputs: Sequence[np.ndarray], o: Sequence[int]):
     raise ValueError(spec.op)
 
 
+def pad_planes(x: np.ndarray, p0: int, p1: int, l: int, kind: int, value: float = 0.0,
+               decay: float = 1.0) -> np.ndarray:
+    """Padded planes p0 .. p1-1 of ``pad1(x, 0, l, *, kind)`` along axis 0,
+    without materialising the rest: padded plane p reads x[h(p - l, n)], the
+    constant, or the nearest plane times decay^d (the same definitions as
+    pad1, readings A1-A5, A29), in fp64."""
+    n = x.shape[0]
+    planes = []
+    for p in range(p0, p1):
+        i = p - l
+        if 0 <= i < n:
+            planes.append(np.asarray(x[i], np.float64))
+        elif kind == CONSTANT:
+            planes.append(np.full(x.shape[1:], np.float64(value)))
+        elif kind == DAMPEN:
+            planes.append(np.asarray(x[int(h_clamp(i, n))], np.float64) *
+                          np.float64(decay) ** int(dampen_distance(i, n)))
+        else:
+            planes.append(np.asarray(x[int(H[kind](i, n))], np.float64))
+    return np.stack(planes, 0)
+
+
+def apply_planes(spec, inputs: Sequence[np.ndarray], z0: int, z1: int):
+    """Output planes [z0, z1) of dimension 0 of ``apply`` (for full-grid checks
+    of grids too large to pad at once).  The same definition restricted to a
+    block of outputs: output plane o reads padded planes o*step_0 + k
+    (slide), so the block needs padded planes
+    [z0*step_0, (z1-1)*step_0 + size_0); those are built by ``pad_planes``
+    (dimension 0 first, as pad_n), the inner dimensions are padded
+    by pad_n, and the map is the same f.  Point-wise grids are taken at the
+    output planes; Acoustic's K uses the global extents and plane index."""
+    _check_op_shape(spec)
+    if spec.op == SRAD:
+        raise ValueError("the SRAD iteration's q0 is a whole-image statistic: use apply")
+    decay = getattr(spec, "pad_decay", 1.0)
+    p0 = z0 * spec.step[0]
+    p1 = (z1 - 1) * spec.step[0] + spec.size[0]
+    inner_lo = (0,) + tuple(spec.pad_lo[1:])
+    inner_hi = (0,) + tuple(spec.pad_hi[1:])
+
+    def pad(x):
+        P0 = pad_planes(x, p0, p1, spec.pad_lo[0], spec.kind[0], spec.pad_value, decay)
+        return pad_n(P0, inner_lo, inner_hi, spec.kind, spec.pad_value, decay)
+
+    sub_step = (spec.step[0],) + tuple(spec.step[1:])
+    tapper = lambda P: (lambda k: slide_tap(P, k, spec.size, sub_step))
+    outs = (z1 - z0,) + tuple(spec.out_extents()[1:])
+    if spec.op == WEIGHTED:
+        Y, A = f_weighted(tapper(pad(inputs[0])), spec.weights)
+    elif spec.op == HOTSPOT3D:
+        Y, A = f_hotspot3d(tapper(pad(inputs[0])), np.asarray(inputs[1][z0:z1], np.float64), spec.params)
+    elif spec.op == SRAD1:
+        Y, A = f_srad1(tapper(pad(inputs[0])), spec.params)
+    elif spec.op == SRAD2:
+        Y, A = f_srad2(tapper(pad(inputs[0])), tapper(pad(inputs[1])), spec.params)
+    elif spec.op == HOTSPOT2D:
+        Y, A = f_hotspot2d(tapper(pad(inputs[0])), tapper(pad(inputs[1])), spec.params)
+    elif spec.op == GRADIENT:
+        Y, A = f_gradient(tapper(pad(inputs[0])), spec.params)
+    elif spec.op == ACOUSTIC:
+        r = spec.size[0] // 2
+        full = spec.out_extents()
+        o = np.meshgrid(np.arange(z0, z1), *[np.arange(n) for n in full[1:]], indexing="ij", sparse=True)
+        K = acoustic_neighbours(o, spec.extents, r)
+        prev, cur = inputs
+        Y, A = f_acoustic(tapper(pad(cur)), np.asarray(prev[z0:z1], np.float64), K, r, spec.params)
+    else:
+        raise ValueError(spec.op)
+    Y = np.broadcast_to(np.asarray(Y, np.float64), outs).copy()
+    A = np.broadcast_to(np.asarray(A, np.float64), outs).copy()
+    return Y, A
+
+
 def iterate(spec, state: Sequence[np.ndarray], aux: Sequence[np.ndarray], n_steps: int,
             round_fp32: bool = False):
     """iterate(in, f, m) with the state rotation of reading
