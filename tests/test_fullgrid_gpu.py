@@ -25,7 +25,9 @@ import torch
 import stencil_inputs as si
 from oracle import stencil_oracle as orc
 
-pytestmark = [pytest.mark.gpu, pytest.mark.slow]
+pytestmark = [pytest.mark.gpu, pytest.mark.slow,
+              # the pool forks a process that has CUDA threads; the children run numpy only
+              pytest.mark.filterwarnings("ignore:This process .* is multi-threaded:DeprecationWarning")]
 
 _JOB = {}
 
