@@ -566,7 +566,14 @@ def main():
                     "sweeps_per_step": steps_per_iter if iterable else sweeps,
                     "ms_per_step": th / args.steps, "l2": "warm (back-to-back sweeps, no flush)"}
         hot = time_hot()
+        # the flush writes 2 x L2, then reads another 2 x L2 buffer: the write
+        # evicts the working set, the read leaves L2 holding CLEAN lines, so
+        # the timed sweep does not pay for writing back the flush buffer's
+        # dirty lines (measured: +2-3 us per cold sweep of an 8 MB grid,
+        # profiles/r02_latency_probe.txt) — the state ncu's cache control gives
         flush = torch.empty(int(2 * L2_BYTES) // 4, dtype=torch.int32, device=dev)
+        flush_rd = torch.ones(int(2 * L2_BYTES) // 4, dtype=torch.int32, device=dev)
+        flush_sink = torch.empty((), dtype=torch.int64, device=dev)
         if not iterable:
             one = None
             if graph is not None:
@@ -599,6 +606,7 @@ def main():
                      for _ in range(args.steps)]
             for k in range(args.steps):
                 flush.fill_(k)              # evict the working set from L2 (not timed)
+                torch.sum(flush_rd, out=flush_sink)   # ... and leave clean lines behind
                 pairs[k][0].record(stream)
                 step()
                 pairs[k][1].record(stream)
@@ -754,9 +762,11 @@ def main():
                        "halo_depth": (args.halo_depth if slabbed else None),
                        "parallelism": f"slab-z x{world}" if slabbed else
                        (f"replicas x{world}" if world > 1 else "single"),
-                       "l2": ("L2 flushed (2 x L2 write) before every timed step; one sweep per step"
+                       "l2": ("L2 flushed (2 x L2 write, then 2 x L2 read: clean lines) before every timed "
+                              "step; one sweep per step"
                               if cold and not iterable else
-                              "L2 flushed (2 x L2 write) before every timed step" if cold else
+                              "L2 flushed (2 x L2 write, then 2 x L2 read: clean lines) before every timed step"
+                              if cold else
                               "inputs larger than L2 (no flush needed)" if npts_local * bpp >= 2 * L2_BYTES
                               else "L2-resident working set, not flushed (--no-flush)"),
                        "variant": {0: "K0 generic",

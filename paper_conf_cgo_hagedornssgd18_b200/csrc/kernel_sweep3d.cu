@@ -998,6 +998,12 @@ Launcher pick(const StencilParams& p) {
   const int pv = e ? atoi(e) : 0;
   if (p.op == OP_HOTSPOT3D) {
     if (pv == 1) return get_launcher_zf<K2_HOTSPOT, 1, 2, 5, 3>(zc, fz);
+    const char* eh = getenv("LIFT_K2_HS");          // A/B: small-nz column shapes
+    const int hs = eh ? atoi(eh) : 0;
+    if (hs == 1) return get_launcher_zf<K2_HOTSPOT, 1, 1, 10, 8>(zc, fz);
+    if (hs == 2) return get_launcher_zf<K2_HOTSPOT, 1, 1, 12, 8>(zc, fz);
+    if (hs == 3) return get_launcher_zf<K2_HOTSPOT, 1, 2, 10, 8>(zc, fz);
+    if (hs == 4) return get_launcher_zf<K2_HOTSPOT, 1, 1, 6, 6>(zc, fz);
     return get_launcher_zf<K2_HOTSPOT, 1, 2, 5, 5>(zc, fz);
   }
   if (R == 1) {
@@ -1061,6 +1067,7 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
                            cudaStream_t stream, int num_sms, std::string* err) {
   const int64_t nz_reg = p.reg1 - p.reg0;
   if (nz_reg <= 0) return cudaSuccess;
+  if (column3d_supported(p, in0, in1)) return launch_column3d(p, in0, in1, out, stream, err);
   const Launcher L = pick(p);
   const int R = p.radius;
   const float* slid = (p.op == OP_ACOUSTIC) ? in1 : in0;

@@ -52,6 +52,12 @@ bool sweep3d_supported(const StencilParams& p);
 cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float* in1, float* out,
                            cudaStream_t stream, int num_sms, std::string* err);
 
+// K2C — whole-column tiles for few-plane 3D grids (nz <= 16; radius-1 star
+// weighted / Hotspot3D); launch_sweep3d routes eligible plans here.
+bool column3d_supported(const StencilParams& p, const float* in0, const float* in1);
+cudaError_t launch_column3d(const StencilParams& p, const float* in0, const float* in1, float* out,
+                            cudaStream_t stream, std::string* err);
+
 // K2T — two weighted 7-point steps per pass (temporal blocking), CLAMP/MIRROR/REFLECT.
 bool sweep3d_t2_supported(const StencilParams& p);
 cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* out, cudaStream_t stream, int num_sms,

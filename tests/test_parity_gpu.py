@@ -627,3 +627,46 @@ def test_wsweep2d_bitwise_vs_k1_k0(lift, case, kind, monkeypatch):
         np.testing.assert_array_equal(y, y0, err_msg=f"hc={hc}")
     Y, A = orc.apply(sp, xs)
     assert orc.max_rel_err(y0, Y, A) <= TOL1
+
+
+# ------------------------------------- K2C whole-column tiles (nz <= 16) ----
+K2C_SHAPES = [(1, 20, 132), (2, 9, 128), (3, 33, 260), (8, 64, 132), (16, 17, 516)]
+
+
+@pytest.mark.parametrize("shape", K2C_SHAPES)
+@pytest.mark.parametrize("kind", KINDS)
+@pytest.mark.parametrize("op", ["j3d7", "hotspot"])
+def test_column3d_few_planes(lift, monkeypatch, shape, kind, op):
+    """Few-plane 3D grids run on K2C (one TMA box per CTA over all nz planes):
+    parity with the oracle, bitwise equal to K0 and to the K2 ring sweep
+    (LIFT_K2C=0), every pad kind, ragged x/y tiles, nz = 1 .. 16."""
+    if op == "j3d7":
+        xs = [rnd(shape, 141)]
+        sp = spec(shape, 3, si.weights_j3d7(), kind, value=0.75)
+    else:
+        xs = [rnd(shape, 142, 300.0, 350.0), rnd(shape, 143, 0.0, 1e-2)]
+        sp = spec(shape, 3, op=si.HOTSPOT3D, params=si.params_hotspot3d(), kind=kind, value=0.75)
+    y, plan = check(lift, sp, xs)
+    assert plan.last_variant == 2
+    y0, _ = run_gpu(lift, sp, xs, "generic")
+    np.testing.assert_array_equal(y, y0)
+    monkeypatch.setenv("LIFT_K2C", "0")
+    y2, _ = run_gpu(lift, sp, xs)
+    np.testing.assert_array_equal(y, y2)
+
+
+def test_column3d_iterate_hotspot(lift, monkeypatch):
+    """Hotspot3D iterate (the x100 workload's structure) on K2C == K2 ring bitwise."""
+    T = rnd((8, 96, 264), 144, 300.0, 350.0)
+    P = rnd(T.shape, 145, 0.0, 1e-2)
+    sp = spec(T.shape, 3, op=si.HOTSPOT3D, params=si.params_hotspot3d())
+    plan = lift.Plan.from_spec(sp)
+    outs = []
+    for env in ("1", "0"):
+        monkeypatch.setenv("LIFT_K2C", env)
+        a, b = torch.from_numpy(T).cuda(), torch.empty(T.shape, device="cuda")
+        ri = plan.iterate([a, b], 9, [torch.from_numpy(P).cuda()])
+        outs.append((a, b)[ri].cpu().numpy())
+    np.testing.assert_array_equal(outs[0], outs[1])
+    ref = orc.iterate(sp, [T], [P], 9)[0]
+    assert np.max(np.abs(outs[0] - ref) / np.abs(ref)) <= TOL10
