@@ -538,11 +538,11 @@ def main():
     for _ in range(args.warmup):
         step()
     barrier()
-    # K4 (persistent iterate of a small L2-resident 3D grid): one launch per step
-    persist = (not slabbed) and iterable and plan.last_variant == 3
+    # K4 / K6 (persistent iterate of a small 3D grid): one launch per bench step
+    persist = (not slabbed) and iterable and plan.last_variant in (3, 5)
     if persist:
         launches_per_step = 1
-    variant_id = 3 if persist else plan.variant
+    variant_id = plan.last_variant if persist else plan.variant
 
     # L2-resident working sets (one sweep's algorithmic bytes < 2 x L2): the
     # timed steps are cold — a 2 x L2 buffer is written before every step,
@@ -606,7 +606,7 @@ def main():
                      for _ in range(args.steps)]
             for k in range(args.steps):
                 flush.fill_(k)              # evict the working set from L2 (not timed)
-                torch.sum(flush_rd, out=flush_sink)   # ... and leave clean lines behind
+                torch.sum(flush_rd, 0, out=flush_sink)   # ... and leave clean lines behind
                 pairs[k][0].record(stream)
                 step()
                 pairs[k][1].record(stream)
@@ -632,7 +632,7 @@ def main():
         # the step is back-to-back launches of the dominant kernel on one stream
         # (SRAD: one iteration = one fused pass; the first iteration's q0 pass is in the time)
         units = args.steps * (steps_per_iter if op == si.SRAD else launches_per_step)
-        if persist:   # K4: one launch per bench step runs all time steps; time per time step
+        if persist:   # K4 / K6: one launch per bench step runs all time steps; time per time step
             units = args.steps * steps_per_iter
         avg_launch_s = (t_ms * 1e-3) / units
         alg_bytes = npts_local * bpp
@@ -774,13 +774,16 @@ def main():
                                        "K1 tile2d (cp.async 8-B pair fill)" if ext1[-1] % 2 == 0 else
                                        "K1 tile2d (cp.async 4-B fill)"),
                                    2: "K2 sweep3d (TMA)",
-                                   3: "K4 persistent iterate (cooperative)"}[variant_id],
+                                   3: "K4 persistent iterate (cooperative)",
+                                   4: "K5 gather tiles",
+                                   5: "K6 shared-memory-resident iterate (cooperative)"}[variant_id],
                        "launch": (f"cuda graph replay ({launches_per_step} launches per graph)" if graph is not None
                                   else "stream launches")},
             "hbm_gbs_per_gpu_whole_step": value * bpp / world,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": ncu_traffic(args.workload),
-                         "kernel": {0: "k0_generic", 1: "k1_tile", 2: "k2_sweep", 3: "k4_iterate"}[variant_id],
+                         "kernel": {0: "k0_generic", 1: "k1_tile", 2: "k2_sweep", 3: "k4_iterate", 4: "k5_gather",
+                                    5: "k6_resident"}[variant_id],
                          "peak_source": peak_src,
                          "alg_bytes_per_launch": alg_bytes, "avg_launch_us": avg_launch_s * 1e6,
                          "frac_of_8TBs": achieved / 8000.0},

@@ -102,10 +102,19 @@ typedef enum {
                                     grids; opt-in with LIFT_K4=1 — measured
                                     slower than K2 steps; reported by
                                     stencil_plan_last_variant, not forceable)  */
-  STENCIL_VARIANT_GATHER = 4     /* K5: WEIGHTED plans the TMA families do not
+  STENCIL_VARIANT_GATHER = 4,    /* K5: WEIGHTED plans the TMA families do not
                                     take (step > 1, even / asymmetric windows,
                                     1D, wide boxes, unaligned 3D) through
                                     shared-memory tiles of the input box        */
+  STENCIL_VARIANT_RESIDENT3D = 5 /* K6: all n steps of stencil_iterate for a
+                                    few-plane (nz <= 16) 3D radius-1 star /
+                                    Hotspot3D grid that fits in the device's
+                                    shared memory (one tile per SM), in one
+                                    cooperative launch with point-to-point
+                                    step flags; opt-in with LIFT_K6=1 (measured
+                                    slower than graph-replayed K2C sweeps);
+                                    reported by stencil_plan_last_variant, not
+                                    forceable                                   */
 } stencil_variant;
 
 /*

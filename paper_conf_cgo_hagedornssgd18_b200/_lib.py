@@ -25,7 +25,8 @@ _lib = C.CDLL(LIB_PATH)
 STENCIL_OK, STENCIL_E_INVALID, STENCIL_E_UNSUPPORTED, STENCIL_E_CUDA, STENCIL_E_NOMEM = range(5)
 PAD_CLAMP, PAD_MIRROR, PAD_WRAP, PAD_CONSTANT, PAD_REFLECT, PAD_DAMPEN = range(6)
 OP_WEIGHTED, OP_HOTSPOT3D, OP_SRAD1, OP_SRAD2, OP_ACOUSTIC, OP_HOTSPOT2D, OP_GRADIENT, OP_SRAD = range(8)
-VARIANT_AUTO, VARIANT_GENERIC, VARIANT_TILE2D, VARIANT_SWEEP3D, VARIANT_PERSIST3D, VARIANT_GATHER = -1, 0, 1, 2, 3, 4
+(VARIANT_AUTO, VARIANT_GENERIC, VARIANT_TILE2D, VARIANT_SWEEP3D, VARIANT_PERSIST3D, VARIANT_GATHER,
+ VARIANT_RESIDENT3D) = -1, 0, 1, 2, 3, 4, 5
 OP_ARITY = {OP_WEIGHTED: 1, OP_HOTSPOT3D: 2, OP_SRAD1: 1, OP_SRAD2: 2, OP_ACOUSTIC: 2, OP_HOTSPOT2D: 2, OP_GRADIENT: 1, OP_SRAD: 1}
 
 _P = C.c_void_p

@@ -645,6 +645,23 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
   if (!state || n_state != 2) return fail(STENCIL_E_INVALID, "iterate needs 2 state buffers");
   if (!state[0] || !state[1] || state[0] == state[1]) return fail(STENCIL_E_INVALID, "bad state buffers");
   int ri = (p.op == OP_ACOUSTIC) ? 1 : 0;
+  // few-plane 3D grids that fit in the device's shared memory: all steps in
+  // one cooperative launch with the grid resident on chip (K6)
+  if ((p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D) && n_steps >= 2 && pl->ndim == 3 && pl->time_block < 2 &&
+      pl->forced_variant == STENCIL_VARIANT_AUTO &&
+      (p.op == OP_WEIGHTED ? n_aux == 0 : (n_aux == 1 && aux && aux[0])) &&
+      resident3d_supported(p, state[0], state[1], p.op == OP_HOTSPOT3D ? aux[0] : nullptr, pl->num_sms)) {
+    DeviceGuard g(pl->device);
+    if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+    std::string err;
+    cudaError_t e = launch_resident3d(p, state[0], state[1], p.op == OP_HOTSPOT3D ? aux[0] : nullptr, n_steps,
+                                      (cudaStream_t)stream, pl->num_sms, &err);
+    if (e != cudaSuccess)
+      return fail(STENCIL_E_CUDA, std::string("K6 launch failed: ") + cudaGetErrorString(e) + " " + err);
+    pl->last_variant = STENCIL_VARIANT_RESIDENT3D;
+    if (result_index) *result_index = n_steps % 2;
+    return STENCIL_OK;
+  }
   // small L2-resident 3D grids: all steps in one persistent launch (K4)
   if ((p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D) && n_steps >= 2 && pl->ndim == 3 && pl->time_block < 2 &&
       pl->forced_variant == STENCIL_VARIANT_AUTO &&

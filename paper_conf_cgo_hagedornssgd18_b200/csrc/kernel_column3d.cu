@@ -26,6 +26,7 @@
 #include "launch.hpp"
 #include "ops.cuh"
 #include "tma.cuh"
+#include "colwin.cuh"
 
 namespace lift {
 namespace {
@@ -36,40 +37,6 @@ constexpr int BX = TX + 2 * XH;
 constexpr int NW = 8;
 constexpr int NT = NW * 32;
 constexpr int kMaxNz = 16;
-constexpr unsigned FULL = 0xffffffffu;
-
-enum K2COp { K2C_WSTAR = 0, K2C_HOTSPOT = 1 };
-
-// the 7-point window of output column I of a lane (x = xo + I), in registers
-struct ColWin {
-  float x[6];     // centre row, x offsets -1 .. 4
-  float ym[4], yp[4], zm[4], zp[4];
-};
-
-template <int I>
-struct ColAcc {
-  const ColWin& w;
-  template <int DZ, int DY, int DX>
-  __device__ __forceinline__ float at() const {
-    static_assert((DZ != 0) + (DY != 0) + (DX != 0) <= 1, "star access only");
-    if constexpr (DZ < 0) return w.zm[I];
-    else if constexpr (DZ > 0) return w.zp[I];
-    else if constexpr (DY < 0) return w.ym[I];
-    else if constexpr (DY > 0) return w.yp[I];
-    else return w.x[I + 1 + DX];
-  }
-};
-
-__device__ __forceinline__ void set4(float (&d)[4], float4 v) {
-  d[0] = v.x; d[1] = v.y; d[2] = v.z; d[3] = v.w;
-}
-
-template <int OP, int I>
-__device__ __forceinline__ float eval(const StencilParams& p, const ColWin& w, const float4& pw) {
-  ColAcc<I> a{w};
-  if constexpr (OP == K2C_WSTAR) return op_weighted<1, 1, 1, true>(a, p.wbox);
-  else return op_hotspot3d(a, f4get(pw, I), p.prm);
-}
 
 template <int OP, int TY>
 __global__ void __launch_bounds__(NT) k2c_column(const __grid_constant__ StencilParams p,
@@ -164,25 +131,14 @@ __global__ void __launch_bounds__(NT) k2c_column(const __grid_constant__ Stencil
     const int zpi = z + 1 < nz ? z + 1 : (kz == PAD_CONSTANT ? -1 : (int)pad_remap(nz, nz, kz));
     const float* pl = tb + z * BY * BX + (yy + 1) * BX + XH + 4 * lane;
     ColWin w;
-    const float4 c = lds128(pl);
-    set4(w.ym, lds128(pl - BX));
-    set4(w.yp, lds128(pl + BX));
-    if (zmi >= 0) set4(w.zm, lds128(pl + (zmi - z) * BY * BX));
-    else w.zm[0] = w.zm[1] = w.zm[2] = w.zm[3] = pv;
-    if (zpi >= 0) set4(w.zp, lds128(pl + (zpi - z) * BY * BX));
-    else w.zp[0] = w.zp[1] = w.zp[2] = w.zp[3] = pv;
-    w.x[1] = c.x; w.x[2] = c.y; w.x[3] = c.z; w.x[4] = c.w;
-    const float left = __shfl_up_sync(FULL, c.w, 1);
-    const float right = __shfl_down_sync(FULL, c.x, 1);
-    w.x[0] = lane == 0 ? pl[-1] : left;
-    w.x[5] = lane == 31 ? pl[4] : right;
+    colwin_load(w, pl, BX, BY * BX, zmi - z, zpi - z, zmi < 0, zpi < 0, pv, lane);
     float4 pw = make_float4(0.f, 0.f, 0.f, 0.f);
     if constexpr (PW) pw = lds128(pb + (z * TY + yy) * TX + 4 * lane);
     float4 res;
-    res.x = eval<OP, 0>(p, w, pw);
-    res.y = eval<OP, 1>(p, w, pw);
-    res.z = eval<OP, 2>(p, w, pw);
-    res.w = eval<OP, 3>(p, w, pw);
+    res.x = colwin_eval<OP, 0>(p, w, pw);
+    res.y = colwin_eval<OP, 1>(p, w, pw);
+    res.z = colwin_eval<OP, 2>(p, w, pw);
+    res.w = colwin_eval<OP, 3>(p, w, pw);
     if (x_ok && gy < ny) stg128(out + ((int64_t)z * ny + gy) * nx + xo, res);
   }
 }

@@ -58,6 +58,14 @@ bool column3d_supported(const StencilParams& p, const float* in0, const float* i
 cudaError_t launch_column3d(const StencilParams& p, const float* in0, const float* in1, float* out,
                             cudaStream_t stream, std::string* err);
 
+// K6 — all n steps of stencil_iterate for a few-plane 3D radius-1 star grid
+// (weighted / Hotspot3D) with the grid resident in shared memory (one tile
+// per SM, one cooperative launch, grid barrier per step).
+bool resident3d_supported(const StencilParams& p, const float* s0, const float* s1, const float* aux,
+                          int num_sms);
+cudaError_t launch_resident3d(const StencilParams& p, float* s0, float* s1, const float* aux, int n_steps,
+                              cudaStream_t stream, int num_sms, std::string* err);
+
 // K2T — two weighted 7-point steps per pass (temporal blocking), CLAMP/MIRROR/REFLECT.
 bool sweep3d_t2_supported(const StencilParams& p);
 cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* out, cudaStream_t stream, int num_sms,

@@ -37,9 +37,11 @@ __device__ __forceinline__ unsigned long long grid_id() {
 }
 
 // Called by one thread per CTA; every CTA of a launch gets the same index.
-__device__ __forceinline__ int claim_launch_slot(LaunchSlot* tab) {
+// ``Slot`` has an ``owner`` word; K (a power of two) entries in ``tab``.
+template <int K, class Slot>
+__device__ __forceinline__ int claim_slot(Slot* tab) {
   const unsigned long long tag = grid_id() + 1ull;
-  const int i = (int)(tag & (unsigned long long)(kLaunchSlots - 1));
+  const int i = (int)(tag & (unsigned long long)(K - 1));
   while (true) {
     unsigned long long o = *reinterpret_cast<volatile unsigned long long*>(&tab[i].owner);
     if (o == tag) return i;
@@ -47,9 +49,11 @@ __device__ __forceinline__ int claim_launch_slot(LaunchSlot* tab) {
       o = atomicCAS(&tab[i].owner, 0ull, tag);
       if (o == 0ull || o == tag) return i;
     }
-    __nanosleep(256);   // held by a launch 65536 ids older that is still running
+    __nanosleep(256);   // held by a launch K ids older that is still running
   }
 }
+
+__device__ __forceinline__ int claim_launch_slot(LaunchSlot* tab) { return claim_slot<kLaunchSlots>(tab); }
 
 // Called by the launch's last CTA (every CTA has finished with the slot):
 // zero the counters, make that visible, then free the slot.

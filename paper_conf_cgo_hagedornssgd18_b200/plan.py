@@ -22,7 +22,7 @@ OPS = {"weighted": L.OP_WEIGHTED, "hotspot3d": L.OP_HOTSPOT3D, "srad1": L.OP_SRA
        "srad": L.OP_SRAD}
 VARIANTS = {"auto": L.VARIANT_AUTO, "generic": L.VARIANT_GENERIC, "tile2d": L.VARIANT_TILE2D,
             "sweep3d": L.VARIANT_SWEEP3D, "persist3d": L.VARIANT_PERSIST3D,
-            "gather": L.VARIANT_GATHER}
+            "gather": L.VARIANT_GATHER, "resident3d": L.VARIANT_RESIDENT3D}
 
 
 def _tuple(v, nd):

@@ -670,3 +670,40 @@ def test_column3d_iterate_hotspot(lift, monkeypatch):
     np.testing.assert_array_equal(outs[0], outs[1])
     ref = orc.iterate(sp, [T], [P], 9)[0]
     assert np.max(np.abs(outs[0] - ref) / np.abs(ref)) <= TOL10
+
+
+# ------------------------------- K6 shared-memory-resident iterate ----------
+K6_SHAPES = [(8, 512, 512), (8, 96, 264), (1, 40, 128), (3, 130, 388), (16, 64, 132)]
+
+
+@pytest.mark.parametrize("shape", K6_SHAPES)
+@pytest.mark.parametrize("kind", KINDS)
+@pytest.mark.parametrize("op", ["j3d7", "hotspot"])
+def test_resident3d_iterate(lift, monkeypatch, shape, kind, op):
+    """K6 (opt-in; the whole grid in shared memory, one cooperative launch,
+    step flags between neighbour tiles): bitwise equal to stepping K2C/K2
+    launches (LIFT_K6=0)
+    for 2, 5 and 9 steps, and within the 10-step tolerance of the oracle."""
+    if op == "j3d7":
+        xs, aux = [rnd(shape, 151)], []
+        sp = spec(shape, 3, si.weights_j3d7(), kind, value=0.75)
+    else:
+        xs, aux = [rnd(shape, 152, 300.0, 350.0)], [rnd(shape, 153, 0.0, 1e-2)]
+        sp = spec(shape, 3, op=si.HOTSPOT3D, params=si.params_hotspot3d(), kind=kind, value=0.75)
+    plan = lift.Plan.from_spec(sp)
+    for n in (2, 5, 9):
+        res = {}
+        for env in ("1", "0"):
+            monkeypatch.setenv("LIFT_K6", env)          # K6 is opt-in
+            a, b = torch.from_numpy(xs[0]).cuda(), torch.empty(shape, device="cuda")
+            ri = plan.iterate([a, b], n, [torch.from_numpy(x).cuda() for x in aux])
+            torch.cuda.synchronize()
+            assert ri == n % 2
+            res[env] = ((a, b)[ri].cpu().numpy(), plan.last_variant)
+        assert res["1"][1] == lift.plan.VARIANTS["resident3d"]
+        assert res["0"][1] != lift.plan.VARIANTS["resident3d"]
+        np.testing.assert_array_equal(res["1"][0], res["0"][0], err_msg=f"{n} steps")
+    if int(np.prod(shape)) <= 1 << 20:
+        ref = orc.iterate(sp, xs, aux, 9)[0]
+        Y = res["1"][0].astype(np.float64)
+        assert np.max(np.abs(Y - ref) / np.maximum(np.abs(ref), 1e-30)) <= TOL10
