@@ -14,7 +14,10 @@ from typing import Optional, Sequence
 import numpy as np
 
 _PKG = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_PKG, "libstencil.so")
+# LIFT_LIB_TAG=x loads the in-tree A/B build libstencil_x.so (build.py with
+# the same variable); the default is the product library
+_TAG = os.environ.get("LIFT_LIB_TAG", "")
+LIB_PATH = os.path.join(_PKG, f"libstencil_{_TAG}.so" if _TAG else "libstencil.so")
 
 if not os.path.exists(LIB_PATH):
     raise ImportError(f"{LIB_PATH} is missing: build it with `python __graft_entry__.py` or "

@@ -22,14 +22,18 @@ import sys
 PKG = os.path.dirname(os.path.abspath(__file__))
 ROOT = os.path.dirname(PKG)
 CSRC = os.path.join(PKG, "csrc")
-BUILD = os.path.join(PKG, "_build")
-LIB = os.path.join(PKG, "libstencil.so")
+# LIFT_LIB_TAG=x builds an A/B variant libstencil_x.so (objects in _build_x)
+# with the extra nvcc flags of LIFT_NVCC_EXTRA (e.g. -DLIFT_MBAR_SPIN); the
+# binding loads it with the same variable
+_TAG = os.environ.get("LIFT_LIB_TAG", "")
+BUILD = os.path.join(PKG, f"_build_{_TAG}" if _TAG else "_build")
+LIB = os.path.join(PKG, f"libstencil_{_TAG}.so" if _TAG else "libstencil.so")
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 CFLAGS = ["-O3", "-std=c++17", "-lineinfo", "-fmad=false", "-Xcompiler", "-fPIC",
           "-Xcompiler", "-Wall", "-I" + os.path.join(ROOT, "include"), "-I" + CSRC,
-          "--expt-relaxed-constexpr"]
+          "--expt-relaxed-constexpr"] + os.environ.get("LIFT_NVCC_EXTRA", "").split()
 
 
 def _sources():

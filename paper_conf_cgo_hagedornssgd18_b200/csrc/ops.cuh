@@ -11,11 +11,42 @@
 // the padded input at offset (DZ, DY, DX) from the window centre (for the
 // centred ops below); point-wise zipped inputs are passed as values.
 #pragma once
+#include <type_traits>
 #include <utility>
 
 #include "common.cuh"
 
 namespace lift {
+
+// ---- scalar and packed arithmetic -----------------------------------------
+// The map functions below are written once over a value type V: float (one
+// output) or float2 (two outputs in the two fp32 lanes of sm_100a's packed
+// FFMA2 / FADD2 / FMUL2 — half the instructions for issue-bound kernels).
+// Each packed lane is the same IEEE round-to-nearest operation as the scalar
+// one, so an output's bits do not depend on which form computed it.
+__device__ __forceinline__ float vfma(float a, float b, float c) { return __fmaf_rn(a, b, c); }
+__device__ __forceinline__ float vadd(float a, float b) { return __fadd_rn(a, b); }
+__device__ __forceinline__ float vsub(float a, float b) { return __fsub_rn(a, b); }
+__device__ __forceinline__ float vmul(float a, float b) { return __fmul_rn(a, b); }
+__device__ __forceinline__ float2 vfma(float2 a, float2 b, float2 c) { return __ffma2_rn(a, b, c); }
+__device__ __forceinline__ float2 vadd(float2 a, float2 b) { return __fadd2_rn(a, b); }
+__device__ __forceinline__ float2 vmul(float2 a, float2 b) { return __fmul2_rn(a, b); }
+__device__ __forceinline__ float2 vsub(float2 a, float2 b) {
+  unsigned long long r;
+  asm("sub.rn.f32x2 %0, %1, %2;"
+      : "=l"(r)
+      : "l"(*reinterpret_cast<const unsigned long long*>(&a)), "l"(*reinterpret_cast<const unsigned long long*>(&b)));
+  return *reinterpret_cast<float2*>(&r);
+}
+template <class V>
+__device__ __forceinline__ V vbc(float s);
+template <>
+__device__ __forceinline__ float vbc<float>(float s) { return s; }
+template <>
+__device__ __forceinline__ float2 vbc<float2>(float s) { return make_float2(s, s); }
+
+template <class Acc>
+using acc_value_t = std::decay_t<decltype(std::declval<const Acc&>().template at<0, 0, 0>())>;
 
 // compile-time loop: f(std::integral_constant<int, 0..N-1>) in order
 template <class F, int... Is>
@@ -69,12 +100,24 @@ __device__ __forceinline__ float op_hotspot3d(const Acc& T, float Pc, const floa
 // slow path: ~10 instructions and a branch per point); within 2 ulp of the
 // exact value for normal inputs — far inside the 1e-5 parity bound — and
 // identical in every kernel family (reading A24b).
-__device__ __forceinline__ float rcp_nr(float x) {
+__device__ __forceinline__ float rcp_approx(float x) {
   float r;
   asm("rcp.approx.ftz.f32 %0, %1;" : "=f"(r) : "f"(x));
+  return r;
+}
+__device__ __forceinline__ float rcp_nr(float x) {
+  const float r = rcp_approx(x);
   const float e = __fmaf_rn(-x, r, 1.0f);
   return __fmaf_rn(r, e, r);
 }
+// two lanes: the same MUFU approximation per lane, the same Newton step packed
+__device__ __forceinline__ float2 rcp_nr(float2 x) {
+  const float2 r = make_float2(rcp_approx(x.x), rcp_approx(x.y));
+  const float2 e = vfma(make_float2(-x.x, -x.y), r, vbc<float2>(1.0f));
+  return vfma(r, e, r);
+}
+__device__ __forceinline__ float clamp01(float c) { return c < 0.0f ? 0.0f : (c > 1.0f ? 1.0f : c); }
+__device__ __forceinline__ float2 clamp01(float2 c) { return make_float2(clamp01(c.x), clamp01(c.y)); }
 __device__ __forceinline__ float rsqrt_nr(float x) {
   float r;
   asm("rsqrt.approx.ftz.f32 %0, %1;" : "=f"(r) : "f"(x));
@@ -92,24 +135,24 @@ __device__ __forceinline__ float rsqrt_nr(float x) {
 //   c = D^2 / (a*D^2 + b*n0),  a = q0/(1+q0),  b = 1/(q0(1+q0))
 // with a, b plan constants (prm[1], prm[2]); then c is clamped to [0, 1].
 template <class Acc>
-__device__ __forceinline__ float op_srad1(const Acc& I, const float* prm) {
-  const float a = prm[1], b = prm[2];
-  const float Ic = I.template at<0, 0, 0>();
-  const float dN = __fsub_rn(I.template at<0, -1, 0>(), Ic);
-  const float dS = __fsub_rn(I.template at<0, 1, 0>(), Ic);
-  const float dW = __fsub_rn(I.template at<0, 0, -1>(), Ic);
-  const float dE = __fsub_rn(I.template at<0, 0, 1>(), Ic);
-  float g = __fmul_rn(dN, dN);
-  g = __fmaf_rn(dS, dS, g);
-  g = __fmaf_rn(dW, dW, g);
-  g = __fmaf_rn(dE, dE, g);
-  const float sd = __fadd_rn(__fadd_rn(__fadd_rn(dN, dS), dW), dE);
-  const float n0 = __fmaf_rn(-0.0625f, __fmul_rn(sd, sd), __fmul_rn(0.5f, g));
-  const float D = __fmaf_rn(0.25f, sd, Ic);
-  const float D2 = __fmul_rn(D, D);
-  float c = __fmul_rn(D2, rcp_nr(__fmaf_rn(a, D2, __fmul_rn(b, n0))));
-  c = c < 0.0f ? 0.0f : (c > 1.0f ? 1.0f : c);
-  return c;
+__device__ __forceinline__ acc_value_t<Acc> op_srad1(const Acc& I, const float* prm) {
+  using V = acc_value_t<Acc>;
+  const V a = vbc<V>(prm[1]), b = vbc<V>(prm[2]);
+  const V Ic = I.template at<0, 0, 0>();
+  const V dN = vsub(I.template at<0, -1, 0>(), Ic);
+  const V dS = vsub(I.template at<0, 1, 0>(), Ic);
+  const V dW = vsub(I.template at<0, 0, -1>(), Ic);
+  const V dE = vsub(I.template at<0, 0, 1>(), Ic);
+  V g = vmul(dN, dN);
+  g = vfma(dS, dS, g);
+  g = vfma(dW, dW, g);
+  g = vfma(dE, dE, g);
+  const V sd = vadd(vadd(vadd(dN, dS), dW), dE);
+  const V n0 = vfma(vbc<V>(-0.0625f), vmul(sd, sd), vmul(vbc<V>(0.5f), g));
+  const V D = vfma(vbc<V>(0.25f), sd, Ic);
+  const V D2 = vmul(D, D);
+  const V c = vmul(D2, rcp_nr(vfma(a, D2, vmul(b, n0))));
+  return clamp01(c);
 }
 
 // SRAD1's constants {q0, a, b} from q0 (the same derivation as the plan's)
@@ -130,21 +173,21 @@ __host__ __device__ inline float srad_q0sqr(double s, double ss, int64_t n) {
 
 // ---- SRAD kernel 2: (c, I) -> I' (Rodinia v3.1 srad; A18) --------
 template <class AccC, class AccI>
-__device__ __forceinline__ float op_srad2(const AccC& C, const AccI& I, const float* prm) {
-  const float lam = prm[0];
-  const float Ic = I.template at<0, 0, 0>();
-  const float dN = __fsub_rn(I.template at<0, -1, 0>(), Ic);
-  const float dS = __fsub_rn(I.template at<0, 1, 0>(), Ic);
-  const float dW = __fsub_rn(I.template at<0, 0, -1>(), Ic);
-  const float dE = __fsub_rn(I.template at<0, 0, 1>(), Ic);
-  const float cC = C.template at<0, 0, 0>();
-  const float cS = C.template at<0, 1, 0>();
-  const float cE = C.template at<0, 0, 1>();
-  float D = __fmul_rn(cC, dN);
-  D = __fmaf_rn(cS, dS, D);
-  D = __fmaf_rn(cC, dW, D);
-  D = __fmaf_rn(cE, dE, D);
-  return __fmaf_rn(__fmul_rn(0.25f, lam), D, Ic);
+__device__ __forceinline__ acc_value_t<AccI> op_srad2(const AccC& C, const AccI& I, const float* prm) {
+  using V = acc_value_t<AccI>;
+  const V Ic = I.template at<0, 0, 0>();
+  const V dN = vsub(I.template at<0, -1, 0>(), Ic);
+  const V dS = vsub(I.template at<0, 1, 0>(), Ic);
+  const V dW = vsub(I.template at<0, 0, -1>(), Ic);
+  const V dE = vsub(I.template at<0, 0, 1>(), Ic);
+  const V cC = C.template at<0, 0, 0>();
+  const V cS = C.template at<0, 1, 0>();
+  const V cE = C.template at<0, 0, 1>();
+  V D = vmul(cC, dN);
+  D = vfma(cS, dS, D);
+  D = vfma(cC, dW, D);
+  D = vfma(cE, dE, D);
+  return vfma(vbc<V>(__fmul_rn(0.25f, prm[0])), D, Ic);
 }
 
 // ---- Hotspot2D (Rodinia v3.1 hotspot; A26) -----------------------

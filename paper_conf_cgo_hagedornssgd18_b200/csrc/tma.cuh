@@ -30,8 +30,13 @@ __device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
   asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
 
+// try_wait with a suspend-time hint: a waiting warp is parked until the phase
+// completes (or the hint elapses) instead of spinning through issue slots
+// that the computing warps of an issue-bound kernel need.  LIFT_MBAR_SPIN
+// (compile-time) restores the plain spin for A/B.
 __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
   const uint32_t addr = smem_u32(bar);
+#ifdef LIFT_MBAR_SPIN
   asm volatile(
       "{\n"
       ".reg .pred p;\n"
@@ -41,6 +46,17 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
       "}\n" ::"r"(addr),
       "r"(parity)
       : "memory");
+#else
+  asm volatile(
+      "{\n"
+      ".reg .pred p;\n"
+      "WAIT_%=:\n"
+      "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1, %2;\n"
+      "@!p bra WAIT_%=;\n"
+      "}\n" ::"r"(addr),
+      "r"(parity), "r"(0x989680u)
+      : "memory");
+#endif
 }
 
 __device__ __forceinline__ void prefetch_tmap(const CUtensorMap* map) {
