@@ -8,18 +8,22 @@ boundary, 100 time steps" — the config the metric's 1/2/4/8-GPU numbers are
 quoted on (north_star: iterated sweeps at 2/4/8 GPUs, weak scaling for the
 iterated 3D Jacobi).  One bench step = one full stencil_iterate of 100 time
 steps (pad -> slide -> map -> store, iterated) over 512^3 points per GPU.
-At N GPUs the global grid is (512*N, 512, 512), slab-decomposed along z with a
-per-time-step halo exchange (NCCL send/recv) overlapped with interior compute
-(weak scaling).  Inputs (512 MiB per grid) are larger than L2 (126 MB), so no
-L2 flush is needed between timed iterations.
+At N GPUs the global grid is (512*N, 512, 512), slab-decomposed along z; ghost
+planes travel by NCCL send/recv overlapped with interior compute, 4 planes
+every 4 time steps by default (deep halos, --halo-depth; weak scaling).
+`python bench.py --gpus N` launches the N ranks itself through
+torch.distributed.run (the driver's launch line) and fails if fewer than N
+GPUs are visible.  Inputs (512 MiB per grid) are larger than L2 (126 MB), so
+no L2 flush is needed between timed iterations.
 
 Other workloads (--workload, stencil_inputs.WORKLOAD_NAMES): the remaining
 BASELINE.json configs (gauss5_8192_mirror, j2d5_256_clamp,
 hotspot3d_8x512x512[_x100], srad1_4096, srad2_4096, srad_iter_4096,
 acoustic7_1024, acoustic13_1024) and the Table-1 workloads (t1_*).
 Workloads whose per-sweep bytes are below 2 x L2 are timed cold: a 2 x L2
-buffer is written before every timed step (outside its event pair) and a
-single-sweep workload's step is one sweep; the warm number is reported as
+buffer is written, then another 2 x L2 buffer read, before every timed step
+(outside its event pair; L2 then holds clean lines) and a single-sweep
+workload's step is one sweep; the warm number is reported as
 "hot" (--no-flush times warm).  --scaling strong splits the single-GPU grid
 over the ranks (Acoustic 1024^3 over 1/2/4/8 GPUs); --halo fused exchanges
 ghosts by peer stores from the boundary kernel instead of NCCL.
@@ -362,12 +366,16 @@ def main():
     ap.add_argument("--halo", default="nccl", choices=["nccl", "fused"],
                     help="multi-GPU ghost exchange: NCCL send/recv overlapped with the interior (default), or the "
                          "fused boundary kernel storing into the neighbours' ghosts over NVLink peer memory")
-    ap.add_argument("--halo-depth", type=int, default=1,
+    ap.add_argument("--halo-depth", type=int, default=None,
                     help="slab path: ghost depth in time steps k (NEXT-3 deep halos): ghosts of r*k planes are "
-                         "exchanged every k time steps and the overlap is recomputed redundantly")
+                         "exchanged every k time steps and the overlap is recomputed redundantly (default 4 on "
+                         "the NCCL path: 797 vs 750 Gpts/s at world size 1, profiles/r02_slab_world1.txt; the "
+                         "fused path exchanges every step)")
     ap.add_argument("--selftest-launch", action="store_true", help=argparse.SUPPRESS)
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
+    if args.halo_depth is None:
+        args.halo_depth = 1 if args.halo == "fused" else 4
 
     # --gpus N without a torchrun environment: launch N ranks ourselves (the
     # same launch line the driver uses), so `python bench.py --gpus N` is a
