@@ -500,17 +500,13 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
         const int crow = y0 + r0 + k - 2;
         // c rows past the bottom edge: WRAP computes them from the box's
         // wrapped I rows (= c(crow - ny)); the others copy the remapped row
-        const bool cval = crow < ny || ky == PAD_WRAP;      // warp-uniform
-        if (cval) {
+        if (crow < ny || ky == PAD_WRAP) {
           static_for<4>([&](auto II) {
             constexpr int ii = decltype(II)::value;
             cr[cs_][ii] = op_srad1(RowsAcc<2, ii>{iw[(k - 2) % 4], iw[(k - 1) % 4], iw[k % 4]}, q);
           });
-        }
-        // shuffles outside the branch: no collective fix-up code around them
-        const float right = __shfl_down_sync(0xffffffffu, cr[cs_][0], 1);
-        const float hcol = __shfl_sync(0xffffffffu, halo_c, k - 2);
-        if (cval) {
+          const float right = __shfl_down_sync(0xffffffffu, cr[cs_][0], 1);
+          const float hcol = __shfl_sync(0xffffffffu, halo_c, k - 2);
           cr[cs_][4] = lane == 31 ? hcol : right;
           cr[cs_][4] = ce == 4 ? cr[cs_][4] : (ce == 3 ? cr[cs_][3] : (ce == 2 ? cr[cs_][2] : cr[cs_][1]));
         } else if constexpr (k >= 3) {
