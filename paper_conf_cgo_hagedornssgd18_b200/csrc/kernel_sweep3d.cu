@@ -609,8 +609,9 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
             }
             if (ok) {
               stg128(orow + jj * nx, res);
-              if constexpr (FZ) {
+              if constexpr (FZ && EDGE) {
                 // fused halo put: boundary planes also go to the neighbour's ghosts
+                // (items of the boundary chunks run this general loop body)
                 if (z < p.ghost && p.put_lo) stg128(p.put_lo + z * p.plane + (int64_t)gy * nx + xo, res);
                 if (z >= p.n[0] - p.ghost && p.put_hi)
                   stg128(p.put_hi + (z - (p.n[0] - p.ghost)) * p.plane + (int64_t)gy * nx + xo, res);
@@ -631,7 +632,11 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
           for (int k = 0; k < 2 * R; ++k) zst[k] = zst[k + 1];
         }
       };
-      if (x_edge || y_edge) plane_loop(std::true_type{});
+      // fused halo put: only the items of the first / last chunk store into the
+      // neighbours' ghosts; they take the general (EDGE) body, every other
+      // item the interior one without the put checks
+      const bool put_item = FZ && (p.put_lo || p.put_hi) && (zs < p.ghost || zs + nzc > p.n[0] - p.ghost);
+      if (x_edge || y_edge || put_item) plane_loop(std::true_type{});
       else plane_loop(std::false_type{});
       // the chunk's last 2R planes (z_end - R .. z_end + R - 1) are still held
       __syncwarp();
