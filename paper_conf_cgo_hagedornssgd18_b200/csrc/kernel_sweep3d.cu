@@ -1156,7 +1156,14 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
   void* args[] = {(void*)&p, (void*)&map, (void*)&pwmap, (void*)&slid, (void*)&out,
                   &ntx_i, &nty_i, &zc_i, &nch_i, &n1_i, &zc2_i};
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
-  return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, !fz);
+  // PDL for the fused halo launches is an A/B knob (LIFT_FUSED_PDL=1): the
+  // kernel's flag spins come after its griddepcontrol.wait, so a dependent
+  // launch cannot run ahead of the step it depends on
+  static const bool fused_pdl = [] {
+    const char* e = getenv("LIFT_FUSED_PDL");
+    return e && e[0] == '1';
+  }();
+  return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, !fz || fused_pdl);
 }
 
 }  // namespace lift
