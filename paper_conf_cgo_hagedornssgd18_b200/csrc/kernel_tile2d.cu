@@ -695,7 +695,13 @@ cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* o
     case 2: L = srad_fused_launcher<4, 3, 2>(); break;
     case 3: L = srad_fused_launcher<6, 3, 2>(); break;
     case 4: L = srad_fused_launcher<4, 2, 3>(); break;
-    default: L = srad_fused_launcher<6, 2, 3>(); break;
+    case 5: L = srad_fused_launcher<8, 2, 3>(); break;
+    case 6: L = srad_fused_launcher<6, 2, 3>(); break;     // round 1's default
+    case 7: L = srad_fused_launcher<12, 2, 2>(); break;
+    // 8 rows per warp (SRAD1 for 9/8 instead of 7/6 of the rows), 96
+    // registers without spills at 2 CTAs/SM: 379 -> 386 Gpts/s
+    // (profiles/r02_ab_srad_shape.txt)
+    default: L = srad_fused_launcher<8, 2, 2>(); break;
   }
   CUtensorMap m0;
   if (!get_map(in0, p.n[2], p.n[1], L.ty + 4, &m0, err)) return cudaErrorInvalidValue;
