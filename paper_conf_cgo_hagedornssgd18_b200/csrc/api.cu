@@ -59,9 +59,10 @@ stencil_status cuda_fail(cudaError_t e, const char* what) {
 }
 
 // ---- bounded halo waits (fused slab path) --------------------------------
-// One process-wide fault word in mapped pinned host memory: a wait that times
-// out ORs a code into it (device store, system scope) and the host reads it
-// without a device round trip.  The timeout is process-wide too.
+// One process-wide fault block in mapped pinned host memory: a wait that
+// times out stores 1 into the word of its code (device store, system scope)
+// and the host reads it without a device round trip.  The timeout is
+// process-wide too.
 std::mutex g_fault_mu;
 unsigned int* g_fault = nullptr;          // host pointer == device pointer (UVA)
 unsigned long long g_wait_timeout_ns = [] {
@@ -88,7 +89,9 @@ stencil_status take_fault() {
   {
     std::lock_guard<std::mutex> lk(g_fault_mu);
     if (!g_fault) return STENCIL_OK;
-    f = __atomic_exchange_n(g_fault, 0u, __ATOMIC_ACQ_REL);
+    // one word per code (the device stores 1, host memory has no device atomics)
+    if (__atomic_exchange_n(&g_fault[kFaultWaitLo - 1], 0u, __ATOMIC_ACQ_REL)) f |= kFaultWaitLo;
+    if (__atomic_exchange_n(&g_fault[kFaultWaitHi - 1], 0u, __ATOMIC_ACQ_REL)) f |= kFaultWaitHi;
   }
   if (!f) return STENCIL_OK;
   std::string which = (f & kFaultWaitLo) && (f & kFaultWaitHi) ? "lower and upper"

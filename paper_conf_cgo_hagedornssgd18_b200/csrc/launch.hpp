@@ -109,7 +109,7 @@ cudaError_t launch_persist3d(const StencilParams& p, float* s0, float* s1, const
                              cudaStream_t stream, int num_sms, std::string* err);
 
 // wait (one thread, acquire.sys) until *a >= value and *b >= value (NULL =
-// skip); bounded by timeout_ns (0 = none), a timeout ORs into *fault
+// skip); bounded by timeout_ns (0 = none), a timeout sets its fault word
 cudaError_t launch_wait_signals(const unsigned int* a, const unsigned int* b, unsigned int value,
                                 unsigned long long timeout_ns, unsigned int* fault, cudaStream_t stream);
 

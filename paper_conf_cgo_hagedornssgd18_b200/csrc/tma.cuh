@@ -152,9 +152,12 @@ __device__ __forceinline__ unsigned long long globaltimer_ns() {
 
 // Waits (acquire, system scope) until *f >= v in wrap-around order.  A
 // neighbour that never raises its flag (a dead or stalled rank) must not hang
-// the GPU: after timeout_ns (0 = no limit) the wait gives up, ORs ``code``
-// into the host-visible fault word (stencil_device_fault reports it) and
-// returns false; the launch then completes with stale ghost data.
+// the GPU: after timeout_ns (0 = no limit) the wait gives up, stores 1 into
+// the host-visible fault word of ``code`` (fault[code - 1];
+// stencil_device_fault reports it) and returns false; the launch then
+// completes with stale ghost data.  A plain system-scope store, not an
+// atomic: the word is mapped host memory, where device atomics are not
+// supported over PCIe.
 __device__ __forceinline__ bool spin_until_bounded(const unsigned int* f, unsigned int v,
                                                    unsigned long long timeout_ns, unsigned int* fault,
                                                    unsigned int code) {
@@ -162,7 +165,10 @@ __device__ __forceinline__ bool spin_until_bounded(const unsigned int* f, unsign
   const unsigned long long t0 = globaltimer_ns();
   while ((int)(ld_acquire_sys(f) - v) < 0) {
     if (timeout_ns && globaltimer_ns() - t0 > timeout_ns) {
-      if (fault) atomicOr_system(fault, code);
+      if (fault) {
+        asm volatile("st.relaxed.sys.global.u32 [%0], %1;" ::"l"(fault + (code - 1)), "r"(1u) : "memory");
+        __threadfence_system();
+      }
       return false;
     }
     __nanosleep(64);
