@@ -296,6 +296,42 @@ def reference_arm(args, workload):
     print(json.dumps(line), flush=True)
 
 
+class HostStagedExchange:
+    """Test transport (--test-transport staged): the slab's ghost exchange with
+    DistExchange's neighbour pairing, the planes staged through host memory
+    over gloo (ranks sharing one GPU cannot use NCCL)."""
+
+    def __init__(self, rank, world, n, g, wrap, group=None):
+        from paper_conf_cgo_hagedornssgd18_b200.slab import DistExchange
+        self.inner = DistExchange(rank, world, n, g, wrap, group)
+
+    def post(self, buf):
+        import torch
+        import torch.distributed as dist
+        ex = self.inner
+        n, g = ex.n, ex.g
+        if ex.self_wrap or (ex.lo is None and ex.hi is None):
+            return ex.post(buf)
+        low, high = buf[g:2 * g].cpu(), buf[n:n + g].cpu()
+        rlo, rhi = torch.empty_like(low), torch.empty_like(high)
+        ops = []
+        if ex.lo is not None:
+            ops.append(dist.P2POp(dist.isend, low, ex.lo, tag=0))
+        if ex.hi is not None:
+            ops.append(dist.P2POp(dist.irecv, rhi, ex.hi, tag=0))
+        if ex.hi is not None:
+            ops.append(dist.P2POp(dist.isend, high, ex.hi, tag=1))
+        if ex.lo is not None:
+            ops.append(dist.P2POp(dist.irecv, rlo, ex.lo, tag=1))
+        for w in dist.batch_isend_irecv(ops):
+            w.wait()
+        if ex.lo is not None:
+            buf[0:g].copy_(rlo)
+        if ex.hi is not None:
+            buf[n + g:n + 2 * g].copy_(rhi)
+        return []
+
+
 # ----------------------------------------------------------------------------
 # launcher: --gpus N without torchrun re-executes through torch.distributed.run
 # ----------------------------------------------------------------------------
@@ -372,6 +408,11 @@ def main():
                          "the NCCL path: 797 vs 750 Gpts/s at world size 1, profiles/r02_slab_world1.txt; the "
                          "fused path exchanges every step)")
     ap.add_argument("--selftest-launch", action="store_true", help=argparse.SUPPRESS)
+    # test-only transport: N ranks share cuda:0 over gloo, ghost planes staged
+    # through host memory (NCCL refuses two ranks on one GPU) — exercises the
+    # whole multi-rank bench path (partition, exchange schedule, timing, the
+    # JSON line) on a one-GPU box
+    ap.add_argument("--test-transport", default=None, choices=["staged"], help=argparse.SUPPRESS)
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
     if args.halo_depth is None:
@@ -381,7 +422,7 @@ def main():
     # same launch line the driver uses), so `python bench.py --gpus N` is a
     # real N-process run; N = 1 runs in this process (the same code path)
     if args.gpus > 1 and "WORLD_SIZE" not in os.environ and args.impl == "ours":
-        if not args.selftest_launch:
+        if not args.selftest_launch and not args.test_transport:
             import torch
             have = torch.cuda.device_count()
             if have < args.gpus:
@@ -407,6 +448,11 @@ def main():
     sym, fused = None, None
     rank = env_int("RANK", 0)
     local = env_int("LOCAL_RANK", 0)
+    staged = args.test_transport == "staged"
+    if staged:
+        local = 0                                   # every rank on cuda:0 (test transport)
+        if args.halo == "fused":
+            raise SystemExit("bench.py: the staged test transport exchanges through host memory (no --halo fused)")
     if world != args.gpus:
         raise SystemExit(f"bench.py: --gpus {args.gpus} but the launch has WORLD_SIZE={world} ranks")
     if torch.cuda.device_count() <= local:
@@ -414,11 +460,21 @@ def main():
     torch.cuda.set_device(local)
     use_pg = world > 1 or (args.force_slab and "MASTER_ADDR" in os.environ)
     if use_pg:
-        os.environ.setdefault("NCCL_DEBUG", "INFO")        # communicator nranks in the log (stderr)
-        os.environ.setdefault("NCCL_DEBUG_FILE", "/dev/stderr")
-        dist.init_process_group("nccl", device_id=torch.device(f"cuda:{local}"))
+        if staged:
+            dist.init_process_group("gloo")
+        else:
+            os.environ.setdefault("NCCL_DEBUG", "INFO")        # communicator nranks in the log (stderr)
+            os.environ.setdefault("NCCL_DEBUG_FILE", "/dev/stderr")
+            dist.init_process_group("nccl", device_id=torch.device(f"cuda:{local}"))
         if dist.get_world_size() != args.gpus:
             raise SystemExit(f"bench.py: process group has {dist.get_world_size()} ranks, --gpus {args.gpus}")
+
+    def max_over_ranks(v: float) -> float:
+        if not use_pg:
+            return v
+        tt = torch.tensor([v], dtype=torch.float64, device="cpu" if staged else dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        return float(tt.item())
     dev = torch.device(f"cuda:{local}")
 
     w = si.workload(args.workload)
@@ -453,7 +509,8 @@ def main():
 
     if slabbed:
         sp = SlabPlan(gext, rank, world, spec.size, spec.pad_lo, list(spec.kind), spec.pad_value, spec.op,
-                      spec.weights, spec.params, device=local, depth=args.halo_depth)
+                      spec.weights, spec.params, device=local, depth=args.halo_depth,
+                      exchange_factory=HostStagedExchange if staged else None)
         plan = sp.plan
         host = [torch.from_numpy(x).pin_memory() for x in xs]
         bufs = []
@@ -625,11 +682,7 @@ def main():
             ev1.record(stream)
         barrier()
     t_ms = sum(a.elapsed_time(b) for a, b in pairs) if cold else ev0.elapsed_time(ev1)
-    t_max = t_ms
-    if use_pg:
-        tt = torch.tensor([t_ms], device=dev)
-        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
-        t_max = float(tt.item())
+    t_max = max_over_ranks(t_ms)
     ms_per_step = t_max / args.steps
     points = npts_local * world * steps_per_iter * sweeps * args.steps
     value = points / (t_max * 1e-3) / 1e9
@@ -684,9 +737,7 @@ def main():
                 sp._join(sp._on_comm(lambda: sp._post(exb)))
             x1.record(stream)
             barrier()
-            tt = torch.tensor([x0.elapsed_time(x1) / nrep], device=dev)
-            dist.all_reduce(tt, op=dist.ReduceOp.MAX)
-            ex_us = float(tt.item()) * 1e3
+            ex_us = max_over_ranks(x0.elapsed_time(x1) / nrep) * 1e3
         nvl_gbs = per_nb / (ex_us * 1e-6) / 1e9 if ex_us else None
         halo = {"path": args.halo, "depth_steps": k, "ghost_planes": sp.g, "grids_per_exchange": grids,
                 "neighbours": n_nb, "bytes_per_neighbour_per_exchange": per_nb,
@@ -739,10 +790,7 @@ def main():
             e2e_step()
         q1.record(stream)
         barrier()
-        te = q0.elapsed_time(q1)
-        tt = torch.tensor([te], device=dev)
-        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
-        te = float(tt.item()) / n_e2e
+        te = max_over_ranks(q0.elapsed_time(q1)) / n_e2e
         h2d = sum(int(x.numel()) * 4 for x in host)
         e2e = {"value": npts_local * world * steps_per_iter / (te * 1e-3) / 1e9, "unit": "Gpoints/s",
                "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": int(res_h.numel()) * 4, "ms_per_step": te,
