@@ -116,7 +116,15 @@ __device__ __forceinline__ float2 rcp_nr(float2 x) {
   const float2 e = vfma(make_float2(-x.x, -x.y), r, vbc<float2>(1.0f));
   return vfma(r, e, r);
 }
-__device__ __forceinline__ float clamp01(float c) { return c < 0.0f ? 0.0f : (c > 1.0f ? 1.0f : c); }
+// c clamped to [0, 1]; a NaN stays NaN (as the select form c < 0 ? 0 :
+// (c > 1 ? 1 : c) does): max.NaN / min.NaN, two FMNMX instead of a
+// compare-select chain
+__device__ __forceinline__ float clamp01(float c) {
+  float r;
+  asm("max.NaN.f32 %0, %1, 0f00000000;" : "=f"(r) : "f"(c));
+  asm("min.NaN.f32 %0, %0, 0f3F800000;" : "+f"(r));
+  return r;
+}
 __device__ __forceinline__ float2 clamp01(float2 c) { return make_float2(clamp01(c.x), clamp01(c.y)); }
 __device__ __forceinline__ float rsqrt_nr(float x) {
   float r;
