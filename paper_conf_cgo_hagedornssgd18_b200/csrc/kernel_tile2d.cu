@@ -507,8 +507,9 @@ __global__ void __launch_bounds__(NCONS + 32, MINB)
           });
           const float right = __shfl_down_sync(0xffffffffu, cr[cs_][0], 1);
           const float hcol = __shfl_sync(0xffffffffu, halo_c, k - 2);
-          cr[cs_][4] = lane == 31 ? hcol : right;
-          cr[cs_][4] = ce == 4 ? cr[cs_][4] : (ce == 3 ? cr[cs_][3] : (ce == 2 ? cr[cs_][2] : cr[cs_][1]));
+          float e4 = lane == 31 ? hcol : right;
+          if (ce != 4) e4 = ce == 3 ? cr[cs_][3] : (ce == 2 ? cr[cs_][2] : cr[cs_][1]);   // the grid's last column
+          cr[cs_][4] = e4;
         } else if constexpr (k >= 3) {
           // c row outside the grid: the remapped row (one or two above)
           const int d = crow - (int)pad_remap(crow, ny, ky);
