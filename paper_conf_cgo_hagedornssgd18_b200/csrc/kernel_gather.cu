@@ -123,10 +123,25 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
             for (int b = lane; b < ncopy; b += 32) cp_async4(dst + b, s0 + b);
           }
         } else {
-          for (int b = lane; b < T.bx; b += 32) {
-            const int64_t ix = remap_or_const(gxa + b, p.n[2], p.kind[2]);
-            if (ix < 0) dst[b] = p.pad_value;
-            else cp_async4(dst + b, in + o + ix);
+          // a tile touching the x edges: the in-grid columns [blo, bhi) of the
+          // row are copied like an interior row (16-byte pieces: gxa and nx are
+          // multiples of 4, so the range is quad-aligned), only the
+          // out-of-grid columns are remapped one by one
+          const int64_t nx = p.n[2];
+          const int blo = (int)(gxa < 0 ? -gxa : 0);
+          const int64_t hi_ = nx - gxa < (int64_t)T.bx ? nx - gxa : (int64_t)T.bx;
+          const int bhi = hi_ > blo ? (int)hi_ : blo;
+          const float* s0 = in + o + gxa;
+          if (quads) {
+            for (int b = blo + 4 * lane; b < bhi; b += 128) cp_async16(dst + b, s0 + b);
+          } else {
+            for (int b = blo + lane; b < bhi; b += 32) cp_async4(dst + b, s0 + b);
+          }
+          for (int b = lane; b < blo + (T.bx - bhi); b += 32) {
+            const int bb = b < blo ? b : bhi + (b - blo);
+            const int64_t ix = remap_or_const(gxa + bb, nx, p.kind[2]);
+            if (ix < 0) dst[bb] = p.pad_value;
+            else cp_async4(dst + bb, in + o + ix);
           }
         }
       } else {
