@@ -172,14 +172,24 @@ __device__ __forceinline__ void fill_box(const StencilParams& p, const Tile& T, 
 template <int SZ, int SY, int SX>
 __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__ StencilParams p, Tile T,
                                                       const float* __restrict__ in, float* __restrict__ out,
-                                                      int64_t ntz, int64_t nty, int64_t ntx, int nbuf) {
-  extern __shared__ __align__(16) float box[];
+                                                      int64_t ntz, int64_t nty, int64_t ntx, int nbuf,
+                                                      const __grid_constant__ CUtensorMap tmap, int use_tma) {
+  extern __shared__ __align__(128) float box[];
   __shared__ int toff[kMaxTaps];
+  __shared__ uint64_t tbar[2];
   pdl_launch_dependents();
   const int BYX = T.by * T.bx;
   const int box_floats = T.bz * BYX;
+  const int buf_floats = (box_floats + 31) & ~31;     // buffers 128-B aligned (TMA destinations)
   for (int t = threadIdx.x; t < p.ntaps; t += kThreads)
     toff[t] = p.tap[t][0] * BYX + p.tap[t][1] * T.bx + p.tap[t][2];
+  if (threadIdx.x == 0) {
+    mbar_init(&tbar[0], 1);
+    mbar_init(&tbar[1], 1);
+    fence_mbar_init();
+    if (use_tma) prefetch_tmap(&tmap);
+  }
+  __syncthreads();
   pdl_wait();
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t oz_n = p.reg1 - p.reg0, oy_n = p.o[1], ox_n = p.o[2];
@@ -196,13 +206,38 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
     oy0 = (int64_t)ty * T.oty;
     ox0 = (int64_t)tx * T.otx;
   };
+  // Interior boxes (every cell the outputs read inside the grid, so no pad)
+  // arrive as ONE TMA box load issued by one thread (use_tma: 16-B aligned
+  // rows, box dims <= 256); edge boxes are filled by the warps (fill_box).
+  // tma_mask / tma_phase: per buffer, whether its pending fill is a TMA load
+  // and the parity of its barrier.
+  unsigned tma_mask = 0u, tma_phase = 0u;      // bit b: buffer b (no local-memory arrays)
   auto fill = [&](int64_t tile, int buf) {
     int64_t oz0, oy0, ox0;
     origin(tile, oz0, oy0, ox0);
     // unpadded coordinates of the box origin (global z)
-    fill_box(p, T, in, box + buf * box_floats, p.z_off + oz0 * p.step[0] - p.lo[0], oy0 * p.step[1] - p.lo[1],
-             ox0 * p.step[2] - p.lo[2], warp, lane);
-    cp_async_commit();
+    const int64_t gz0 = p.z_off + oz0 * p.step[0] - p.lo[0], gy0 = oy0 * p.step[1] - p.lo[1];
+    const int64_t gx0 = ox0 * p.step[2] - p.lo[2];
+    const int64_t lz0 = gz0 - p.z_off + p.ghost;
+    const bool interior = use_tma && gx0 >= 0 && gx0 + T.wx <= p.n[2] && gy0 >= 0 && gy0 + T.by <= p.n[1] &&
+                          gz0 >= 0 && gz0 + T.bz <= p.gnz && lz0 >= 0 && lz0 + T.bz <= p.n[0] + 2 * p.ghost;
+    tma_mask = interior ? (tma_mask | (1u << buf)) : (tma_mask & ~(1u << buf));
+    if (interior) {
+      if (threadIdx.x == 0) {
+        fence_proxy_async_smem();     // the buffer's earlier generic-proxy accesses before the async-proxy write
+        mbar_arrive_expect_tx(&tbar[buf], (uint32_t)(box_floats * 4));
+        tma_load_3d(box + buf * buf_floats, &tmap, &tbar[buf], (int)(gx0 & ~(int64_t)3), (int)gy0, (int)lz0);
+      }
+    } else {
+      fill_box(p, T, in, box + buf * buf_floats, gz0, gy0, gx0, warp, lane);
+    }
+    cp_async_commit();                // (an empty group for a TMA fill keeps the group count per tile)
+  };
+  auto wait_tma = [&](int buf) {
+    if ((tma_mask >> buf) & 1u) {
+      mbar_wait(&tbar[buf], (tma_phase >> buf) & 1u);
+      tma_phase ^= 1u << buf;
+    }
   };
   // this thread's outputs within a tile (tile-invariant: no per-tile division):
   // k = tid + (pass * NJ + j) * kThreads, at most NP passes (nout <= NP*NJ*kThreads)
@@ -222,7 +257,7 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
   if ((int64_t)blockIdx.x < ntiles) fill(blockIdx.x, 0);
   for (int64_t tile = blockIdx.x; tile < ntiles; tile += gridDim.x) {
     const int64_t next = tile + gridDim.x;
-    float* bcur = box + cur * box_floats;
+    float* bcur = box + cur * buf_floats;
     if (nbuf == 2) {
       if (next < ntiles) fill(next, cur ^ 1);
       else cp_async_commit();
@@ -230,6 +265,7 @@ __global__ void __launch_bounds__(kThreads, 3) k5_gather(const __grid_constant__
     } else {
       cp_async_wait<0>();
     }
+    wait_tma(cur);
     __syncthreads();
     int64_t oz0, oy0, ox0;
     origin(tile, oz0, oy0, ox0);
@@ -353,7 +389,7 @@ struct Shape {
 
 // output tile per dimensionality: 3D (2, 4, 128), 2D (1, 16, 128), 1D (1, 1, 1024),
 // halved (largest first) until the box fits
-bool choose(const StencilParams& p, Tile* T) {
+bool choose(const StencilParams& p, Tile* T, bool tma = false) {
   const bool d3 = p.o[0] > 1 || p.size[0] > 1;
   const bool d2 = p.o[1] > 1 || p.size[1] > 1;
   // 3D: long box rows amortise the per-row work of the fill (measured on 512^3
@@ -367,10 +403,25 @@ bool choose(const StencilParams& p, Tile* T) {
       if (v == 3) s = Shape{4, 8, 32};
     }
   }
-  for (int it = 0; it < 16; ++it) {
+  // TMA boxes are at most 256 per dimension: narrower, taller tiles (3D
+  // (2, 8, 64), 2D (1, 32, 64)) — with the fill in one instruction there is no
+  // per-row cost to amortise
+  if (tma) {
+    if (d3) s = Shape{2, 8, 64};
+    else if (d2) s = Shape{1, 32, 64};
+    if (const char* e = getenv("LIFT_K5_TMA_SHAPE")) {   // A/B hook
+      const int v = atoi(e);
+      if (v == 1) s = d3 ? Shape{2, 4, 124} : Shape{1, 16, 124};
+      if (v == 2) s = d3 ? Shape{4, 8, 32} : Shape{1, 64, 32};
+      if (v == 3) s = d3 ? Shape{1, 16, 64} : Shape{1, 16, 64};
+      if (v == 4) s = d3 ? Shape{2, 16, 32} : Shape{1, 32, 32};
+    }
+  }
+  for (int it = 0; it < 24; ++it) {
     const Tile t = tile_of(p, s.otz, s.oty, s.otx);
+    const bool tma_fits = !tma || (t.bx <= 256 && t.by <= 256 && t.bz <= 256);
     if ((int64_t)t.bz * t.by * t.bx <= kMaxSmemFloats && s.otz * s.oty * s.otx <= NP * NJ * kThreads &&
-        t.bz * t.by <= kMaxRows) {
+        t.bz * t.by <= kMaxRows && tma_fits) {
       *T = t;
       return true;
     }
@@ -393,16 +444,32 @@ bool gather_supported(const StencilParams& p) {
 
 cudaError_t launch_gather(const StencilParams& p, const float* in0, float* out, cudaStream_t stream, int num_sms,
                           std::string* err) {
+  // TMA box fills for the interior tiles: 16-B aligned rows (nx % 4 == 0, an
+  // aligned base); LIFT_K5_TMA=0 keeps the cp.async fill everywhere (A/B)
+  // (measured, profiles/r02_k5_tma.txt: 2D windows and 3D windows of depth <= 2
+  // gain 36-62%; the 3x3x3 box is compute-bound and runs faster on the
+  // cp.async path's (2, 4, 128) tiles than on any TMA-sized tile)
+  const char* et = getenv("LIFT_K5_TMA");
+  const bool deep3d = (p.o[0] > 1 || p.size[0] > 1) && p.size[0] >= 3;
+  bool tma = !(et && et[0] == '0') && (!deep3d || (et && et[0] == '1')) && p.n[2] % 4 == 0 &&
+             (reinterpret_cast<uintptr_t>(in0) & 15u) == 0;
   Tile T;
-  if (!choose(p, &T)) {
-    *err = "gather: window box exceeds shared memory";
-    return cudaErrorInvalidConfiguration;
+  if (!(tma && choose(p, &T, true))) {
+    tma = false;
+    if (!choose(p, &T)) {
+      *err = "gather: window box exceeds shared memory";
+      return cudaErrorInvalidConfiguration;
+    }
   }
+  CUtensorMap tmap{};
+  if (tma && !encode_tensor_map_3d(&tmap, in0, p.n[2], p.n[1], p.n[0] + 2 * p.ghost, (uint32_t)T.bx, (uint32_t)T.by,
+                                   (uint32_t)T.bz, err))
+    return cudaErrorInvalidValue;
   const int64_t oz_n = p.reg1 - p.reg0;
   if (oz_n <= 0 || p.o[1] <= 0 || p.o[2] <= 0) return cudaSuccess;
   const int64_t ntz = (oz_n + T.otz - 1) / T.otz, nty = (p.o[1] + T.oty - 1) / T.oty;
   const int64_t ntx = (p.o[2] + T.otx - 1) / T.otx;
-  const size_t box_bytes = (size_t)T.bz * T.by * T.bx * sizeof(float);
+  const size_t box_bytes = (size_t)(((int64_t)T.bz * T.by * T.bx + 31) & ~31ll) * sizeof(float);
   const int nbuf = 2 * box_bytes <= (size_t)kMaxSmemFloats * 4 ? 2 : 1;
   const size_t smem = nbuf * box_bytes;
   // compile-time windows for the common shapes when every tap is non-zero
@@ -436,8 +503,9 @@ cudaError_t launch_gather(const StencilParams& p, const float* in0, float* out, 
   }
   if (grid > ntiles) grid = ntiles;
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
-  int nb = nbuf;
-  void* args[] = {(void*)&p, (void*)&T, (void*)&in0, (void*)&out, (void*)&ntz, (void*)&nty, (void*)&ntx, (void*)&nb};
+  int nb = nbuf, ut = tma ? 1 : 0;
+  void* args[] = {(void*)&p,   (void*)&T,   (void*)&in0, (void*)&out, (void*)&ntz,
+                  (void*)&nty, (void*)&ntx, (void*)&nb,  (void*)&tmap, (void*)&ut};
   return launch_kernel(fn, dim3((unsigned)grid), dim3(kThreads), args, smem, stream, !fz);
 }
 

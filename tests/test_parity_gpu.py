@@ -707,3 +707,33 @@ def test_resident3d_iterate(lift, monkeypatch, shape, kind, op):
         ref = orc.iterate(sp, xs, aux, 9)[0]
         Y = res["1"][0].astype(np.float64)
         assert np.max(np.abs(Y - ref) / np.maximum(np.abs(ref), 1e-30)) <= TOL10
+
+
+# --------------------------- K5 TMA box fill (interior tiles) ---------------
+K5_TMA_CASES = {
+    "2d_3x3_s2": ((260, 520), (3, 3), (2, 2), (1, 1), (1, 1), (MIRROR, CLAMP)),
+    "2d_5x5_s2": ((300, 1032), (5, 5), (2, 2), (2, 2), (2, 2), (REFLECT, WRAP)),
+    "2d_2x2_s2": ((256, 512), (2, 2), (2, 2), (0, 0), (1, 1), (CLAMP, CLAMP)),
+    "2d_4x3_s3x2": ((301, 516), (4, 3), (3, 2), (1, 1), (2, 1), (CONSTANT, MIRROR)),
+    "3d_2x2x2_s2": ((40, 72, 264), (2, 2, 2), (2, 2, 2), (0, 0, 0), (1, 1, 1), (CLAMP, WRAP, MIRROR)),
+    "3d_3x2x4_s1x2x2": ((20, 40, 520), (3, 2, 4), (1, 2, 2), (1, 0, 1), (1, 1, 2), (REFLECT, CLAMP, CONSTANT)),
+}
+
+
+@pytest.mark.parametrize("case", list(K5_TMA_CASES))
+def test_k5_tma_interior_tiles(lift, monkeypatch, case):
+    """K5 boxes fully inside the grid arrive as one TMA load, edge boxes
+    through the warps' cp.async fill: both are bitwise K0 and the cp.async-only
+    build (LIFT_K5_TMA=0), and match the oracle (grids several tiles wide,
+    nx % 4 == 0 so TMA applies; mixed pads; strided and asymmetric windows)."""
+    ext, size, step, lo, hi, kinds = K5_TMA_CASES[case]
+    w = np.random.default_rng(161).standard_normal(size).astype(np.float32)
+    sp = spec(ext, size, w, kinds, lo=lo, hi=hi, step=step, value=0.3)
+    xs = [rnd(ext, 162)]
+    y, plan = check(lift, sp, xs)
+    assert plan.last_variant == lift.plan.VARIANTS["gather"]
+    y0, _ = run_gpu(lift, sp, xs, "generic")
+    np.testing.assert_array_equal(y, y0)
+    monkeypatch.setenv("LIFT_K5_TMA", "0")
+    y1, _ = run_gpu(lift, sp, xs)
+    np.testing.assert_array_equal(y, y1)
