@@ -797,6 +797,8 @@ __global__ void __launch_bounds__(NCONS + 32, 2)
       const int nzc = (int)(min(zs + (int64_t)zc, p.reg1) - zs);
       const int xo = x0 - 4 + 4 * lane;                 // this lane's X_{t+1} / output columns
       const bool pl = xo == 0, pr = xo + 4 == nx;       // x-halo out of grid for this lane
+      // (clamp / mirror / reflect: the x = -1 / nx tap is one of the lane's
+      // own 4 values; a float4 element index, resolved by selects)
       // X rows (box origin y0-2) and X_{t+1} rows (tile origin y0-1) of this
       // warp's two rows, with the pad redirect folded into the row offsets
       int xm[2], xq[2], ym_[2], yq[2];
@@ -831,8 +833,10 @@ __global__ void __launch_bounds__(NCONS + 32, 2)
         if (++sn == S) { sn = 0; ++pn; }
         const int ys = i & 3;
         const bool inside = yz >= 0 && yz < gnz;
-        if (inside) {
-          // ---- step 1: X_{t+1} plane yz on the extended tile ----
+        {
+          // ---- step 1: X_{t+1} plane yz on the extended tile (computed for a
+          // plane outside the grid too — from the producer's remapped planes —
+          // and never read: its slot is aliased away below; no branch) ----
 #pragma unroll
           for (int jj = 0; jj < 2; ++jj) {
             const int rr = warp * 2 + jj;
@@ -874,13 +878,20 @@ __global__ void __launch_bounds__(NCONS + 32, 2)
         // ---- step 2: X_{t+2} plane oz = yz - 1 from X_{t+1} planes oz-1..oz+1 ----
         const int oz = yz - 1;
         // ring slots with the pad of X_{t+1} in z (a plane outside the grid
-        // aliases the remapped plane, which is one of the three)
+        // aliases the remapped plane, which is one of the three); interior
+        // planes (all but the first and last of the grid) take the fast path
+        if (oz >= 1 && oz + 1 < gnz) {
+          yslot[0] = yreal[0];
+          yslot[1] = yreal[1];
+          yslot[2] = yreal[2];
+        } else {
 #pragma unroll
-        for (int k = 0; k < 3; ++k) {
-          const int gzk = oz - 1 + k;
-          int src = k;
-          if (gzk < 0 || gzk >= gnz) src = (int)pad_remap(gzk, gnz, kz) - (oz - 1);
-          yslot[k] = (src == 0 ? yreal[0] : (src == 1 ? yreal[1] : yreal[2]));
+          for (int k = 0; k < 3; ++k) {
+            const int gzk = oz - 1 + k;
+            int src = k;
+            if (gzk < 0 || gzk >= gnz) src = (int)pad_remap(gzk, gnz, kz) - (oz - 1);
+            yslot[k] = (src == 0 ? yreal[0] : (src == 1 ? yreal[1] : yreal[2]));
+          }
         }
         float* op = out + ((int64_t)(oz - p.z_off) + p.ghost) * p.plane;
 #pragma unroll
