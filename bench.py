@@ -713,6 +713,7 @@ def main():
         alg_bytes = npts_local * bpp
     peak, peak_src = peaks()
     achieved = alg_bytes / avg_launch_s / 1e9
+    kernel_name = plan.last_kernel          # the kernel function the timed step launched (stencil_plan_last_kernel)
 
     # ---- halo exchange (slab path): bytes per rank, exchange time, NVLink fraction
     halo = None
@@ -838,8 +839,7 @@ def main():
             "hbm_gbs_per_gpu_whole_step": value * bpp / world,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": ncu_traffic(args.workload),
-                         "kernel": {0: "k0_generic", 1: "k1_tile", 2: "k2_sweep", 3: "k4_iterate", 4: "k5_gather",
-                                    5: "k6_resident"}[variant_id],
+                         "kernel": kernel_name,
                          "peak_source": peak_src,
                          "alg_bytes_per_launch": alg_bytes, "avg_launch_us": avg_launch_s * 1e6,
                          "frac_of_8TBs": achieved / 8000.0},

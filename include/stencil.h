@@ -186,6 +186,12 @@ stencil_status stencil_plan_set_pad_decay(stencil_plan plan, float decay);
 /* The family that ran the plan's most recent apply / iterate launch
  * (STENCIL_VARIANT_PERSIST3D after a K4 iterate; GENERIC before any launch). */
 int32_t stencil_plan_last_variant(stencil_plan plan);
+/* The kernel function of the plan's most recent launch within its family
+ * ("k2_sweep", "k2c_column", "k2t_sweep", "k1_tile", "k1_srad_fused",
+ * "k3_wsweep", "k5_gather", "k5_gather (TMA)", "k0_generic", "k4_iterate",
+ * "k6_resident"; "none" before any launch).  A static string owned by the
+ * library. */
+const char* stencil_plan_last_kernel(stencil_plan plan);
 
 /*
  * out = map(f, slide(pad(inputs))) — one application.

@@ -13,7 +13,8 @@ from ._lib import (StencilError, stencil_apply, stencil_apply_region, stencil_ap
                    stencil_last_error, stencil_plan_create, stencil_plan_destroy,
                    stencil_plan_output_extents, stencil_plan_set_slab, stencil_plan_set_time_block,
                    stencil_plan_set_variant, stencil_plan_time_block,
-                   stencil_plan_variant, stencil_plan_last_variant, stencil_plan_set_pad_decay,
+                   stencil_plan_variant, stencil_plan_last_variant, stencil_plan_last_kernel,
+                   stencil_plan_set_pad_decay,
                    stencil_run_host, stencil_status_string,
                    stencil_version)
 from .plan import Plan  # noqa: F401

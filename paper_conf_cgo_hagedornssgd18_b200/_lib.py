@@ -68,13 +68,14 @@ _set_wait_timeout = _sig("stencil_set_wait_timeout_ms", C.c_int, [C.c_uint32])
 _device_fault = _sig("stencil_device_fault", C.c_int, [])
 _run_host = _sig("stencil_run_host", C.c_int, [_P, _FPP, C.c_int32, _FPP, C.c_int32, C.c_int32, _P, _P])
 _destroy = _sig("stencil_plan_destroy", None, [_P])
+_last_kernel = _sig("stencil_plan_last_kernel", C.c_char_p, [_P])
 _status_string = _sig("stencil_status_string", C.c_char_p, [C.c_int])
 _last_error = _sig("stencil_last_error", C.c_char_p, [])
 _version = _sig("stencil_version", C.c_char_p, [])
 
 EXPORTED = ("stencil_plan_create", "stencil_plan_output_extents", "stencil_plan_set_slab",
             "stencil_plan_set_variant", "stencil_plan_variant", "stencil_plan_last_variant",
-            "stencil_plan_set_pad_decay",
+            "stencil_plan_set_pad_decay", "stencil_plan_last_kernel",
             "stencil_plan_set_time_block",
             "stencil_plan_time_block", "stencil_apply", "stencil_apply_region",
             "stencil_apply_region_put", "stencil_slab_step_fused", "stencil_wait_signals",
@@ -208,6 +209,10 @@ def stencil_iterate(plan: int, state: Sequence[int], aux: Sequence[int], n_steps
     _check(_iterate(plan, _ptrs(state), len(state), _ptrs(aux), len(aux), int(n_steps), C.c_void_p(int(stream)),
                     C.byref(ri)), "stencil_iterate")
     return ri.value
+
+
+def stencil_plan_last_kernel(plan: int) -> str:
+    return _last_kernel(plan).decode()
 
 
 def stencil_set_wait_timeout_ms(ms: int):

@@ -28,6 +28,7 @@ struct stencil_plan_s {
   int32_t forced_variant = STENCIL_VARIANT_AUTO;
   int32_t time_block = 1;          // stencil_iterate: time steps per pass where K2T applies (opt-in, see DESIGN)
   int32_t last_variant = STENCIL_VARIANT_GENERIC;
+  const char* last_kernel = "none";  // kernel function of the most recent launch (stencil_plan_last_kernel)
   // OP_SRAD: device workspace {2 x partials of the q0 reduction, q0 constants}
   void* srad_ws = nullptr;
   // OP_SRAD inside stencil_iterate: the fused pass left the statistics of the
@@ -211,6 +212,7 @@ stencil_status launch(stencil_plan_s* pl, const StencilParams& p_in, const float
       std::string err;
       int n_out = 0;
       cudaError_t e = launch_srad_fused(p, in0, out, stream, pl->num_sms, &err, &n_out);
+      pl->last_kernel = g_last_kernel;
       if (e != cudaSuccess)
         return fail(STENCIL_E_CUDA, std::string("kernel launch failed: ") + cudaGetErrorString(e) + " " + err);
       if (pl->srad_chain) {
@@ -227,6 +229,7 @@ stencil_status launch(stencil_plan_s* pl, const StencilParams& p_in, const float
   }
   std::string err;
   cudaError_t e;
+  set_last_kernel("none");
   switch (v) {
     case STENCIL_VARIANT_SWEEP3D:
       e = launch_sweep3d(p, in0, in1, out, stream, pl->num_sms, &err);
@@ -240,6 +243,7 @@ stencil_status launch(stencil_plan_s* pl, const StencilParams& p_in, const float
     default:
       e = launch_generic(p, in0, in1, out, stream, pl->num_sms);
   }
+  pl->last_kernel = g_last_kernel;
   if (e != cudaSuccess) {
     g_last_error = std::string("kernel launch failed: ") + cudaGetErrorString(e) + (err.empty() ? "" : " (" + err + ")");
     return STENCIL_E_CUDA;
@@ -508,6 +512,8 @@ int32_t stencil_plan_time_block(stencil_plan pl) {
 
 int32_t stencil_plan_last_variant(stencil_plan pl) { return pl ? pl->last_variant : -1; }
 
+const char* stencil_plan_last_kernel(stencil_plan pl) { return pl ? pl->last_kernel : "none"; }
+
 stencil_status stencil_plan_set_pad_decay(stencil_plan pl, float decay) {
   if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
   if (!(decay >= 0.0f && decay <= 1.0f)) return fail(STENCIL_E_INVALID, "pad decay must be in [0, 1]");
@@ -662,6 +668,7 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
     if (e != cudaSuccess)
       return fail(STENCIL_E_CUDA, std::string("K6 launch failed: ") + cudaGetErrorString(e) + " " + err);
     pl->last_variant = STENCIL_VARIANT_RESIDENT3D;
+    pl->last_kernel = g_last_kernel;
     if (result_index) *result_index = n_steps % 2;
     return STENCIL_OK;
   }
@@ -678,6 +685,7 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
     if (e != cudaSuccess)
       return fail(STENCIL_E_CUDA, std::string("K4 launch failed: ") + cudaGetErrorString(e) + " " + err);
     pl->last_variant = STENCIL_VARIANT_PERSIST3D;
+    pl->last_kernel = g_last_kernel;
     if (result_index) *result_index = n_steps % 2;
     return STENCIL_OK;
   }
@@ -693,6 +701,8 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
       for (; t + 2 <= n_steps; t += 2) {
         std::string err;
         cudaError_t e = launch_sweep3d_t2(p, state[ri], state[1 - ri], (cudaStream_t)stream, pl->num_sms, &err);
+        pl->last_kernel = g_last_kernel;
+        pl->last_variant = STENCIL_VARIANT_SWEEP3D;
         if (e != cudaSuccess)
           return fail(STENCIL_E_CUDA, std::string("K2T launch failed: ") + cudaGetErrorString(e) + " " + err);
         ri = 1 - ri;

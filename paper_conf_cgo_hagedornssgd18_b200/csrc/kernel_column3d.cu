@@ -236,6 +236,7 @@ cudaError_t launch_column3d(const StencilParams& p, const float* in0, const floa
                       (p.op == OP_HOTSPOT3D ? (size_t)TX * L.ty * nz * 4 : 0);
   int ntx_i = ntx;
   void* args[] = {(void*)&p, (void*)&map, (void*)&pwmap, (void*)&in0, (void*)&out, &ntx_i};
+  set_last_kernel("k2c_column");
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NT), args, smem, stream, true);
 }
 

@@ -506,6 +506,7 @@ cudaError_t launch_gather(const StencilParams& p, const float* in0, float* out, 
   int nb = nbuf, ut = tma ? 1 : 0;
   void* args[] = {(void*)&p,   (void*)&T,   (void*)&in0, (void*)&out, (void*)&ntz,
                   (void*)&nty, (void*)&ntx, (void*)&nb,  (void*)&tmap, (void*)&ut};
+  set_last_kernel(tma ? "k5_gather (TMA)" : "k5_gather");
   return launch_kernel(fn, dim3((unsigned)grid), dim3(kThreads), args, smem, stream, !fz);
 }
 

@@ -175,6 +175,7 @@ cudaError_t launch_generic(const StencilParams& p, const float* in0, const float
   if (blocks > cap) blocks = cap;
   const bool fz = p.put_lo || p.put_hi || p.fused_step || p.wait_lo || p.wait_hi;
   void* args[] = {(void*)&p, (void*)&in0, (void*)&in1, (void*)&out};
+  set_last_kernel("k0_generic");
   return launch_kernel(reinterpret_cast<const void*>(&k0_generic), dim3((unsigned)blocks), dim3(threads), args, 0,
                        stream, !fz);
 }

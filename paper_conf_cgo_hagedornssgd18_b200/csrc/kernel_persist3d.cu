@@ -259,6 +259,7 @@ cudaError_t launch_persist3d(const StencilParams& p, float* s0, float* s1, const
   at[0].val.cooperative = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
+  set_last_kernel("k4_iterate");
   return cudaLaunchKernelExC(&cfg, L.fn, args);
 }
 

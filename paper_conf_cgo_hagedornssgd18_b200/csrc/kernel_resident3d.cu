@@ -377,6 +377,7 @@ cudaError_t launch_resident3d(const StencilParams& p, float* s0, float* s1, cons
   at[0].val.cooperative = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
+  set_last_kernel("k6_resident");
   return cudaLaunchKernelExC(&cfg, L.fn, args);
 }
 

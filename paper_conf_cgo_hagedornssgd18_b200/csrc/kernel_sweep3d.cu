@@ -1174,6 +1174,7 @@ cudaError_t launch_sweep3d(const StencilParams& p, const float* in0, const float
     const char* e = getenv("LIFT_FUSED_PDL");
     return e && e[0] == '1';
   }();
+  set_last_kernel("k2_sweep");
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, !fz || fused_pdl);
 }
 
@@ -1223,6 +1224,7 @@ cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* ou
   int64_t grid = slots < items ? slots : items;
   int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk;
   void* args[] = {(void*)&p, (void*)&map, (void*)&out, &ntx_i, &nty_i, &zc_i, &nch_i};
+  set_last_kernel("k2t_sweep");
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, true);
 }
 

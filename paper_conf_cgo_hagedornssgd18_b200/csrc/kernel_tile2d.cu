@@ -716,6 +716,7 @@ cudaError_t launch_srad_fused(const StencilParams& p, const float* in0, float* o
   }
   if (nparts_out) *nparts_out = (int)grid;
   void* args[] = {(void*)&p, (void*)&m0, (void*)&in0, (void*)&out, (void*)&ntx, (void*)&nty};
+  set_last_kernel("k1_srad_fused");
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, true);
 }
 
@@ -767,6 +768,7 @@ cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float*
   if (grid > ntiles) grid = ntiles;
   const float* s1 = L.nin > 1 ? in1 : in0;
   void* args[] = {(void*)&p, (void*)&m0, (void*)&m1, (void*)&in0, (void*)&s1, (void*)&out, (void*)&ntx, (void*)&nty};
+  set_last_kernel("k1_tile");
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(NCONS + 32), args, (size_t)L.smem, stream, true);
 }
 

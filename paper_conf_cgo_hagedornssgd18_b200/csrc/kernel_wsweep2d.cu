@@ -579,6 +579,7 @@ cudaError_t launch_wsweep2d(const StencilParams& p, const float* in0, const floa
   if (grid > need) grid = need;
   int ns = nstrips, hci = (int)hc, ni = (int)nitems;
   void* args[] = {(void*)&p, (void*)&m0, (void*)&m1, (void*)&in0, (void*)&s1, (void*)&out, &ns, &hci, &ni};
+  set_last_kernel("k3_wsweep");
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(L.wpc * 32), args, (size_t)L.smem, stream, true);
 }
 

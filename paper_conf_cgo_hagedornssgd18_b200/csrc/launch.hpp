@@ -23,6 +23,11 @@ inline bool pdl_enabled() {
   return on;
 }
 
+// The kernel function the calling thread's most recent launch used (for
+// stencil_plan_last_kernel: which kernel of a family ran, e.g. K2 or K2C).
+inline thread_local const char* g_last_kernel = "none";
+inline void set_last_kernel(const char* name) { g_last_kernel = name; }
+
 inline cudaError_t launch_kernel(const void* fn, dim3 grid, dim3 block, void** args, size_t smem,
                                  cudaStream_t stream, bool pdl) {
   cudaLaunchConfig_t cfg{};

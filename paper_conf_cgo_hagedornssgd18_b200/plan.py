@@ -106,6 +106,11 @@ class Plan:
         return L.stencil_plan_variant(self.handle)
 
     @property
+    def last_kernel(self) -> str:
+        """Kernel function of the most recent launch (e.g. 'k2_sweep', 'k2c_column')."""
+        return L.stencil_plan_last_kernel(self.handle)
+
+    @property
     def last_variant(self) -> int:
         """Kernel family of the most recent apply / iterate launch."""
         return L.stencil_plan_last_variant(self.handle)

@@ -737,3 +737,26 @@ def test_k5_tma_interior_tiles(lift, monkeypatch, case):
     monkeypatch.setenv("LIFT_K5_TMA", "0")
     y1, _ = run_gpu(lift, sp, xs)
     np.testing.assert_array_equal(y, y1)
+
+
+def test_last_kernel_names(lift, monkeypatch):
+    """stencil_plan_last_kernel names the kernel function within a family."""
+    T = rnd((8, 64, 132), 171, 300.0, 350.0)
+    P = rnd(T.shape, 172, 0.0, 1e-2)
+    sp = spec(T.shape, 3, op=si.HOTSPOT3D, params=si.params_hotspot3d())
+    y, plan = run_gpu(lift, sp, [T, P])
+    assert plan.last_kernel == "k2c_column"
+    monkeypatch.setenv("LIFT_K2C", "0")
+    y, plan = run_gpu(lift, sp, [T, P])
+    assert plan.last_kernel == "k2_sweep"
+    x = rnd((40, 48, 136), 173)
+    y, plan = run_gpu(lift, spec(x.shape, 3, si.weights_j3d7()), [x])
+    assert plan.last_kernel == "k2_sweep"
+    y, plan = run_gpu(lift, spec(x.shape, 3, si.weights_j3d7()), [x], "generic")
+    assert plan.last_kernel == "k0_generic"
+    x2 = rnd((260, 520), 174)
+    y, plan = run_gpu(lift, spec(x2.shape, (3, 3), np.ones((3, 3), np.float32) / 9, step=(2, 2)), [x2])
+    assert plan.last_kernel == "k5_gather (TMA)"
+    I = np.exp(rnd((150, 388), 175, 0.0, 1.0)).astype(np.float32)
+    y, plan = run_gpu(lift, spec(I.shape, 3, op=si.SRAD, params=si.params_srad2()), [I])
+    assert plan.last_kernel == "k1_srad_fused"
