@@ -171,6 +171,18 @@ DEEP_CASES = {
     "acoustic13": lambda: (si.StencilSpec((48, 36, 132), (5,) * 3, (1,) * 3, (2,) * 3, (2,) * 3,
                                           (si.CONSTANT,) * 3, 0.0, si.ACOUSTIC, None, si.params_acoustic(13)),
                            [si.uniform((48, 36, 132), 98, -1, 1), si.uniform((48, 36, 132), 99, -1, 1)], []),
+    # a 5x5x5 box (K5 gather tiles) and an odd-width 3x3x3 box (K0 rows / K5):
+    # the regions reaching into the ghosts on the non-TMA kernel families
+    "box5_k5": lambda: (si.StencilSpec((48, 20, 36), (5,) * 3, (1,) * 3, (2,) * 3, (2,) * 3, (si.REFLECT,) * 3, 0.0,
+                                       si.WEIGHTED, (np.random.default_rng(5).random((5, 5, 5)) / 125).astype(np.float32),
+                                       ()), [si.uniform((48, 20, 36), 102)], []),
+    "box3_odd_width": lambda: (si.StencilSpec((40, 24, 37), (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.WRAP,) * 3, 0.0,
+                                              si.WEIGHTED, (np.random.default_rng(6).random((3, 3, 3)) / 27).astype(
+                                                  np.float32), ()), [si.uniform((40, 24, 37), 103)], []),
+    # Acoustic on an odd width runs on K0 (one thread per output)
+    "acoustic7_k0": lambda: (si.StencilSpec((40, 20, 37), (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.CONSTANT,) * 3,
+                                            0.0, si.ACOUSTIC, None, si.params_acoustic(7)),
+                             [si.uniform((40, 20, 37), 104, -1, 1), si.uniform((40, 20, 37), 105, -1, 1)], []),
     "hotspot3d": lambda: (si.StencilSpec((40, 64, 128), (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.CLAMP,) * 3,
                                          0.0, si.HOTSPOT3D, None, si.params_hotspot3d()),
                           [si.uniform((40, 64, 128), 100, 300, 350)], [si.uniform((40, 64, 128), 101, 0, 0.01)]),
