@@ -1194,6 +1194,7 @@ bool sweep3d_t2_supported(const StencilParams& p) {
 
 cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* out, cudaStream_t stream, int num_sms,
                               std::string* err) {
+  if (sweep3d_r2_supported(p)) return launch_sweep3d_r2(p, in, out, stream, num_sms, err);
   const int64_t nz_reg = p.reg1 - p.reg0;
   if (nz_reg <= 0) return cudaSuccess;
   constexpr int S = 5;

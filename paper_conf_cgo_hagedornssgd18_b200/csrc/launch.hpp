@@ -76,6 +76,13 @@ bool sweep3d_t2_supported(const StencilParams& p);
 cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* out, cudaStream_t stream, int num_sms,
                               std::string* err);
 
+// K2R — two weighted 7-point steps per pass with X_{t+1} in registers
+// (temporal blocking; x/y CLAMP/MIRROR/REFLECT, z CLAMP/MIRROR); the K2T
+// entry point routes eligible plans here.
+bool sweep3d_r2_supported(const StencilParams& p);
+cudaError_t launch_sweep3d_r2(const StencilParams& p, const float* in, float* out, cudaStream_t stream, int num_sms,
+                              std::string* err);
+
 // K1 — 2D TMA halo-tile kernel (weighted box r<=4, srad1, srad2).
 bool tile2d_supported(const StencilParams& p);
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,

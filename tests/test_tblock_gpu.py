@@ -1,0 +1,130 @@
+"""K2R — two weighted 7-point steps per pass with X_{t+1} in registers
+(temporal blocking; tiling preserves semantics, PAPER.md
+P:771-791): bitwise equal to single steps and within the iterate tolerance of
+the fp64 oracle, over tile / chunk / boundary cases.
+
+Tiles are 128 columns x 8*RPW rows (RPW = 8 by default; LIFT_K2R_SHAPE=4/6
+picks the other instantiations), z-chunks are chosen by the launcher
+(LIFT_K2R_ZC / LIFT_K2R_ZC2 force them: every chunk boundary recomputes two
+X_{t+1} planes).
+"""
+import os
+
+import numpy as np
+import pytest
+import torch
+
+import stencil_inputs as si
+from oracle import stencil_oracle as orc
+from stencil_inputs import CLAMP, MIRROR, REFLECT, WRAP
+
+pytestmark = pytest.mark.gpu
+
+TOL10 = 1e-4
+
+
+@pytest.fixture(scope="module")
+def lift():
+    import __graft_entry__
+    __graft_entry__.build()
+    import paper_conf_cgo_hagedornssgd18_b200 as m
+    torch.cuda.set_device(0)
+    return m
+
+
+def rnd(shape, seed):
+    return np.random.default_rng(seed).uniform(0.5, 1.5, size=shape).astype(np.float32)
+
+
+def spec(extents, kind):
+    kind = (kind,) * 3 if isinstance(kind, int) else tuple(kind)
+    return si.StencilSpec(tuple(extents), (3, 3, 3), (1, 1, 1), (1, 1, 1), (1, 1, 1), kind, 0.0,
+                          si.WEIGHTED, si.f32(si.weights_j3d7()), ())
+
+
+def run(lift, sp, x, steps, tb, env=None):
+    old = {}
+    for k, v in (env or {}).items():
+        old[k] = os.environ.get(k)
+        os.environ[k] = v
+    try:
+        plan = lift.Plan.from_spec(sp)
+        plan.set_time_block(tb)
+        a = torch.from_numpy(x).cuda()
+        b = torch.empty_like(a)
+        ri = plan.iterate([a, b], steps)
+        torch.cuda.synchronize()
+        return (a, b)[ri].cpu().numpy(), plan
+    finally:
+        for k, v in old.items():
+            if v is None:
+                os.environ.pop(k, None)
+            else:
+                os.environ[k] = v
+
+
+SHAPES = [(37, 70, 260), (3, 15, 124), (1, 14, 120), (2, 129, 244), (40, 8, 516), (5, 1, 128),
+          (4, 2, 132), (9, 65, 128), (6, 64, 256), (17, 130, 388), (2, 3, 4)]
+
+
+@pytest.mark.parametrize("kind", [CLAMP, MIRROR, (CLAMP, REFLECT, REFLECT), (MIRROR, CLAMP, REFLECT),
+                                  (CLAMP, MIRROR, CLAMP)])
+@pytest.mark.parametrize("shape", SHAPES)
+def test_k2r_bitwise_equal_single_steps(lift, kind, shape):
+    x = rnd(shape, 70)
+    sp = spec(shape, kind)
+    y1, _ = run(lift, sp, x, 6, 1)
+    y2, plan = run(lift, sp, x, 6, 2)
+    assert plan.time_block == 2
+    assert plan.last_kernel == "k2r_sweep"
+    np.testing.assert_array_equal(y2, y1)
+
+
+@pytest.mark.parametrize("rpw", ["4", "6", "8"])
+@pytest.mark.parametrize("zc", [("1", "0"), ("2", "0"), ("3", "1"), ("5", "2"), ("64", "0")])
+def test_k2r_shapes_and_chunks(lift, rpw, zc):
+    shape = (23, 70, 260)
+    x = rnd(shape, 71)
+    for kind in (CLAMP, (MIRROR, REFLECT, MIRROR)):
+        sp = spec(shape, kind)
+        y1, _ = run(lift, sp, x, 4, 1)
+        y2, plan = run(lift, sp, x, 4, 2, {"LIFT_K2R_SHAPE": rpw, "LIFT_K2R_ZC": zc[0], "LIFT_K2R_ZC2": zc[1]})
+        assert plan.last_kernel == "k2r_sweep"
+        np.testing.assert_array_equal(y2, y1)
+
+
+def test_k2r_odd_steps_vs_oracle(lift):
+    shape = (19, 37, 132)
+    x = rnd(shape, 72)
+    sp = spec(shape, CLAMP)
+    y2, _ = run(lift, sp, x, 7, 2)            # three K2R passes + one single step
+    ref = orc.iterate(sp, [x], [], 7)[0]
+    assert np.max(np.abs(y2 - ref) / np.abs(ref)) <= TOL10
+    y1, _ = run(lift, sp, x, 7, 1)
+    np.testing.assert_array_equal(y2, y1)
+
+
+def test_k2r_not_taken(lift):
+    """z REFLECT (the out-of-grid X_{t+1} plane is not the edge plane) keeps
+    the shared-memory two-step kernel; WRAP keeps single steps."""
+    shape = (12, 20, 128)
+    x = rnd(shape, 73)
+    sp = spec(shape, (REFLECT, CLAMP, CLAMP))
+    y2, plan = run(lift, sp, x, 4, 2)
+    assert plan.last_kernel == "k2t_sweep"
+    y1, _ = run(lift, sp, x, 4, 1)
+    np.testing.assert_array_equal(y2, y1)
+    sp = spec(shape, WRAP)
+    plan = lift.Plan.from_spec(sp)
+    plan.set_time_block(2)
+    assert plan.time_block == 1
+
+
+def test_k2r_j3d7_512_sampled(lift):
+    """BASELINE C3 size (512^3, clamp), 10 steps as 5 K2R passes: bitwise equal
+    to single steps over the whole grid."""
+    xs, sp = si.make_workload_inputs(si.workload("j3d7_512_clamp"))
+    y1, _ = run(lift, sp, xs[0], 10, 1)
+    y2, plan = run(lift, sp, xs[0], 10, 2)
+    assert plan.last_kernel == "k2r_sweep"
+    assert np.array_equal(y2, y1)
