@@ -138,20 +138,23 @@ __device__ __forceinline__ ItemGeom item_geom(const StencilParams& p, int item, 
 }
 
 // One X_t plane step of a warp: X_{t+1}(q) on its RPW+2 rows, then the
-// X_{t+2} accumulators.  YE: the warp's rows touch a y boundary.
-template <int RPW, bool YE>
+// X_{t+2} accumulators.  YE: the warp's rows touch a y boundary.  RAG: x = nx
+// falls inside the tile (nx % 128 != 0; the lane holding column nx-1 is not
+// lane 31).
+template <int RPW, bool YE, bool RAG>
 __device__ __forceinline__ void plane_step(const StencilParams& p, const float* __restrict__ Pm,
                                            const float* __restrict__ Pc, const float* __restrict__ Pp, int lane,
                                            int rb0, int lcol, int rcol, bool useR, int hofs_c, int hofs_m,
                                            int hofs_p, int hofs_xm, int hofs_xp, int jlo, int jhi, int ylo_src,
-                                           int yhi_src, bool ragged, bool pr, int rex,
+                                           int yhi_src, bool pr, int rex,
                                            float4 (&accA)[RPW], float4 (&accB)[RPW], bool fin_prev, bool mid,
                                            bool first_plane, bool top_plane, float* oprev, float* ocur,
                                            int row_ok, int rowp) {
   constexpr int J = RPW + 2;
   const float* w = p.wbox;
   // ---- halo columns x0-1 (lanes 0..J-1) and x0+128 (lanes 16..16+J-1) ----
-  const float hv = star7(w, Pm[hofs_c], Pc[hofs_m], Pc[hofs_xm], Pc[hofs_c], Pc[hofs_xp], Pc[hofs_p], Pp[hofs_c]);
+  const float hcen = Pc[hofs_c];      // X_t at the halo column (lane 0 / 31's outer x tap of step 1)
+  const float hv = star7(w, Pm[hofs_c], Pc[hofs_m], Pc[hofs_xm], hcen, Pc[hofs_xp], Pc[hofs_p], Pp[hofs_c]);
   float h[J];
 #pragma unroll
   for (int j = 0; j < J; ++j) h[j] = __shfl_sync(RX_FULL, hv, lane < 16 ? j : 16 + j);
@@ -165,10 +168,17 @@ __device__ __forceinline__ void plane_step(const StencilParams& p, const float* 
     const float4 rnext = lds4(Pc, br + 1, lane);
     float l = __shfl_up_sync(RX_FULL, rcur.w, 1);
     float r = __shfl_down_sync(RX_FULL, rcur.x, 1);
-    const float le = Pc[br * RX_BX + lcol];
-    const float re = Pc[br * RX_BX + rcol];
-    if (lane == 0) l = le;
-    if (useR) r = re;
+    if constexpr (RAG) {
+      const float le = Pc[br * RX_BX + lcol];
+      const float re = Pc[br * RX_BX + rcol];
+      if (lane == 0) l = le;
+      if (useR) r = re;
+    } else {
+      // lanes 0 / 31: X_t at the halo columns, from the halo lanes of row j
+      const float e = __shfl_sync(RX_FULL, hcen, lane < 16 ? j : 16 + j);
+      l = lane == 0 ? e : l;
+      r = lane == 31 ? e : r;
+    }
     const float4 zm = lds4(Pm, br, lane);
     const float4 zp = lds4(Pp, br, lane);
     float4 ym = rprev, yp = rnext;
@@ -242,7 +252,7 @@ __device__ __forceinline__ void plane_step(const StencilParams& p, const float* 
       // the remapped column, so the pad of X_{t+1} in x costs nothing here)
       l = lane == 0 ? h[i + 1] : l;
       r = lane == 31 ? h[i + 1] : r;
-      if (ragged) r = pr ? pick4r(rex, c) : r;     // nx % 128 != 0: x = nx inside the tile
+      if constexpr (RAG) r = pr ? pick4r(rex, c) : r;     // x = nx inside the tile
       const float4 ym = s1[i], yp = s1[i + 2];
       float4 a;
       a.x = __fmaf_rn(w10, ym.x, accB[i].x);
@@ -380,6 +390,7 @@ __global__ void __launch_bounds__(nthreads_r<NW, WS>(), 1)
     const int ylo_src = (int)pad_remap(-1, ny, ky);                   // row of y = -1 (0 or 1)
     const int yhi_src = (int)(ny - 1 - pad_remap(ny, ny, ky));        // y = ny is row ny-1-yhi_src
     const int rb0 = warp * RPW;                  // box row of gy = yw - 2
+    const uint32_t full_a = smem_u32(full), empty_a = smem_u32(empty);
     int sn = 0;
     uint32_t pn = 0;
     float4 accA[RPW], accB[RPW];
@@ -446,30 +457,33 @@ __global__ void __launch_bounds__(nthreads_r<NW, WS>(), 1)
       mbar_wait(&full[sn], pn & 1);
       int xs1 = sn;
       if (++sn == S) { sn = 0; ++pn; }
+      float* oprev = obase + (int64_t)(g.qa - 1) * plane;     // output plane q-1
       for (int q = (int)g.qa; q <= (int)g.qb; ++q) {
-        mbar_wait(&full[sn], pn & 1);
+        mbar_wait_a(full_a + 8 * sn, pn & 1);
         const int xs2 = sn;
         if (++sn == S) { sn = 0; ++pn; }
         const bool fin_prev = q - 1 >= g.gzs;
         const bool mid = q >= g.gzs && q < g.gze;
         const bool first_plane = q == 0, top_plane = q == gnz - 1;
-        float* oprev = obase + (int64_t)(q - 1) * plane;
-        float* ocur = oprev + plane;
         const float* Pm = dsm + xs0 * SF;
         const float* Pc = dsm + xs1 * SF;
         const float* Pp = dsm + xs2 * SF;
-        if (yedge) {
-          plane_step<RPW, true>(p, Pm, Pc, Pp, lane, rb0, lcol, rcol, useR, hofs_c, hofs_m, hofs_p, hofs_xm,
-                                hofs_xp, jlo, jhi, ylo_src, yhi_src, ragged, pr, rex, accA, accB,
-                                fin_prev, mid, first_plane, top_plane, oprev, ocur, rows_store, nx);
+#define K2R_STEP(YE, RAG)                                                                                    \
+  plane_step<RPW, YE, RAG>(p, Pm, Pc, Pp, lane, rb0, lcol, rcol, useR, hofs_c, hofs_m, hofs_p, hofs_xm, hofs_xp, \
+                           jlo, jhi, ylo_src, yhi_src, pr, rex, accA, accB, fin_prev, mid, first_plane, top_plane, \
+                           oprev, oprev + plane, rows_store, nx)
+        if (ragged) {
+          if (yedge) K2R_STEP(true, true);
+          else K2R_STEP(false, true);
         } else {
-          plane_step<RPW, false>(p, Pm, Pc, Pp, lane, rb0, lcol, rcol, useR, hofs_c, hofs_m, hofs_p, hofs_xm,
-                                 hofs_xp, jlo, jhi, ylo_src, yhi_src, ragged, pr, rex, accA, accB,
-                                 fin_prev, mid, first_plane, top_plane, oprev, ocur, rows_store, nx);
+          if (yedge) K2R_STEP(true, false);
+          else K2R_STEP(false, false);
         }
+#undef K2R_STEP
+        oprev += plane;
         // X_t plane q-1 is done
         __syncwarp();
-        if (lane == 0) mbar_arrive(&empty[xs0]);
+        if (lane == 0) mbar_arrive_a(empty_a + 8 * xs0);
         xs0 = xs1;
         xs1 = xs2;
       }
