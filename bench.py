@@ -73,14 +73,19 @@ def peaks():
     return 6650.0, "fallback (B200_PROFILING.md)"
 
 
-def ncu_traffic(workload):
-    """dram bytes per launch of the dominant kernel from the committed ncu capture."""
+def ncu_traffic(workload, kernel=None):
+    """dram bytes per launch of the dominant kernel from the committed ncu capture
+    (the entry "workload:kernel" when the step's kernel has its own capture)."""
     p = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     if not os.path.exists(p):
         return None
     with open(p) as f:
         d = json.load(f)
-    v = d.get(workload)
+    v = d.get(f"{workload}:{kernel}") if kernel else None
+    if v is None:
+        v = d.get(workload)
+        if v is not None and kernel and kernel not in v.get("kernel", kernel):
+            return None          # the capture is of another kernel
     return None if v is None else v.get("dram_bytes_per_launch")
 
 
@@ -394,6 +399,9 @@ def main():
     ap.add_argument("--no-flush", action="store_true",
                     help="L2-resident workloads: time L2-warm back-to-back sweeps instead of cold flushed steps")
     ap.add_argument("--no-graph", action="store_true", help="launch single sweeps eagerly instead of a CUDA graph")
+    ap.add_argument("--time-block", type=int, default=0, choices=[0, 1, 2],
+                    help="iterate time steps per pass: 0 = AUTO (two where the register two-step kernel K2R "
+                         "applies), 1 = single steps, 2 = two steps where K2R/K2T apply")
     ap.add_argument("--scaling", default="weak", choices=["weak", "strong"],
                     help="multi-GPU iterated sweeps: weak = the single-GPU grid per rank (default), "
                          "strong = the single-GPU grid split over the ranks")
@@ -525,6 +533,7 @@ def main():
             bufs.append(b)
     else:
         plan = lift.Plan.from_spec(spec, device=local)
+        plan.set_time_block(args.time_block)
         host = [torch.from_numpy(x).pin_memory() for x in xs]
         bufs = [x.to(dev, non_blocking=True) for x in host]
     torch.cuda.synchronize()
@@ -557,6 +566,9 @@ def main():
     else:
         out = plan.empty_output()
         launches_per_step = 1
+    tb = plan.time_block if (iterable and not slabbed) else 1     # time steps per launch (K2R / K2T: 2)
+    if tb == 2:
+        launches_per_step = steps_per_iter // 2 + steps_per_iter % 2
     # a bench step of a single-sweep workload is a CUDA graph of `sweeps` full
     # sweeps (each reads the whole input and writes the whole output): small
     # grids (J2D5 256^2) take microseconds per sweep, so one graph launch per
@@ -812,6 +824,7 @@ def main():
             "config": {"workload": args.workload, "extents_per_gpu": list(spec.extents),
                        "global_extents": list(gext) if slabbed else list(ext1),
                        "time_steps_per_bench_step": steps_per_iter if iterable else 1,
+                       "time_steps_per_pass": tb,
                        "sweeps_per_bench_step": steps_per_iter if iterable else sweeps,
                        "op": si.OP_NAMES[op], "boundary": [si.KIND_NAMES[k] for k in spec.kind],
                        "window": list(spec.size),
@@ -836,10 +849,12 @@ def main():
                                    5: "K6 shared-memory-resident iterate (cooperative)"}[variant_id],
                        "launch": (f"cuda graph replay ({launches_per_step} launches per graph)" if graph is not None
                                   else "stream launches")},
-            "hbm_gbs_per_gpu_whole_step": value * bpp / world,
+            "hbm_gbs_per_gpu_whole_step": value * bpp / tb / world,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                         "frac": achieved / peak, "traffic": ncu_traffic(args.workload),
+                         "frac": achieved / peak, "traffic": ncu_traffic(args.workload, kernel_name),
                          "kernel": kernel_name,
+                         "time_steps_per_launch": tb,
+                         "single_step_roofline_gpts": peak / bpp,
                          "peak_source": peak_src,
                          "alg_bytes_per_launch": alg_bytes, "avg_launch_us": avg_launch_s * 1e6,
                          "frac_of_8TBs": achieved / 8000.0},

@@ -164,13 +164,17 @@ stencil_status stencil_plan_output_extents(stencil_plan plan, int64_t* out_exten
 stencil_status stencil_plan_set_slab(stencil_plan plan, int64_t z_offset,
                                      int64_t global_n0, int32_t ghost);
 
-/* Temporal blocking for stencil_iterate: 2 lets iterate
- * advance two time steps per pass over HBM where the TMA sweep's two-step
- * kernel applies (WEIGHTED 7-point star, CLAMP/MIRROR/REFLECT); the result is
- * bitwise identical to single steps.  1 (default) takes one step per pass:
- * on B200 the single-step sweep already reaches ~0.9 of the HBM roofline and
- * the two-step kernel is instruction-bound.
- * stencil_plan_time_block returns the steps per pass iterate will use. */
+/* Temporal blocking for stencil_iterate (overlapped tiling
+ * applied to iterate): steps = 2 lets iterate
+ * advance two time steps per pass over HBM where a two-step kernel applies
+ * (WEIGHTED 7-point star; K2R with X_{t+1} in registers for x/y CLAMP /
+ * MIRROR / REFLECT and z CLAMP / MIRROR, else the shared-memory K2T for z
+ * REFLECT); the result is bitwise identical to single steps (an odd step
+ * count ends with one single step).  1 forces one step per pass.  0 (the
+ * default, AUTO) takes two steps per pass exactly where K2R applies (J3D7
+ * 512^3: ~1.5x the single-step rate).  Returns
+ * STENCIL_E_INVALID for steps outside 0..2.  stencil_plan_time_block returns
+ * the steps per pass iterate will use (1 or 2). */
 stencil_status stencil_plan_set_time_block(stencil_plan plan, int32_t steps);
 int32_t stencil_plan_time_block(stencil_plan plan);
 

@@ -26,7 +26,7 @@ struct stencil_plan_s {
   StencilParams p{};
   int64_t user_out_ext[3] = {0, 0, 0};
   int32_t forced_variant = STENCIL_VARIANT_AUTO;
-  int32_t time_block = 1;          // stencil_iterate: time steps per pass where K2T applies (opt-in, see DESIGN)
+  int32_t time_block = 0;          // stencil_iterate steps per pass: 0 AUTO (2 where K2R applies), 1, 2
   int32_t last_variant = STENCIL_VARIANT_GENERIC;
   const char* last_kernel = "none";  // kernel function of the most recent launch (stencil_plan_last_kernel)
   // OP_SRAD: device workspace {2 x partials of the q0 reduction, q0 constants}
@@ -500,13 +500,14 @@ stencil_status stencil_plan_set_variant(stencil_plan pl, int32_t variant) {
 
 stencil_status stencil_plan_set_time_block(stencil_plan pl, int32_t steps) {
   if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
-  if (steps != 1 && steps != 2) return fail(STENCIL_E_INVALID, "time block must be 1 or 2");
+  if (steps < 0 || steps > 2) return fail(STENCIL_E_INVALID, "time block must be 0 (auto), 1 or 2");
   pl->time_block = steps;
   return STENCIL_OK;
 }
 
 int32_t stencil_plan_time_block(stencil_plan pl) {
   if (!pl) return -1;
+  if (pl->time_block == 0) return (pl->ndim == 3 && sweep3d_r2_supported(pl->p)) ? 2 : 1;
   return (pl->time_block >= 2 && sweep3d_t2_supported(pl->p)) ? 2 : 1;
 }
 
@@ -654,9 +655,10 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
   if (!state || n_state != 2) return fail(STENCIL_E_INVALID, "iterate needs 2 state buffers");
   if (!state[0] || !state[1] || state[0] == state[1]) return fail(STENCIL_E_INVALID, "bad state buffers");
   int ri = (p.op == OP_ACOUSTIC) ? 1 : 0;
+  const int32_t tb = stencil_plan_time_block(pl);     // steps per pass (K2R / K2T when 2)
   // few-plane 3D grids that fit in the device's shared memory: all steps in
   // one cooperative launch with the grid resident on chip (K6)
-  if ((p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D) && n_steps >= 2 && pl->ndim == 3 && pl->time_block < 2 &&
+  if ((p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D) && n_steps >= 2 && pl->ndim == 3 && pl->time_block != 2 &&
       pl->forced_variant == STENCIL_VARIANT_AUTO &&
       (p.op == OP_WEIGHTED ? n_aux == 0 : (n_aux == 1 && aux && aux[0])) &&
       resident3d_supported(p, state[0], state[1], p.op == OP_HOTSPOT3D ? aux[0] : nullptr, pl->num_sms)) {
@@ -673,7 +675,7 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
     return STENCIL_OK;
   }
   // small L2-resident 3D grids: all steps in one persistent launch (K4)
-  if ((p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D) && n_steps >= 2 && pl->ndim == 3 && pl->time_block < 2 &&
+  if ((p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D) && n_steps >= 2 && pl->ndim == 3 && pl->time_block != 2 &&
       pl->forced_variant == STENCIL_VARIANT_AUTO &&
       (p.op == OP_WEIGHTED ? n_aux == 0 : (n_aux == 1 && aux && aux[0])) &&
       persist3d_supported(p, state[0], state[1], p.op == OP_HOTSPOT3D ? aux[0] : nullptr)) {
@@ -693,7 +695,7 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
     if (n_aux != 0) return fail(STENCIL_E_INVALID, "WEIGHTED/GRADIENT/SRAD iterate takes no aux grids");
     int t = 0;
     // temporal blocking: two steps per pass (K2T) while at least two remain
-    if (pl->time_block >= 2 && n_steps >= 2 && sweep3d_t2_supported(p) &&
+    if (tb >= 2 && n_steps >= 2 &&
         (pl->forced_variant == STENCIL_VARIANT_AUTO || pl->forced_variant == STENCIL_VARIANT_SWEEP3D) &&
         aligned16(state[0]) && aligned16(state[1])) {
       DeviceGuard g(pl->device);

@@ -24,7 +24,7 @@ out = {}
 for wl in WORKLOADS:
     w = si.workload(wl)
     npts = int(np.prod(w.spec.out_extents()))
-    kern = "regex:k1_srad|k1_tile|k2_sweep|k2c_column|k2t|k0_generic|k3_wsweep|k4_iterate|k6_resident|k5_gather"
+    kern = "regex:k1_srad|k1_tile|k2_sweep|k2c_column|k2t|k2r|k0_generic|k3_wsweep|k4_iterate|k6_resident|k5_gather"
     skip = "6" if w.steps > 1 else "2"     # single sweeps: 3 warm-up + 1 timed launch
     cmd = ["ncu", "--metrics", "dram__bytes_read.sum,dram__bytes_write.sum,gpu__time_duration.sum",
            "--clock-control", "none", "-k", kern, "-s", skip, "-c", "2", "--csv",
