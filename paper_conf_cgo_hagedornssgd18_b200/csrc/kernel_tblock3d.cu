@@ -68,17 +68,23 @@ constexpr int smem_r() {
   return S * CfgR<RPW, NW>::STAGE_FLOATS * 4 + 2 * S * 8 + S * 4 + 64;
 }
 
-// the weighted 7-point star in op_weighted's tap order (w = the dense 3x3x3
-// window: z-1 = 4, y-1 = 10, x-1 = 12, centre 13, x+1 = 14, y+1 = 16, z+1 = 22)
-__device__ __forceinline__ float star7(const float* w, float zm, float ym, float xl, float c, float xr, float yp,
+// the 7 star weights of the dense 3x3x3 window, held in registers for the
+// whole launch (z-1 = 4, y-1 = 10, x-1 = 12, centre 13, x+1 = 14, y+1 = 16,
+// z+1 = 22)
+struct W7 {
+  float zm, ym, xl, c, xr, yp, zp;
+};
+
+// the weighted 7-point star in op_weighted's tap order
+__device__ __forceinline__ float star7(const W7& w, float zm, float ym, float xl, float c, float xr, float yp,
                                        float zp) {
-  float a = __fmaf_rn(w[4], zm, 0.0f);
-  a = __fmaf_rn(w[10], ym, a);
-  a = __fmaf_rn(w[12], xl, a);
-  a = __fmaf_rn(w[13], c, a);
-  a = __fmaf_rn(w[14], xr, a);
-  a = __fmaf_rn(w[16], yp, a);
-  return __fmaf_rn(w[22], zp, a);
+  float a = __fmaf_rn(w.zm, zm, 0.0f);
+  a = __fmaf_rn(w.ym, ym, a);
+  a = __fmaf_rn(w.xl, xl, a);
+  a = __fmaf_rn(w.c, c, a);
+  a = __fmaf_rn(w.xr, xr, a);
+  a = __fmaf_rn(w.yp, yp, a);
+  return __fmaf_rn(w.zp, zp, a);
 }
 
 __device__ __forceinline__ float4 lds4(const float* base, int row, int lane) {
@@ -142,7 +148,7 @@ __device__ __forceinline__ ItemGeom item_geom(const StencilParams& p, int item, 
 // falls inside the tile (nx % 128 != 0; the lane holding column nx-1 is not
 // lane 31).
 template <int RPW, bool YE, bool RAG>
-__device__ __forceinline__ void plane_step(const StencilParams& p, const float* __restrict__ Pm,
+__device__ __forceinline__ void plane_step(const W7& w, const float* __restrict__ Pm,
                                            const float* __restrict__ Pc, const float* __restrict__ Pp, int lane,
                                            int rb0, int lcol, int rcol, bool useR, int hofs_c, int hofs_m,
                                            int hofs_p, int hofs_xm, int hofs_xp, int jlo, int jhi, int ylo_src,
@@ -151,7 +157,6 @@ __device__ __forceinline__ void plane_step(const StencilParams& p, const float* 
                                            bool first_plane, bool top_plane, float* oprev, float* ocur,
                                            int row_ok, int rowp) {
   constexpr int J = RPW + 2;
-  const float* w = p.wbox;
   // ---- halo columns x0-1 (lanes 0..J-1) and x0+128 (lanes 16..16+J-1) ----
   const float hcen = Pc[hofs_c];      // X_t at the halo column (lane 0 / 31's outer x tap of step 1)
   const float hv = star7(w, Pm[hofs_c], Pc[hofs_m], Pc[hofs_xm], hcen, Pc[hofs_xp], Pc[hofs_p], Pp[hofs_c]);
@@ -218,7 +223,7 @@ __device__ __forceinline__ void plane_step(const StencilParams& p, const float* 
     });
   }
   // ---- X_{t+2}: finish plane q-1, accumulate plane q, start plane q+1 ----
-  const float w4 = w[4], w22 = w[22];
+  const float w4 = w.zm, w22 = w.zp;
   if (fin_prev) {
     float* op = oprev;
 #pragma unroll
@@ -242,7 +247,7 @@ __device__ __forceinline__ void plane_step(const StencilParams& p, const float* 
         accB[i].w = __fmaf_rn(w4, s1[i + 1].w, 0.0f);
       }
     }
-    const float w10 = w[10], w12 = w[12], w13 = w[13], w14 = w[14], w16 = w[16];
+    const float w10 = w.ym, w12 = w.xl, w13 = w.c, w14 = w.xr, w16 = w.yp;
 #pragma unroll
     for (int i = 0; i < RPW; ++i) {
       const float4 c = s1[i + 1];
@@ -391,6 +396,7 @@ __global__ void __launch_bounds__(nthreads_r<NW, WS>(), 1)
     const int yhi_src = (int)(ny - 1 - pad_remap(ny, ny, ky));        // y = ny is row ny-1-yhi_src
     const int rb0 = warp * RPW;                  // box row of gy = yw - 2
     const uint32_t full_a = smem_u32(full), empty_a = smem_u32(empty);
+    const W7 w7{p.wbox[4], p.wbox[10], p.wbox[12], p.wbox[13], p.wbox[14], p.wbox[16], p.wbox[22]};
     int sn = 0;
     uint32_t pn = 0;
     float4 accA[RPW], accB[RPW];
@@ -447,6 +453,7 @@ __global__ void __launch_bounds__(nthreads_r<NW, WS>(), 1)
         hofs_xp = hr * RX_BX + hxp;
       }
       const int row_ok = min(RPW, ny - yw);      // output rows of this warp inside the grid
+      const bool idle = yw - 1 >= ny;
       const bool col_ok = xo < nx;
       const int rows_store = col_ok ? row_ok : 0;
       const int64_t plane = p.plane;
@@ -465,11 +472,18 @@ __global__ void __launch_bounds__(nthreads_r<NW, WS>(), 1)
         const bool fin_prev = q - 1 >= g.gzs;
         const bool mid = q >= g.gzs && q < g.gze;
         const bool first_plane = q == 0, top_plane = q == gnz - 1;
+        if (idle) {            // every row of this warp is outside the grid (ragged last tile row)
+          __syncwarp();
+          if (lane == 0) mbar_arrive_a(empty_a + 8 * xs0);
+          xs0 = xs1;
+          xs1 = xs2;
+          continue;
+        }
         const float* Pm = dsm + xs0 * SF;
         const float* Pc = dsm + xs1 * SF;
         const float* Pp = dsm + xs2 * SF;
 #define K2R_STEP(YE, RAG)                                                                                    \
-  plane_step<RPW, YE, RAG>(p, Pm, Pc, Pp, lane, rb0, lcol, rcol, useR, hofs_c, hofs_m, hofs_p, hofs_xm, hofs_xp, \
+  plane_step<RPW, YE, RAG>(w7, Pm, Pc, Pp, lane, rb0, lcol, rcol, useR, hofs_c, hofs_m, hofs_p, hofs_xm, hofs_xp, \
                            jlo, jhi, ylo_src, yhi_src, pr, rex, accA, accB, fin_prev, mid, first_plane, top_plane, \
                            oprev, oprev + plane, rows_store, nx)
         if (ragged) {
@@ -534,6 +548,8 @@ LauncherR pick_r() {
   if (v == 8) return get_launcher_r<8, 8, 5, false>();
   if (v == 104) return get_launcher_r<4, 8, 6, true>();
   if (v == 108) return get_launcher_r<8, 8, 5, true>();
+  if (v == 1086) return get_launcher_r<8, 8, 6, true>();
+  if (v == 1064) return get_launcher_r<6, 8, 4, true>();
   if (v == 204) return get_launcher_r<4, 16, 5, true>();
   if (v == 203) return get_launcher_r<3, 16, 6, true>();
   return get_launcher_r<6, 8, 6, true>();
@@ -566,18 +582,30 @@ cudaError_t launch_sweep3d_r2(const StencilParams& p, const float* in, float* ou
   const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);
   const int64_t tiles = (int64_t)ntx * nty;
   const int64_t slots = (int64_t)num_sms * L.ctas_per_sm;
-  // chunks: ~6 items per CTA of at least 8 planes (each chunk recomputes 2
-  // X_{t+1} planes), the last ~2 waves in short chunks (guided tail)
+  // z-chunks (items are (chunk, tile), chunk-major): long chunks of zc planes
+  // (each chunk recomputes 2 X_{t+1} planes and refills the ring), then ~2
+  // waves of items in short chunks of zc2 planes so the launch's tail is
+  // short.  Measured on J3D7 512^3 (profiles/r02_k2r_chunks.txt): (128, 16),
+  // (112, 16), (64, 16) and (48, 8) all ~1290 Gpts/s; pairs whose long items
+  // leave a partial wave of long items after the whole waves lost up to 17%
+  // ((64, 8) 1096, (96, 16) 1078), and so did plans with < 2 long items per
+  // CTA and no short tail ((160, -) 1106) or 4-plane tails (1200-1240).
+  // LIFT_K2R_ZC / LIFT_K2R_ZC2 override the pair.
   const int64_t work = nz_reg * tiles;
-  int64_t zc = (work + 6 * slots - 1) / (6 * slots);
-  if (zc < 8) zc = 8;
-  int64_t want2 = 4;
-  if (const char* e = getenv("LIFT_K2R_ZC")) zc = std::max<int64_t>(1, atoll(e));
-  if (const char* e = getenv("LIFT_K2R_ZC2")) want2 = std::max<int64_t>(0, atoll(e));
+  const char* ez = getenv("LIFT_K2R_ZC");
+  const char* ez2 = getenv("LIFT_K2R_ZC2");
+  int64_t zc = std::min<int64_t>(128, std::max<int64_t>(16, nz_reg / 4));
+  int64_t want2 = 16;
+  if (work < 16 * slots) {       // small grids: ~6 items per CTA
+    zc = std::max<int64_t>(4, (work + 6 * slots - 1) / (6 * slots));
+    want2 = 0;
+  }
+  if (ez) zc = std::max<int64_t>(1, atoll(ez));
+  if (ez2) want2 = std::max<int64_t>(0, atoll(ez2));
   if (zc > nz_reg) zc = nz_reg;
   int64_t nchunk = (nz_reg + zc - 1) / zc;
   int64_t n1 = nchunk, zc2 = zc;
-  if (want2 > 0 && want2 < zc && work >= 16 * slots) {
+  if (want2 > 0 && want2 < zc) {
     const int64_t nsmall = (2 * slots + tiles - 1) / tiles;     // short chunks per tile column
     const int64_t z2 = nsmall * want2;
     if (z2 < nz_reg) {
