@@ -547,6 +547,9 @@ def main():
     if iterable:
         if op == si.ACOUSTIC:
             state = [bufs[0], bufs[1]]          # prev, cur
+            if not slabbed and args.time_block != 1:
+                # two spare grids: two steps per pass where K2RA applies
+                state += [torch.empty_like(bufs[0]), torch.empty_like(bufs[0])]
             aux = []
         elif op == si.HOTSPOT3D:
             state = [bufs[0], sym[1] if (slabbed and fused is not None) else torch.empty_like(bufs[0])]
@@ -627,6 +630,10 @@ def main():
     # sweep per step; the hot number (graph of back-to-back sweeps, L2-warm)
     # is reported beside it as "hot"
     bpp = BYTES_PER_POINT[op]
+    # algorithmic bytes of one launch: a two-step Acoustic pass (K2RA) reads
+    # u^{n-1}, u^n and writes u^{n+1}, u^{n+2}; a two-step weighted pass (K2R)
+    # reads X_t and writes X_{t+2}
+    bpp_launch = 16 if (tb == 2 and op == si.ACOUSTIC) else bpp
     cold = (not slabbed) and npts_local * bpp < 2 * L2_BYTES and not args.no_flush
     hot = None
     if cold:
@@ -708,7 +715,7 @@ def main():
         if persist:   # K4 / K6: one launch per bench step runs all time steps; time per time step
             units = args.steps * steps_per_iter
         avg_launch_s = (t_ms * 1e-3) / units
-        alg_bytes = npts_local * bpp
+        alg_bytes = npts_local * bpp_launch
     else:
         # time the owned-slab sweep alone (all planes in one launch) on this rank
         e0 = torch.cuda.Event(enable_timing=True)
@@ -849,7 +856,7 @@ def main():
                                    5: "K6 shared-memory-resident iterate (cooperative)"}[variant_id],
                        "launch": (f"cuda graph replay ({launches_per_step} launches per graph)" if graph is not None
                                   else "stream launches")},
-            "hbm_gbs_per_gpu_whole_step": value * bpp / tb / world,
+            "hbm_gbs_per_gpu_whole_step": value * bpp_launch / tb / world,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": ncu_traffic(args.workload, kernel_name),
                          "kernel": kernel_name,

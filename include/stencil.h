@@ -172,7 +172,8 @@ stencil_status stencil_plan_set_slab(stencil_plan plan, int64_t z_offset,
  * REFLECT); the result is bitwise identical to single steps (an odd step
  * count ends with one single step).  1 forces one step per pass.  0 (the
  * default, AUTO) takes two steps per pass exactly where K2R applies (J3D7
- * 512^3: ~1.5x the single-step rate).  Returns
+ * 512^3: ~1.5x the single-step rate), and for ACOUSTIC with
+ * zero padding where K2RA applies (iterate with four state buffers).  Returns
  * STENCIL_E_INVALID for steps outside 0..2.  stencil_plan_time_block returns
  * the steps per pass iterate will use (1 or 2). */
 stencil_status stencil_plan_set_time_block(stencil_plan plan, int32_t steps);
@@ -286,7 +287,15 @@ stencil_status stencil_device_fault(void);
  *     reduces those instead of re-reading the image; only the first pass
  *     reads X0 once more for its q0)
  *   ACOUSTIC  : state {prev, cur}         next overwrites prev; roles swap
- * *result_index receives the index into ``state`` holding the newest grid.
+ *     or {prev, cur, spare, spare} (n_state 4, four distinct grids): where
+ *     the two-step kernel K2RA applies (zero padding, 7/13-point, not a slab,
+ *     time block 0 or 2) each pass reads prev and cur once and writes
+ *     u^{n+1} and u^{n+2} into the other pair (16 B per point for two steps
+ *     instead of 24), bitwise equal to single steps; an odd remainder runs
+ *     one single step.  The grid before the newest is state[*result_index ^ 1].
+ * *result_index receives the index into ``state`` holding the newest grid
+ * (with two-step passes not necessarily n_steps % 2).  n_state must be 2
+ * (ACOUSTIC: 2 or 4), else E_INVALID.
  * Requires output extents == input extents.
  */
 stencil_status stencil_iterate(stencil_plan plan, float* const* state, int32_t n_state,

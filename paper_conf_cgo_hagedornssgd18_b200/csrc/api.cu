@@ -10,6 +10,7 @@
 #include <mutex>
 #include <new>
 #include <string>
+#include <utility>
 #include <vector>
 
 #include "../../include/stencil.h"
@@ -507,8 +508,11 @@ stencil_status stencil_plan_set_time_block(stencil_plan pl, int32_t steps) {
 
 int32_t stencil_plan_time_block(stencil_plan pl) {
   if (!pl) return -1;
-  if (pl->time_block == 0) return (pl->ndim == 3 && sweep3d_r2_supported(pl->p)) ? 2 : 1;
-  return (pl->time_block >= 2 && sweep3d_t2_supported(pl->p)) ? 2 : 1;
+  if (pl->time_block == 0)
+    return (pl->ndim == 3 && (sweep3d_r2_supported(pl->p) || acoustic_r2_auto(pl->p))) ? 2 : 1;
+  return (pl->time_block >= 2 && pl->ndim == 3 && (sweep3d_t2_supported(pl->p) || acoustic_r2_supported(pl->p)))
+             ? 2
+             : 1;
 }
 
 int32_t stencil_plan_last_variant(stencil_plan pl) { return pl ? pl->last_variant : -1; }
@@ -652,8 +656,13 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
   const StencilParams& p = pl->p;
   if (!same_extents(p)) return fail(STENCIL_E_INVALID, "iterate needs output extents == input extents");
   if (n_steps < 0) return fail(STENCIL_E_INVALID, "n_steps < 0");
-  if (!state || n_state != 2) return fail(STENCIL_E_INVALID, "iterate needs 2 state buffers");
-  if (!state[0] || !state[1] || state[0] == state[1]) return fail(STENCIL_E_INVALID, "bad state buffers");
+  if (!state || !(n_state == 2 || (n_state == 4 && p.op == OP_ACOUSTIC)))
+    return fail(STENCIL_E_INVALID, "iterate needs 2 state buffers (ACOUSTIC: 2 or 4)");
+  for (int i = 0; i < n_state; ++i) {
+    if (!state[i]) return fail(STENCIL_E_INVALID, "bad state buffers");
+    for (int k = 0; k < i; ++k)
+      if (state[k] == state[i]) return fail(STENCIL_E_INVALID, "bad state buffers");
+  }
   int ri = (p.op == OP_ACOUSTIC) ? 1 : 0;
   const int32_t tb = stencil_plan_time_block(pl);     // steps per pass (K2R / K2T when 2)
   // few-plane 3D grids that fit in the device's shared memory: all steps in
@@ -738,14 +747,35 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
     }
   } else if (p.op == OP_ACOUSTIC) {
     if (n_aux != 0) return fail(STENCIL_E_INVALID, "ACOUSTIC iterate takes no aux grids");
-    // state {prev, cur}: next overwrites prev, then roles swap (A21)
-    for (int t = 0; t < n_steps; ++t) {
-      const int prev = 1 - ri;
-      const float* in[2] = {state[prev], state[ri]};
-      stencil_status s = stencil_apply(pl, in, 2, state[prev], stream);
-      if (s != STENCIL_OK) return s;
-      ri = prev;
+    // state {prev, cur} (+ two spare grids): (a, b) = (prev, cur)
+    int a = 0, b = 1, t = 0;
+    if (n_state == 4 && tb == 2 && n_steps >= 2 && pl->ndim == 3 && acoustic_r2_supported(p) &&
+        (pl->forced_variant == STENCIL_VARIANT_AUTO || pl->forced_variant == STENCIL_VARIANT_SWEEP3D) &&
+        aligned16(state[0]) && aligned16(state[1]) && aligned16(state[2]) && aligned16(state[3])) {
+      // K2RA: two steps per pass, (prev, cur) -> (u^{n+1}, u^{n+2}) in the spare pair
+      DeviceGuard g(pl->device);
+      if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+      int c = 2, d = 3;
+      for (; t + 2 <= n_steps; t += 2) {
+        std::string err;
+        cudaError_t e = launch_acoustic_r2(p, state[a], state[b], state[c], state[d], (cudaStream_t)stream,
+                                           pl->num_sms, &err);
+        pl->last_kernel = g_last_kernel;
+        pl->last_variant = STENCIL_VARIANT_SWEEP3D;
+        if (e != cudaSuccess)
+          return fail(STENCIL_E_CUDA, std::string("K2RA launch failed: ") + cudaGetErrorString(e) + " " + err);
+        std::swap(a, c);
+        std::swap(b, d);
+      }
     }
+    // single steps: next overwrites prev, then roles swap (A21)
+    for (; t < n_steps; ++t) {
+      const float* in[2] = {state[a], state[b]};
+      stencil_status s = stencil_apply(pl, in, 2, state[a], stream);
+      if (s != STENCIL_OK) return s;
+      std::swap(a, b);
+    }
+    ri = b;
   } else {
     return fail(STENCIL_E_UNSUPPORTED, "iterate is built for WEIGHTED, HOTSPOT3D/2D, GRADIENT and ACOUSTIC");
   }
@@ -792,11 +822,13 @@ stencil_status stencil_run_host(stencil_plan pl, const float* const* host_state,
   const bool iterable = (p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D || p.op == OP_ACOUSTIC ||
                          p.op == OP_HOTSPOT2D || p.op == OP_GRADIENT || p.op == OP_SRAD) && same_extents(p);
   if (iterable && (p.op != OP_ACOUSTIC || n_state == 2)) {
-    // WEIGHTED/HOTSPOT3D: state {X, scratch}; ACOUSTIC: state {prev, cur}
-    float* state[2] = {pl->ws[0], pl->ws[1]};
+    // WEIGHTED/HOTSPOT3D: state {X, scratch}; ACOUSTIC: state {prev, cur} plus
+    // the two other workspace grids (two steps per pass where K2RA applies)
+    float* state[4] = {pl->ws[0], pl->ws[1], pl->ws[2], pl->ws[3]};
     const float* aux[1] = {pl->ws[2]};
     int32_t ri = 0;
-    stencil_status s = stencil_iterate(pl, state, 2, aux, n_aux, n_steps, stream, &ri);
+    const int ns = p.op == OP_ACOUSTIC ? 4 : 2;
+    stencil_status s = stencil_iterate(pl, state, ns, aux, n_aux, n_steps, stream, &ri);
     if (s != STENCIL_OK) return s;
     result = state[ri];
   } else {

@@ -516,6 +516,453 @@ __global__ void __launch_bounds__(nthreads_r<NW, WS>(), 1)
   }
 }
 
+// ---------------------------------------------------------------------------
+// K2RA: two Acoustic time steps per pass (Listing 3; iterate
+// rotation A21), X_{t+1} in registers — the K2R design for the leapfrog update
+//   u^{n+1} = combine(star sum of u^n, u^n centre, u^{n-1}, K)
+// with zero padding (CONSTANT 0: every grid, u^{n+1} included, is 0 outside).
+// A pass reads u^{n-1} (point-wise, "P") and u^n (slid, "C") and writes
+// u^{n+1} and u^{n+2}: 16 B per point for two steps instead of 24.  The star
+// sum's tap order (z-R .. z-1, in-plane y/x, z+1 .. z+R) lets u^{n+2}'s sum be
+// accumulated across planes like K2R's weighted sum; u^{n+2}'s centre and
+// "previous" terms are X1 = u^{n+1} of its own plane (kept for R planes in
+// registers) and u^n of its plane (still in the C ring).  Planes outside the
+// grid are zero planes (TMA out-of-bounds fill for C; X1 forced to 0), so the
+// operation sequence is exactly two single steps' (bitwise equal, tested).
+// ---------------------------------------------------------------------------
+template <int R, int RPW>
+struct CfgA {
+  static constexpr int TY = 8 * RPW;
+  static constexpr int J = RPW + 2 * R;               // X1 rows per warp
+  static constexpr int BYC = TY + 4 * R;              // u^n rows y0-2R ..
+  static constexpr int BYP = TY + 2 * R;              // u^{n-1} rows y0-R ..
+  static constexpr int C_BYTES = RX_BX * BYC * 4;
+  static constexpr int P_BYTES = RX_BX * BYP * 4;
+  static constexpr int SFC = ((C_BYTES + 127) / 128) * 128 / 4;
+  static constexpr int SFP = ((P_BYTES + 127) / 128) * 128 / 4;
+};
+template <int R, int RPW, int S, int SP>
+constexpr int smem_a() {
+  return S * CfgA<R, RPW>::SFC * 4 + SP * CfgA<R, RPW>::SFP * 4 + (2 * S + 2 * SP) * 8 + S * 4 + 64;
+}
+
+struct AcConst {
+  float l2, c0;          // lambda^2, 2 - lambda^2 * 6R (the interior K)
+  const float* prm;
+};
+
+// u^{n+1} from the ordered star sum (FAST: K = 6R, cf1 = cf2 = 1; the same
+// operations as acoustic_combine, whose product by cf1 = 1 is exact)
+template <int R, bool FAST>
+__device__ __forceinline__ float ac_comb(const AcConst& a, float s, float uc, float prev, int K) {
+  if constexpr (FAST) {
+    float t = __fmul_rn(a.c0, uc);
+    t = __fmaf_rn(a.l2, s, t);
+    return __fmaf_rn(-1.0f, prev, t);
+  } else {
+    return acoustic_combine<R>(s, uc, prev, K, a.prm);
+  }
+}
+
+// K's y part for global row gy, z part for plane gz (in-domain neighbours)
+template <int R>
+__device__ __forceinline__ int ac_k1(int g, int n) {
+  int k = 0;
+#pragma unroll
+  for (int o = 1; o <= R; ++o) k += (g - o >= 0) + (g + o < n);
+  return k;
+}
+
+__device__ __forceinline__ float f4e(const float4& v, int e) {
+  return e == 0 ? v.x : (e == 1 ? v.y : (e == 2 ? v.z : v.w));
+}
+__device__ __forceinline__ void f4s(float4& v, int e, float x) {
+  if (e == 0) v.x = x;
+  else if (e == 1) v.y = x;
+  else if (e == 2) v.z = x;
+  else v.w = x;
+}
+
+// One X1 plane of a warp.  Cq[k] = u^n stage of plane q-R+k (k = 0..2R),
+// Pq = u^{n-1} stage of plane q.  EDGE: K per element and zero outside the
+// grid (y / x / ragged); otherwise every point of the warp is interior.
+template <int R, int RPW, bool EDGE>
+__device__ __forceinline__ void ac_plane(const AcConst& a, const float* const (&Cq)[2 * R + 1],
+                                         const float* __restrict__ Pq, int lane, int rb0, int hofs, int hpofs,
+                                         int hK, bool hin, bool qin, int kzq, int kzo, int yw, int ny, int kxp,
+                                         bool colin, float4 (&acc)[R][RPW], float4 (&hist)[R][RPW], bool st1,
+                                         bool fin, bool newacc, float* o1, float* o2, int row_ok, int rowp) {
+  constexpr int J = RPW + 2 * R;
+  // ---- halo lanes: X1 at columns x0-R+k (lanes k*J+j) and x0+128+k (16+k*J+j) ----
+  float hcen, hv;
+  {
+    const float* c = Cq[R];
+    hcen = c[hofs];
+    float sh = Cq[0][hofs];
+#pragma unroll
+    for (int k = 1; k < R; ++k) sh = __fadd_rn(sh, Cq[k][hofs]);
+#pragma unroll
+    for (int k = R; k >= 1; --k) sh = __fadd_rn(sh, c[hofs - k * RX_BX]);
+#pragma unroll
+    for (int k = R; k >= 1; --k) sh = __fadd_rn(sh, c[hofs - k]);
+#pragma unroll
+    for (int k = 1; k <= R; ++k) sh = __fadd_rn(sh, c[hofs + k]);
+#pragma unroll
+    for (int k = 1; k <= R; ++k) sh = __fadd_rn(sh, c[hofs + k * RX_BX]);
+#pragma unroll
+    for (int k = R + 1; k <= 2 * R; ++k) sh = __fadd_rn(sh, Cq[k][hofs]);
+    hv = acoustic_combine<R>(sh, hcen, Pq[hpofs], hK, a.prm);
+    if (!(hin && qin)) hv = 0.0f;
+  }
+  // ---- X1(q) rows j = 0..J-1 (gy = yw-R+j; u^n box row rb0+R+j; u^{n-1} box row rb0+j) ----
+  float4 s1[J];
+  float4 win[2 * R + 1];                 // u^n rows br-R .. br+R of plane q
+#pragma unroll
+  for (int k = 0; k < 2 * R; ++k) win[k] = lds4(Cq[R], rb0 + k, lane);
+#pragma unroll
+  for (int j = 0; j < J; ++j) {
+    const int br = rb0 + R + j;
+    win[2 * R] = lds4(Cq[R], br + R, lane);
+    const float4 c = win[R];
+    float xw[4 + 2 * R];
+    xw[R + 0] = c.x; xw[R + 1] = c.y; xw[R + 2] = c.z; xw[R + 3] = c.w;
+    // in-row neighbours: adjacent lanes; lanes 0 / 31 from the halo lanes' u^n
+#pragma unroll
+    for (int k = 0; k < R; ++k) {
+      const float e = __shfl_sync(RX_FULL, hcen, lane < 16 ? k * J + j : 16 + k * J + j);
+      const float lv = __shfl_up_sync(RX_FULL, f4e(c, 4 - R + k), 1);
+      const float rv = __shfl_down_sync(RX_FULL, f4e(c, k), 1);
+      xw[k] = lane == 0 ? e : lv;
+      xw[R + 4 + k] = lane == 31 ? e : rv;
+    }
+    float4 zs[2 * R];
+#pragma unroll
+    for (int k = 0; k < R; ++k) zs[k] = lds4(Cq[k], br, lane);
+#pragma unroll
+    for (int k = 0; k < R; ++k) zs[R + k] = lds4(Cq[R + 1 + k], br, lane);
+    const float4 pv = lds4(Pq, rb0 + j, lane);
+    float4 v;
+    int ky = 0;
+    if constexpr (EDGE) ky = kzq + ac_k1<R>(yw - R + j, ny);
+#pragma unroll
+    for (int e = 0; e < 4; ++e) {
+      float sm = f4e(zs[0], e);
+#pragma unroll
+      for (int k = 1; k < R; ++k) sm = __fadd_rn(sm, f4e(zs[k], e));
+#pragma unroll
+      for (int k = R; k >= 1; --k) sm = __fadd_rn(sm, f4e(win[R - k], e));
+#pragma unroll
+      for (int k = R; k >= 1; --k) sm = __fadd_rn(sm, xw[R + e - k]);
+#pragma unroll
+      for (int k = 1; k <= R; ++k) sm = __fadd_rn(sm, xw[R + e + k]);
+#pragma unroll
+      for (int k = 1; k <= R; ++k) sm = __fadd_rn(sm, f4e(win[R + k], e));
+#pragma unroll
+      for (int k = 0; k < R; ++k) sm = __fadd_rn(sm, f4e(zs[R + k], e));
+      const int K = EDGE ? ky + ((kxp >> (4 * e)) & 15) : 0;
+      f4s(v, e, ac_comb<R, !EDGE>(a, sm, f4e(c, e), f4e(pv, e), K));
+    }
+    if constexpr (EDGE) {
+      const int gy = yw - R + j;
+      if (!(qin && colin && gy >= 0 && gy < ny)) v = make_float4(0.f, 0.f, 0.f, 0.f);
+    }
+    s1[j] = v;
+#pragma unroll
+    for (int k = 0; k < 2 * R; ++k) win[k] = win[k + 1];
+  }
+  // halo X1 for lanes 0 / 31, row by row below
+  // ---- u^{n+1} of the output rows (plane q) ----
+  if (st1) {
+    float* op = o1;
+#pragma unroll
+    for (int i = 0; i < RPW; ++i) {
+      stg128_if(op, s1[R + i], i < row_ok);
+      op += rowp;
+    }
+  }
+  // ---- u^{n+2}: finish plane q-R, accumulate plane q ----
+  if (fin) {
+    float* op = o2;
+#pragma unroll
+    for (int i = 0; i < RPW; ++i) {
+      float4 sm = acc[0][i];
+      sm.x = __fadd_rn(sm.x, s1[R + i].x);
+      sm.y = __fadd_rn(sm.y, s1[R + i].y);
+      sm.z = __fadd_rn(sm.z, s1[R + i].z);
+      sm.w = __fadd_rn(sm.w, s1[R + i].w);
+      const float4 uc = hist[0][i];
+      const float4 pr = lds4(Cq[0], rb0 + 2 * R + i, lane);     // u^n of plane q-R at the output rows
+      int ko = 0;
+      if constexpr (EDGE) ko = kzo + ac_k1<R>(yw + i, ny);
+      float4 v;
+#pragma unroll
+      for (int e = 0; e < 4; ++e)
+        f4s(v, e, ac_comb<R, !EDGE>(a, f4e(sm, e), f4e(uc, e), f4e(pr, e), EDGE ? ko + ((kxp >> (4 * e)) & 15) : 0));
+      stg128_if(op, v, i < row_ok);
+      op += rowp;
+    }
+  }
+  if constexpr (R == 2) {
+    // the plane before: its z+1 tap
+#pragma unroll
+    for (int i = 0; i < RPW; ++i) {
+      acc[0][i].x = __fadd_rn(acc[1][i].x, s1[R + i].x);
+      acc[0][i].y = __fadd_rn(acc[1][i].y, s1[R + i].y);
+      acc[0][i].z = __fadd_rn(acc[1][i].z, s1[R + i].z);
+      acc[0][i].w = __fadd_rn(acc[1][i].w, s1[R + i].w);
+    }
+  }
+  if (newacc) {
+#pragma unroll
+    for (int i = 0; i < RPW; ++i) {
+      const int j = R + i;                 // X1 row of output row i
+      float4 sm = hist[0][i];              // z-R
+#pragma unroll
+      for (int k = 1; k < R; ++k) {
+        sm.x = __fadd_rn(sm.x, hist[k][i].x);
+        sm.y = __fadd_rn(sm.y, hist[k][i].y);
+        sm.z = __fadd_rn(sm.z, hist[k][i].z);
+        sm.w = __fadd_rn(sm.w, hist[k][i].w);
+      }
+#pragma unroll
+      for (int k = R; k >= 1; --k) {
+        sm.x = __fadd_rn(sm.x, s1[j - k].x);
+        sm.y = __fadd_rn(sm.y, s1[j - k].y);
+        sm.z = __fadd_rn(sm.z, s1[j - k].z);
+        sm.w = __fadd_rn(sm.w, s1[j - k].w);
+      }
+      const float4 c = s1[j];
+      float xw[4 + 2 * R];
+      xw[R + 0] = c.x; xw[R + 1] = c.y; xw[R + 2] = c.z; xw[R + 3] = c.w;
+#pragma unroll
+      for (int k = 0; k < R; ++k) {
+        const float e = __shfl_sync(RX_FULL, hv, lane < 16 ? k * J + j : 16 + k * J + j);
+        const float lv = __shfl_up_sync(RX_FULL, f4e(c, 4 - R + k), 1);
+        const float rv = __shfl_down_sync(RX_FULL, f4e(c, k), 1);
+        xw[k] = lane == 0 ? e : lv;
+        xw[R + 4 + k] = lane == 31 ? e : rv;
+      }
+#pragma unroll
+      for (int e = 0; e < 4; ++e) {
+        float t = f4e(sm, e);
+#pragma unroll
+        for (int k = R; k >= 1; --k) t = __fadd_rn(t, xw[R + e - k]);
+#pragma unroll
+        for (int k = 1; k <= R; ++k) t = __fadd_rn(t, xw[R + e + k]);
+        f4s(sm, e, t);
+      }
+#pragma unroll
+      for (int k = 1; k <= R; ++k) {
+        sm.x = __fadd_rn(sm.x, s1[j + k].x);
+        sm.y = __fadd_rn(sm.y, s1[j + k].y);
+        sm.z = __fadd_rn(sm.z, s1[j + k].z);
+        sm.w = __fadd_rn(sm.w, s1[j + k].w);
+      }
+      acc[R - 1][i] = sm;
+    }
+  }
+  // X1 history: hist[k] = X1(q-R+k+1) after this plane
+#pragma unroll
+  for (int i = 0; i < RPW; ++i) {
+#pragma unroll
+    for (int k = 0; k + 1 < R; ++k) hist[k][i] = hist[k + 1][i];
+    hist[R - 1][i] = s1[R + i];
+  }
+}
+
+template <int R, int RPW, int S, int SP>
+__global__ void __launch_bounds__(384, 1)
+    k2ra_sweep(const __grid_constant__ StencilParams p, const __grid_constant__ CUtensorMap tmc,
+               const __grid_constant__ CUtensorMap tmp, float* out1, float* out2, int ntx, int nty, int zc,
+               int nchunk, int n1, int zc2) {
+  using C = CfgA<R, RPW>;
+  constexpr int TY = C::TY, J = C::J, SFC = C::SFC, SFP = C::SFP;
+  static_assert(R * J <= 16, "halo lanes: R * J <= 16");
+  extern __shared__ __align__(128) float dsm[];
+  float* psm = dsm + S * SFC;
+  uint64_t* fullc = reinterpret_cast<uint64_t*>(psm + SP * SFP);
+  uint64_t* emptyc = fullc + S;
+  uint64_t* fullp = emptyc + S;
+  uint64_t* emptyp = fullp + SP;
+  int* stage_item = reinterpret_cast<int*>(emptyp + SP);
+  int* slot_sm = stage_item + S;
+  const int ntile = ntx * nty;
+  const int nitems = ntile * nchunk;
+  const int lane = threadIdx.x & 31;
+  const int warp = (int)(threadIdx.x >> 5) - 4;
+  if (threadIdx.x == 0) {
+    for (int s = 0; s < S; ++s) {
+      mbar_init(&fullc[s], 1);
+      mbar_init(&emptyc[s], 8);
+    }
+    for (int s = 0; s < SP; ++s) {
+      mbar_init(&fullp[s], 1);
+      mbar_init(&emptyp[s], 8);
+    }
+    fence_mbar_init();
+    *slot_sm = claim_launch_slot(g_launch_r);
+  }
+  __syncthreads();
+  const int slot = *slot_sm;
+  pdl_launch_dependents();
+  pdl_wait();
+  if (warp < 0) asm volatile("setmaxnreg.dec.sync.aligned.u32 56;\n" ::: "memory");
+  else asm volatile("setmaxnreg.inc.sync.aligned.u32 224;\n" ::: "memory");
+
+  if (warp == -4) {
+    if (lane == 0) {
+      prefetch_tmap(&tmc);
+      prefetch_tmap(&tmp);
+      int s = 0, sp = 0;
+      uint32_t pass = 0, passp = 0;
+      while (true) {
+        const int item = (int)atomicAdd(&g_launch_r[slot].c[0], 1u);
+        const bool done = item >= nitems;
+        int nc = 1, x0 = 0, y0 = 0;
+        int64_t gzs = 0;
+        if (!done) {
+          const ItemGeom g = item_geom(p, item, ntx, ntile, TY, zc, n1, zc2);
+          x0 = g.x0;
+          y0 = g.y0;
+          gzs = g.gzs;
+          nc = (int)(g.gze - g.gzs) + 4 * R;        // u^n planes gzs-2R .. gze-1+2R
+        }
+        for (int i = 0; i < nc; ++i) {
+          if (pass > 0) mbar_wait(&emptyc[s], (pass - 1) & 1);
+          if (i == 0) stage_item[s] = done ? -1 : item;
+          if (!done) {
+            // planes outside the grid: TMA's out-of-bounds fill (zero padding)
+            mbar_arrive_expect_tx(&fullc[s], C::C_BYTES);
+            tma_load_3d(dsm + s * SFC, &tmc, &fullc[s], x0 - 4, y0 - 2 * R, (int)(gzs - 2 * R + i));
+          } else {
+            mbar_arrive(&fullc[s]);
+          }
+          if (++s == S) { s = 0; ++pass; }
+          if (!done && i >= 2 * R) {                // u^{n-1} plane q = gzs - 3R + i
+            if (passp > 0) mbar_wait(&emptyp[sp], (passp - 1) & 1);
+            mbar_arrive_expect_tx(&fullp[sp], C::P_BYTES);
+            tma_load_3d(psm + sp * SFP, &tmp, &fullp[sp], x0 - 4, y0 - R, (int)(gzs - 3 * R + i));
+            if (++sp == SP) { sp = 0; ++passp; }
+          }
+        }
+        if (done) break;
+      }
+    }
+  } else if (warp >= 0) {
+    const int nx = (int)p.n[2], ny = (int)p.n[1];
+    const int gnz = (int)p.gnz;
+    const int rb0 = warp * RPW;
+    const uint32_t fullc_a = smem_u32(fullc), emptyc_a = smem_u32(emptyc);
+    const uint32_t fullp_a = smem_u32(fullp), emptyp_a = smem_u32(emptyp);
+    AcConst ac;
+    ac.l2 = p.prm[0];
+    ac.c0 = __fsub_rn(2.0f, __fmul_rn(p.prm[0], (float)(6 * R)));
+    ac.prm = p.prm;
+    int sn = 0, spn = 0;
+    uint32_t pn = 0, ppn = 0;
+    float4 acc[R][RPW], hist[R][RPW];
+#pragma unroll
+    for (int k = 0; k < R; ++k)
+#pragma unroll
+      for (int i = 0; i < RPW; ++i) {
+        acc[k][i] = make_float4(0.f, 0.f, 0.f, 0.f);
+        hist[k][i] = acc[k][i];
+      }
+    while (true) {
+      mbar_wait(&fullc[sn], pn & 1);
+      const int item = stage_item[sn];
+      if (item < 0) {
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&emptyc[sn]);
+        break;
+      }
+      const ItemGeom g = item_geom(p, item, ntx, ntile, TY, zc, n1, zc2);
+      const int x0 = g.x0, y0 = g.y0;
+      const int gzs = (int)g.gzs, gze = (int)g.gze;
+      const int yw = y0 + warp * RPW;
+      const int xo = x0 + 4 * lane;
+      const bool colin = xo < nx;
+      // K's x part of the lane's 4 columns, 4 bits each
+      int kxp = 0;
+#pragma unroll
+      for (int e = 0; e < 4; ++e) kxp |= ac_k1<R>(xo + e, nx) << (4 * e);
+      const bool rows_int = yw - 2 * R >= 0 && yw + RPW + 2 * R <= ny;      // X1 rows and their K interior
+      const bool cols_int = x0 >= R && x0 + RX_TX + R <= nx;
+      // halo lane: X1 at (row hj, column hx)
+      int hofs, hpofs, hKyx;
+      bool hin;
+      {
+        const int idx = min(lane & 15, R * J - 1);
+        const int hk = idx / J, hj = idx % J;
+        const int hx = lane < 16 ? x0 - R + hk : x0 + RX_TX + hk;
+        const int hgy = yw - R + hj;
+        hin = hx >= 0 && hx < nx && hgy >= 0 && hgy < ny;
+        hofs = (rb0 + R + hj) * RX_BX + 4 + hx - x0;
+        hpofs = (rb0 + hj) * RX_BX + 4 + hx - x0;
+        hKyx = ac_k1<R>(hgy, ny) + ac_k1<R>(hx, nx);
+      }
+      const int row_ok = colin ? min(RPW, ny - yw) : 0;
+      const int64_t plane = p.plane;
+      float* ob1 = out1 + (int64_t)yw * nx + xo;
+      float* ob2 = out2 + (int64_t)yw * nx + xo;
+      // u^n stages of planes q-R .. q+R (ring positions)
+      int cs[2 * R + 1];
+      cs[0] = sn;
+      if (++sn == S) { sn = 0; ++pn; }
+#pragma unroll
+      for (int k = 1; k < 2 * R; ++k) {
+        mbar_wait_a(fullc_a + 8 * sn, pn & 1);
+        cs[k] = sn;
+        if (++sn == S) { sn = 0; ++pn; }
+      }
+      for (int q = gzs - R; q < gze + R; ++q) {
+        mbar_wait_a(fullc_a + 8 * sn, pn & 1);
+        cs[2 * R] = sn;
+        if (++sn == S) { sn = 0; ++pn; }
+        mbar_wait_a(fullp_a + 8 * spn, ppn & 1);
+        const int ps = spn;
+        if (++spn == SP) { spn = 0; ++ppn; }
+        const float* Cq[2 * R + 1];
+#pragma unroll
+        for (int k = 0; k <= 2 * R; ++k) Cq[k] = dsm + cs[k] * SFC;
+        const float* Pq = psm + ps * SFP;
+        const bool qin = q >= 0 && q < gnz;
+        const int kzq = ac_k1<R>(q, gnz), kzo = ac_k1<R>(q - R, gnz);
+        const bool st1 = q >= gzs && q < gze;
+        const bool fin = q - R >= gzs;
+        const bool newacc = q >= gzs && q < gze;
+        const bool fast = rows_int && cols_int && q >= R && q + R < gnz && (q - R >= R || !fin);
+        float* o1 = ob1 + (int64_t)q * plane;
+        float* o2 = ob2 + (int64_t)(q - R) * plane;
+        if (fast)
+          ac_plane<R, RPW, false>(ac, Cq, Pq, lane, rb0, hofs, hpofs, kzq + hKyx, hin, qin, kzq, kzo, yw, ny,
+                                  kxp, colin, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
+        else
+          ac_plane<R, RPW, true>(ac, Cq, Pq, lane, rb0, hofs, hpofs, kzq + hKyx, hin, qin, kzq, kzo, yw, ny,
+                                 kxp, colin, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
+        __syncwarp();
+        if (lane == 0) {
+          mbar_arrive_a(emptyc_a + 8 * cs[0]);
+          mbar_arrive_a(emptyp_a + 8 * ps);
+        }
+#pragma unroll
+        for (int k = 0; k < 2 * R; ++k) cs[k] = cs[k + 1];
+      }
+      __syncwarp();
+      if (lane == 0) {
+#pragma unroll
+        for (int k = 0; k < 2 * R; ++k) mbar_arrive_a(emptyc_a + 8 * cs[k]);
+      }
+    }
+  }
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    __threadfence();
+    const unsigned prev = atomicAdd(&g_launch_r[slot].c[1], 1u);
+    if (prev == gridDim.x - 1) release_launch_slot(g_launch_r, slot);
+  }
+}
+
 struct LauncherR {
   const void* fn;
   int smem;
@@ -555,6 +1002,78 @@ LauncherR pick_r() {
   return get_launcher_r<6, 8, 6, true>();
 }
 
+// z-chunks (items are (chunk, tile), chunk-major) of the two-step kernels:
+// long chunks of zc planes (each chunk recomputes the X_{t+1} planes next to
+// it and refills the ring), then ~2 waves of items in short chunks of zc2
+// planes so the launch's tail is short.  Measured on J3D7 512^3
+// (profiles/r02_k2r_chunks.txt): (128, 16), (112, 16), (64, 16) and (48, 8)
+// all ~1290 Gpts/s; pairs whose long items leave a partial wave of long items
+// after the whole waves lost up to 17% ((64, 8) 1096, (96, 16) 1078), and so
+// did plans with < 2 long items per CTA and no short tail ((160, -) 1106) or
+// 4-plane tails (1200-1240).  Environment hooks override the pair.
+void chunk_plan(int64_t nz_reg, int64_t tiles, int64_t slots, const char* env_zc, const char* env_zc2,
+                int64_t* zc_out, int64_t* n1_out, int64_t* zc2_out, int64_t* nchunk_out, int64_t zc_max = 128,
+                int64_t tail = 16) {
+  const int64_t work = nz_reg * tiles;
+  const char* ez = getenv(env_zc);
+  const char* ez2 = getenv(env_zc2);
+  int64_t zc = std::min<int64_t>(zc_max, std::max<int64_t>(16, nz_reg / 4));
+  int64_t want2 = tail;
+  if (work < 16 * slots) {       // small grids: ~6 items per CTA
+    zc = std::max<int64_t>(4, (work + 6 * slots - 1) / (6 * slots));
+    want2 = 0;
+  }
+  if (ez) zc = std::max<int64_t>(1, atoll(ez));
+  if (ez2) want2 = std::max<int64_t>(0, atoll(ez2));
+  if (zc > nz_reg) zc = nz_reg;
+  int64_t nchunk = (nz_reg + zc - 1) / zc;
+  int64_t n1 = nchunk, zc2 = zc;
+  if (want2 > 0 && want2 < zc) {
+    const int64_t nsmall = (2 * slots + tiles - 1) / tiles;     // short chunks per tile column
+    const int64_t z2 = nsmall * want2;
+    if (z2 < nz_reg) {
+      n1 = (nz_reg - z2) / zc;
+      zc2 = want2;
+      nchunk = n1 + (nz_reg - n1 * zc + zc2 - 1) / zc2;
+    }
+  }
+  *zc_out = zc;
+  *n1_out = n1;
+  *zc2_out = zc2;
+  *nchunk_out = nchunk;
+}
+
+template <int R, int RPW, int S, int SP>
+LauncherR get_launcher_a() {
+  static LauncherR L{};
+  static std::once_flag once;
+  std::call_once(once, [] {
+    auto fn = k2ra_sweep<R, RPW, S, SP>;
+    constexpr int smem = smem_a<R, RPW, S, SP>();
+    cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    int occ = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, 384, smem) != cudaSuccess) occ = 1;
+    cudaGetLastError();
+    L = LauncherR{reinterpret_cast<const void*>(fn), smem, CfgA<R, RPW>::TY, occ > 0 ? occ : 1, 384};
+  });
+  return L;
+}
+
+LauncherR pick_a(int R) {
+  const char* e = getenv("LIFT_K2RA_SHAPE");     // A/B: rows per warp
+  const int v = e ? atoi(e) : 0;
+  if (R == 2) {
+    if (v == 3) return get_launcher_a<2, 3, 6, 3>();
+    if (v == 2) return get_launcher_a<2, 2, 7, 3>();
+    return get_launcher_a<2, 4, 6, 3>();
+  }
+  // (rows per warp, u^n stages, u^{n-1} slots); Acoustic-7 1024^3
+  // (profiles/r02_k2ra_probe.txt): 4 rows 729-744, 6 rows 714, 8 rows 684 Gpts/s
+  if (v == 6) return get_launcher_a<1, 6, 4, 3>();
+  if (v == 8) return get_launcher_a<1, 8, 4, 2>();
+  return get_launcher_a<1, 4, 5, 3>();
+}
+
 }  // namespace
 
 bool sweep3d_r2_supported(const StencilParams& p) {
@@ -582,44 +1101,67 @@ cudaError_t launch_sweep3d_r2(const StencilParams& p, const float* in, float* ou
   const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);
   const int64_t tiles = (int64_t)ntx * nty;
   const int64_t slots = (int64_t)num_sms * L.ctas_per_sm;
-  // z-chunks (items are (chunk, tile), chunk-major): long chunks of zc planes
-  // (each chunk recomputes 2 X_{t+1} planes and refills the ring), then ~2
-  // waves of items in short chunks of zc2 planes so the launch's tail is
-  // short.  Measured on J3D7 512^3 (profiles/r02_k2r_chunks.txt): (128, 16),
-  // (112, 16), (64, 16) and (48, 8) all ~1290 Gpts/s; pairs whose long items
-  // leave a partial wave of long items after the whole waves lost up to 17%
-  // ((64, 8) 1096, (96, 16) 1078), and so did plans with < 2 long items per
-  // CTA and no short tail ((160, -) 1106) or 4-plane tails (1200-1240).
-  // LIFT_K2R_ZC / LIFT_K2R_ZC2 override the pair.
-  const int64_t work = nz_reg * tiles;
-  const char* ez = getenv("LIFT_K2R_ZC");
-  const char* ez2 = getenv("LIFT_K2R_ZC2");
-  int64_t zc = std::min<int64_t>(128, std::max<int64_t>(16, nz_reg / 4));
-  int64_t want2 = 16;
-  if (work < 16 * slots) {       // small grids: ~6 items per CTA
-    zc = std::max<int64_t>(4, (work + 6 * slots - 1) / (6 * slots));
-    want2 = 0;
-  }
-  if (ez) zc = std::max<int64_t>(1, atoll(ez));
-  if (ez2) want2 = std::max<int64_t>(0, atoll(ez2));
-  if (zc > nz_reg) zc = nz_reg;
-  int64_t nchunk = (nz_reg + zc - 1) / zc;
-  int64_t n1 = nchunk, zc2 = zc;
-  if (want2 > 0 && want2 < zc) {
-    const int64_t nsmall = (2 * slots + tiles - 1) / tiles;     // short chunks per tile column
-    const int64_t z2 = nsmall * want2;
-    if (z2 < nz_reg) {
-      n1 = (nz_reg - z2) / zc;
-      zc2 = want2;
-      nchunk = n1 + (nz_reg - n1 * zc + zc2 - 1) / zc2;
-    }
-  }
+  int64_t zc, n1, zc2, nchunk;
+  chunk_plan(nz_reg, tiles, slots, "LIFT_K2R_ZC", "LIFT_K2R_ZC2", &zc, &n1, &zc2, &nchunk);
   const int64_t items = tiles * nchunk;
   if (items > 0x7fffffff) return cudaErrorInvalidConfiguration;
   const int64_t grid = slots < items ? slots : items;
   int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk, n1_i = (int)n1, zc2_i = (int)zc2;
   void* args[] = {(void*)&p, (void*)&map, (void*)&out, &ntx_i, &nty_i, &zc_i, &nch_i, &n1_i, &zc2_i};
   set_last_kernel("k2r_sweep");
+  return launch_kernel(L.fn, dim3((unsigned)grid), dim3(L.threads), args, (size_t)L.smem, stream, true);
+}
+
+}  // namespace lift
+
+namespace lift {
+
+bool acoustic_r2_auto(const StencilParams& p) {
+  // radius 2 (Acoustic-13): measured 487-497 vs 491-522 Gpts/s for single
+  // steps (its X1 rows are recomputed 2x per warp), so AUTO keeps single steps
+  return p.radius == 1 && acoustic_r2_supported(p);
+}
+
+bool acoustic_r2_supported(const StencilParams& p) {
+  if (p.op != OP_ACOUSTIC || (p.radius != 1 && p.radius != 2) || !sweep3d_supported(p)) return false;
+  for (int d = 0; d < 3; ++d)
+    if (p.kind[d] != PAD_CONSTANT) return false;
+  if (p.pad_value != 0.0f) return false;              // zero padding: TMA's out-of-bounds fill
+  if (p.slab || p.ghost != 0 || p.put_lo || p.put_hi || p.fused_step) return false;
+  if (p.n[2] < 4 || p.gnz >= (1ll << 30)) return false;
+  static const bool off = [] {
+    const char* e = getenv("LIFT_K2RA");
+    return e && e[0] == '0';
+  }();
+  return !off;
+}
+
+cudaError_t launch_acoustic_r2(const StencilParams& p, const float* prev, const float* cur, float* out1, float* out2,
+                               cudaStream_t stream, int num_sms, std::string* err) {
+  const int64_t nz_reg = p.reg1 - p.reg0;
+  if (nz_reg <= 0) return cudaSuccess;
+  const int R = p.radius;
+  const LauncherR L = pick_a(R);
+  CUtensorMap mc, mp;
+  if (!encode_tensor_map_3d(&mc, cur, p.n[2], p.n[1], p.n[0], (uint32_t)RX_BX, (uint32_t)(L.ty + 4 * R), 1, err) ||
+      !encode_tensor_map_3d(&mp, prev, p.n[2], p.n[1], p.n[0], (uint32_t)RX_BX, (uint32_t)(L.ty + 2 * R), 1, err))
+    return cudaErrorInvalidValue;
+  const int ntx = (int)((p.n[2] + RX_TX - 1) / RX_TX);
+  const int nty = (int)((p.n[1] + L.ty - 1) / L.ty);
+  const int64_t tiles = (int64_t)ntx * nty;
+  const int64_t slots = (int64_t)num_sms * L.ctas_per_sm;
+  int64_t zc, n1, zc2, nchunk;
+  // chunks (32, tail 8): the u^n / u^{n-1} halo rows of neighbouring tiles stay
+  // L2 hits when the CTAs in flight keep to a narrower z window (Acoustic-7
+  // 729 -> 744 Gpts/s vs (128, 16))
+  chunk_plan(nz_reg, tiles, slots, "LIFT_K2RA_ZC", "LIFT_K2RA_ZC2", &zc, &n1, &zc2, &nchunk, 32, 8);
+  const int64_t items = tiles * nchunk;
+  if (items > 0x7fffffff) return cudaErrorInvalidConfiguration;
+  const int64_t grid = slots < items ? slots : items;
+  int ntx_i = ntx, nty_i = nty, zc_i = (int)zc, nch_i = (int)nchunk, n1_i = (int)n1, zc2_i = (int)zc2;
+  void* args[] = {(void*)&p, (void*)&mc, (void*)&mp, (void*)&out1, (void*)&out2,
+                  &ntx_i, &nty_i, &zc_i, &nch_i, &n1_i, &zc2_i};
+  set_last_kernel("k2ra_sweep");
   return launch_kernel(L.fn, dim3((unsigned)grid), dim3(L.threads), args, (size_t)L.smem, stream, true);
 }
 

@@ -83,6 +83,14 @@ bool sweep3d_r2_supported(const StencilParams& p);
 cudaError_t launch_sweep3d_r2(const StencilParams& p, const float* in, float* out, cudaStream_t stream, int num_sms,
                               std::string* err);
 
+// K2RA — two Acoustic (7 / 13-point, zero pad) steps per pass: reads u^{n-1}
+// (prev) and u^n (cur), writes u^{n+1} (out1) and u^{n+2} (out2); four
+// distinct buffers.
+bool acoustic_r2_supported(const StencilParams& p);
+bool acoustic_r2_auto(const StencilParams& p);        // the plans AUTO time blocking sends to K2RA
+cudaError_t launch_acoustic_r2(const StencilParams& p, const float* prev, const float* cur, float* out1, float* out2,
+                               cudaStream_t stream, int num_sms, std::string* err);
+
 // K1 — 2D TMA halo-tile kernel (weighted box r<=4, srad1, srad2).
 bool tile2d_supported(const StencilParams& p);
 cudaError_t launch_tile2d(const StencilParams& p, const float* in0, const float* in1, float* out,

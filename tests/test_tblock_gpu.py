@@ -128,3 +128,119 @@ def test_k2r_j3d7_512_sampled(lift):
     y2, plan = run(lift, sp, xs[0], 10, 2)
     assert plan.last_kernel == "k2r_sweep"
     assert np.array_equal(y2, y1)
+
+
+# ------------------------------------------------------------------ K2RA ----
+# Two Acoustic steps per pass (Listing 3; zero padding): iterate
+# with four state buffers {prev, cur, spare, spare}; the newest grid is
+# state[ri], the one before it state[ri ^ 1].
+
+def ac_spec(extents, pts):
+    return si.StencilSpec(tuple(extents), (5, 5, 5) if pts == 13 else (3, 3, 3), (1, 1, 1),
+                          (2, 2, 2) if pts == 13 else (1, 1, 1), (2, 2, 2) if pts == 13 else (1, 1, 1),
+                          (si.CONSTANT,) * 3, 0.0, si.ACOUSTIC, None, si.params_acoustic(pts))
+
+
+def ac_run(lift, sp, u0, u1, steps, nbuf, env=None, tb=2):
+    old = {}
+    for k, v in (env or {}).items():
+        old[k] = os.environ.get(k)
+        os.environ[k] = v
+    try:
+        plan = lift.Plan.from_spec(sp)
+        plan.set_time_block(tb)
+        bufs = [torch.from_numpy(u0.copy()).cuda(), torch.from_numpy(u1.copy()).cuda()]
+        bufs += [torch.full_like(bufs[0], float("nan")) for _ in range(nbuf - 2)]
+        ri = plan.iterate(bufs, steps)
+        torch.cuda.synchronize()
+        return bufs[ri].cpu().numpy(), bufs[ri ^ 1].cpu().numpy(), plan
+    finally:
+        for k, v in old.items():
+            if v is None:
+                os.environ.pop(k, None)
+            else:
+                os.environ[k] = v
+
+
+AC_SHAPES = [(20, 36, 132), (5, 64, 256), (1, 9, 128), (3, 1, 4), (2, 50, 260), (9, 33, 516), (40, 8, 128),
+             (6, 70, 388)]
+
+
+@pytest.mark.parametrize("pts", [7, 13])
+@pytest.mark.parametrize("shape", AC_SHAPES)
+def test_k2ra_bitwise_equal_single_steps(lift, pts, shape):
+    rng = np.random.default_rng(80)
+    u0 = rng.uniform(-1, 1, size=shape).astype(np.float32)
+    u1 = rng.uniform(-1, 1, size=shape).astype(np.float32)
+    sp = ac_spec(shape, pts)
+    n1, p1, _ = ac_run(lift, sp, u0, u1, 6, 2)
+    n2, p2, plan = ac_run(lift, sp, u0, u1, 6, 4)
+    assert plan.last_kernel == "k2ra_sweep"
+    np.testing.assert_array_equal(n2, n1)
+    np.testing.assert_array_equal(p2, p1)
+
+
+@pytest.mark.parametrize("pts,shape_env", [(7, "4"), (7, "8"), (7, "6"), (13, "2"), (13, "3"), (13, "4")])
+@pytest.mark.parametrize("zc", [("1", "0"), ("3", "1"), ("64", "0"), ("5", "2")])
+def test_k2ra_shapes_and_chunks(lift, pts, shape_env, zc):
+    shape = (17, 70, 260)
+    rng = np.random.default_rng(81)
+    u0 = rng.uniform(-1, 1, size=shape).astype(np.float32)
+    u1 = rng.uniform(-1, 1, size=shape).astype(np.float32)
+    sp = ac_spec(shape, pts)
+    n1, p1, _ = ac_run(lift, sp, u0, u1, 4, 2)
+    n2, p2, plan = ac_run(lift, sp, u0, u1, 4, 4, {"LIFT_K2RA_SHAPE": shape_env, "LIFT_K2RA_ZC": zc[0],
+                                                   "LIFT_K2RA_ZC2": zc[1]})
+    assert plan.last_kernel == "k2ra_sweep"
+    np.testing.assert_array_equal(n2, n1)
+    np.testing.assert_array_equal(p2, p1)
+
+
+@pytest.mark.parametrize("pts", [7, 13])
+def test_k2ra_vs_oracle_odd_steps(lift, pts):
+    """7 steps = three K2RA passes + one single step, against the fp64 oracle
+    (prev = cur initial condition as the BASELINE C5 recipe)."""
+    shape = (14, 30, 132)
+    u = np.random.default_rng(82).uniform(-1, 1, size=shape).astype(np.float32)
+    sp = ac_spec(shape, pts)
+    n2, p2, _ = ac_run(lift, sp, u, u, 7, 4)
+    ref = orc.iterate(sp, [u, u], [], 7)
+    assert np.max(np.abs(n2 - ref[1])) <= TOL10 * np.max(np.abs(ref[1]))
+    assert np.max(np.abs(p2 - ref[0])) <= TOL10 * np.max(np.abs(ref[0]))
+    n1, p1, _ = ac_run(lift, sp, u, u, 7, 2)
+    np.testing.assert_array_equal(n2, n1)
+
+
+def test_k2ra_time_block_1_and_two_buffers(lift):
+    shape = (8, 20, 128)
+    u = np.random.default_rng(83).uniform(-1, 1, size=shape).astype(np.float32)
+    sp = ac_spec(shape, 7)
+    _, _, plan = ac_run(lift, sp, u, u, 4, 4, tb=1)
+    assert plan.last_kernel != "k2ra_sweep"
+    _, _, plan = ac_run(lift, sp, u, u, 4, 2)
+    assert plan.last_kernel != "k2ra_sweep"
+    # AUTO (time block 0): two-step passes for the 7-point update only
+    _, _, plan = ac_run(lift, sp, u, u, 4, 4, tb=0)
+    assert plan.time_block == 2 and plan.last_kernel == "k2ra_sweep"
+    _, _, plan = ac_run(lift, ac_spec(shape, 13), u, u, 4, 4, tb=0)
+    assert plan.time_block == 1 and plan.last_kernel != "k2ra_sweep"
+    _, _, plan = ac_run(lift, ac_spec(shape, 13), u, u, 4, 4, tb=2)
+    assert plan.time_block == 2 and plan.last_kernel == "k2ra_sweep"
+
+
+def test_k2ra_acoustic13_1024_whole_grid(lift):
+    """BASELINE C5b size (1024^3), 4 steps as two K2RA passes: bitwise equal to
+    single steps over the whole grid (compared on the device)."""
+    xs, sp = si.make_workload_inputs(si.workload("acoustic13_1024"))
+    res = []
+    for nbuf in (2, 4):
+        plan = lift.Plan.from_spec(sp)
+        plan.set_time_block(2)
+        bufs = [torch.from_numpy(xs[0]).cuda(), torch.from_numpy(xs[1]).cuda()]
+        bufs += [torch.empty_like(bufs[0]) for _ in range(nbuf - 2)]
+        ri = plan.iterate(bufs, 4)
+        torch.cuda.synchronize()
+        res.append((bufs[ri], bufs[ri ^ 1], plan.last_kernel))
+        del bufs
+    assert res[1][2] == "k2ra_sweep"
+    assert torch.equal(res[0][0], res[1][0]) and torch.equal(res[0][1], res[1][1])
