@@ -344,10 +344,13 @@ __global__ void __launch_bounds__(nthreads_r<NW, WS>(), 1)
   pdl_launch_dependents();   // PDL: let the next launch ramp up now
   pdl_wait();                // ... and wait for the previous one before any global access
   if constexpr (WS) {
-    static_assert(NW == 8 || NW == 16, "register split for 8 or 16 consumer warps");
+    static_assert(NW == 8 || NW == 12 || NW == 16, "register split for 8, 12 or 16 consumer warps");
     if constexpr (NW == 8) {       // launched at 168: 128 x (168 - 56) == 256 x (224 - 168)
       if (warp < 0) asm volatile("setmaxnreg.dec.sync.aligned.u32 56;\n" ::: "memory");
       else asm volatile("setmaxnreg.inc.sync.aligned.u32 224;\n" ::: "memory");
+    } else if constexpr (NW == 12) {   // launched at 128: 128 x (128 - 24) >= 384 x (160 - 128)
+      if (warp < 0) asm volatile("setmaxnreg.dec.sync.aligned.u32 24;\n" ::: "memory");
+      else asm volatile("setmaxnreg.inc.sync.aligned.u32 160;\n" ::: "memory");
     } else {                       // registers come from the CTA's own pool: 128 x (96 - 24) >= 512 x (112 - 96)
       if (warp < 0) asm volatile("setmaxnreg.dec.sync.aligned.u32 24;\n" ::: "memory");
       else asm volatile("setmaxnreg.inc.sync.aligned.u32 112;\n" ::: "memory");
@@ -586,18 +589,31 @@ __device__ __forceinline__ void f4s(float4& v, int e, float x) {
 // One X1 plane of a warp.  Cq[k] = u^n stage of plane q-R+k (k = 0..2R),
 // Pq = u^{n-1} stage of plane q.  EDGE: K per element and zero outside the
 // grid (y / x / ragged); otherwise every point of the warp is interior.
+// halo point of a lane in one round: X1 at (row j, column x0-R+k or x0+128+k),
+// point index i = k*J + j, round i / 16, lane i % 16 (left) / 16 + i % 16 (right)
+struct HaloA {
+  int ofs, pofs, kyx;
+  bool in;
+};
+template <int R, int RPW>
+constexpr int halo_rounds() { return (R * (RPW + 2 * R) + 15) / 16; }
+
 template <int R, int RPW, bool EDGE>
 __device__ __forceinline__ void ac_plane(const AcConst& a, const float* const (&Cq)[2 * R + 1],
-                                         const float* __restrict__ Pq, int lane, int rb0, int hofs, int hpofs,
-                                         int hK, bool hin, bool qin, int kzq, int kzo, int yw, int ny, int kxp,
+                                         const float* __restrict__ Pq, int lane, int rb0,
+                                         const HaloA (&hl)[halo_rounds<R, RPW>()], bool qin, int kzq, int kzo,
+                                         int yw, int ny, int kxp,
                                          bool colin, float4 (&acc)[R][RPW], float4 (&hist)[R][RPW], bool st1,
                                          bool fin, bool newacc, float* o1, float* o2, int row_ok, int rowp) {
   constexpr int J = RPW + 2 * R;
-  // ---- halo lanes: X1 at columns x0-R+k (lanes k*J+j) and x0+128+k (16+k*J+j) ----
-  float hcen, hv;
-  {
+  // ---- halo lanes: X1 at columns x0-R+k and x0+128+k, rows 0..J-1 ----
+  constexpr int NR = halo_rounds<R, RPW>();
+  float hcen[NR], hv[NR];
+#pragma unroll
+  for (int r = 0; r < NR; ++r) {
     const float* c = Cq[R];
-    hcen = c[hofs];
+    const int hofs = hl[r].ofs;
+    hcen[r] = c[hofs];
     float sh = Cq[0][hofs];
 #pragma unroll
     for (int k = 1; k < R; ++k) sh = __fadd_rn(sh, Cq[k][hofs]);
@@ -611,8 +627,8 @@ __device__ __forceinline__ void ac_plane(const AcConst& a, const float* const (&
     for (int k = 1; k <= R; ++k) sh = __fadd_rn(sh, c[hofs + k * RX_BX]);
 #pragma unroll
     for (int k = R + 1; k <= 2 * R; ++k) sh = __fadd_rn(sh, Cq[k][hofs]);
-    hv = acoustic_combine<R>(sh, hcen, Pq[hpofs], hK, a.prm);
-    if (!(hin && qin)) hv = 0.0f;
+    hv[r] = acoustic_combine<R>(sh, hcen[r], Pq[hl[r].pofs], kzq + hl[r].kyx, a.prm);
+    if (!(hl[r].in && qin)) hv[r] = 0.0f;
   }
   // ---- X1(q) rows j = 0..J-1 (gy = yw-R+j; u^n box row rb0+R+j; u^{n-1} box row rb0+j) ----
   float4 s1[J];
@@ -629,7 +645,8 @@ __device__ __forceinline__ void ac_plane(const AcConst& a, const float* const (&
     // in-row neighbours: adjacent lanes; lanes 0 / 31 from the halo lanes' u^n
 #pragma unroll
     for (int k = 0; k < R; ++k) {
-      const float e = __shfl_sync(RX_FULL, hcen, lane < 16 ? k * J + j : 16 + k * J + j);
+      const int hi = k * J + j;       // (a constant after unrolling)
+      const float e = __shfl_sync(RX_FULL, hcen[hi / 16], lane < 16 ? hi % 16 : 16 + hi % 16);
       const float lv = __shfl_up_sync(RX_FULL, f4e(c, 4 - R + k), 1);
       const float rv = __shfl_down_sync(RX_FULL, f4e(c, k), 1);
       xw[k] = lane == 0 ? e : lv;
@@ -736,7 +753,8 @@ __device__ __forceinline__ void ac_plane(const AcConst& a, const float* const (&
       xw[R + 0] = c.x; xw[R + 1] = c.y; xw[R + 2] = c.z; xw[R + 3] = c.w;
 #pragma unroll
       for (int k = 0; k < R; ++k) {
-        const float e = __shfl_sync(RX_FULL, hv, lane < 16 ? k * J + j : 16 + k * J + j);
+        const int hi = k * J + j;
+        const float e = __shfl_sync(RX_FULL, hv[hi / 16], lane < 16 ? hi % 16 : 16 + hi % 16);
         const float lv = __shfl_up_sync(RX_FULL, f4e(c, 4 - R + k), 1);
         const float rv = __shfl_down_sync(RX_FULL, f4e(c, k), 1);
         xw[k] = lane == 0 ? e : lv;
@@ -777,7 +795,7 @@ __global__ void __launch_bounds__(384, 1)
                int nchunk, int n1, int zc2) {
   using C = CfgA<R, RPW>;
   constexpr int TY = C::TY, J = C::J, SFC = C::SFC, SFP = C::SFP;
-  static_assert(R * J <= 16, "halo lanes: R * J <= 16");
+  constexpr int NR = halo_rounds<R, RPW>();
   extern __shared__ __align__(128) float dsm[];
   float* psm = dsm + S * SFC;
   uint64_t* fullc = reinterpret_cast<uint64_t*>(psm + SP * SFP);
@@ -888,18 +906,18 @@ __global__ void __launch_bounds__(384, 1)
       for (int e = 0; e < 4; ++e) kxp |= ac_k1<R>(xo + e, nx) << (4 * e);
       const bool rows_int = yw - 2 * R >= 0 && yw + RPW + 2 * R <= ny;      // X1 rows and their K interior
       const bool cols_int = x0 >= R && x0 + RX_TX + R <= nx;
-      // halo lane: X1 at (row hj, column hx)
-      int hofs, hpofs, hKyx;
-      bool hin;
-      {
-        const int idx = min(lane & 15, R * J - 1);
+      // halo lanes: X1 at (row hj, column hx), NR rounds of 16 points per side
+      HaloA hl[NR];
+#pragma unroll
+      for (int r = 0; r < NR; ++r) {
+        const int idx = min((lane & 15) + 16 * r, R * J - 1);
         const int hk = idx / J, hj = idx % J;
         const int hx = lane < 16 ? x0 - R + hk : x0 + RX_TX + hk;
         const int hgy = yw - R + hj;
-        hin = hx >= 0 && hx < nx && hgy >= 0 && hgy < ny;
-        hofs = (rb0 + R + hj) * RX_BX + 4 + hx - x0;
-        hpofs = (rb0 + hj) * RX_BX + 4 + hx - x0;
-        hKyx = ac_k1<R>(hgy, ny) + ac_k1<R>(hx, nx);
+        hl[r].in = hx >= 0 && hx < nx && hgy >= 0 && hgy < ny;
+        hl[r].ofs = (rb0 + R + hj) * RX_BX + 4 + hx - x0;
+        hl[r].pofs = (rb0 + hj) * RX_BX + 4 + hx - x0;
+        hl[r].kyx = ac_k1<R>(hgy, ny) + ac_k1<R>(hx, nx);
       }
       const int row_ok = colin ? min(RPW, ny - yw) : 0;
       const int64_t plane = p.plane;
@@ -935,10 +953,10 @@ __global__ void __launch_bounds__(384, 1)
         float* o1 = ob1 + (int64_t)q * plane;
         float* o2 = ob2 + (int64_t)(q - R) * plane;
         if (fast)
-          ac_plane<R, RPW, false>(ac, Cq, Pq, lane, rb0, hofs, hpofs, kzq + hKyx, hin, qin, kzq, kzo, yw, ny,
+          ac_plane<R, RPW, false>(ac, Cq, Pq, lane, rb0, hl, qin, kzq, kzo, yw, ny,
                                   kxp, colin, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
         else
-          ac_plane<R, RPW, true>(ac, Cq, Pq, lane, rb0, hofs, hpofs, kzq + hKyx, hin, qin, kzq, kzo, yw, ny,
+          ac_plane<R, RPW, true>(ac, Cq, Pq, lane, rb0, hl, qin, kzq, kzo, yw, ny,
                                  kxp, colin, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
         __syncwarp();
         if (lane == 0) {
@@ -999,6 +1017,8 @@ LauncherR pick_r() {
   if (v == 1064) return get_launcher_r<6, 8, 4, true>();
   if (v == 204) return get_launcher_r<4, 16, 5, true>();
   if (v == 203) return get_launcher_r<3, 16, 6, true>();
+  if (v == 304) return get_launcher_r<4, 12, 6, true>();
+  if (v == 303) return get_launcher_r<3, 12, 6, true>();
   return get_launcher_r<6, 8, 6, true>();
 }
 

@@ -22,6 +22,7 @@ spare = [torch.empty_like(bufs[0]) for _ in range(2)]
 
 def timed(nbuf, steps=20):
     plan = lift.Plan.from_spec(spec)
+    plan.set_time_block(2 if nbuf == 4 else 1)
     st = bufs + (spare if nbuf == 4 else [])
     plan.iterate(st, 4)
     torch.cuda.synchronize()
@@ -38,6 +39,9 @@ def timed(nbuf, steps=20):
 
 v, k = timed(2)
 print(f"acoustic{pts} {n}^3 single steps: {v:7.1f} Gpts/s ({k})", flush=True)
+if os.environ.get("K2RA_SINGLE_AGAIN"):
+    v, k = timed(2)
+    print(f"acoustic{pts} {n}^3 single steps (again): {v:7.1f} Gpts/s ({k})", flush=True)
 for arg in sys.argv[2:] or ["::"]:
     parts = (arg.split(":") + ["", "", ""])[:3]
     for key, val in zip(("LIFT_K2RA_SHAPE", "LIFT_K2RA_ZC", "LIFT_K2RA_ZC2"), parts):
