@@ -1015,6 +1015,8 @@ LauncherR pick_r() {
   if (v == 108) return get_launcher_r<8, 8, 5, true>();
   if (v == 1086) return get_launcher_r<8, 8, 6, true>();
   if (v == 1064) return get_launcher_r<6, 8, 4, true>();
+  if (v == 1067) return get_launcher_r<6, 8, 7, true>();
+  if (v == 1045) return get_launcher_r<4, 8, 8, true>();
   if (v == 204) return get_launcher_r<4, 16, 5, true>();
   if (v == 203) return get_launcher_r<3, 16, 6, true>();
   if (v == 304) return get_launcher_r<4, 12, 6, true>();
