@@ -508,9 +508,14 @@ stencil_status stencil_plan_set_time_block(stencil_plan pl, int32_t steps) {
 
 int32_t stencil_plan_time_block(stencil_plan pl) {
   if (!pl) return -1;
+  const bool hs2 = pl->p.op == OP_HOTSPOT3D && column3d_t2_supported(pl->p, nullptr, nullptr);
+  // (K2CT, two Hotspot3D steps per launch of a few-plane grid, measured no
+  // faster than K2C single steps — 6.75 vs 6.53 us per step — so AUTO keeps
+  // single steps for it; time block 2 forces it)
   if (pl->time_block == 0)
     return (pl->ndim == 3 && (sweep3d_r2_supported(pl->p) || acoustic_r2_auto(pl->p))) ? 2 : 1;
-  return (pl->time_block >= 2 && pl->ndim == 3 && (sweep3d_t2_supported(pl->p) || acoustic_r2_supported(pl->p)))
+  return (pl->time_block >= 2 && pl->ndim == 3 &&
+          (sweep3d_t2_supported(pl->p) || acoustic_r2_supported(pl->p) || hs2))
              ? 2
              : 1;
 }
@@ -739,7 +744,24 @@ stencil_status stencil_iterate(stencil_plan pl, float* const* state, int32_t n_s
     }
   } else if (p.op == OP_HOTSPOT3D || p.op == OP_HOTSPOT2D) {
     if (n_aux != 1 || !aux || !aux[0]) return fail(STENCIL_E_INVALID, "HOTSPOT iterate needs aux {P}");
-    for (int t = 0; t < n_steps; ++t) {
+    int t = 0;
+    // two steps per launch (K2CT) for few-plane Hotspot3D grids
+    if (p.op == OP_HOTSPOT3D && tb == 2 && n_steps >= 2 && pl->ndim == 3 &&
+        (pl->forced_variant == STENCIL_VARIANT_AUTO || pl->forced_variant == STENCIL_VARIANT_SWEEP3D) &&
+        column3d_t2_supported(p, state[0], aux[0]) && column3d_t2_supported(p, state[1], aux[0])) {
+      DeviceGuard g(pl->device);
+      if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+      for (; t + 2 <= n_steps; t += 2) {
+        std::string err;
+        cudaError_t e = launch_column3d_t2(p, state[ri], aux[0], state[1 - ri], (cudaStream_t)stream, &err);
+        pl->last_kernel = g_last_kernel;
+        pl->last_variant = STENCIL_VARIANT_SWEEP3D;
+        if (e != cudaSuccess)
+          return fail(STENCIL_E_CUDA, std::string("K2CT launch failed: ") + cudaGetErrorString(e) + " " + err);
+        ri = 1 - ri;
+      }
+    }
+    for (; t < n_steps; ++t) {
       const float* in[2] = {state[ri], aux[0]};
       stencil_status s = stencil_apply(pl, in, 2, state[1 - ri], stream);
       if (s != STENCIL_OK) return s;

@@ -63,6 +63,12 @@ bool column3d_supported(const StencilParams& p, const float* in0, const float* i
 cudaError_t launch_column3d(const StencilParams& p, const float* in0, const float* in1, float* out,
                             cudaStream_t stream, std::string* err);
 
+// K2CT — two steps per launch of a few-plane grid (Hotspot3D, reindexing
+// pads): in0 = X_t, in1 = the point-wise grid, out = X_{t+2}.
+bool column3d_t2_supported(const StencilParams& p, const float* in0, const float* in1);
+cudaError_t launch_column3d_t2(const StencilParams& p, const float* in0, const float* in1, float* out,
+                               cudaStream_t stream, std::string* err);
+
 // K6 — all n steps of stencil_iterate for a few-plane 3D radius-1 star grid
 // (weighted / Hotspot3D) with the grid resident in shared memory (one tile
 // per SM, one cooperative launch, grid barrier per step).

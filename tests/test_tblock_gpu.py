@@ -244,3 +244,78 @@ def test_k2ra_acoustic13_1024_whole_grid(lift):
         del bufs
     assert res[1][2] == "k2ra_sweep"
     assert torch.equal(res[0][0], res[1][0]) and torch.equal(res[0][1], res[1][1])
+
+
+# ------------------------------------------------------------------ K2CT ----
+# Two Hotspot3D steps per launch for few-plane grids (whole-column tiles, the
+# slid box with two halo rows/columns, X_{t+1} through registers into the
+# same shared box; reindexing pads).
+
+def hs_spec(extents, kind):
+    kind = (kind,) * 3 if isinstance(kind, int) else tuple(kind)
+    return si.StencilSpec(tuple(extents), (3, 3, 3), (1, 1, 1), (1, 1, 1), (1, 1, 1), kind, 0.0,
+                          si.HOTSPOT3D, None, si.params_hotspot3d())
+
+
+def hs_run(lift, sp, T, P, steps, tb, env=None):
+    old = {}
+    for k, v in (env or {}).items():
+        old[k] = os.environ.get(k)
+        os.environ[k] = v
+    try:
+        plan = lift.Plan.from_spec(sp)
+        plan.set_time_block(tb)
+        a = torch.from_numpy(T.copy()).cuda()
+        b = torch.empty_like(a)
+        pw = torch.from_numpy(P).cuda()
+        ri = plan.iterate([a, b], steps, aux=[pw])
+        torch.cuda.synchronize()
+        return (a, b)[ri].cpu().numpy(), plan
+    finally:
+        for k, v in old.items():
+            if v is None:
+                os.environ.pop(k, None)
+            else:
+                os.environ[k] = v
+
+
+HS_SHAPES = [(8, 64, 256), (8, 37, 260), (1, 9, 128), (2, 5, 132), (3, 1, 4), (16, 23, 388), (5, 70, 128),
+             (8, 2, 516)]
+
+
+@pytest.mark.parametrize("kind", [CLAMP, MIRROR, REFLECT, (CLAMP, REFLECT, MIRROR)])
+@pytest.mark.parametrize("shape", HS_SHAPES)
+def test_k2ct_bitwise_equal_single_steps(lift, kind, shape):
+    rng = np.random.default_rng(90)
+    T = rng.uniform(300, 350, size=shape).astype(np.float32)
+    P = rng.uniform(0, 1e-2, size=shape).astype(np.float32)
+    sp = hs_spec(shape, kind)
+    y1, _ = hs_run(lift, sp, T, P, 6, 1)
+    y2, plan = hs_run(lift, sp, T, P, 6, 2)
+    assert plan.time_block == 2 and plan.last_kernel == "k2ct_column"
+    np.testing.assert_array_equal(y2, y1)
+
+
+@pytest.mark.parametrize("ty", ["4", "5"])
+def test_k2ct_tile_heights_and_odd_steps(lift, ty):
+    shape = (8, 41, 260)
+    rng = np.random.default_rng(91)
+    T = rng.uniform(300, 350, size=shape).astype(np.float32)
+    P = rng.uniform(0, 1e-2, size=shape).astype(np.float32)
+    sp = hs_spec(shape, CLAMP)
+    y1, _ = hs_run(lift, sp, T, P, 7, 1)
+    y2, plan = hs_run(lift, sp, T, P, 7, 2, {"LIFT_K2CT_TY": ty})
+    np.testing.assert_array_equal(y2, y1)
+    ref = orc.iterate(sp, [T], [P], 7)[0]
+    assert np.max(np.abs(y2 - ref) / np.abs(ref)) <= TOL10
+
+
+def test_k2ct_hotspot3d_8x512x512_whole_grid(lift):
+    """BASELINE C4a size, 10 steps as 5 K2CT launches: bitwise equal to single steps."""
+    xs, sp = si.make_workload_inputs(si.workload("hotspot3d_8x512x512_x100"))
+    y1, _ = hs_run(lift, sp, xs[0], xs[1], 10, 1)
+    y2, plan = hs_run(lift, sp, xs[0], xs[1], 10, 2)
+    assert plan.last_kernel == "k2ct_column"
+    _, plan = hs_run(lift, sp, xs[0], xs[1], 2, 0)
+    assert plan.time_block == 1 and plan.last_kernel == "k2c_column"     # AUTO: single steps
+    assert np.array_equal(y2, y1)
