@@ -220,6 +220,21 @@ stencil_status stencil_apply_region(stencil_plan plan, const float* const* input
                                     int32_t n_inputs, float* out, int64_t o0_begin,
                                     int64_t o0_end, void* stream);
 
+/* TWO time steps of a WEIGHTED 3D plan in one pass over HBM (the two-step
+ * kernels of stencil_plan_set_time_block: K2R, or K2T for z REFLECT) on
+ * output planes [o0_begin, o0_end): out = S(S(in)) there, bitwise equal to
+ * two stencil_apply_region steps (the first over [o0_begin - pad_lo[0],
+ * o0_end + pad_hi[0])).  in: 1 device pointer, out: a different buffer of the
+ * same layout, both 16-byte aligned.  Slab plans may reach into the ghosts
+ * as far as the first step's input stays inside them: o0_begin >= -(ghost -
+ * 2 pad_lo[0]), o0_end <= n0_local + ghost - 2 pad_hi[0] (deep halos with
+ * two steps per pass).  E_UNSUPPORTED if no two-step kernel
+ * takes the plan (stencil_plan_time_block would return 1 for time block 2);
+ * E_INVALID for a region outside those limits, bad pointers or aliasing;
+ * E_CUDA on launch failure. */
+stencil_status stencil_apply2_region(stencil_plan plan, const float* in, float* out, int64_t o0_begin,
+                                     int64_t o0_end, void* stream);
+
 /*
  * Fused halo put (slab mode, 3D plans on the TMA sweep kernel): like
  * stencil_apply_region, and every output plane z < ghost is ALSO stored to

@@ -8,6 +8,7 @@ tensors, ``slab`` adds the multi-GPU slab decomposition.
 """
 from . import _lib
 from ._lib import (StencilError, stencil_apply, stencil_apply_region, stencil_apply_region_put,  # noqa: F401
+                   stencil_apply2_region,
                    stencil_iterate, stencil_slab_step_fused, stencil_wait_signals,
                    stencil_set_wait_timeout_ms, stencil_device_fault,
                    stencil_last_error, stencil_plan_create, stencil_plan_destroy,

@@ -58,6 +58,7 @@ _set_tb = _sig("stencil_plan_set_time_block", C.c_int, [_P, C.c_int32])
 _tb = _sig("stencil_plan_time_block", C.c_int32, [_P])
 _apply = _sig("stencil_apply", C.c_int, [_P, _FPP, C.c_int32, _P, _P])
 _apply_region = _sig("stencil_apply_region", C.c_int, [_P, _FPP, C.c_int32, _P, C.c_int64, C.c_int64, _P])
+_apply2_region = _sig("stencil_apply2_region", C.c_int, [_P, _P, _P, C.c_int64, C.c_int64, _P])
 _apply_region_put = _sig("stencil_apply_region_put", C.c_int, [_P, _FPP, C.c_int32, _P, C.c_int64, C.c_int64, _P, _P,
                                                               _P, _P, C.c_uint32, _P])
 _slab_step_fused = _sig("stencil_slab_step_fused", C.c_int, [_P, _FPP, C.c_int32, _P, _P, _P, _P, _P, C.c_uint32,
@@ -77,7 +78,7 @@ EXPORTED = ("stencil_plan_create", "stencil_plan_output_extents", "stencil_plan_
             "stencil_plan_set_variant", "stencil_plan_variant", "stencil_plan_last_variant",
             "stencil_plan_set_pad_decay", "stencil_plan_last_kernel",
             "stencil_plan_set_time_block",
-            "stencil_plan_time_block", "stencil_apply", "stencil_apply_region",
+            "stencil_plan_time_block", "stencil_apply", "stencil_apply_region", "stencil_apply2_region",
             "stencil_apply_region_put", "stencil_slab_step_fused", "stencil_wait_signals",
             "stencil_set_wait_timeout_ms", "stencil_device_fault",
             "stencil_iterate", "stencil_run_host", "stencil_plan_destroy", "stencil_status_string",
@@ -178,6 +179,11 @@ def stencil_apply_region(plan: int, inputs: Sequence[int], out: int, o0_begin: i
                          stream: int = 0):
     _check(_apply_region(plan, _ptrs(inputs), len(inputs), C.c_void_p(int(out)), int(o0_begin), int(o0_end),
                          C.c_void_p(int(stream))), "stencil_apply_region")
+
+
+def stencil_apply2_region(plan: int, inp: int, out: int, o0_begin: int, o0_end: int, stream: int = 0):
+    _check(_apply2_region(plan, C.c_void_p(int(inp)), C.c_void_p(int(out)), int(o0_begin), int(o0_end),
+                          C.c_void_p(int(stream))), "stencil_apply2_region")
 
 
 def stencil_apply_region_put(plan: int, inputs: Sequence[int], out: int, o0_begin: int, o0_end: int,

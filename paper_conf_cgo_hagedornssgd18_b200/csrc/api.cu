@@ -573,6 +573,34 @@ stencil_status stencil_apply_region(stencil_plan pl, const float* const* inputs,
   return launch(pl, p, inputs[0], n_inputs > 1 ? inputs[1] : nullptr, out, (cudaStream_t)stream);
 }
 
+stencil_status stencil_apply2_region(stencil_plan pl, const float* in, float* out, int64_t o0_begin, int64_t o0_end,
+                                     void* stream) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  if (!in || !out || in == out) return fail(STENCIL_E_INVALID, "apply2_region: bad or aliasing buffers");
+  if (pl->ndim != 3 || !sweep3d_t2_supported(pl->p))
+    return fail(STENCIL_E_UNSUPPORTED, "apply2_region: no two-step kernel takes this plan");
+  if (!aligned16(in) || !aligned16(out)) return fail(STENCIL_E_INVALID, "apply2_region: buffers must be 16-B aligned");
+  int64_t lo_lim = 0, hi_lim = pl->p.o[0];
+  if (pl->p.slab) {
+    lo_lim = -(int64_t)(pl->p.ghost - 2 * pl->p.lo[0]);
+    hi_lim = pl->p.o[0] + (pl->p.ghost - 2 * pl->p.hi[0]);
+  }
+  if (o0_begin < lo_lim || o0_end > hi_lim || o0_begin > o0_end)
+    return fail(STENCIL_E_INVALID, "apply2_region: region outside the output extents (slab: ghosts minus 2 pads)");
+  if (o0_begin == o0_end) return STENCIL_OK;
+  DeviceGuard g(pl->device);
+  if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+  StencilParams p = pl->p;
+  p.reg0 = o0_begin;
+  p.reg1 = o0_end;
+  std::string err;
+  cudaError_t e = launch_sweep3d_t2(p, in, out, (cudaStream_t)stream, pl->num_sms, &err);
+  pl->last_kernel = g_last_kernel;
+  pl->last_variant = STENCIL_VARIANT_SWEEP3D;
+  if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("two-step launch failed: ") + cudaGetErrorString(e) + " " + err);
+  return STENCIL_OK;
+}
+
 stencil_status stencil_apply_region_put(stencil_plan pl, const float* const* inputs, int32_t n_inputs, float* out,
                                         int64_t o0_begin, int64_t o0_end, float* put_lo, float* put_hi,
                                         uint32_t* sig_lo, uint32_t* sig_hi, uint32_t sig_value, void* stream) {

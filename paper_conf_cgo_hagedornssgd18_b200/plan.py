@@ -145,6 +145,14 @@ class Plan:
                                _stream_handle(stream))
         return out
 
+    def apply2_region(self, x: torch.Tensor, out: torch.Tensor, begin: int, end: int,
+                      stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+        """Two time steps in one pass on output planes [begin, end) (stencil_apply2_region)."""
+        self._check(x, self.alloc_extents, "input")
+        self._check(out, self.out_alloc_extents, "out")
+        L.stencil_apply2_region(self.handle, x.data_ptr(), out.data_ptr(), begin, end, _stream_handle(stream))
+        return out
+
     def iterate(self, state: Sequence[torch.Tensor], n_steps: int, aux: Sequence[torch.Tensor] = (),
                 stream: Optional[torch.cuda.Stream] = None) -> int:
         for i, x in enumerate(list(state) + list(aux)):

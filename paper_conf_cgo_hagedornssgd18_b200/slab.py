@@ -107,7 +107,7 @@ def slab_step(compute: Callable[[int, int], None], exchange_post: Callable[[], l
 
 
 def deep_halo_iterate(n_steps: int, k: int, r: int, n: int, g: int, extension, compute, post, on_comm, join,
-                      acoustic: bool, ri: int, aux=()) -> int:
+                      acoustic: bool, ri: int, aux=(), compute2=None) -> int:
     """The time-step schedule of a slab with ghosts of g = r*k planes (k = 1:
     the plain per-step exchange).  ``compute(src, dst, a, b)`` writes output
     planes [a, b) (slab-local, may reach into the ghosts) of state ``dst`` from
@@ -115,7 +115,11 @@ def deep_halo_iterate(n_steps: int, k: int, r: int, n: int, g: int, extension, c
     indices / tensors and returns its works; ``on_comm`` runs a post on the
     side stream, ``join`` waits for its works; ``extension(e)`` is the output
     range reaching e planes into the ghosts on the sides that have a
-    neighbour.  Returns the index of the newest state."""
+    neighbour.  ``compute2(src, dst, a, b)`` (optional) advances TWO steps in
+    one pass on output planes [a, b) (stencil_apply2_region): a block then runs
+    its steps in pairs — a pair's region is that of its second step, the first
+    step's wider region being implied — and an odd block starts with one
+    single step.  Returns the index of the newest state."""
     first = [ri]
     if k > 1:
         first += [1 - ri] if acoustic else list(aux)
@@ -123,6 +127,27 @@ def deep_halo_iterate(n_steps: int, k: int, r: int, n: int, g: int, extension, c
     t = 0
     while t < n_steps:
         kb = min(k, n_steps - t)
+        if compute2 is not None and kb >= 2:
+            j = 1
+            if kb % 2:                      # odd block: one single extended step first
+                a, b = extension((kb - 1) * r)
+                compute(ri, 1 - ri, a, b)
+                ri = 1 - ri
+                j = 2
+            while j <= kb:
+                dst = 1 - ri
+                if j + 1 < kb:              # steps j, j+1 before the block's last pair
+                    a, b = extension((kb - j - 1) * r)
+                    compute2(ri, dst, a, b)
+                else:                       # the block's last two steps: boundary, (exchange || interior)
+                    src = ri
+                    works = slab_step(lambda a, b: compute2(src, dst, a, b), lambda: post([dst]), n, g,
+                                      on_comm=on_comm)
+                    join(works)
+                ri = dst
+                j += 2
+            t += kb
+            continue
         for j in range(1, kb + 1):
             dst = 1 - ri
             if j < kb:
@@ -253,8 +278,14 @@ class SlabPlan:
         def post(grids):
             return self._post([state[i] if isinstance(i, int) else i for i in grids])
 
+        compute2 = None
+        if op == 0 and self.plan.time_block == 2 and self.r == 1:
+            # weighted 7-point star: two steps per pass (K2R) inside the blocks
+            def compute2(src, dst, a, b):
+                self.plan.apply2_region(state[src], out=state[dst], begin=a, end=b)
+
         return deep_halo_iterate(n_steps, self.depth, self.r, self.n, self.g, self.extension, compute, post,
-                                 self._on_comm, self._join, acoustic, ri, aux)
+                                 self._on_comm, self._join, acoustic, ri, aux, compute2=compute2)
 
 
 def _iterate_fused_impl(slab, state, n_steps, aux, fused, ri, acoustic):
@@ -378,16 +409,26 @@ def virtual_slab_iterate(global_extents, world: int, state_global: Sequence[torc
             ex.fill([b[1 - ri] for b in bufs])
         for k in range(len(aux_global)):
             ex.fill([a[k] for a in auxs])
+    # weighted 7-point star with ghosts >= 2: two steps per pass inside the
+    # blocks, paired as deep_halo_iterate pairs them (SlabPlan.iterate)
+    two = slabs[0].plan.op == 0 and slabs[0].plan.time_block == 2 and slabs[0].r == 1
     t = 0
     while t < n_steps:
         kb = min(depth, n_steps - t)
-        for j in range(1, kb + 1):
+        j = 1
+        while j <= kb:
             dst = 1 - ri
+            pair = two and kb >= 2 and (kb % 2 == 0 or j > 1)
             for s, b, a in zip(slabs, bufs, auxs):
-                ins = (b[dst], b[ri]) if acoustic else (b[ri],) + tuple(a)
-                lo, hi = s.extension((kb - j) * s.r)
-                s.plan.apply_region(*ins, out=b[dst], begin=lo, end=hi)
+                if pair:
+                    lo, hi = s.extension((kb - j - 1) * s.r)
+                    s.plan.apply2_region(b[ri], out=b[dst], begin=lo, end=hi)
+                else:
+                    ins = (b[dst], b[ri]) if acoustic else (b[ri],) + tuple(a)
+                    lo, hi = s.extension((kb - j) * s.r)
+                    s.plan.apply_region(*ins, out=b[dst], begin=lo, end=hi)
             ri = dst
+            j += 2 if pair else 1
         ex.fill([b[ri] for b in bufs])
         if acoustic and depth > 1:
             ex.fill([b[1 - ri] for b in bufs])

@@ -49,7 +49,10 @@ def test_bench_two_ranks_weak_j3d7():
     assert h["bytes_per_neighbour_per_exchange"] == 4 * 512 * 512 * 4
     assert h["exchanges_per_100_time_steps"] == 25 and h["exchange_us"] > 0
     assert d["value"] > 0 and d["e2e"]["value"] > 0
-    assert d["gpu_launches"] == 1 * (100 + 2 * 25)
+    # 25 blocks of 4 steps, each two-step pass (K2R) + the last pair as
+    # boundary low, boundary high and interior passes
+    assert d["gpu_launches"] == 1 * 25 * 4
+    assert d["roofline"]["time_steps_per_launch"] == 2
 
 
 def test_bench_two_ranks_strong_acoustic13_depth1():

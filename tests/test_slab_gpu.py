@@ -189,7 +189,7 @@ DEEP_CASES = {
 }
 
 
-@pytest.mark.parametrize("depth", [2, 4])
+@pytest.mark.parametrize("depth", [2, 3, 4])
 @pytest.mark.parametrize("world", [1, 2, 3])
 @pytest.mark.parametrize("case", list(DEEP_CASES))
 def test_virtual_slab_deep_halo_bitwise(lift, case, world, depth):
@@ -218,3 +218,61 @@ def test_apply_region_into_ghosts_validation(lift):
         s.plan.apply_region(a, out=b, begin=-4, end=s.n)
     with pytest.raises(StencilError):
         s.plan.apply_region(a, out=b, begin=0, end=s.n + 4)
+
+
+# ------------------------------ two steps per pass inside deep-halo blocks ---
+def _j3d7(ext, kind):
+    return si.StencilSpec(tuple(ext), (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (kind,) * 3, 0.0, si.WEIGHTED,
+                          si.weights_j3d7(), ())
+
+
+def test_apply2_region_bitwise_and_limits(lift):
+    """stencil_apply2_region = two apply_region steps (the first over the
+    region widened by the pad) on an unslabbed plan and on a slab reaching into
+    its ghosts; limits and errors."""
+    from paper_conf_cgo_hagedornssgd18_b200 import StencilError
+    from paper_conf_cgo_hagedornssgd18_b200.slab import SlabPlan, _NoExchange
+    sp = _j3d7((40, 40, 136), si.CLAMP)
+    plan = lift.Plan.from_spec(sp)
+    x = torch.from_numpy(si.uniform((40, 40, 136), 120, 0.5, 1.5)).cuda()
+    ref1, ref2 = torch.zeros_like(x), torch.zeros_like(x)
+    plan.apply_region(x, out=ref1, begin=4, end=31)
+    plan.apply_region(ref1, out=ref2, begin=5, end=30)
+    got = torch.zeros_like(x)
+    plan.apply2_region(x, out=got, begin=5, end=30)
+    assert plan.last_kernel == "k2r_sweep"
+    assert torch.equal(got[5:30], ref2[5:30])
+    with pytest.raises(StencilError):
+        plan.apply2_region(x, out=x, begin=0, end=40)              # aliasing
+    with pytest.raises(StencilError):
+        plan.apply2_region(x, out=got, begin=-1, end=40)           # unslabbed: [0, n) only
+    wrap = lift.Plan.from_spec(_j3d7((40, 40, 136), si.WRAP))
+    with pytest.raises(StencilError):
+        wrap.apply2_region(x, out=got, begin=0, end=40)            # no two-step kernel
+    s = SlabPlan((40, 40, 136), 1, 3, size=3, kind="clamp", weights=si.weights_j3d7(), exchange=_NoExchange(),
+                 depth=4)
+    a, b1, b2, c = s.empty().uniform_(), s.empty().zero_(), s.empty().zero_(), s.empty().zero_()
+    s.plan.apply_region(a, out=b1, begin=-3, end=s.n + 3)
+    s.plan.apply_region(b1, out=b2, begin=-2, end=s.n + 2)
+    s.plan.apply2_region(a, out=c, begin=-2, end=s.n + 2)
+    g = s.g
+    assert torch.equal(c[g - 2:g + s.n + 2], b2[g - 2:g + s.n + 2])
+    with pytest.raises(StencilError):
+        s.plan.apply2_region(a, out=c, begin=-3, end=s.n)          # ghost - 2 pads = 2
+
+
+def test_slabplan_two_step_blocks(lift):
+    """SlabPlan.iterate (world 1, depth 4 and 3) runs the weighted 7-point
+    blocks as two-step passes (K2R) and gives the single-plan bits."""
+    from paper_conf_cgo_hagedornssgd18_b200.slab import SlabPlan, _NoExchange
+    x = si.uniform((40, 40, 136), 121, 0.5, 1.5)
+    sp = _j3d7(x.shape, si.CLAMP)
+    for depth, n in ((4, 8), (3, 9)):            # blocks end with a two-step pair
+        ref = single_iterate(lift, sp, [x], [], n)[0]
+        s = SlabPlan(x.shape, 0, 1, size=3, kind="clamp", weights=si.weights_j3d7(), exchange=_NoExchange(),
+                     depth=depth)
+        a, b = s.scatter(torch.from_numpy(x).cuda()), s.empty()
+        ri = s.iterate([a, b], n)
+        torch.cuda.synchronize()
+        assert s.plan.last_kernel == "k2r_sweep"
+        np.testing.assert_array_equal(s.owned((a, b)[ri]).cpu().numpy(), ref)
