@@ -330,6 +330,24 @@ stencil_status stencil_run_host(stencil_plan plan, const float* const* host_stat
                                 int32_t n_aux, int32_t n_steps, float* host_out,
                                 void* stream);
 
+/*
+ * Batched end-to-end entry: n_jobs independent problems of this plan through
+ * one call that overlaps the host->device copy of job j+1 and the
+ * device->host copy of job j-1 with the compute of job j (three plan-owned
+ * device workspace slots; a copy-in, a compute and a copy-out stream ordered
+ * by events; PCIe copies run in both directions at once).  Job j reads
+ * host_state[j * n_state + s] (s < n_state) and host_aux[j * n_aux + a] and
+ * writes its newest grid to host_out[j] — the same computation as
+ * stencil_run_host per job, bitwise.  Host buffers should be pinned for the
+ * copies to overlap (pageable ones serialise them).  Synchronous: returns
+ * when every output is on the host.  E_INVALID for bad buffers or counts
+ * (n_jobs >= 1), else as stencil_run_host.  ACOUSTIC jobs use four device
+ * grids per slot (two steps per pass where K2RA applies).
+ */
+stencil_status stencil_run_host_batch(stencil_plan plan, const float* const* host_state, int32_t n_state,
+                                      const float* const* host_aux, int32_t n_aux, int32_t n_steps,
+                                      int32_t n_jobs, float* const* host_out);
+
 /* Frees the plan (host memory and any stencil_run_host workspace).  Safe once
  * the caller has synchronised the plan's in-flight work. */
 void stencil_plan_destroy(stencil_plan plan);

@@ -16,7 +16,7 @@ from ._lib import (StencilError, stencil_apply, stencil_apply_region, stencil_ap
                    stencil_plan_set_variant, stencil_plan_time_block,
                    stencil_plan_variant, stencil_plan_last_variant, stencil_plan_last_kernel,
                    stencil_plan_set_pad_decay,
-                   stencil_run_host, stencil_status_string,
+                   stencil_run_host, stencil_run_host_batch, stencil_status_string,
                    stencil_version)
 from .plan import Plan  # noqa: F401
 

@@ -68,6 +68,8 @@ _iterate = _sig("stencil_iterate", C.c_int, [_P, _FPP, C.c_int32, _FPP, C.c_int3
 _set_wait_timeout = _sig("stencil_set_wait_timeout_ms", C.c_int, [C.c_uint32])
 _device_fault = _sig("stencil_device_fault", C.c_int, [])
 _run_host = _sig("stencil_run_host", C.c_int, [_P, _FPP, C.c_int32, _FPP, C.c_int32, C.c_int32, _P, _P])
+_run_host_batch = _sig("stencil_run_host_batch", C.c_int, [_P, _FPP, C.c_int32, _FPP, C.c_int32, C.c_int32,
+                                                         C.c_int32, _FPP])
 _destroy = _sig("stencil_plan_destroy", None, [_P])
 _last_kernel = _sig("stencil_plan_last_kernel", C.c_char_p, [_P])
 _status_string = _sig("stencil_status_string", C.c_char_p, [C.c_int])
@@ -81,7 +83,8 @@ EXPORTED = ("stencil_plan_create", "stencil_plan_output_extents", "stencil_plan_
             "stencil_plan_time_block", "stencil_apply", "stencil_apply_region", "stencil_apply2_region",
             "stencil_apply_region_put", "stencil_slab_step_fused", "stencil_wait_signals",
             "stencil_set_wait_timeout_ms", "stencil_device_fault",
-            "stencil_iterate", "stencil_run_host", "stencil_plan_destroy", "stencil_status_string",
+            "stencil_iterate", "stencil_run_host", "stencil_run_host_batch", "stencil_plan_destroy",
+            "stencil_status_string",
             "stencil_last_error", "stencil_version")
 
 
@@ -239,6 +242,17 @@ def stencil_run_host(plan: int, host_state: Sequence[np.ndarray], host_aux: Sequ
     _check(_run_host(plan, _ptrs([a.ctypes.data for a in host_state]), len(host_state),
                      _ptrs([a.ctypes.data for a in host_aux]), len(host_aux), int(n_steps),
                      C.c_void_p(host_out.ctypes.data), C.c_void_p(int(stream))), "stencil_run_host")
+
+
+def stencil_run_host_batch(plan: int, host_state: Sequence[np.ndarray], n_state: int,
+                           host_aux: Sequence[np.ndarray], n_aux: int, n_steps: int, host_out: Sequence[np.ndarray]):
+    """Jobs j = 0..len(host_out)-1: inputs host_state[j*n_state : (j+1)*n_state], aux host_aux[j*n_aux : ...]."""
+    for a in list(host_state) + list(host_aux) + list(host_out):
+        if a.dtype != np.float32 or not a.flags.c_contiguous:
+            raise ValueError("host buffers must be C-contiguous float32")
+    _check(_run_host_batch(plan, _ptrs([a.ctypes.data for a in host_state]), int(n_state),
+                           _ptrs([a.ctypes.data for a in host_aux]), int(n_aux), int(n_steps), len(host_out),
+                           _ptrs([a.ctypes.data for a in host_out])), "stencil_run_host_batch")
 
 
 def stencil_plan_destroy(plan: int):

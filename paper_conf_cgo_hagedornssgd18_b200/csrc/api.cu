@@ -44,6 +44,9 @@ struct stencil_plan_s {
   // stencil_run_host workspace (device)
   std::vector<float*> ws;
   size_t ws_elems = 0;
+  // stencil_run_host_batch workspace: 3 slots x 4 grids
+  std::vector<float*> wsb;
+  size_t wsb_elems = 0;
 };
 
 namespace {
@@ -896,8 +899,125 @@ stencil_status stencil_run_host(stencil_plan pl, const float* const* host_state,
   return STENCIL_OK;
 }
 
+stencil_status stencil_run_host_batch(stencil_plan pl, const float* const* host_state, int32_t n_state,
+                                      const float* const* host_aux, int32_t n_aux, int32_t n_steps,
+                                      int32_t n_jobs, float* const* host_out) {
+  if (!pl) return fail(STENCIL_E_INVALID, "NULL plan");
+  if (!host_state || !host_out || n_state < 1 || n_state > 2 || n_aux < 0 || n_aux > 1 || n_jobs < 1 ||
+      (n_aux > 0 && !host_aux))
+    return fail(STENCIL_E_INVALID, "bad host buffers or counts");
+  for (int32_t j = 0; j < n_jobs; ++j) {
+    if (!host_out[j]) return fail(STENCIL_E_INVALID, "NULL host_out");
+    for (int32_t s = 0; s < n_state; ++s)
+      if (!host_state[j * n_state + s]) return fail(STENCIL_E_INVALID, "NULL host_state");
+    for (int32_t a = 0; a < n_aux; ++a)
+      if (!host_aux[j * n_aux + a]) return fail(STENCIL_E_INVALID, "NULL host_aux");
+  }
+  const StencilParams& p = pl->p;
+  const bool iterable = (p.op == OP_WEIGHTED || p.op == OP_HOTSPOT3D || p.op == OP_ACOUSTIC ||
+                         p.op == OP_HOTSPOT2D || p.op == OP_GRADIENT || p.op == OP_SRAD) && same_extents(p);
+  if (!(iterable && (p.op != OP_ACOUSTIC || n_state == 2)) && n_steps != 1)
+    return fail(STENCIL_E_UNSUPPORTED, "run_host_batch: op is not iterable; use n_steps = 1");
+  DeviceGuard g(pl->device);
+  if (g.err != cudaSuccess) return cuda_fail(g.err, "cudaSetDevice");
+  const size_t in_elems = (size_t)(p.n[0] + 2 * p.ghost) * p.plane;
+  const size_t out_elems = (size_t)(p.o[0] + 2 * p.ghost) * p.o[1] * p.o[2];
+  const size_t elems = in_elems > out_elems ? in_elems : out_elems;
+  constexpr int kSlots = 3, kGrids = 4;     // per slot: state0, state1, aux0 / spare, out / spare
+  if (pl->wsb_elems < elems) {
+    for (float* b : pl->wsb) cudaFree(b);
+    pl->wsb.clear();
+    pl->wsb_elems = 0;
+    for (int i = 0; i < kSlots * kGrids; ++i) {
+      float* b = nullptr;
+      cudaError_t e = cudaMalloc(&b, elems * sizeof(float));
+      if (e != cudaSuccess) return cuda_fail(e, "cudaMalloc (run_host_batch workspace)");
+      pl->wsb.push_back(b);
+    }
+    pl->wsb_elems = elems;
+  }
+  // streams and events of this call
+  cudaStream_t st_in = nullptr, st_comp = nullptr, st_out = nullptr;
+  std::vector<cudaEvent_t> ev_in(n_jobs, nullptr), ev_comp(n_jobs, nullptr), ev_out(n_jobs, nullptr);
+  struct Cleanup {
+    cudaStream_t* s[3];
+    std::vector<cudaEvent_t>* e[3];
+    ~Cleanup() {
+      for (auto* x : s)
+        if (*x) cudaStreamDestroy(*x);
+      for (auto* v : e)
+        for (cudaEvent_t ev : *v)
+          if (ev) cudaEventDestroy(ev);
+    }
+  } cleanup{{&st_in, &st_comp, &st_out}, {&ev_in, &ev_comp, &ev_out}};
+  cudaError_t e = cudaStreamCreateWithFlags(&st_in, cudaStreamNonBlocking);
+  if (e == cudaSuccess) e = cudaStreamCreateWithFlags(&st_comp, cudaStreamNonBlocking);
+  if (e == cudaSuccess) e = cudaStreamCreateWithFlags(&st_out, cudaStreamNonBlocking);
+  for (int32_t j = 0; j < n_jobs && e == cudaSuccess; ++j) {
+    e = cudaEventCreateWithFlags(&ev_in[j], cudaEventDisableTiming);
+    if (e == cudaSuccess) e = cudaEventCreateWithFlags(&ev_comp[j], cudaEventDisableTiming);
+    if (e == cudaSuccess) e = cudaEventCreateWithFlags(&ev_out[j], cudaEventDisableTiming);
+  }
+  if (e != cudaSuccess) return cuda_fail(e, "run_host_batch: streams / events");
+  for (int32_t j = 0; j < n_jobs; ++j) {
+    float* const* slot = pl->wsb.data() + (j % kSlots) * kGrids;
+    // copy in (after the slot's previous job has been copied out)
+    if (j >= kSlots) {
+      e = cudaStreamWaitEvent(st_in, ev_out[j - kSlots], 0);
+      if (e != cudaSuccess) return cuda_fail(e, "run_host_batch: wait");
+    }
+    for (int32_t s = 0; s < n_state; ++s) {
+      e = cudaMemcpyAsync(slot[s], host_state[j * n_state + s], in_elems * sizeof(float), cudaMemcpyHostToDevice,
+                          st_in);
+      if (e != cudaSuccess) return cuda_fail(e, "H2D copy");
+    }
+    for (int32_t a = 0; a < n_aux; ++a) {
+      e = cudaMemcpyAsync(slot[2], host_aux[j * n_aux + a], in_elems * sizeof(float), cudaMemcpyHostToDevice, st_in);
+      if (e != cudaSuccess) return cuda_fail(e, "H2D copy");
+    }
+    e = cudaEventRecord(ev_in[j], st_in);
+    if (e == cudaSuccess) e = cudaStreamWaitEvent(st_comp, ev_in[j], 0);
+    if (e != cudaSuccess) return cuda_fail(e, "run_host_batch: events");
+    // compute
+    const float* result = nullptr;
+    if (iterable && (p.op != OP_ACOUSTIC || n_state == 2)) {
+      float* state[4] = {slot[0], slot[1], slot[2], slot[3]};
+      const float* aux[1] = {slot[2]};
+      int32_t ri = 0;
+      const int ns = p.op == OP_ACOUSTIC ? 4 : 2;
+      stencil_status s = stencil_iterate(pl, state, ns, aux, n_aux, n_steps, st_comp, &ri);
+      if (s != STENCIL_OK) return s;
+      result = state[ri];
+    } else {
+      const float* in[2] = {slot[0], n_state > 1 ? slot[1] : (n_aux ? slot[2] : nullptr)};
+      stencil_status s = stencil_apply(pl, in, op_arity(p.op), slot[3], st_comp);
+      if (s != STENCIL_OK) return s;
+      result = slot[3];
+    }
+    e = cudaEventRecord(ev_comp[j], st_comp);
+    if (e == cudaSuccess) e = cudaStreamWaitEvent(st_out, ev_comp[j], 0);
+    if (e != cudaSuccess) return cuda_fail(e, "run_host_batch: events");
+    // copy out
+    e = cudaMemcpyAsync(host_out[j], result, out_elems * sizeof(float), cudaMemcpyDeviceToHost, st_out);
+    if (e != cudaSuccess) return cuda_fail(e, "D2H copy");
+    e = cudaEventRecord(ev_out[j], st_out);
+    if (e != cudaSuccess) return cuda_fail(e, "run_host_batch: events");
+    // the next job's compute must not overwrite this slot before its copy-out:
+    // slots are reused only kSlots jobs later, after ev_out (copy-in waits)
+  }
+  e = cudaStreamSynchronize(st_out);
+  if (e == cudaSuccess) e = cudaStreamSynchronize(st_comp);
+  if (e == cudaSuccess) e = cudaStreamSynchronize(st_in);
+  if (e != cudaSuccess) return cuda_fail(e, "stream synchronize");
+  return STENCIL_OK;
+}
+
 void stencil_plan_destroy(stencil_plan pl) {
   if (!pl) return;
+  if (!pl->wsb.empty()) {
+    DeviceGuard g(pl->device);
+    for (float* b : pl->wsb) cudaFree(b);
+  }
   if (!pl->ws.empty() || pl->srad_ws) {
     DeviceGuard g(pl->device);
     for (float* b : pl->ws) cudaFree(b);

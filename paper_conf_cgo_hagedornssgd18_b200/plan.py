@@ -176,6 +176,34 @@ class Plan:
         L.stencil_run_host(self.handle, list(host_state), list(host_aux), n_steps, out, _stream_handle(stream))
         return out
 
+    def run_host_batch(self, jobs: Sequence[Sequence[np.ndarray]], n_steps: int = 1,
+                       aux: Sequence[Sequence[np.ndarray]] = (), outs: Optional[Sequence[np.ndarray]] = None):
+        """Independent jobs (each a list of host state grids, plus its aux grids)
+        with copy-in / compute / copy-out overlapped across jobs
+        (stencil_run_host_batch); returns the list of output arrays."""
+        n_in = int(np.prod(self.alloc_extents))
+        n_out = int(np.prod(self.out_alloc_extents))
+        if outs is None:
+            outs = [np.empty(self.out_alloc_extents, np.float32) for _ in jobs]
+        if len(outs) != len(jobs) or (aux and len(aux) != len(jobs)):
+            raise ValueError("run_host_batch: one output (and aux list) per job")
+        n_state = len(jobs[0])
+        n_aux = len(aux[0]) if aux else 0
+        flat, flat_aux = [], []
+        for j, st in enumerate(jobs):
+            if len(st) != n_state or (aux and len(aux[j]) != n_aux):
+                raise ValueError("run_host_batch: every job needs the same number of grids")
+            for a in list(st) + (list(aux[j]) if aux else []):
+                if np.asarray(a).size != n_in:
+                    raise ValueError(f"run_host_batch: input of {np.asarray(a).size} elements, plan needs {n_in}")
+            flat += list(st)
+            flat_aux += list(aux[j]) if aux else []
+        for o in outs:
+            if o.size != n_out:
+                raise ValueError(f"run_host_batch: out has {o.size} elements, plan writes {n_out}")
+        L.stencil_run_host_batch(self.handle, flat, n_state, flat_aux, n_aux, n_steps, list(outs))
+        return list(outs)
+
     def close(self):
         if getattr(self, "handle", None):
             L.stencil_plan_destroy(self.handle)

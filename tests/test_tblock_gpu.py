@@ -319,3 +319,31 @@ def test_k2ct_hotspot3d_8x512x512_whole_grid(lift):
     _, plan = hs_run(lift, sp, xs[0], xs[1], 2, 0)
     assert plan.time_block == 1 and plan.last_kernel == "k2c_column"     # AUTO: single steps
     assert np.array_equal(y2, y1)
+
+
+# ------------------------------------------------------- run_host_batch ----
+@pytest.mark.parametrize("case", ["j3d7", "acoustic7", "hotspot"])
+def test_run_host_batch_matches_run_host(lift, case):
+    """stencil_run_host_batch: every job's output equals stencil_run_host's
+    (bitwise), with jobs of different inputs, more jobs than workspace slots."""
+    rng = np.random.default_rng(130)
+    if case == "j3d7":
+        shape = (20, 40, 136)
+        sp = spec(shape, CLAMP)
+        jobs = [[rng.uniform(0.5, 1.5, size=shape).astype(np.float32)] for _ in range(5)]
+        aux = ()
+    elif case == "acoustic7":
+        shape = (12, 30, 132)
+        sp = ac_spec(shape, 7)
+        jobs = [[rng.uniform(-1, 1, size=shape).astype(np.float32) for _ in range(2)] for _ in range(5)]
+        aux = ()
+    else:
+        shape = (8, 30, 128)
+        sp = hs_spec(shape, CLAMP)
+        jobs = [[rng.uniform(300, 350, size=shape).astype(np.float32)] for _ in range(5)]
+        aux = [[rng.uniform(0, 1e-2, size=shape).astype(np.float32)] for _ in range(5)]
+    plan = lift.Plan.from_spec(sp)
+    outs = plan.run_host_batch(jobs, 6, aux)
+    for j in range(5):
+        ref = plan.run_host(jobs[j], n_steps=6, host_aux=aux[j] if aux else ())
+        np.testing.assert_array_equal(outs[j], ref)
