@@ -103,30 +103,36 @@ class ClockSampler:
         self.samples = []
         self.stop = threading.Event()
         self.t = threading.Thread(target=self.run, daemon=True)
-
-    def run_nvml(self):
-        import pynvml as nv
-        nv.nvmlInit()
+        # NVML is initialised here, before the timed region (nvmlInit can take
+        # longer than a short timed region: the sampler thread would start late)
+        self.nv = self.h = None
         try:
+            import pynvml as nv
+            nv.nvmlInit()
             vis = os.environ.get("CUDA_VISIBLE_DEVICES")
             idx = int(vis.split(",")[self.idx]) if vis and vis.split(",")[self.idx].isdigit() else self.idx
-            h = nv.nvmlDeviceGetHandleByIndex(idx)
-            mx = nv.nvmlDeviceGetMaxClockInfo(h, nv.NVML_CLOCK_SM)
-            bits = [0x8, 0x40, 0x20, 0x4]    # hw_slowdown, hw_thermal, sw_thermal, sw_power_cap
-            while not self.stop.is_set():
-                sm = nv.nvmlDeviceGetClockInfo(h, nv.NVML_CLOCK_SM)
-                rs = nv.nvmlDeviceGetCurrentClocksEventReasons(h)
-                self.samples.append([str(sm), str(mx)] + ["Active" if rs & b else "Not Active" for b in bits])
-                self.stop.wait(0.02)
-        finally:
-            nv.nvmlShutdown()
+            self.h = nv.nvmlDeviceGetHandleByIndex(idx)
+            self.mx = nv.nvmlDeviceGetMaxClockInfo(self.h, nv.NVML_CLOCK_SM)
+            self.nv = nv
+        except Exception:
+            self.nv = None
+
+    def sample_nvml(self):
+        nv, h = self.nv, self.h
+        bits = [0x8, 0x40, 0x20, 0x4]    # hw_slowdown, hw_thermal, sw_thermal, sw_power_cap
+        sm = nv.nvmlDeviceGetClockInfo(h, nv.NVML_CLOCK_SM)
+        rs = nv.nvmlDeviceGetCurrentClocksEventReasons(h)
+        self.samples.append([str(sm), str(self.mx)] + ["Active" if rs & b else "Not Active" for b in bits])
 
     def run(self):
-        try:
-            self.run_nvml()
-            return
-        except Exception:
-            pass
+        if self.nv is not None:
+            try:
+                while not self.stop.is_set():
+                    self.sample_nvml()
+                    self.stop.wait(0.02)
+                return
+            except Exception:
+                pass
         while not self.stop.is_set():
             try:
                 r = subprocess.run(["nvidia-smi", "-i", str(self.idx), f"--query-gpu={self.Q}",
@@ -143,8 +149,20 @@ class ClockSampler:
         return self
 
     def __exit__(self, *a):
+        # one more sample at the end of the timed region (before the sync's
+        # return lets the clocks drop), then stop
+        if self.nv is not None:
+            try:
+                self.sample_nvml()
+            except Exception:
+                pass
         self.stop.set()
         self.t.join(timeout=10)
+        if self.nv is not None:
+            try:
+                self.nv.nvmlShutdown()
+            except Exception:
+                pass
 
     def summary(self):
         if not self.samples:
