@@ -872,6 +872,44 @@ def main():
                "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": int(res_h.numel()) * 4, "ms_per_step": te,
                "timing": "CUDA events, max over ranks, pinned host buffers"}
 
+    # ---- the same workload with one step per pass (temporal
+    # blocking raises Gpts/s above the per-sweep HBM roofline, so the per-sweep
+    # rate and its bandwidth fraction are reported beside it)
+    single_step = None
+    if tb == 2 and not slabbed and iterable:
+        p1 = lift.Plan.from_spec(spec, device=local)
+        p1.set_time_block(1)
+        st1 = [torch.empty_like(x) for x in state]
+        for a_, b_ in zip(st1, state):
+            a_.copy_(b_)
+
+        def step1():
+            return p1.iterate(st1, steps_per_iter, aux)
+        side = torch.cuda.Stream()
+        side.wait_stream(torch.cuda.current_stream())
+        with torch.cuda.stream(side):
+            step1()
+        torch.cuda.current_stream().wait_stream(side)
+        g1 = torch.cuda.CUDAGraph()
+        with torch.cuda.graph(g1):
+            step1()
+        for _ in range(max(1, args.warmup)):
+            g1.replay()
+        torch.cuda.synchronize()
+        f0, f1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        f0.record(stream)
+        for _ in range(args.steps):
+            g1.replay()
+        f1.record(stream)
+        torch.cuda.synchronize()
+        t1_ms = f0.elapsed_time(f1)
+        launch1 = t1_ms * 1e-3 / (args.steps * steps_per_iter)
+        single_step = {"value": npts_local * steps_per_iter * args.steps / (t1_ms * 1e-3) / 1e9,
+                       "ms_per_step": t1_ms / args.steps, "kernel": p1.last_kernel,
+                       "roofline_frac": npts_local * bpp / launch1 / 1e9 / peak,
+                       "avg_launch_us": launch1 * 1e6}
+        del st1, g1
+
     # ---- cpu baseline: the oracle on a bounded sample (rank 0, N=1 only)
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu:
@@ -924,6 +962,7 @@ def main():
             "cpu_baseline": cpu,
             "halo": halo,
             "hot": hot,
+            "single_step": single_step,
             "e2e": e2e,
             "gpu_launches": int(args.steps * launches_per_step),
             "clocks": clocks,
