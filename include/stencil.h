@@ -172,8 +172,11 @@ stencil_status stencil_plan_set_slab(stencil_plan plan, int64_t z_offset,
  * REFLECT); the result is bitwise identical to single steps (an odd step
  * count ends with one single step).  1 forces one step per pass.  0 (the
  * default, AUTO) takes two steps per pass exactly where K2R applies (J3D7
- * 512^3: ~1.5x the single-step rate), and for ACOUSTIC with
- * zero padding where K2RA applies (iterate with four state buffers).  Returns
+ * 512^3: ~1.5x the single-step rate), and for the 7-point
+ * ACOUSTIC update with zero padding where K2RA applies (iterate with four
+ * state buffers).  2 also forces K2RA for the 13-point update and K2CT (two
+ * Hotspot3D steps per launch of a few-plane grid, nz <= 16, reindexing pads),
+ * which measured no faster than single steps and are not in AUTO.  Returns
  * STENCIL_E_INVALID for steps outside 0..2.  stencil_plan_time_block returns
  * the steps per pass iterate will use (1 or 2). */
 stencil_status stencil_plan_set_time_block(stencil_plan plan, int32_t steps);
@@ -341,8 +344,10 @@ stencil_status stencil_run_host(stencil_plan plan, const float* const* host_stat
  * stencil_run_host per job, bitwise.  Host buffers should be pinned for the
  * copies to overlap (pageable ones serialise them).  Synchronous: returns
  * when every output is on the host.  E_INVALID for bad buffers or counts
- * (n_jobs >= 1), else as stencil_run_host.  ACOUSTIC jobs use four device
- * grids per slot (two steps per pass where K2RA applies).
+ * (n_jobs >= 1), else as stencil_run_host.  Device memory: 12 grid-sized
+ * buffers (3 slots x 4 grids), allocated on first use, kept by the plan and
+ * freed by stencil_plan_destroy.  ACOUSTIC jobs use the four grids of a slot
+ * as its state (two steps per pass where K2RA applies).
  */
 stencil_status stencil_run_host_batch(stencil_plan plan, const float* const* host_state, int32_t n_state,
                                       const float* const* host_aux, int32_t n_aux, int32_t n_steps,
