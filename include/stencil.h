@@ -195,7 +195,8 @@ stencil_status stencil_plan_set_pad_decay(stencil_plan plan, float decay);
  * (STENCIL_VARIANT_PERSIST3D after a K4 iterate; GENERIC before any launch). */
 int32_t stencil_plan_last_variant(stencil_plan plan);
 /* The kernel function of the plan's most recent launch within its family
- * ("k2_sweep", "k2c_column", "k2t_sweep", "k1_tile", "k1_srad_fused",
+ * ("k2_sweep", "k2c_column", "k2t_sweep", "k2r_sweep", "k2ra_sweep",
+ * "k2ct_column", "k1_tile", "k1_srad_fused",
  * "k3_wsweep", "k5_gather", "k5_gather (TMA)", "k0_generic", "k4_iterate",
  * "k6_resident"; "none" before any launch).  A static string owned by the
  * library. */
