@@ -943,6 +943,10 @@ stencil_status stencil_run_host_batch(stencil_plan pl, const float* const* host_
     cudaStream_t* s[3];
     std::vector<cudaEvent_t>* e[3];
     ~Cleanup() {
+      // (an early error return must not leave copies into / out of the
+      // caller's host buffers in flight)
+      for (auto* x : s)
+        if (*x) cudaStreamSynchronize(*x);
       for (auto* x : s)
         if (*x) cudaStreamDestroy(*x);
       for (auto* v : e)
