@@ -151,7 +151,7 @@ def _region_compute(spec, gext, rank, world, n, g, inp, out, a, b):
     out[g + a:g + b] = torch.from_numpy(Y.astype(np.float32))
 
 
-def _deep_worker(rank, world, port, kind, size, steps, depth, q):
+def _deep_worker(rank, world, port, kind, size, steps, depth, q, two=False):
     from paper_conf_cgo_hagedornssgd18_b200.slab import deep_halo_iterate
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
@@ -188,7 +188,18 @@ def _deep_worker(rank, world, port, kind, size, steps, depth, q):
             for w in works:
                 w.wait()
 
-        ri = deep_halo_iterate(steps, depth, r, n, g, extension, compute, post, lambda f: f(), join, False, 0)
+        def compute2(src, dst, a, b):
+            # two steps over [a, b): the first over the region widened by r,
+            # except at a global non-periodic edge (there the intermediate grid
+            # is padded instead), as stencil_apply2_region does
+            tmp = torch.zeros_like(bufs[0])
+            a1 = a if (a == 0 and lo_nb is None) else a - r
+            b1 = b if (b == n and hi_nb is None) else b + r
+            _region_compute(spec, gext, rank, world, n, g, bufs[src], tmp, a1, b1)
+            _region_compute(spec, gext, rank, world, n, g, tmp, bufs[dst], a, b)
+
+        ri = deep_halo_iterate(steps, depth, r, n, g, extension, compute, post, lambda f: f(), join, False, 0,
+                               compute2=compute2 if two else None)
         q.put((rank, z0, bufs[ri][g:g + n].numpy().copy(), len(posts)))
     finally:
         dist.destroy_process_group()
@@ -206,6 +217,33 @@ def test_gloo_deep_halo_matches_global_oracle(world, kind, size, depth):
     q = ctx.Queue()
     port = _free_port()
     procs = [ctx.Process(target=_deep_worker, args=(r, world, port, kind, size, steps, depth, q))
+             for r in range(world)]
+    for p in procs:
+        p.start()
+    res = sorted(q.get(timeout=240) for _ in range(world))
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    got = np.concatenate([r[2] for r in res], 0)
+    gext = (23, 6, 8)
+    ref = orc.iterate(_spec(gext, kind, size), [si.uniform(gext, 2025, 0.5, 1.5)], [], steps, round_fp32=True)[0]
+    np.testing.assert_array_equal(got, ref.astype(np.float32))
+    assert all(r[3] == -(-steps // depth) + 1 for r in res)
+
+
+@pytest.mark.parametrize("depth", [2, 3, 4])
+@pytest.mark.parametrize("world,kind,size", [(2, si.CLAMP, 3), (3, si.WRAP, 3), (2, si.MIRROR, 5)])
+def test_gloo_deep_halo_two_step_pairs_match_global_oracle(world, kind, size, depth):
+    """The deep-halo schedule with two-step passes (compute2: the pairing used
+    with stencil_apply2_region on the GPU — pairs of steps over the second
+    step's region, an odd block starting with one single step, the block's
+    last pair split into boundary / exchange || interior): bit-for-bit the
+    oracle's global iterate, same exchange count."""
+    steps = 7
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_deep_worker, args=(r, world, port, kind, size, steps, depth, q, True))
              for r in range(world)]
     for p in procs:
         p.start()
