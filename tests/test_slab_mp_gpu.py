@@ -62,6 +62,11 @@ class StagedExchange:
 
 
 def _case(name):
+    if name == "j3d7_clamp":          # two-step passes (K2R) inside the deep-halo blocks
+        ext = (26, 40, 136)
+        sp = si.StencilSpec(ext, (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.CLAMP,) * 3, 0.0, si.WEIGHTED,
+                            si.weights_j3d7(), ())
+        return sp, [si.uniform(ext, 94, 0.5, 1.5)], []
     if name == "j3d7_wrap":
         ext = (24, 40, 136)
         sp = si.StencilSpec(ext, (3,) * 3, (1,) * 3, (1,) * 3, (1,) * 3, (si.WRAP,) * 3, 0.0, si.WEIGHTED,
@@ -111,7 +116,8 @@ def _worker(rank, world, port, name, steps, q, depth=1):
 
 @pytest.mark.parametrize("name,world,depth", [("j3d7_wrap", 2, 1), ("j3d7_wrap", 3, 1), ("j3d13_mirror", 2, 1),
                                               ("acoustic13", 3, 1), ("j3d7_wrap", 2, 2), ("j3d7_wrap", 3, 4),
-                                              ("j3d13_mirror", 2, 2), ("acoustic13", 2, 2)])
+                                              ("j3d13_mirror", 2, 2), ("acoustic13", 2, 2), ("j3d7_clamp", 2, 2),
+                                              ("j3d7_clamp", 3, 3), ("j3d7_clamp", 2, 4)])
 def test_multiprocess_slab_bitwise(name, world, depth):
     """depth k > 1: deep halos (r*k ghost planes every k steps); the number of
     exchanges per rank is ceil(6/k) + 1 (the first fills the initial ghosts)."""
