@@ -16,6 +16,16 @@ torch.distributed.run (the driver's launch line) and fails if fewer than N
 GPUs are visible.  Inputs (512 MiB per grid) are larger than L2 (126 MB), so
 no L2 flush is needed between timed iterations.
 
+Iterated workloads use the plan's AUTO time blocking (--time-block 0): the
+7-point weighted star (J3D7) and the 7-point Acoustic update advance two time
+steps per pass (K2R / K2RA, bitwise equal to single steps); --time-block 1
+forces one step per pass, and the line's "single_step" object reports that
+rate and its HBM fraction beside the headline.  roofline.time_steps_per_launch
+says how many time steps one launch's algorithmic bytes cover.  "e2e" is the
+batched end-to-end call (stencil_run_host_batch: one job per bench step with
+its own host->device input copy and device->host result copy, the copies of
+neighbouring jobs overlapped with compute).
+
 Other workloads (--workload, stencil_inputs.WORKLOAD_NAMES): the remaining
 BASELINE.json configs (gauss5_8192_mirror, j2d5_256_clamp,
 hotspot3d_8x512x512[_x100], srad1_4096, srad2_4096, srad_iter_4096,
