@@ -567,6 +567,25 @@ __device__ __forceinline__ float ac_comb(const AcConst& a, float s, float uc, fl
   }
 }
 
+// x-edge tiles whose rows and planes are interior: K = 4R + Kx per lane
+// element, so the update's K-dependent factors are per-lane constants
+// (computed once per item with acoustic_combine's own operations)
+struct AcLane {
+  float a[4], ncf2[4], cf1[4];     // 2 - l2*K, -cf2, cf1
+};
+
+template <int R>
+__device__ __forceinline__ float ac_comb_x(const AcConst& a, const AcLane& L, int e, float s, float uc,
+                                           float prev) {
+  const float a_e = e == 0 ? L.a[0] : (e == 1 ? L.a[1] : (e == 2 ? L.a[2] : L.a[3]));
+  const float n_e = e == 0 ? L.ncf2[0] : (e == 1 ? L.ncf2[1] : (e == 2 ? L.ncf2[2] : L.ncf2[3]));
+  const float c_e = e == 0 ? L.cf1[0] : (e == 1 ? L.cf1[1] : (e == 2 ? L.cf1[2] : L.cf1[3]));
+  float t = __fmul_rn(a_e, uc);
+  t = __fmaf_rn(a.l2, s, t);
+  t = __fmaf_rn(n_e, prev, t);
+  return __fmul_rn(c_e, t);
+}
+
 // K's y part for global row gy, z part for plane gz (in-domain neighbours)
 template <int R>
 __device__ __forceinline__ int ac_k1(int g, int n) {
@@ -598,14 +617,16 @@ struct HaloA {
 template <int R, int RPW>
 constexpr int halo_rounds() { return (R * (RPW + 2 * R) + 15) / 16; }
 
-template <int R, int RPW, bool EDGE>
+template <int R, int RPW, int MODE>       // 0 interior, 1 x-edge tile (rows / plane interior), 2 general
 __device__ __forceinline__ void ac_plane(const AcConst& a, const float* const (&Cq)[2 * R + 1],
                                          const float* __restrict__ Pq, int lane, int rb0,
                                          const HaloA (&hl)[halo_rounds<R, RPW>()], bool qin, int kzq, int kzo,
                                          int yw, int ny, int kxp,
-                                         bool colin, float4 (&acc)[R][RPW], float4 (&hist)[R][RPW], bool st1,
+                                         bool colin, const AcLane& xl, float4 (&acc)[R][RPW],
+                                         float4 (&hist)[R][RPW], bool st1,
                                          bool fin, bool newacc, float* o1, float* o2, int row_ok, int rowp) {
   constexpr int J = RPW + 2 * R;
+  constexpr bool EDGE = MODE == 2;
   // ---- halo lanes: X1 at columns x0-R+k and x0+128+k, rows 0..J-1 ----
   constexpr int NR = halo_rounds<R, RPW>();
   float hcen[NR], hv[NR];
@@ -676,12 +697,18 @@ __device__ __forceinline__ void ac_plane(const AcConst& a, const float* const (&
       for (int k = 1; k <= R; ++k) sm = __fadd_rn(sm, f4e(win[R + k], e));
 #pragma unroll
       for (int k = 0; k < R; ++k) sm = __fadd_rn(sm, f4e(zs[R + k], e));
-      const int K = EDGE ? ky + ((kxp >> (4 * e)) & 15) : 0;
-      f4s(v, e, ac_comb<R, !EDGE>(a, sm, f4e(c, e), f4e(pv, e), K));
+      if constexpr (MODE == 1) {
+        f4s(v, e, ac_comb_x<R>(a, xl, e, sm, f4e(c, e), f4e(pv, e)));
+      } else {
+        const int K = EDGE ? ky + ((kxp >> (4 * e)) & 15) : 0;
+        f4s(v, e, ac_comb<R, !EDGE>(a, sm, f4e(c, e), f4e(pv, e), K));
+      }
     }
     if constexpr (EDGE) {
       const int gy = yw - R + j;
       if (!(qin && colin && gy >= 0 && gy < ny)) v = make_float4(0.f, 0.f, 0.f, 0.f);
+    } else if constexpr (MODE == 1) {
+      if (!colin) v = make_float4(0.f, 0.f, 0.f, 0.f);     // ragged tile: columns past nx
     }
     s1[j] = v;
 #pragma unroll
@@ -714,7 +741,9 @@ __device__ __forceinline__ void ac_plane(const AcConst& a, const float* const (&
       float4 v;
 #pragma unroll
       for (int e = 0; e < 4; ++e)
-        f4s(v, e, ac_comb<R, !EDGE>(a, f4e(sm, e), f4e(uc, e), f4e(pr, e), EDGE ? ko + ((kxp >> (4 * e)) & 15) : 0));
+        f4s(v, e, MODE == 1 ? ac_comb_x<R>(a, xl, e, f4e(sm, e), f4e(uc, e), f4e(pr, e))
+                            : ac_comb<R, !EDGE>(a, f4e(sm, e), f4e(uc, e), f4e(pr, e),
+                                                EDGE ? ko + ((kxp >> (4 * e)) & 15) : 0));
       stg128_if(op, v, i < row_ok);
       op += rowp;
     }
@@ -904,6 +933,14 @@ __global__ void __launch_bounds__(384, 1)
       int kxp = 0;
 #pragma unroll
       for (int e = 0; e < 4; ++e) kxp |= ac_k1<R>(xo + e, nx) << (4 * e);
+      AcLane xl;
+#pragma unroll
+      for (int e = 0; e < 4; ++e) {
+        const int K = 4 * R + ((kxp >> (4 * e)) & 15);
+        xl.a[e] = __fsub_rn(2.0f, __fmul_rn(p.prm[0], (float)K));
+        xl.ncf2[e] = -(K < 6 * R ? p.prm[2] : 1.0f);
+        xl.cf1[e] = K < 6 * R ? p.prm[1] : 1.0f;
+      }
       const bool rows_int = yw - 2 * R >= 0 && yw + RPW + 2 * R <= ny;      // X1 rows and their K interior
       const bool cols_int = x0 >= R && x0 + RX_TX + R <= nx;
       // halo lanes: X1 at (row hj, column hx), NR rounds of 16 points per side
@@ -949,15 +986,18 @@ __global__ void __launch_bounds__(384, 1)
         const bool st1 = q >= gzs && q < gze;
         const bool fin = q - R >= gzs;
         const bool newacc = q >= gzs && q < gze;
-        const bool fast = rows_int && cols_int && q >= R && q + R < gnz && (q - R >= R || !fin);
+        const bool zint = q >= R && q + R < gnz && (q - R >= R || !fin);   // K's z part is 2R
         float* o1 = ob1 + (int64_t)q * plane;
         float* o2 = ob2 + (int64_t)(q - R) * plane;
-        if (fast)
-          ac_plane<R, RPW, false>(ac, Cq, Pq, lane, rb0, hl, qin, kzq, kzo, yw, ny,
-                                  kxp, colin, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
+        if (rows_int && zint && cols_int)
+          ac_plane<R, RPW, 0>(ac, Cq, Pq, lane, rb0, hl, qin, kzq, kzo, yw, ny,
+                              kxp, colin, xl, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
+        else if (rows_int && zint)
+          ac_plane<R, RPW, 1>(ac, Cq, Pq, lane, rb0, hl, qin, kzq, kzo, yw, ny,
+                              kxp, colin, xl, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
         else
-          ac_plane<R, RPW, true>(ac, Cq, Pq, lane, rb0, hl, qin, kzq, kzo, yw, ny,
-                                 kxp, colin, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
+          ac_plane<R, RPW, 2>(ac, Cq, Pq, lane, rb0, hl, qin, kzq, kzo, yw, ny,
+                              kxp, colin, xl, acc, hist, st1, fin, newacc, o1, o2, row_ok, nx);
         __syncwarp();
         if (lane == 0) {
           mbar_arrive_a(emptyc_a + 8 * cs[0]);
