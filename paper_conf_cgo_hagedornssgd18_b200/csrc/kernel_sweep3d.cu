@@ -343,6 +343,9 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
       // Acoustic: x part of the in-domain neighbour count of the lane's 4
       // outputs, packed 4 bits each (computed once per item)
       int kxp = 0;
+      // and its y part per output row (the z part comes per plane): K = Kz +
+      // Ky + Kx with one add per row instead of 4R compares
+      int kyr[RPW];
       if constexpr (OP == K2_ACOUSTIC) {
 #pragma unroll
         for (int i = 0; i < 4; ++i) {
@@ -350,6 +353,14 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
 #pragma unroll
           for (int o = 1; o <= R; ++o) kxi += (xo + i - o >= 0) + (xo + i + o < nx);
           kxp |= kxi << (4 * i);
+        }
+#pragma unroll
+        for (int jj = 0; jj < RPW; ++jj) {
+          const int gy = y0 + warp * RPW + jj;
+          int k = 0;
+#pragma unroll
+          for (int o = 1; o <= R; ++o) k += (gy - o >= 0) + (gy + o < ny);
+          kyr[jj] = k;
         }
       }
       // float4 offset of the warp's row d - R (d = 0 .. RPW-1+2R) relative to
@@ -492,6 +503,11 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
           zst[2 * R] = zenc(sn);
           const int64_t z = zs + j;                  // local output plane
           const int gz = (int)(p.z_off + z);
+          int kzp = 0;             // Acoustic: z part of K for this output plane
+          if constexpr (OP == K2_ACOUSTIC) {
+#pragma unroll
+            for (int o = 1; o <= R; ++o) kzp += (gz - o >= 0) + (gz + o < (int)p.gnz);
+          }
           if constexpr (FIX_ON_ARRIVAL && EDGE) {
             if (fix) {
               fix_plane(sn, p.z_off + z + R);
@@ -565,13 +581,7 @@ __global__ void __launch_bounds__(NCONS + 32, (!is_box(OP) && (R == 1 || RPW == 
                 for (int k = 1; k <= R; ++k) add4(cr[jj + R + k]);
 #pragma unroll
                 for (int k = 1; k <= R; ++k) add4(zrow(k));
-                const int Kzy = [&] {
-                  int K = 0;
-#pragma unroll
-                  for (int o = 1; o <= R; ++o)
-                    K += (gz - o >= 0) + (gz + o < (int)p.gnz) + (gy - o >= 0) + (gy + o < ny);
-                  return K;
-                }();
+                const int Kzy = kzp + kyr[jj];
                 const float pwv[4] = {pw.x, pw.y, pw.z, pw.w};
                 float rv[4];
                 if (Kzy == 4 * R && kxp == kx_full) {
