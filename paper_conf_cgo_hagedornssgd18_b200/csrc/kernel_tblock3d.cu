@@ -1213,10 +1213,11 @@ cudaError_t launch_acoustic_r2(const StencilParams& p, const float* prev, const 
   const int64_t tiles = (int64_t)ntx * nty;
   const int64_t slots = (int64_t)num_sms * L.ctas_per_sm;
   int64_t zc, n1, zc2, nchunk;
-  // chunks (32, tail 8): the u^n / u^{n-1} halo rows of neighbouring tiles stay
-  // L2 hits when the CTAs in flight keep to a narrower z window (Acoustic-7
-  // 729 -> 744 Gpts/s vs (128, 16))
-  chunk_plan(nz_reg, tiles, slots, "LIFT_K2RA_ZC", "LIFT_K2RA_ZC2", &zc, &n1, &zc2, &nchunk, 32, 8);
+  // chunks (128, tail 16) as K2R: in short runs (32, 8) measured 729 -> 744
+  // Gpts/s, but in the sustained, power-capped bench the fewer recomputed
+  // X1 planes of long chunks win (699 vs 714-716 Gpts/s,
+  // profiles/r02_k2ra_chunks_sustained.txt)
+  chunk_plan(nz_reg, tiles, slots, "LIFT_K2RA_ZC", "LIFT_K2RA_ZC2", &zc, &n1, &zc2, &nchunk);
   const int64_t items = tiles * nchunk;
   if (items > 0x7fffffff) return cudaErrorInvalidConfiguration;
   const int64_t grid = slots < items ? slots : items;
