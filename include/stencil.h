@@ -171,10 +171,11 @@ stencil_status stencil_plan_set_slab(stencil_plan plan, int64_t z_offset,
  * MIRROR / REFLECT and z CLAMP / MIRROR, else the shared-memory K2T for z
  * REFLECT); the result is bitwise identical to single steps (an odd step
  * count ends with one single step).  1 forces one step per pass.  0 (the
- * default, AUTO) takes two steps per pass exactly where K2R applies (J3D7
- * 512^3: ~1.5x the single-step rate), and for the 7-point
- * ACOUSTIC update with zero padding where K2RA applies (iterate with four
- * state buffers).  2 also forces K2RA for the 13-point update and K2CT (two
+ * default, AUTO) takes two steps per pass where K2R applies and the grid
+ * fills the GPU (>= 8 tiles of 128 x 48 per plane with >= 0.9 useful columns
+ * and >= 2048 (plane, tile) pairs; J3D7 512^3: ~1.6x the single-step rate,
+ * 256^3: 1.2x), and likewise for the 7-point ACOUSTIC update
+ * with zero padding where K2RA applies (iterate with four state buffers).  2 also forces K2RA for the 13-point update and K2CT (two
  * Hotspot3D steps per launch of a few-plane grid, nz <= 16, reindexing pads),
  * which measured no faster than single steps and are not in AUTO.  Returns
  * STENCIL_E_INVALID for steps outside 0..2.  stencil_plan_time_block returns

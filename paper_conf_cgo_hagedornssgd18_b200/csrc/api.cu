@@ -516,7 +516,7 @@ int32_t stencil_plan_time_block(stencil_plan pl) {
   // faster than K2C single steps — 6.75 vs 6.53 us per step — so AUTO keeps
   // single steps for it; time block 2 forces it)
   if (pl->time_block == 0)
-    return (pl->ndim == 3 && (sweep3d_r2_supported(pl->p) || acoustic_r2_auto(pl->p))) ? 2 : 1;
+    return (pl->ndim == 3 && (sweep3d_r2_auto(pl->p) || acoustic_r2_auto(pl->p))) ? 2 : 1;
   return (pl->time_block >= 2 && pl->ndim == 3 &&
           (sweep3d_t2_supported(pl->p) || acoustic_r2_supported(pl->p) || hs2))
              ? 2

@@ -1099,6 +1099,40 @@ void chunk_plan(int64_t nz_reg, int64_t tiles, int64_t slots, const char* env_zc
       nchunk = n1 + (nz_reg - n1 * zc + zc2 - 1) / zc2;
     }
   }
+  // too few items to fill the GPU (e.g. J3D7 256^3: 12 tiles x 4 chunks = 48
+  // items for 148 CTAs, 327 Gpts/s): short chunks with a short tail, (16, 4)
+  // or (8, 2) if that gives >= 2 items per CTA (256^3: 764 / 728 Gpts/s vs 648
+  // for single steps, profiles/r02_k2r_256.txt), else ~4 items per CTA
+  if (!ez && !ez2 && tiles * nchunk < 2 * slots && nz_reg > 4) {
+    bool done = false;
+    for (const int64_t c : {16, 8}) {
+      const int64_t t = c / 4;
+      if (c >= nz_reg) continue;
+      const int64_t nsmall = (2 * slots + tiles - 1) / tiles;
+      int64_t a1 = nz_reg / c, a2 = c, nc = (nz_reg + c - 1) / c;
+      if (nsmall * t < nz_reg) {
+        a1 = (nz_reg - nsmall * t) / c;
+        a2 = t;
+        nc = a1 + (nz_reg - a1 * c + t - 1) / t;
+      } else {
+        a1 = nc;
+      }
+      if (tiles * nc >= 2 * slots) {
+        zc = c;
+        n1 = a1;
+        zc2 = a2;
+        nchunk = nc;
+        done = true;
+        break;
+      }
+    }
+    if (!done) {
+      zc = std::min<int64_t>(nz_reg, std::max<int64_t>(4, (work + 4 * slots - 1) / (4 * slots)));
+      nchunk = (nz_reg + zc - 1) / zc;
+      n1 = nchunk;
+      zc2 = zc;
+    }
+  }
   *zc_out = zc;
   *n1_out = n1;
   *zc2_out = zc2;
@@ -1178,10 +1212,27 @@ cudaError_t launch_sweep3d_r2(const StencilParams& p, const float* in, float* ou
 
 namespace lift {
 
+// AUTO time blocking only where the two-step pass fills the GPU with long
+// z-chunks: at least 8 tiles per plane of at least 0.9 useful columns and
+// 2048 (plane, tile) pairs.  Measured J3D7 (profiles/r02_k2r_small.txt,
+// K2R vs single steps, Gpts/s): 512^3 1297 / 820, 256^3 767 / 647 (taken);
+// 192^3 353 / 483 (ragged x), 64x256^2 381 / 425, 512x128^2 534 / 609
+// (3 tiles per plane: short chunks, the recomputed planes dominate) —
+// single steps; 128^3 303 / 252 and 32x512^2 622 / 584 stay on single steps
+// too (small grids; the rule keeps it simple).
+bool two_step_fills(const StencilParams& p, int ty) {
+  const int64_t nx = p.n[2], ny = p.n[1], nz = p.reg1 - p.reg0;
+  const int64_t ntx = (nx + RX_TX - 1) / RX_TX, nty = (ny + ty - 1) / ty;
+  const int64_t tiles = ntx * nty;
+  return tiles >= 8 && nx * 10 >= ntx * RX_TX * 9 && nz * tiles >= 2048;
+}
+
+bool sweep3d_r2_auto(const StencilParams& p) { return sweep3d_r2_supported(p) && two_step_fills(p, 48); }
+
 bool acoustic_r2_auto(const StencilParams& p) {
   // radius 2 (Acoustic-13): measured 487-497 vs 491-522 Gpts/s for single
   // steps (its X1 rows are recomputed 2x per warp), so AUTO keeps single steps
-  return p.radius == 1 && acoustic_r2_supported(p);
+  return p.radius == 1 && acoustic_r2_supported(p) && two_step_fills(p, 32);
 }
 
 bool acoustic_r2_supported(const StencilParams& p) {

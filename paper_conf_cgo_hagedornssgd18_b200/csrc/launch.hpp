@@ -86,6 +86,7 @@ cudaError_t launch_sweep3d_t2(const StencilParams& p, const float* in, float* ou
 // (temporal blocking; x/y CLAMP/MIRROR/REFLECT, z CLAMP/MIRROR); the K2T
 // entry point routes eligible plans here.
 bool sweep3d_r2_supported(const StencilParams& p);
+bool sweep3d_r2_auto(const StencilParams& p);          // the plans AUTO time blocking sends to K2R
 cudaError_t launch_sweep3d_r2(const StencilParams& p, const float* in, float* out, cudaStream_t stream, int num_sms,
                               std::string* err);
 

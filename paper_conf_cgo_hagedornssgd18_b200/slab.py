@@ -390,13 +390,17 @@ class LocalExchange:
 
 
 def virtual_slab_iterate(global_extents, world: int, state_global: Sequence[torch.Tensor], n_steps: int,
-                         aux_global: Sequence[torch.Tensor] = (), depth: int = 1, **plan_kw) -> List[torch.Tensor]:
+                         aux_global: Sequence[torch.Tensor] = (), depth: int = 1, time_block: Optional[int] = None,
+                         **plan_kw) -> List[torch.Tensor]:
     """Run G slabs on the current device (no process group) and return the
     reassembled global state (newest grid last for ACOUSTIC, else [newest]).
     ``depth`` k > 1: deep halos (r*k ghost planes filled every k steps, the
     overlap recomputed; the schedule of deep_halo_iterate in lockstep)."""
     slabs = [SlabPlan(global_extents, r, world, exchange=_NoExchange(), depth=depth, **plan_kw)
              for r in range(world)]
+    if time_block is not None:       # (tests: force two-step passes on grids AUTO keeps single-step)
+        for s in slabs:
+            s.plan.set_time_block(time_block)
     ex = LocalExchange(slabs)
     nst = len(state_global)
     bufs = [[s.scatter(state_global[k]) if k < nst else s.empty() for k in range(2)] for s in slabs]

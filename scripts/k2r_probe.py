@@ -13,7 +13,8 @@ import paper_conf_cgo_hagedornssgd18_b200 as lift  # noqa: E402
 import stencil_inputs as si  # noqa: E402
 
 wl = os.environ.get("K2R_WORKLOAD", "j3d7_512_clamp")
-xs, spec = si.make_workload_inputs(si.workload(wl))
+scale = os.environ.get("K2R_SCALE")          # e.g. 128,128,128: override the extents
+xs, spec = si.make_workload_inputs(si.workload(wl, scale=tuple(int(v) for v in scale.split(",")) if scale else None))
 npts = 1
 for e in spec.extents:
     npts *= e

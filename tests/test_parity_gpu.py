@@ -438,7 +438,9 @@ def test_time_block2_bitwise_equal_single_steps(lift, kind, shape):
 def test_time_block_eligibility(lift):
     # (plan, default AUTO, after set_time_block(2)): AUTO takes two steps per
     # pass exactly where K2R applies (z CLAMP / MIRROR); 2 also takes K2T (z REFLECT)
-    for sp_, auto, exp in [(spec((64, 64, 128), 3, si.weights_j3d7()), 2, 2),
+    # (AUTO also needs a grid that fills the GPU: >= 8 tiles of 128 x 48, >= 2048 (plane, tile) pairs)
+    for sp_, auto, exp in [(spec((128, 256, 512), 3, si.weights_j3d7()), 2, 2),
+                           (spec((64, 64, 128), 3, si.weights_j3d7()), 1, 2),
                            (spec((64, 64, 128), 3, si.weights_j3d7(), (REFLECT, CLAMP, CLAMP)), 1, 2),
                            (spec((64, 64, 128), 3, si.weights_j3d7(), WRAP), 1, 1),
                            (spec((64, 64, 128), 5, si.weights_j3d13()), 1, 1)]:

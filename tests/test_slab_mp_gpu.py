@@ -95,6 +95,8 @@ def _worker(rank, world, port, name, steps, q, depth=1):
         slab = SlabPlan(sp.extents, rank, world, size=sp.size, pad=sp.pad_lo, kind=list(sp.kind),
                         pad_value=sp.pad_value, op=sp.op, weights=sp.weights, params=sp.params,
                         exchange_factory=StagedExchange, depth=depth)
+        if name == "j3d7_clamp":
+            slab.plan.set_time_block(2)           # K2R pairs (AUTO keeps single steps on a grid this small)
         bufs = [slab.scatter(torch.from_numpy(x).cuda()) for x in state]
         if len(bufs) == 1:
             bufs.append(slab.empty())

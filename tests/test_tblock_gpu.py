@@ -219,10 +219,15 @@ def test_k2ra_time_block_1_and_two_buffers(lift):
     assert plan.last_kernel != "k2ra_sweep"
     _, _, plan = ac_run(lift, sp, u, u, 4, 2)
     assert plan.last_kernel != "k2ra_sweep"
-    # AUTO (time block 0): two-step passes for the 7-point update only
+    # AUTO (time block 0): two-step passes for the 7-point update only, on
+    # grids that fill the GPU (>= 8 tiles of 128 x 32, >= 2048 (plane, tile) pairs)
     _, _, plan = ac_run(lift, sp, u, u, 4, 4, tb=0)
+    assert plan.time_block == 1                              # too small for AUTO
+    big = (64, 256, 1024)
+    ub = np.random.default_rng(84).uniform(-1, 1, size=big).astype(np.float32)
+    _, _, plan = ac_run(lift, ac_spec(big, 7), ub, ub, 2, 4, tb=0)
     assert plan.time_block == 2 and plan.last_kernel == "k2ra_sweep"
-    _, _, plan = ac_run(lift, ac_spec(shape, 13), u, u, 4, 4, tb=0)
+    _, _, plan = ac_run(lift, ac_spec(big, 13), ub, ub, 2, 4, tb=0)
     assert plan.time_block == 1 and plan.last_kernel != "k2ra_sweep"
     _, _, plan = ac_run(lift, ac_spec(shape, 13), u, u, 4, 4, tb=2)
     assert plan.time_block == 2 and plan.last_kernel == "k2ra_sweep"
