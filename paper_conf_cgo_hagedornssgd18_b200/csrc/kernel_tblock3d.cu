@@ -87,6 +87,35 @@ __device__ __forceinline__ float star7(const W7& w, float zm, float ym, float xl
   return __fmaf_rn(w.zp, zp, a);
 }
 
+// the same star on two adjacent points in the two lanes of FFMA2 (per-lane
+// rounding identical to FFMA: the same bits), weights broadcast.  K2R uses
+// the packed forms by default: they take half the FMA issue slots of this
+// issue-bound kernel (same-box A/B 1302 -> 1332 Gpts/s J3D7 512^3,
+// profiles/r02_k2r_ffma2_ab.txt); -DLIFT_K2R_SCALAR restores scalar FFMA
+__device__ __forceinline__ float2 star7p(const W7& w, float2 zm, float2 ym, float2 xl, float2 c, float2 xr, float2 yp,
+                                         float2 zp) {
+  float2 a = __ffma2_rn(make_float2(w.zm, w.zm), zm, make_float2(0.0f, 0.0f));
+  a = __ffma2_rn(make_float2(w.ym, w.ym), ym, a);
+  a = __ffma2_rn(make_float2(w.xl, w.xl), xl, a);
+  a = __ffma2_rn(make_float2(w.c, w.c), c, a);
+  a = __ffma2_rn(make_float2(w.xr, w.xr), xr, a);
+  a = __ffma2_rn(make_float2(w.yp, w.yp), yp, a);
+  return __ffma2_rn(make_float2(w.zp, w.zp), zp, a);
+}
+
+__device__ __forceinline__ float2 lo2(const float4& v) { return make_float2(v.x, v.y); }
+__device__ __forceinline__ float2 hi2(const float4& v) { return make_float2(v.z, v.w); }
+__device__ __forceinline__ float2 bc2(float w) { return make_float2(w, w); }
+// fma(w, s, a) on the four points of a lane as two FFMA2
+__device__ __forceinline__ float4 fma4(float w, const float4& s, const float4& a) {
+#ifndef LIFT_K2R_SCALAR
+  const float2 l = __ffma2_rn(bc2(w), lo2(s), lo2(a)), h = __ffma2_rn(bc2(w), hi2(s), hi2(a));
+  return make_float4(l.x, l.y, h.x, h.y);
+#else
+  return make_float4(__fmaf_rn(w, s.x, a.x), __fmaf_rn(w, s.y, a.y), __fmaf_rn(w, s.z, a.z), __fmaf_rn(w, s.w, a.w));
+#endif
+}
+
 __device__ __forceinline__ float4 lds4(const float* base, int row, int lane) {
   return *reinterpret_cast<const float4*>(base + row * RX_BX + 4 + 4 * lane);
 }
@@ -191,10 +220,20 @@ __device__ __forceinline__ void plane_step(const W7& w, const float* __restrict_
       if (j == jlo) ym = ylo_src ? rnext : rcur;      // y = -1 of X_t -> remapped row (0 or 1)
       if (j == jhi) yp = yhi_src ? rprev : rcur;      // y = ny of X_t -> ny-1 or ny-2
     }
+#ifndef LIFT_K2R_SCALAR
+    const float2 lo = star7p(w, make_float2(zm.x, zm.y), make_float2(ym.x, ym.y), make_float2(l, rcur.x),
+                             make_float2(rcur.x, rcur.y), make_float2(rcur.y, rcur.z), make_float2(yp.x, yp.y),
+                             make_float2(zp.x, zp.y));
+    const float2 hi = star7p(w, make_float2(zm.z, zm.w), make_float2(ym.z, ym.w), make_float2(rcur.y, rcur.z),
+                             make_float2(rcur.z, rcur.w), make_float2(rcur.w, r), make_float2(yp.z, yp.w),
+                             make_float2(zp.z, zp.w));
+    s1[j] = make_float4(lo.x, lo.y, hi.x, hi.y);
+#else
     s1[j].x = star7(w, zm.x, ym.x, l, rcur.x, rcur.y, yp.x, zp.x);
     s1[j].y = star7(w, zm.y, ym.y, rcur.x, rcur.y, rcur.z, yp.y, zp.y);
     s1[j].z = star7(w, zm.z, ym.z, rcur.y, rcur.z, rcur.w, yp.z, zp.z);
     s1[j].w = star7(w, zm.w, ym.w, rcur.z, rcur.w, r, yp.w, zp.w);
+#endif
     rprev = rcur;
     rcur = rnext;
   }
@@ -228,24 +267,16 @@ __device__ __forceinline__ void plane_step(const W7& w, const float* __restrict_
     float* op = oprev;
 #pragma unroll
     for (int i = 0; i < RPW; ++i) {
-      float4 v;
-      v.x = __fmaf_rn(w22, s1[i + 1].x, accA[i].x);
-      v.y = __fmaf_rn(w22, s1[i + 1].y, accA[i].y);
-      v.z = __fmaf_rn(w22, s1[i + 1].z, accA[i].z);
-      v.w = __fmaf_rn(w22, s1[i + 1].w, accA[i].w);
+      const float4 v = fma4(w22, s1[i + 1], accA[i]);
       stg128_if(op, v, i < row_ok);
       op += rowp;
     }
   }
+  const float4 zero4 = make_float4(0.0f, 0.0f, 0.0f, 0.0f);
   if (mid) {
     if (first_plane) {      // plane -1 of X_{t+1} is plane 0 (CLAMP / MIRROR in z)
 #pragma unroll
-      for (int i = 0; i < RPW; ++i) {
-        accB[i].x = __fmaf_rn(w4, s1[i + 1].x, 0.0f);
-        accB[i].y = __fmaf_rn(w4, s1[i + 1].y, 0.0f);
-        accB[i].z = __fmaf_rn(w4, s1[i + 1].z, 0.0f);
-        accB[i].w = __fmaf_rn(w4, s1[i + 1].w, 0.0f);
-      }
+      for (int i = 0; i < RPW; ++i) accB[i] = fma4(w4, s1[i + 1], zero4);
     }
     const float w10 = w.ym, w12 = w.xl, w13 = w.c, w14 = w.xr, w16 = w.yp;
 #pragma unroll
@@ -259,6 +290,19 @@ __device__ __forceinline__ void plane_step(const W7& w, const float* __restrict_
       r = lane == 31 ? h[i + 1] : r;
       if constexpr (RAG) r = pr ? pick4r(rex, c) : r;     // x = nx inside the tile
       const float4 ym = s1[i], yp = s1[i + 2];
+#ifndef LIFT_K2R_SCALAR
+      float2 al = __ffma2_rn(bc2(w10), lo2(ym), lo2(accB[i]));
+      float2 ah = __ffma2_rn(bc2(w10), hi2(ym), hi2(accB[i]));
+      al = __ffma2_rn(bc2(w12), make_float2(l, c.x), al);
+      ah = __ffma2_rn(bc2(w12), make_float2(c.y, c.z), ah);
+      al = __ffma2_rn(bc2(w13), lo2(c), al);
+      ah = __ffma2_rn(bc2(w13), hi2(c), ah);
+      al = __ffma2_rn(bc2(w14), make_float2(c.y, c.z), al);
+      ah = __ffma2_rn(bc2(w14), make_float2(c.w, r), ah);
+      al = __ffma2_rn(bc2(w16), lo2(yp), al);
+      ah = __ffma2_rn(bc2(w16), hi2(yp), ah);
+      accA[i] = make_float4(al.x, al.y, ah.x, ah.y);
+#else
       float4 a;
       a.x = __fmaf_rn(w10, ym.x, accB[i].x);
       a.y = __fmaf_rn(w10, ym.y, accB[i].y);
@@ -281,28 +325,20 @@ __device__ __forceinline__ void plane_step(const W7& w, const float* __restrict_
       a.z = __fmaf_rn(w16, yp.z, a.z);
       a.w = __fmaf_rn(w16, yp.w, a.w);
       accA[i] = a;
+#endif
     }
     if (top_plane) {        // plane gnz of X_{t+1} is plane gnz-1 (CLAMP / MIRROR in z)
       float* op = ocur;
 #pragma unroll
       for (int i = 0; i < RPW; ++i) {
-        float4 v;
-        v.x = __fmaf_rn(w22, s1[i + 1].x, accA[i].x);
-        v.y = __fmaf_rn(w22, s1[i + 1].y, accA[i].y);
-        v.z = __fmaf_rn(w22, s1[i + 1].z, accA[i].z);
-        v.w = __fmaf_rn(w22, s1[i + 1].w, accA[i].w);
+        const float4 v = fma4(w22, s1[i + 1], accA[i]);
         stg128_if(op, v, i < row_ok);
         op += rowp;
       }
     }
   }
 #pragma unroll
-  for (int i = 0; i < RPW; ++i) {
-    accB[i].x = __fmaf_rn(w4, s1[i + 1].x, 0.0f);
-    accB[i].y = __fmaf_rn(w4, s1[i + 1].y, 0.0f);
-    accB[i].z = __fmaf_rn(w4, s1[i + 1].z, 0.0f);
-    accB[i].w = __fmaf_rn(w4, s1[i + 1].w, 0.0f);
-  }
+  for (int i = 0; i < RPW; ++i) accB[i] = fma4(w4, s1[i + 1], zero4);
 }
 
 // WS: 12 warps — a producer warpgroup (one lane streams, the group gives its
