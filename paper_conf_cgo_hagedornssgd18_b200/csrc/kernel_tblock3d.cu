@@ -1097,7 +1097,10 @@ LauncherR pick_r() {
   if (v == 203) return get_launcher_r<3, 16, 6, true>();
   if (v == 304) return get_launcher_r<4, 12, 6, true>();
   if (v == 303) return get_launcher_r<3, 12, 6, true>();
-  return get_launcher_r<6, 8, 6, true>();
+  if (v == 1066) return get_launcher_r<6, 8, 6, true>();
+  // default: 6 rows per warp, 7-stage ring (with the FFMA2 stars, 1349 vs
+  // 1334 Gpts/s for 6 stages, profiles/r02_k2r_s7_ab.txt)
+  return get_launcher_r<6, 8, 7, true>();
 }
 
 // z-chunks (items are (chunk, tile), chunk-major) of the two-step kernels:
